@@ -1,0 +1,141 @@
+/*
+ * hj.h -- C-ABI of the B200-native radix-partitioned hash join (Sioulas et al., ICDE 2019).
+ *
+ * The hot path behind this boundary (every step runs in hand-written sm_100a CUDA kernels):
+ *   a1 radix histogram of the co-partition id p = key & (2^B - 1)      (north star; the paper
+ *      has none)
+ *   a2 device-wide exclusive scan -> partition offsets, pass cursors, pass-2 chunk list, join
+ *      work list
+ *   a3 pass-1 scatter on digit d1 (low ceil(B/2) bits), staged through a shared-memory tile
+ *      so HBM writes are contiguous runs (P:265-275 metadata + shuffle space in smem)
+ *   a4 pass-2 scatter on digit d2 (next floor(B/2) bits), fixed-size chunks of each pass-1
+ *      partition assigned to blocks (bucket-at-a-time analogue)
+ *   a5 work planning: oversized co-partitions split into (R chunk x S chunk) items
+ *      (P:306-308 long chains decomposed; P:1470-1473 block nested loops)
+ *   a6 build a shared-memory chained hash table on the R chunk with atomicExch and 16-bit
+ *      offsets (Listing 2)
+ *   a7 probe with the S chunk following the chains
+ *   a8 aggregate (count + pair checksum) or materialize (r_pay, s_pay) pairs through
+ *      a shared-memory output buffer with one global atomic per flush
+ *
+ * Result definition (identical for every radix_bits):
+ *   J = multiset {(r_pay, s_pay) : r_key == s_key}  (keys compared as unsigned bit patterns,
+ *       every value legal, bag semantics for duplicates on both sides)
+ *   matches  = |J|
+ *   checksum = sum over J of sig(r_pay, s_pay) mod 2^64,
+ *              sig(p, q) = fmix64(p ^ (q * 0x9E3779B97F4A7C15)), payloads zero-extended,
+ *              fmix64 = splitmix64 finalizer.
+ *   The build side is always R as passed (no swap); pairs are (r_pay, s_pay); pair order is
+ *   unspecified (compare after sorting).
+ *
+ * Status codes: every int-returning entry point returns HJ_OK or a negative HJ_ERR_*;
+ * hj_last_error() gives the message of the last failure on that context.
+ */
+#ifndef HJ_H_
+#define HJ_H_
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+typedef struct hj_ctx hj_ctx; /* opaque; not thread-safe; use one per stream / thread */
+
+enum hj_out_mode {
+  HJ_OUT_COUNT_CHECKSUM = 0, /* matches + checksum only (the paper's aggregation) */
+  HJ_OUT_MATERIALIZE = 1     /* also the pairs, SoA r_pay_out[] / s_pay_out[]   */
+};
+
+enum hj_status {
+  HJ_OK = 0,
+  HJ_ERR_INVALID = -1,     /* bad argument (null pointer with n > 0, bad mode, bad width ...) */
+  HJ_ERR_UNSUPPORTED = -2, /* key/payload widths other than 4/4 and 8/8; radix_bits > 20     */
+  HJ_ERR_OOM = -3,         /* device or pinned-host allocation failed                         */
+  HJ_ERR_CUDA = -4,        /* any CUDA runtime error; message in hj_last_error()              */
+  HJ_ERR_COMM = -5         /* reserved for the multi-GPU exchange                             */
+};
+
+enum hj_option {
+  HJ_OPT_CAP_R = 1,        /* max R tuples per join item (shared-memory build capacity C_R);
+                              0 = auto (1.25x the mean R partition, >= 512)                  */
+  HJ_OPT_CHUNK_S = 2,      /* max S tuples per join item (C_S); 0 = auto                      */
+  HJ_OPT_OUT_CAPACITY = 3, /* initial materialization capacity in pairs; 0 = max(nS, 1M)      */
+  HJ_OPT_TIMING = 4,       /* 1 = record per-phase CUDA events into hj_result (default 1)     */
+  HJ_OPT_BLOCKS_PER_SM = 5 /* persistent-grid residency override for the passes (0 = auto)    */
+};
+
+typedef struct hj_result {
+  uint64_t matches;      /* |R ⋈ S| (always filled)                                              */
+  uint64_t checksum;     /* sum of sig(r_pay, s_pay) mod 2^64 (always filled)                    */
+  const void* r_pay_out; /* MATERIALIZE: `matches` payloads of R, pay_bytes each (device memory
+                            for hj_join, pinned host memory for hj_join_host); owned by the ctx,
+                            valid until the next join on this ctx or hj_destroy                   */
+  const void* s_pay_out; /* same, payloads of S                                                  */
+  uint64_t n_items;      /* join work items executed (co-partition x R chunk x S chunk)          */
+  int radix_bits;        /* B actually used                                                      */
+  int passes;            /* partitioning passes (2 for B >= 2)                                   */
+  float ms_total;        /* CUDA-event time of the whole call (first kernel -> result ready)     */
+  float ms_partition;    /* histogram + scan + both passes                                      */
+  float ms_join;         /* build + probe + output                                              */
+} hj_result;
+
+/* Create a context on CUDA device `device` for key/payload widths 4/4 or 8/8 bytes.
+ * cuda_stream: a cudaStream_t to issue all work on (NULL = a ctx-owned non-blocking stream).
+ * Returns HJ_OK and *out, or HJ_ERR_INVALID / HJ_ERR_UNSUPPORTED / HJ_ERR_CUDA. */
+int hj_create(hj_ctx** out, int device, int key_bytes, int pay_bytes, void* cuda_stream);
+
+/* Free every ctx-owned device and host allocation. NULL-safe. */
+void hj_destroy(hj_ctx* ctx);
+
+/* Message of the last failure on ctx ("" if none). NULL ctx -> message of the last hj_create. */
+const char* hj_last_error(const hj_ctx* ctx);
+
+/* Re-target the context to another stream (NULL = the ctx-owned stream). */
+int hj_set_stream(hj_ctx* ctx, void* cuda_stream);
+
+/* Set a tuning / test knob (enum hj_option). Results never depend on knobs. */
+int hj_set_option(hj_ctx* ctx, int option, int64_t value);
+
+/* R ⋈ S on GPU-resident columns. All four column pointers are DEVICE pointers on ctx's device,
+ * caller-owned, read-only, 16-byte alignment recommended (else a scalar-load path is used),
+ * and must stay valid until the call returns. Widths are those given to hj_create.
+ *   radix_bits: B < 0 = auto (mean R partition ~4096 tuples), 0 = one co-partition (pure
+ *               block-nested-loop smem join), 1..20 = 2^B co-partitions in two passes.
+ *   out_mode:   enum hj_out_mode.
+ * Synchronous: returns once *res is valid (matches/checksum copied to the host, pairs in HBM).
+ * nR == 0 or nS == 0 -> HJ_OK with zero results. */
+int hj_join(hj_ctx* ctx,
+            const void* R_keys, const void* R_pay, uint64_t nR,
+            const void* S_keys, const void* S_pay, uint64_t nS,
+            int radix_bits, int out_mode, hj_result* res);
+
+/* Same join from HOST columns (pageable or pinned): copies the inputs host->device on the ctx
+ * stream, runs hj_join's pipeline, and copies the result back (matches/checksum, and for
+ * MATERIALIZE the pairs into ctx-owned pinned host memory returned in res->*_pay_out). */
+int hj_join_host(hj_ctx* ctx,
+                 const void* R_keys, const void* R_pay, uint64_t nR,
+                 const void* S_keys, const void* S_pay, uint64_t nS,
+                 int radix_bits, int out_mode, hj_result* res);
+
+/* Steps a1-a4 alone on one relation (for parity tests and the multi-GPU exchange): radix
+ * partition n device tuples into 2^B co-partitions with the same two passes hj_join uses.
+ * Outputs (ctx-owned, valid until the next call on ctx):
+ *   *tuples_out: device pointer to n AoS tuples (4/4: uint64 = key | pay << 32;
+ *                8/8: {uint64 key; uint64 pay}), co-partition p stored contiguously at
+ *                [part_start[p], part_start[p] + part_count[p]), order inside a partition
+ *                unspecified.
+ *   part_start, part_count: HOST arrays of 2^B entries (caller-allocated), indexed by
+ *                p = key & (2^B - 1).
+ * B must be 0..20. */
+int hj_partition(hj_ctx* ctx, const void* keys, const void* pays, uint64_t n, int radix_bits,
+                 const void** tuples_out, uint64_t* part_start, uint64_t* part_count);
+
+/* Library build string (compile flags, arch). */
+const char* hj_version(void);
+
+#ifdef __cplusplus
+}
+#endif
+
+#endif /* HJ_H_ */

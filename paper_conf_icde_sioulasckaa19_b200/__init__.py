@@ -1,0 +1,266 @@
+"""B200-native radix-partitioned hash join (Sioulas et al., ICDE 2019) -- Python binding.
+
+Argument marshalling only: every step of the join runs in the sm_100a kernels of
+``libhj.so`` behind the C-ABI of ``include/hj.h``. There is no CPU fallback: importing
+this package without the built library raises, and so does calling it without a CUDA
+device. PyTorch supplies device memory and streams.
+
+    import paper_conf_icde_sioulasckaa19_b200 as hj
+    res = hj.join(R_keys, R_pay, S_keys, S_pay, radix_bits=-1, out_mode=hj.OUT_COUNT_CHECKSUM)
+    res.matches, res.checksum                      # python ints (uint64 semantics)
+    res = hj.join(..., out_mode=hj.OUT_MATERIALIZE)
+    res.r_pay, res.s_pay                           # torch CUDA tensors of `matches` payloads
+
+Columns are 1-D contiguous CUDA tensors of 4-byte (int32/uint32 bits) or 8-byte
+(int64/uint64 bits) elements; key and payload widths must match (4/4 or 8/8).
+"""
+from __future__ import annotations
+
+import ctypes
+import dataclasses
+import os
+import threading
+
+import numpy as np
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+LIB_PATH = os.path.join(_HERE, "libhj.so")
+
+OUT_COUNT_CHECKSUM = 0
+OUT_MATERIALIZE = 1
+
+OPT_CAP_R = 1
+OPT_CHUNK_S = 2
+OPT_OUT_CAPACITY = 3
+OPT_TIMING = 4
+OPT_BLOCKS_PER_SM = 5
+
+_ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4: "HJ_ERR_CUDA", -5: "HJ_ERR_COMM"}
+
+# every symbol include/hj.h declares (checked by tests/test_abi.py)
+EXPORTS = ("hj_create", "hj_destroy", "hj_last_error", "hj_set_stream", "hj_set_option", "hj_join",
+           "hj_join_host", "hj_partition", "hj_version")
+
+
+class HJError(RuntimeError):
+    def __init__(self, code: int, msg: str):
+        super().__init__(f"{_ERRORS.get(code, code)}: {msg}")
+        self.code = code
+
+
+class _Result(ctypes.Structure):
+    _fields_ = [("matches", ctypes.c_uint64), ("checksum", ctypes.c_uint64), ("r_pay_out", ctypes.c_void_p),
+                ("s_pay_out", ctypes.c_void_p), ("n_items", ctypes.c_uint64), ("radix_bits", ctypes.c_int),
+                ("passes", ctypes.c_int), ("ms_total", ctypes.c_float), ("ms_partition", ctypes.c_float),
+                ("ms_join", ctypes.c_float)]
+
+
+def _load_lib():
+    if not os.path.exists(LIB_PATH):
+        raise ImportError(f"{LIB_PATH} is missing: build it with `make` or __graft_entry__.build() "
+                          "(there is no CPU fallback)")
+    lib = ctypes.CDLL(LIB_PATH)
+    vp, u64, i32, i64 = ctypes.c_void_p, ctypes.c_uint64, ctypes.c_int, ctypes.c_int64
+    lib.hj_create.argtypes = [ctypes.POINTER(vp), i32, i32, i32, vp]
+    lib.hj_create.restype = i32
+    lib.hj_destroy.argtypes = [vp]
+    lib.hj_destroy.restype = None
+    lib.hj_last_error.argtypes = [vp]
+    lib.hj_last_error.restype = ctypes.c_char_p
+    lib.hj_set_stream.argtypes = [vp, vp]
+    lib.hj_set_stream.restype = i32
+    lib.hj_set_option.argtypes = [vp, i32, i64]
+    lib.hj_set_option.restype = i32
+    for f in (lib.hj_join, lib.hj_join_host):
+        f.argtypes = [vp, vp, vp, u64, vp, vp, u64, i32, i32, ctypes.POINTER(_Result)]
+        f.restype = i32
+    lib.hj_partition.argtypes = [vp, vp, vp, u64, i32, ctypes.POINTER(vp), ctypes.POINTER(u64), ctypes.POINTER(u64)]
+    lib.hj_partition.restype = i32
+    lib.hj_version.argtypes = []
+    lib.hj_version.restype = ctypes.c_char_p
+    return lib
+
+
+_lib = _load_lib()
+
+
+def lib():
+    return _lib
+
+
+def version() -> str:
+    return _lib.hj_version().decode()
+
+
+@dataclasses.dataclass
+class JoinResult:
+    matches: int
+    checksum: int
+    r_pay: object = None  # torch tensor (device) or numpy array (host) when materialized
+    s_pay: object = None
+    n_items: int = 0
+    radix_bits: int = 0
+    passes: int = 0
+    ms_total: float = 0.0
+    ms_partition: float = 0.0
+    ms_join: float = 0.0
+
+
+class Context:
+    """One hj_ctx (device, widths). Not thread-safe; the module keeps one per thread."""
+
+    def __init__(self, device: int = 0, key_bytes: int = 4, pay_bytes: int = 4, stream: int | None = None):
+        h = ctypes.c_void_p()
+        rc = _lib.hj_create(ctypes.byref(h), device, key_bytes, pay_bytes, stream)
+        if rc != 0:
+            raise HJError(rc, _lib.hj_last_error(None).decode())
+        self._h = h
+        self.device = device
+        self.key_bytes = key_bytes
+        self.pay_bytes = pay_bytes
+
+    def close(self):
+        if getattr(self, "_h", None):
+            _lib.hj_destroy(self._h)
+            self._h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+    def _check(self, rc):
+        if rc != 0:
+            raise HJError(rc, _lib.hj_last_error(self._h).decode())
+
+    def set_option(self, opt: int, value: int):
+        self._check(_lib.hj_set_option(self._h, opt, int(value)))
+
+    def set_stream(self, stream_handle: int | None):
+        self._check(_lib.hj_set_stream(self._h, stream_handle))
+
+    def join(self, Rk, Rp, Sk, Sp, radix_bits: int = -1, out_mode: int = OUT_COUNT_CHECKSUM) -> JoinResult:
+        import torch
+
+        cols = [_as_device_col(t, self.key_bytes if i % 2 == 0 else self.pay_bytes) for i, t in enumerate((Rk, Rp, Sk, Sp))]
+        if cols[0].numel() != cols[1].numel() or cols[2].numel() != cols[3].numel():
+            raise ValueError("key and payload columns differ in length")
+        self.set_stream(torch.cuda.current_stream(cols[0].device).cuda_stream)
+        res = _Result()
+        rc = _lib.hj_join(self._h, _ptr(cols[0]), _ptr(cols[1]), cols[0].numel(), _ptr(cols[2]), _ptr(cols[3]),
+                          cols[2].numel(), radix_bits, out_mode, ctypes.byref(res))
+        self._check(rc)
+        out = _result(res)
+        if out_mode == OUT_MATERIALIZE and res.matches:
+            out.r_pay = _wrap_device(res.r_pay_out, res.matches, self.pay_bytes, cols[0].device)
+            out.s_pay = _wrap_device(res.s_pay_out, res.matches, self.pay_bytes, cols[0].device)
+        return out
+
+    def join_host(self, Rk, Rp, Sk, Sp, radix_bits: int = -1, out_mode: int = OUT_COUNT_CHECKSUM) -> JoinResult:
+        """End-to-end call from host numpy columns (H2D copies, join, D2H of the result)."""
+        cols = [np.ascontiguousarray(a) for a in (Rk, Rp, Sk, Sp)]
+        for i, a in enumerate(cols):
+            want = self.key_bytes if i % 2 == 0 else self.pay_bytes
+            if a.dtype.itemsize != want:
+                raise ValueError(f"column {i} has {a.dtype.itemsize}-byte elements, expected {want}")
+        self.set_stream(None)
+        res = _Result()
+        rc = _lib.hj_join_host(self._h, _nptr(cols[0]), _nptr(cols[1]), len(cols[0]), _nptr(cols[2]), _nptr(cols[3]),
+                               len(cols[2]), radix_bits, out_mode, ctypes.byref(res))
+        self._check(rc)
+        out = _result(res)
+        if out_mode == OUT_MATERIALIZE and res.matches:
+            dt = np.uint32 if self.pay_bytes == 4 else np.uint64
+            n = res.matches
+            buf_r = (ctypes.c_char * (n * self.pay_bytes)).from_address(res.r_pay_out)
+            buf_s = (ctypes.c_char * (n * self.pay_bytes)).from_address(res.s_pay_out)
+            out.r_pay = np.frombuffer(buf_r, dtype=dt).copy()
+            out.s_pay = np.frombuffer(buf_s, dtype=dt).copy()
+        return out
+
+    def partition(self, keys, pays, radix_bits: int):
+        """Steps a1-a4 on one relation. Returns (tuples, part_start, part_count): tuples is a
+        torch tensor view of the ctx-owned AoS buffer (int64 per 4/4 tuple, or [n, 2] int64 for
+        8/8), valid until the next call on this context."""
+        import torch
+
+        k = _as_device_col(keys, self.key_bytes)
+        p = _as_device_col(pays, self.pay_bytes)
+        self.set_stream(torch.cuda.current_stream(k.device).cuda_stream)
+        np_ = 1 << radix_bits
+        start = (ctypes.c_uint64 * np_)()
+        count = (ctypes.c_uint64 * np_)()
+        out = ctypes.c_void_p()
+        self._check(_lib.hj_partition(self._h, _ptr(k), _ptr(p), k.numel(), radix_bits, ctypes.byref(out), start, count))
+        n = k.numel()
+        tw = self.key_bytes + self.pay_bytes
+        t = _wrap_device(out.value, n * tw // 8, 8, k.device) if n else torch.zeros(0, dtype=torch.int64, device=k.device)
+        if self.key_bytes == 8:
+            t = t.view(n, 2)
+        return t, np.frombuffer(start, dtype=np.uint64).copy(), np.frombuffer(count, dtype=np.uint64).copy()
+
+
+def _result(res: _Result) -> JoinResult:
+    return JoinResult(matches=int(res.matches), checksum=int(res.checksum), n_items=int(res.n_items),
+                      radix_bits=res.radix_bits, passes=res.passes, ms_total=res.ms_total,
+                      ms_partition=res.ms_partition, ms_join=res.ms_join)
+
+
+def _as_device_col(t, width: int):
+    import torch
+
+    if not isinstance(t, torch.Tensor) or not t.is_cuda:
+        raise TypeError("columns must be CUDA tensors (use join_host for host arrays)")
+    if t.dim() != 1 or not t.is_contiguous():
+        raise ValueError("columns must be 1-D contiguous tensors")
+    if t.element_size() != width:
+        raise ValueError(f"column has {t.element_size()}-byte elements, expected {width}")
+    return t
+
+
+def _ptr(t):
+    return ctypes.c_void_p(t.data_ptr()) if t.numel() else None
+
+
+def _nptr(a):
+    return a.ctypes.data_as(ctypes.c_void_p) if a.size else None
+
+
+def _wrap_device(addr: int, n: int, width: int, device):
+    """Non-owning torch view of ctx-owned device memory (valid until the next call on the ctx)."""
+    import torch
+
+    dtype = torch.int32 if width == 4 else torch.int64
+
+    class _CAI:
+        __cuda_array_interface__ = {"shape": (int(n),), "typestr": "<i4" if width == 4 else "<i8",
+                                    "data": (int(addr), False), "version": 3, "strides": None}
+
+    return torch.as_tensor(_CAI(), device=device).view(dtype)
+
+
+_tls = threading.local()
+
+
+def context(device: int = 0, key_bytes: int = 4, pay_bytes: int = 4) -> Context:
+    cache = getattr(_tls, "ctx", None)
+    if cache is None:
+        cache = _tls.ctx = {}
+    key = (device, key_bytes, pay_bytes)
+    if key not in cache:
+        cache[key] = Context(device, key_bytes, pay_bytes)
+    return cache[key]
+
+
+def join(Rk, Rp, Sk, Sp, radix_bits: int = -1, out_mode: int = OUT_COUNT_CHECKSUM) -> JoinResult:
+    """R ⋈ S on CUDA tensors with the thread's cached context for (device, widths)."""
+    return context(Rk.device.index or 0, Rk.element_size(), Rp.element_size()).join(Rk, Rp, Sk, Sp, radix_bits, out_mode)
+
+
+def join_host(Rk, Rp, Sk, Sp, radix_bits: int = -1, out_mode: int = OUT_COUNT_CHECKSUM, device: int = 0) -> JoinResult:
+    return context(device, Rk.dtype.itemsize, Rp.dtype.itemsize).join_host(Rk, Rp, Sk, Sp, radix_bits, out_mode)
+
+
+def partition(keys, pays, radix_bits: int):
+    return context(keys.device.index or 0, keys.element_size(), pays.element_size()).partition(keys, pays, radix_bits)

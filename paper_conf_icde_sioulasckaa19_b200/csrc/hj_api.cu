@@ -1,0 +1,595 @@
+// hj_api.cu -- the C-ABI of include/hj.h: context, workspace, planning of launch shapes and
+// the launch sequence of one join. Single translation unit (kernels in the .cuh headers).
+#include <cuda_runtime.h>
+
+#include <algorithm>
+#include <cstdarg>
+#include <cstdio>
+#include <cstring>
+#include <string>
+
+#include "../../include/hj.h"
+#include "hj_join.cuh"
+#include "hj_partition.cuh"
+
+using namespace hj;
+
+#define HJ_STR2(x) #x
+#define HJ_STR(x) HJ_STR2(x)
+
+namespace {
+
+thread_local std::string g_create_error;
+
+constexpr int PASS_NT = 512;   // threads per partition-pass block
+constexpr int JOIN_NT = 512;   // threads per join block (the paper used 512)
+constexpr int JOIN_SPT = 4;    // S tuples per thread per probe round
+constexpr int HIST_NT = 1024;
+
+struct DevBuf {
+  void* p = nullptr;
+  size_t bytes = 0;
+};
+
+struct Ctx {
+  int device = 0;
+  int key_bytes = 4, pay_bytes = 4;
+  cudaStream_t stream = nullptr;
+  cudaStream_t own_stream = nullptr;
+  int num_sms = 148;
+  size_t smem_optin = 0;
+  std::string err;
+  // options
+  int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0;
+  // workspace
+  DevBuf t1[2], t2[2], meta, out_r, out_s, in[4];
+  void* h_res = nullptr;  // pinned host: results readback
+  void* h_out = nullptr;  // pinned host: materialized pairs (hj_join_host)
+  size_t h_out_bytes = 0;
+  DevBuf part_off_host_dummy;
+  cudaEvent_t ev[4] = {nullptr, nullptr, nullptr, nullptr};
+};
+
+int fail(Ctx* c, int code, const char* fmt, ...) {
+  char buf[512];
+  va_list ap;
+  va_start(ap, fmt);
+  vsnprintf(buf, sizeof buf, fmt, ap);
+  va_end(ap);
+  if (c) c->err = buf;
+  else g_create_error = buf;
+  return code;
+}
+
+#define CUDA_TRY(c, expr)                                                                         \
+  do {                                                                                            \
+    cudaError_t e_ = (expr);                                                                      \
+    if (e_ != cudaSuccess)                                                                        \
+      return fail((c), e_ == cudaErrorMemoryAllocation ? HJ_ERR_OOM : HJ_ERR_CUDA, "%s: %s (%s:%d)", \
+                  #expr, cudaGetErrorString(e_), __FILE__, __LINE__);                             \
+  } while (0)
+
+int ensure(Ctx* c, DevBuf& b, size_t bytes) {
+  if (b.bytes >= bytes && b.p) return HJ_OK;
+  if (b.p) cudaFree(b.p);
+  b.p = nullptr;
+  b.bytes = 0;
+  if (bytes == 0) return HJ_OK;
+  CUDA_TRY(c, cudaMalloc(&b.p, bytes));
+  b.bytes = bytes;
+  return HJ_OK;
+}
+
+size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
+
+int ilog2_ceil(unsigned long long x) {
+  int l = 0;
+  while ((1ull << l) < x) ++l;
+  return l;
+}
+
+// Host-side plan of one call: radix bits, capacities, launch shapes, metadata layout.
+struct HostPlan {
+  int B = 0, b1 = 0, b2 = 0;
+  uint32_t CR = 0, CS = 0, C2 = 0;
+  int lg_nb = 6;
+  size_t join_smem = 0;
+  uint32_t ob_cap = 0;
+  size_t pass_smem = 0;
+  int tile = 0;
+  // metadata offsets (bytes) inside ctx->meta
+  size_t o_cnt[2], o_off[2], o_cur1[2], o_cur2[2], o_cst[2], o_ist, o_counters, o_results;
+  size_t zero_bytes = 0;  // [0, zero_bytes) is memset to 0 per call
+  size_t meta_bytes = 0;
+};
+
+template <typename K>
+constexpr int pass_items() {
+  return sizeof(K) == 4 ? 16 : 8;  // 8192-tuple tiles of 8 B, 4096-tuple tiles of 16 B (64 KB)
+}
+
+int choose_bits(unsigned long long nR) {
+  // mean R co-partition ~4096 tuples: the paper's shared-memory reservation
+  if (nR <= 4096) return 0;
+  int B = ilog2_ceil((nR + 4095) / 4096);
+  return std::min(B, 20);
+}
+
+int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat) {
+  const size_t tb = (size_t)c->key_bytes + c->pay_bytes;  // AoS tuple bytes
+  hp.B = radix_bits < 0 ? choose_bits(nR) : radix_bits;
+  if (hp.B > 20) return fail(c, HJ_ERR_UNSUPPORTED, "radix_bits %d > 20", hp.B);
+  hp.b1 = (hp.B + 1) / 2;
+  hp.b2 = hp.B / 2;
+  hp.tile = PASS_NT * (c->key_bytes == 4 ? pass_items<uint32_t>() : pass_items<uint64_t>());
+  hp.C2 = (uint32_t)hp.tile;
+  const uint32_t F = 1u << std::max(hp.b1, hp.b2);
+  hp.pass_smem = (size_t)hp.tile * tb + (size_t)F * (8 + 4 + 4);
+
+  // join capacities
+  const unsigned long long mean = (nR + (1ull << hp.B) - 1) >> hp.B;
+  size_t cap_max_smem = c->smem_optin ? c->smem_optin : 227 * 1024;
+  uint32_t CR;
+  if (c->opt_cap_r > 0) CR = (uint32_t)std::min<int64_t>(c->opt_cap_r, 65534);
+  else CR = (uint32_t)std::min<unsigned long long>(align_up(mean + mean / 4 + 64, 256), 16384);
+  CR = std::max<uint32_t>(CR, c->opt_cap_r > 0 ? 1 : 512);
+  uint32_t CS;
+  if (c->opt_chunk_s > 0) CS = (uint32_t)std::min<int64_t>(c->opt_chunk_s, 1ll << 30);
+  else CS = std::max<uint32_t>(8 * CR, 32768);
+  int lg_nb = std::max(6, ilog2_ceil(CR) - 1);
+  hp.ob_cap = mat ? 2048 : 0;
+  auto join_smem = [&](uint32_t cr, int lg) {
+    size_t s = (size_t)cr * tb + ((size_t)4 << lg) + (size_t)cr * 2;
+    s = align_up(s, 16) + (size_t)2 * hp.ob_cap * c->pay_bytes;
+    return s;
+  };
+  while (join_smem(CR, lg_nb) > cap_max_smem - 8 * 1024 && CR > 256) {
+    CR /= 2;
+    lg_nb = std::max(6, ilog2_ceil(CR) - 1);
+  }
+  hp.CR = CR;
+  hp.CS = CS;
+  hp.lg_nb = lg_nb;
+  hp.join_smem = join_smem(CR, lg_nb);
+
+  // metadata layout
+  const size_t np = (size_t)1 << hp.B, F1 = (size_t)1 << hp.b1;
+  size_t o = 0;
+  auto take = [&](size_t bytes) {
+    size_t r = o;
+    o = align_up(o + bytes, 256);
+    return r;
+  };
+  // zeroed region first
+  hp.o_counters = take(64);
+  hp.o_results = take(64);
+  hp.o_cnt[0] = take(np * 4);
+  hp.o_cnt[1] = take(np * 4);
+  hp.zero_bytes = o;
+  for (int r = 0; r < 2; ++r) {
+    hp.o_off[r] = take((np + 1) * 8);
+    hp.o_cur1[r] = take(F1 * 8);
+    hp.o_cur2[r] = take(np * 8);
+    hp.o_cst[r] = take((F1 + 1) * 4);
+  }
+  hp.o_ist = take((np + 1) * 4);
+  hp.meta_bytes = o;
+  (void)nS;
+  return HJ_OK;
+}
+
+template <typename K>
+int set_kernel_attrs(Ctx* c) {
+  int rc = 0;
+  auto attr = [&](const void* f) {
+    cudaFuncAttributes fa;
+    if (cudaFuncGetAttributes(&fa, f) != cudaSuccess ||
+        cudaFuncSetAttribute(f, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                             (int)(c->smem_optin - fa.sharedSizeBytes)) != cudaSuccess)
+      rc = -1;
+  };
+  attr((const void*)k_hist<K, true>);
+  attr((const void*)k_pass<K, 1, PASS_NT, pass_items<K>()>);
+  attr((const void*)k_pass<K, 2, PASS_NT, pass_items<K>()>);
+  attr((const void*)k_join<K, JOIN_NT, JOIN_SPT, false>);
+  attr((const void*)k_join<K, JOIN_NT, JOIN_SPT, true>);
+  return rc;
+}
+
+int grid_for(Ctx* c, const void* f, int nt, size_t smem, unsigned long long units) {
+  int per_sm = 0;
+  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, f, nt, smem);
+  if (per_sm < 1) per_sm = 1;
+  if (c->opt_bps > 0) per_sm = std::min<int>(per_sm, (int)c->opt_bps);
+  unsigned long long g = (unsigned long long)per_sm * c->num_sms;
+  if (units < g) g = units;
+  return (int)std::max<unsigned long long>(g, 1);
+}
+
+// Fill the device Plan for one call; rel 1 may be empty (hj_partition).
+Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk,
+                 const void* Sp, unsigned long long nS) {
+  Plan P;
+  memset(&P, 0, sizeof P);
+  char* m = (char*)c->meta.p;
+  const void* ks[2] = {Rk, Sk};
+  const void* ps[2] = {Rp, Sp};
+  const unsigned long long ns[2] = {nR, nS};
+  for (int r = 0; r < 2; ++r) {
+    RelDev& d = P.rel[r];
+    d.keys = ks[r];
+    d.pays = ps[r];
+    d.n = ns[r];
+    d.t1 = c->t1[r].p;
+    d.t2 = c->t2[r].p;
+    d.cnt = (uint32_t*)(m + hp.o_cnt[r]);
+    d.off = (unsigned long long*)(m + hp.o_off[r]);
+    d.cur1 = (unsigned long long*)(m + hp.o_cur1[r]);
+    d.cur2 = (unsigned long long*)(m + hp.o_cur2[r]);
+    d.cst = (uint32_t*)(m + hp.o_cst[r]);
+    P.tiles1[r] = (ns[r] + hp.tile - 1) / hp.tile;
+  }
+  P.B = hp.B;
+  P.b1 = hp.b1;
+  P.b2 = hp.b2;
+  P.C2 = hp.C2;
+  P.CR = hp.CR;
+  P.CS = hp.CS;
+  P.ist = (uint32_t*)(m + hp.o_ist);
+  P.counters = (uint32_t*)(m + hp.o_counters);
+  P.results = (unsigned long long*)(m + hp.o_results);
+  P.out_r = c->out_r.p;
+  P.out_s = c->out_s.p;
+  P.out_cap = c->out_r.bytes / c->pay_bytes;
+  P.lg_nb = hp.lg_nb;
+  return P;
+}
+
+// a1-a4 on the relations of P (both, or R only when nS == 0)
+template <typename K>
+int launch_partition(Ctx* c, const HostPlan& hp, const Plan& P) {
+  cudaStream_t st = c->stream;
+  CUDA_TRY(c, cudaMemsetAsync(c->meta.p, 0, hp.zero_bytes, st));
+  // a1 histogram
+  {
+    const bool smem = hp.B <= 15;
+    const size_t sm = smem ? ((size_t)4 << hp.B) : 0;
+    const unsigned long long nmax = std::max(P.rel[0].n, P.rel[1].n);
+    const void* f = smem ? (const void*)k_hist<K, true> : (const void*)k_hist<K, false>;
+    int g = grid_for(c, f, HIST_NT, sm, (nmax + 4095) / 4096);
+    dim3 grid((unsigned)std::max(1, g / 2), 2);
+    if (smem) k_hist<K, true><<<grid, HIST_NT, sm, st>>>(P);
+    else k_hist<K, false><<<grid, HIST_NT, 0, st>>>(P);
+    CUDA_TRY(c, cudaGetLastError());
+  }
+  // a2 + a5 planner
+  k_plan<<<1, 1024, 0, st>>>(P);
+  CUDA_TRY(c, cudaGetLastError());
+  // a3 pass 1
+  {
+    constexpr int IT = pass_items<K>();
+    const void* f = (const void*)k_pass<K, 1, PASS_NT, IT>;
+    const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.b1) * 16;
+    int g = grid_for(c, f, PASS_NT, sm, P.tiles1[0] + P.tiles1[1]);
+    k_pass<K, 1, PASS_NT, IT><<<g, PASS_NT, sm, st>>>(P, hp.b1);
+    CUDA_TRY(c, cudaGetLastError());
+  }
+  // a4 pass 2
+  {
+    constexpr int IT = pass_items<K>();
+    const void* f = (const void*)k_pass<K, 2, PASS_NT, IT>;
+    const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.b2) * 16;
+    // chunks: at most tiles1 + 2^b1 per relation
+    unsigned long long units = P.tiles1[0] + P.tiles1[1] + 2 * (1ull << hp.b1);
+    int g = grid_for(c, f, PASS_NT, sm, units);
+    k_pass<K, 2, PASS_NT, IT><<<g, PASS_NT, sm, st>>>(P, hp.b2);
+    CUDA_TRY(c, cudaGetLastError());
+  }
+  return HJ_OK;
+}
+
+template <typename K>
+int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
+  cudaStream_t st = c->stream;
+  // upper bound of items: ~(nR/CR + 2^B) * ... ; grid capped by residency
+  const void* f = mat ? (const void*)k_join<K, JOIN_NT, JOIN_SPT, true> : (const void*)k_join<K, JOIN_NT, JOIN_SPT, false>;
+  int g = grid_for(c, f, JOIN_NT, hp.join_smem, 1ull << 40);
+  if (mat) k_join<K, JOIN_NT, JOIN_SPT, true><<<g, JOIN_NT, hp.join_smem, st>>>(P, hp.ob_cap);
+  else k_join<K, JOIN_NT, JOIN_SPT, false><<<g, JOIN_NT, hp.join_smem, st>>>(P, 0);
+  CUDA_TRY(c, cudaGetLastError());
+  return HJ_OK;
+}
+
+int prepare(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat) {
+  int rc = make_plan(c, hp, nR, nS, radix_bits, mat);
+  if (rc) return rc;
+  const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
+  const unsigned long long ns[2] = {nR, nS};
+  for (int r = 0; r < 2; ++r) {
+    if ((rc = ensure(c, c->t1[r], ns[r] * tb))) return rc;
+    if ((rc = ensure(c, c->t2[r], ns[r] * tb))) return rc;
+  }
+  if ((rc = ensure(c, c->meta, hp.meta_bytes))) return rc;
+  if (mat) {
+    unsigned long long cap = c->opt_out_cap > 0 ? (unsigned long long)c->opt_out_cap : std::max<unsigned long long>(nS, 1 << 20);
+    if (c->out_r.bytes < cap * c->pay_bytes) {
+      if ((rc = ensure(c, c->out_r, cap * c->pay_bytes))) return rc;
+      if ((rc = ensure(c, c->out_s, cap * c->pay_bytes))) return rc;
+    }
+  }
+  return HJ_OK;
+}
+
+int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk, const void* Sp,
+             unsigned long long nS, int radix_bits, int out_mode, hj_result* res) {
+  const bool mat = out_mode == HJ_OUT_MATERIALIZE;
+  HostPlan hp;
+  int rc = prepare(c, hp, nR, nS, radix_bits, mat);
+  if (rc) return rc;
+  Plan P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
+  cudaStream_t st = c->stream;
+  const bool timing = c->opt_timing != 0;
+  if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[0], st));
+  if (c->key_bytes == 4) rc = launch_partition<uint32_t>(c, hp, P);
+  else rc = launch_partition<uint64_t>(c, hp, P);
+  if (rc) return rc;
+  if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[1], st));
+  if (c->key_bytes == 4) rc = launch_join<uint32_t>(c, hp, P, mat);
+  else rc = launch_join<uint64_t>(c, hp, P, mat);
+  if (rc) return rc;
+  unsigned long long* h = (unsigned long long*)c->h_res;
+  CUDA_TRY(c, cudaMemcpyAsync(h, P.results, 4 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st));
+  CUDA_TRY(c, cudaMemcpyAsync(h + 4, P.ist + (1ull << hp.B), sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
+  if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[2], st));
+  CUDA_TRY(c, cudaStreamSynchronize(st));
+  unsigned long long matches = h[RES_MATCHES];
+  if (mat && matches > P.out_cap) {
+    // materialization overflow (reading S11): grow to the exact size and re-run only the join
+    if ((rc = ensure(c, c->out_r, matches * c->pay_bytes))) return rc;
+    if ((rc = ensure(c, c->out_s, matches * c->pay_bytes))) return rc;
+    P.out_r = c->out_r.p;
+    P.out_s = c->out_s.p;
+    P.out_cap = matches;
+    CUDA_TRY(c, cudaMemsetAsync(P.results, 0, 4 * sizeof(unsigned long long), st));
+    CUDA_TRY(c, cudaMemsetAsync(P.counters, 0, 8 * sizeof(uint32_t), st));
+    if (c->key_bytes == 4) rc = launch_join<uint32_t>(c, hp, P, mat);
+    else rc = launch_join<uint64_t>(c, hp, P, mat);
+    if (rc) return rc;
+    CUDA_TRY(c, cudaMemcpyAsync(h, P.results, 4 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st));
+    if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[2], st));
+    CUDA_TRY(c, cudaStreamSynchronize(st));
+    matches = h[RES_MATCHES];
+  }
+  memset(res, 0, sizeof *res);
+  res->matches = matches;
+  res->checksum = h[RES_CHECKSUM];
+  res->n_items = (uint32_t)h[4];
+  res->radix_bits = hp.B;
+  res->passes = hp.B >= 2 ? 2 : (hp.B == 1 ? 1 : 0);
+  if (mat) {
+    res->r_pay_out = c->out_r.p;
+    res->s_pay_out = c->out_s.p;
+  }
+  if (timing) {
+    cudaEventElapsedTime(&res->ms_total, c->ev[0], c->ev[2]);
+    cudaEventElapsedTime(&res->ms_partition, c->ev[0], c->ev[1]);
+    cudaEventElapsedTime(&res->ms_join, c->ev[1], c->ev[2]);
+  }
+  return HJ_OK;
+}
+
+int check_args(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk, const void* Sp,
+               unsigned long long nS, int radix_bits, int out_mode) {
+  if (out_mode != HJ_OUT_COUNT_CHECKSUM && out_mode != HJ_OUT_MATERIALIZE)
+    return fail(c, HJ_ERR_INVALID, "bad out_mode %d", out_mode);
+  if (radix_bits > 20) return fail(c, HJ_ERR_UNSUPPORTED, "radix_bits %d > 20", radix_bits);
+  if (nR && (!Rk || !Rp)) return fail(c, HJ_ERR_INVALID, "null R column with nR > 0");
+  if (nS && (!Sk || !Sp)) return fail(c, HJ_ERR_INVALID, "null S column with nS > 0");
+  if (nR >= (1ull << 40) || nS >= (1ull << 40)) return fail(c, HJ_ERR_UNSUPPORTED, "relation too large");
+  return HJ_OK;
+}
+
+}  // namespace
+
+struct hj_ctx {
+  Ctx c;
+};
+
+extern "C" {
+
+const char* hj_version(void) {
+  return "hj-b200 0.1 (sm_100a; nvcc " HJ_STR(__CUDACC_VER_MAJOR__) ")";
+}
+
+int hj_create(hj_ctx** out, int device, int key_bytes, int pay_bytes, void* cuda_stream) {
+  if (!out) return fail(nullptr, HJ_ERR_INVALID, "out is NULL");
+  *out = nullptr;
+  if (!((key_bytes == 4 && pay_bytes == 4) || (key_bytes == 8 && pay_bytes == 8)))
+    return fail(nullptr, HJ_ERR_UNSUPPORTED, "key/payload widths %d/%d (supported: 4/4, 8/8)", key_bytes, pay_bytes);
+  int ndev = 0;
+  cudaError_t e = cudaGetDeviceCount(&ndev);
+  if (e != cudaSuccess || ndev == 0) return fail(nullptr, HJ_ERR_CUDA, "no CUDA device: %s", cudaGetErrorString(e));
+  if (device < 0 || device >= ndev) return fail(nullptr, HJ_ERR_INVALID, "device %d out of range", device);
+  hj_ctx* h = new hj_ctx();
+  Ctx* c = &h->c;
+  c->device = device;
+  c->key_bytes = key_bytes;
+  c->pay_bytes = pay_bytes;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(device);
+  cudaDeviceProp prop;
+  cudaGetDeviceProperties(&prop, device);
+  c->num_sms = prop.multiProcessorCount;
+  c->smem_optin = prop.sharedMemPerBlockOptin;
+  if (prop.major < 10) {
+    cudaSetDevice(prev);
+    delete h;
+    return fail(nullptr, HJ_ERR_UNSUPPORTED, "device %d is sm_%d%d; this library is built for sm_100a", device,
+                prop.major, prop.minor);
+  }
+  int rc = key_bytes == 4 ? set_kernel_attrs<uint32_t>(c) : set_kernel_attrs<uint64_t>(c);
+  e = cudaGetLastError();
+  if (rc || e != cudaSuccess) {
+    cudaSetDevice(prev);
+    delete h;
+    return fail(nullptr, HJ_ERR_CUDA, "kernel attribute setup failed: %s", cudaGetErrorString(e));
+  }
+  if (cudaStreamCreateWithFlags(&c->own_stream, cudaStreamNonBlocking) != cudaSuccess ||
+      cudaMallocHost(&c->h_res, 64) != cudaSuccess) {
+    cudaSetDevice(prev);
+    delete h;
+    return fail(nullptr, HJ_ERR_CUDA, "stream / pinned allocation failed");
+  }
+  c->stream = cuda_stream ? (cudaStream_t)cuda_stream : c->own_stream;
+  for (auto& ev : c->ev) cudaEventCreate(&ev);
+  cudaSetDevice(prev);
+  *out = h;
+  return HJ_OK;
+}
+
+void hj_destroy(hj_ctx* h) {
+  if (!h) return;
+  Ctx* c = &h->c;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  if (c->stream) cudaStreamSynchronize(c->stream);
+  DevBuf* bufs[] = {&c->t1[0], &c->t1[1], &c->t2[0], &c->t2[1], &c->meta, &c->out_r, &c->out_s,
+                    &c->in[0], &c->in[1], &c->in[2], &c->in[3]};
+  for (DevBuf* b : bufs)
+    if (b->p) cudaFree(b->p);
+  if (c->h_res) cudaFreeHost(c->h_res);
+  if (c->h_out) cudaFreeHost(c->h_out);
+  for (auto& ev : c->ev)
+    if (ev) cudaEventDestroy(ev);
+  if (c->own_stream) cudaStreamDestroy(c->own_stream);
+  cudaSetDevice(prev);
+  delete h;
+}
+
+const char* hj_last_error(const hj_ctx* h) { return h ? h->c.err.c_str() : g_create_error.c_str(); }
+
+int hj_set_stream(hj_ctx* h, void* s) {
+  if (!h) return HJ_ERR_INVALID;
+  h->c.stream = s ? (cudaStream_t)s : h->c.own_stream;
+  return HJ_OK;
+}
+
+int hj_set_option(hj_ctx* h, int opt, int64_t v) {
+  if (!h) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  if (v < 0) return fail(c, HJ_ERR_INVALID, "negative option value");
+  switch (opt) {
+    case HJ_OPT_CAP_R: c->opt_cap_r = v; break;
+    case HJ_OPT_CHUNK_S: c->opt_chunk_s = v; break;
+    case HJ_OPT_OUT_CAPACITY: c->opt_out_cap = v; break;
+    case HJ_OPT_TIMING: c->opt_timing = v; break;
+    case HJ_OPT_BLOCKS_PER_SM: c->opt_bps = v; break;
+    default: return fail(c, HJ_ERR_INVALID, "unknown option %d", opt);
+  }
+  return HJ_OK;
+}
+
+int hj_join(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const void* Sk, const void* Sp, uint64_t nS,
+            int radix_bits, int out_mode, hj_result* res) {
+  if (!h || !res) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  int rc = check_args(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode);
+  if (rc) return rc;
+  memset(res, 0, sizeof *res);
+  if (nR == 0 || nS == 0) return HJ_OK;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  rc = run_join(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
+  cudaSetDevice(prev);
+  return rc;
+}
+
+int hj_join_host(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const void* Sk, const void* Sp, uint64_t nS,
+                 int radix_bits, int out_mode, hj_result* res) {
+  if (!h || !res) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  int rc = check_args(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode);
+  if (rc) return rc;
+  memset(res, 0, sizeof *res);
+  if (nR == 0 || nS == 0) return HJ_OK;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  const size_t kb = c->key_bytes, pb = c->pay_bytes;
+  cudaStream_t st = c->stream;
+  const void* src[4] = {Rk, Rp, Sk, Sp};
+  const size_t bytes[4] = {nR * kb, nR * pb, nS * kb, nS * pb};
+  for (int i = 0; i < 4 && rc == HJ_OK; ++i) {
+    rc = ensure(c, c->in[i], bytes[i]);
+    if (rc == HJ_OK && cudaMemcpyAsync(c->in[i].p, src[i], bytes[i], cudaMemcpyHostToDevice, st) != cudaSuccess)
+      rc = fail(c, HJ_ERR_CUDA, "H2D copy failed");
+  }
+  if (rc == HJ_OK)
+    rc = run_join(c, c->in[0].p, c->in[1].p, nR, c->in[2].p, c->in[3].p, nS, radix_bits, out_mode, res);
+  if (rc == HJ_OK && out_mode == HJ_OUT_MATERIALIZE && res->matches) {
+    const size_t need = 2 * res->matches * pb;
+    if (c->h_out_bytes < need) {
+      if (c->h_out) cudaFreeHost(c->h_out);
+      c->h_out = nullptr;
+      c->h_out_bytes = 0;
+      if (cudaMallocHost(&c->h_out, need) != cudaSuccess) rc = fail(c, HJ_ERR_OOM, "pinned host alloc of %zu B", need);
+      else c->h_out_bytes = need;
+    }
+    if (rc == HJ_OK) {
+      char* ho = (char*)c->h_out;
+      if (cudaMemcpyAsync(ho, res->r_pay_out, res->matches * pb, cudaMemcpyDeviceToHost, st) != cudaSuccess ||
+          cudaMemcpyAsync(ho + res->matches * pb, res->s_pay_out, res->matches * pb, cudaMemcpyDeviceToHost, st) !=
+              cudaSuccess ||
+          cudaStreamSynchronize(st) != cudaSuccess)
+        rc = fail(c, HJ_ERR_CUDA, "D2H copy of pairs failed");
+      res->r_pay_out = ho;
+      res->s_pay_out = ho + res->matches * pb;
+    }
+  }
+  cudaSetDevice(prev);
+  return rc;
+}
+
+int hj_partition(hj_ctx* h, const void* keys, const void* pays, uint64_t n, int radix_bits, const void** tuples_out,
+                 uint64_t* part_start, uint64_t* part_count) {
+  if (!h || !tuples_out || !part_start || !part_count) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  if (radix_bits < 0 || radix_bits > 20) return fail(c, HJ_ERR_INVALID, "radix_bits must be 0..20");
+  if (n && (!keys || !pays)) return fail(c, HJ_ERR_INVALID, "null column with n > 0");
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  HostPlan hp;
+  int rc = prepare(c, hp, n, 0, radix_bits, false);
+  if (rc == HJ_OK) {
+    Plan P = device_plan(c, hp, keys, pays, n, nullptr, nullptr, 0);
+    rc = c->key_bytes == 4 ? launch_partition<uint32_t>(c, hp, P) : launch_partition<uint64_t>(c, hp, P);
+    if (rc == HJ_OK) {
+      const size_t np = (size_t)1 << hp.B;
+      unsigned long long* off = new unsigned long long[np + 1];
+      cudaError_t e = cudaMemcpyAsync(off, P.rel[0].off, (np + 1) * 8, cudaMemcpyDeviceToHost, c->stream);
+      if (e == cudaSuccess) e = cudaStreamSynchronize(c->stream);
+      if (e != cudaSuccess) rc = fail(c, HJ_ERR_CUDA, "partition: %s", cudaGetErrorString(e));
+      else {
+        for (size_t q = 0; q < np; ++q) {
+          const size_t d1 = q >> hp.b2, d2 = q & ((1ull << hp.b2) - 1);
+          const size_t p = (d2 << hp.b1) | d1;
+          part_start[p] = off[q];
+          part_count[p] = off[q + 1] - off[q];
+        }
+        *tuples_out = c->t2[0].p;
+      }
+      delete[] off;
+    }
+  }
+  cudaSetDevice(prev);
+  return rc;
+}
+
+}  // extern "C"

@@ -1,0 +1,297 @@
+// hj_partition.cuh -- steps a1-a4 of the hot path:
+//   k_hist   a1: histogram of p = key & (2^B-1) for both relations (shared-memory counters)
+//   k_plan   a2/a5: one-block scan -> co-partition offsets, pass cursors, pass-2 chunk list,
+//            join work list
+//   k_pass   a3 (MODE 1, SoA tiles -> T1 by d1) and a4 (MODE 2, chunks of each pass-1
+//            partition -> T2 by d2)
+//
+// Partitioning follows PAPER.md §III-A: a multi-pass radix partition whose
+// fan-out per pass is bounded by the shared memory holding per-partition metadata and the
+// shuffle space used to make the device-memory writes coalesced. Each pass
+// stages a whole tile in shared memory sorted by digit, then writes every digit's run to a
+// range reserved with one global atomic per (tile, digit) -- the histogram-derived cursors
+// replace the paper's bucket chains (reading D2 in DESIGN.md).
+#pragma once
+#include "hj_common.cuh"
+#include "hj_plan.cuh"
+
+namespace hj {
+
+// ------------------------------------------------------------------------------------------
+// a1: histogram. grid = (blocks_per_rel, 2). Each block counts a contiguous, 16-byte aligned
+// range of one relation's keys in 2^B shared-memory counters (smem atomics measured at ~6
+// tuples/clk/SM on B200, tools/microbench/mb_rank.cu), then merges non-zero counters with
+// one global RED each. For B > 15 (more than 128 KB of counters) SMEM = false counts with
+// global atomics directly (correct, slower; not used by the benchmark configs).
+// ------------------------------------------------------------------------------------------
+template <typename K, bool SMEM>
+__global__ void __launch_bounds__(1024) k_hist(Plan P) {
+  extern __shared__ uint32_t s_hist[];
+  const int rel = blockIdx.y;
+  const RelDev& R = P.rel[rel];
+  const unsigned long long n = R.n;
+  const uint32_t np = 1u << P.B;
+  const uint32_t mask = np - 1;
+  if (SMEM) {
+    for (uint32_t i = threadIdx.x; i < np; i += blockDim.x) s_hist[i] = 0;
+    __syncthreads();
+  }
+  uint32_t* h = SMEM ? s_hist : R.cnt;
+  constexpr int VEC = 16 / sizeof(K);
+  unsigned long long per = (n + gridDim.x - 1) / gridDim.x;
+  per = (per + VEC - 1) / VEC * VEC;
+  const unsigned long long lo = (unsigned long long)blockIdx.x * per;
+  const unsigned long long hi = lo + per < n ? lo + per : n;
+  const K* keys = (const K*)R.keys;
+  if (lo < hi) {
+    const bool aligned = ((reinterpret_cast<uintptr_t>(keys) & 15) == 0);
+    unsigned long long i = lo;
+    if (aligned) {
+      const unsigned long long nvec = (hi - lo) / VEC;
+      const uint4* kv = reinterpret_cast<const uint4*>(keys + lo);
+      for (unsigned long long v = threadIdx.x; v < nvec; v += blockDim.x) {
+        uint4 x = __ldcs(kv + v);  // streaming: keys are read again by pass 1 from HBM anyway
+        const K* e = reinterpret_cast<const K*>(&x);
+        #pragma unroll
+        for (int t = 0; t < VEC; ++t) atomicAdd(&h[(uint32_t)(e[t]) & mask], 1u);
+      }
+      i = lo + nvec * VEC;
+    }
+    for (unsigned long long j = i + threadIdx.x; j < hi; j += blockDim.x) atomicAdd(&h[(uint32_t)keys[j] & mask], 1u);
+  }
+  if (SMEM) {
+    __syncthreads();
+    for (uint32_t i = threadIdx.x; i < np; i += blockDim.x) {
+      uint32_t c = s_hist[i];
+      if (c) atomicAdd(&R.cnt[i], c);
+    }
+  }
+}
+
+// ------------------------------------------------------------------------------------------
+// a2 + a5: the planner. One block of 1024 threads; 2^B <= 2^20 entries per relation.
+//   off[q]  = exclusive scan of cnt[p(q)] in q-order          (co-partition starts, T2)
+//   cur1[d1] = off[d1 << b2], cur2[q] = off[q]                (pass reservation cursors)
+//   cst[d1]  = exclusive scan of ceil(|partition d1| / C2)    (pass-2 chunk list)
+//   ist[q]   = exclusive scan of items(q),  items(q) = ceil(|R_q|/CR) * ceil(|S_q|/CS) if both
+//              non-empty else 0                                (join work list)
+// ------------------------------------------------------------------------------------------
+__device__ __forceinline__ uint32_t q_to_p(uint32_t q, int b1, int b2) {
+  const uint32_t d1 = q >> b2, d2 = q & ((1u << b2) - 1);
+  return (d2 << b1) | d1;
+}
+
+__global__ void __launch_bounds__(1024) k_plan(Plan P) {
+  constexpr int NT = 1024;
+  __shared__ unsigned long long s_tmp[NT / 32 + 1];
+  const uint32_t np = 1u << P.B;
+  const uint32_t F1 = 1u << P.b1;
+  const uint32_t per = (np + NT - 1) / NT;
+  const uint32_t q0 = threadIdx.x * per;
+  const uint32_t q1 = min(q0 + per, np);
+  for (int rel = 0; rel < 2; ++rel) {
+    const RelDev& R = P.rel[rel];
+    unsigned long long local = 0;
+    for (uint32_t q = q0; q < q1; ++q) local += R.cnt[q_to_p(q, P.b1, P.b2)];
+    unsigned long long tot;
+    unsigned long long base = block_exclusive_scan64<NT>(local, s_tmp, &tot);
+    for (uint32_t q = q0; q < q1; ++q) {
+      R.off[q] = base;
+      R.cur2[q] = base;
+      base += R.cnt[q_to_p(q, P.b1, P.b2)];
+    }
+    if (threadIdx.x == 0) R.off[np] = tot;
+    __syncthreads();
+    // pass-2 chunk list over the 2^b1 pass-1 partitions (b1 <= 10 -> at most one per thread)
+    unsigned long long nch = 0;
+    if (threadIdx.x < F1) {
+      const unsigned long long a = R.off[(unsigned long long)threadIdx.x << P.b2];
+      const unsigned long long b = R.off[(unsigned long long)(threadIdx.x + 1) << P.b2];
+      R.cur1[threadIdx.x] = a;
+      nch = (b - a + P.C2 - 1) / P.C2;
+    }
+    unsigned long long cbase = block_exclusive_scan64<NT>(nch, s_tmp, &tot);
+    if (threadIdx.x < F1) R.cst[threadIdx.x] = (uint32_t)cbase;
+    if (threadIdx.x == 0) R.cst[F1] = (uint32_t)tot;
+    __syncthreads();
+  }
+  // join work list
+  {
+    const RelDev& R = P.rel[0];
+    const RelDev& S = P.rel[1];
+    unsigned long long local = 0;
+    for (uint32_t q = q0; q < q1; ++q) {
+      const unsigned long long cr = R.off[q + 1] - R.off[q], cs = S.off[q + 1] - S.off[q];
+      if (cr && cs) local += ((cr + P.CR - 1) / P.CR) * ((cs + P.CS - 1) / P.CS);
+    }
+    unsigned long long tot;
+    unsigned long long base = block_exclusive_scan64<NT>(local, s_tmp, &tot);
+    for (uint32_t q = q0; q < q1; ++q) {
+      P.ist[q] = (uint32_t)base;
+      const unsigned long long cr = R.off[q + 1] - R.off[q], cs = S.off[q + 1] - S.off[q];
+      if (cr && cs) base += ((cr + P.CR - 1) / P.CR) * ((cs + P.CS - 1) / P.CS);
+    }
+    if (threadIdx.x == 0) P.ist[np] = (uint32_t)tot;
+  }
+}
+
+// ------------------------------------------------------------------------------------------
+// a3 / a4: one partition pass. Persistent blocks loop over work units:
+//   MODE 1: unit = a tile of TILE consecutive rows of the SoA input of R or S; digit
+//           d1 = key & (2^b1 - 1); output T1 at cur1[d1] reservations.
+//   MODE 2: unit = chunk k of pass-1 partition d1 (T1[off + k*TILE, ...)); digit
+//           d2 = (key >> b1) & (2^b2 - 1); output T2 at cur2[d1 << b2 | d2] reservations.
+// Per unit: rank every tuple within its digit with a shared-memory atomicAdd (returning the
+// rank), scan the per-digit counts, reserve each digit's run in the output with one global
+// atomicAdd, shuffle the tile into digit order in shared memory, then stream it out so each
+// warp writes consecutive addresses inside a run (P:142-148 coalescing, P:269-272 shuffle
+// space). Every output location is written exactly once; the tile order inside a run is
+// whatever the smem atomics produced (partitions are multisets, reading S9).
+// ------------------------------------------------------------------------------------------
+template <typename K, int MODE, int NT, int ITEMS>
+__global__ void __launch_bounds__(NT, 2) k_pass(Plan P, int fanout_bits) {
+  using TT = Tup<K>;
+  using T = typename TT::T;
+  constexpr int TILE = NT * ITEMS;
+  extern __shared__ __align__(16) unsigned char s_raw[];
+  const uint32_t F = 1u << fanout_bits;
+  T* s_buf = reinterpret_cast<T*>(s_raw);                                        // TILE tuples
+  unsigned long long* s_gb = reinterpret_cast<unsigned long long*>(s_buf + TILE); // F
+  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gb + F);                         // F
+  uint32_t* s_loc = s_cnt + F;                                                     // F
+  __shared__ uint32_t s_tmp[NT / 32 + 1];
+
+  const int b1 = P.b1, b2 = P.b2;
+  const uint32_t dmask = F - 1;
+  const int dshift = (MODE == 1) ? 0 : b1;
+  const uint32_t E = (F + NT - 1) / NT;  // digits per thread in the scan
+
+  for (uint32_t d = threadIdx.x; d < F; d += NT) s_cnt[d] = 0;
+  __syncthreads();
+
+  unsigned long long units0, units1;
+  if (MODE == 1) {
+    units0 = P.tiles1[0];
+    units1 = P.tiles1[1];
+  } else {
+    units0 = P.rel[0].cst[1u << b1];
+    units1 = P.rel[1].cst[1u << b1];
+  }
+  const unsigned long long units = units0 + units1;
+
+  for (unsigned long long u = blockIdx.x; u < units; u += gridDim.x) {
+    const int rel = (u < units0) ? 0 : 1;
+    const RelDev& R = P.rel[rel];
+    const unsigned long long ul = (rel == 0) ? u : u - units0;
+    unsigned long long src0, len;
+    uint32_t d1 = 0;
+    if (MODE == 1) {
+      src0 = ul * TILE;
+      len = min((unsigned long long)TILE, R.n - src0);
+    } else {
+      // chunk -> pass-1 partition d1 by binary search over cst[0..2^b1]
+      uint32_t lo = 0, hi = 1u << b1;  // invariant cst[lo] <= ul < cst[hi]
+      while (hi - lo > 1) {
+        uint32_t mid = (lo + hi) >> 1;
+        if (R.cst[mid] <= ul) lo = mid; else hi = mid;
+      }
+      d1 = lo;
+      const unsigned long long pa = R.off[(unsigned long long)d1 << b2];
+      const unsigned long long pb = R.off[(unsigned long long)(d1 + 1) << b2];
+      src0 = pa + (ul - R.cst[d1]) * TILE;
+      len = min((unsigned long long)TILE, pb - src0);
+    }
+
+    // ---- load + rank ---------------------------------------------------------------------
+    K kk[ITEMS], pp[ITEMS];
+    uint32_t rk[ITEMS];
+    if (MODE == 1) {
+      const K* keys = (const K*)R.keys + src0;
+      const K* pays = (const K*)R.pays + src0;
+      constexpr int VEC = 16 / sizeof(K);
+      const bool vec_ok = (len == TILE) && ((reinterpret_cast<uintptr_t>(keys) & 15) == 0) &&
+                          ((reinterpret_cast<uintptr_t>(pays) & 15) == 0);
+      if (vec_ok) {
+        #pragma unroll
+        for (int j = 0; j < ITEMS / VEC; ++j) {
+          uint4 kv = __ldcs(reinterpret_cast<const uint4*>(keys) + j * NT + threadIdx.x);
+          uint4 pv = __ldcs(reinterpret_cast<const uint4*>(pays) + j * NT + threadIdx.x);
+          const K* ke = reinterpret_cast<const K*>(&kv);
+          const K* pe = reinterpret_cast<const K*>(&pv);
+          #pragma unroll
+          for (int t = 0; t < VEC; ++t) {
+            kk[j * VEC + t] = ke[t];
+            pp[j * VEC + t] = pe[t];
+          }
+        }
+      } else {
+        #pragma unroll
+        for (int j = 0; j < ITEMS; ++j) {
+          // same element->thread map as the vector path: element (j/VEC)*NT*VEC + tid*VEC + j%VEC
+          const unsigned long long e = (unsigned long long)(j / VEC) * NT * VEC + threadIdx.x * VEC + (j % VEC);
+          if (e < len) {
+            kk[j] = keys[e];
+            pp[j] = pays[e];
+          }
+        }
+      }
+      #pragma unroll
+      for (int j = 0; j < ITEMS; ++j) {
+        const unsigned long long e = (unsigned long long)(j / VEC) * NT * VEC + threadIdx.x * VEC + (j % VEC);
+        rk[j] = (e < len) ? atomicAdd(&s_cnt[(uint32_t)(kk[j] >> dshift) & dmask], 1u) : 0xffffffffu;
+      }
+    } else {
+      const T* src = (const T*)R.t1 + src0;
+      #pragma unroll
+      for (int j = 0; j < ITEMS; ++j) {
+        const unsigned long long e = (unsigned long long)j * NT + threadIdx.x;
+        if (e < len) {
+          T t = __ldcs(src + e);
+          kk[j] = TT::key(t);
+          pp[j] = TT::pay(t);
+          rk[j] = atomicAdd(&s_cnt[(uint32_t)(kk[j] >> dshift) & dmask], 1u);
+        } else {
+          rk[j] = 0xffffffffu;
+        }
+      }
+    }
+    __syncthreads();
+
+    // ---- scan digit counts, reserve output runs ---------------------------------------------
+    {
+      const uint32_t d0 = threadIdx.x * E;
+      uint32_t local = 0;
+      for (uint32_t d = d0; d < d0 + E && d < F; ++d) local += s_cnt[d];
+      uint32_t tot;
+      uint32_t base = block_exclusive_scan<NT>(local, s_tmp, &tot);
+      for (uint32_t d = d0; d < d0 + E && d < F; ++d) {
+        const uint32_t c = s_cnt[d];
+        s_loc[d] = base;
+        if (c) {
+          unsigned long long* cur = (MODE == 1) ? &R.cur1[d] : &R.cur2[((unsigned long long)d1 << b2) | d];
+          s_gb[d] = atomicAdd(cur, (unsigned long long)c);
+        }
+        s_cnt[d] = 0;
+        base += c;
+      }
+    }
+    __syncthreads();
+
+    // ---- shuffle into digit order in shared memory ------------------------------------------
+    #pragma unroll
+    for (int j = 0; j < ITEMS; ++j)
+      if (rk[j] != 0xffffffffu) s_buf[s_loc[(uint32_t)(kk[j] >> dshift) & dmask] + rk[j]] = TT::make(kk[j], pp[j]);
+    __syncthreads();
+
+    // ---- stream runs out (consecutive threads -> consecutive addresses within a run) -------
+    T* dst = (T*)((MODE == 1) ? R.t1 : R.t2);
+    for (uint32_t i = threadIdx.x; i < (uint32_t)len; i += NT) {
+      const T t = s_buf[i];
+      const uint32_t d = (uint32_t)(TT::key(t) >> dshift) & dmask;
+      __stcs(dst + s_gb[d] + (i - s_loc[d]), t);
+    }
+    // the next unit rewrites s_loc / s_gb / s_buf only after its own first __syncthreads
+  }
+}
+
+}  // namespace hj

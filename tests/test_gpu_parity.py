@@ -1,0 +1,235 @@
+"""GPU parity: the CUDA path (through the C-ABI) vs the CPU oracle, element by element.
+
+Integer work, so the bar is bit-exact: matches and checksum equal, materialized pairs equal
+after a lexicographic sort (reading S9), partitions equal as multisets. Inputs are the seeded
+generator's (workloads/) or small adversarial arrays; expected values come only from oracle/
+or from the generator's closed forms, never from the CUDA path.
+"""
+import numpy as np
+import pytest
+import torch
+
+import oracle
+import workloads as W
+
+pytestmark = pytest.mark.gpu
+
+M64 = (1 << 64) - 1
+GOLDEN = 0x9E3779B97F4A7C15
+
+
+@pytest.fixture(scope="module")
+def hj():
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_icde_sioulasckaa19_b200 as m
+
+    return m
+
+
+def dev(a: np.ndarray):
+    t = torch.from_numpy(np.ascontiguousarray(a).view(np.int32 if a.dtype.itemsize == 4 else np.int64))
+    return t.cuda()
+
+
+def np_sig(p, q):
+    with np.errstate(over="ignore"):
+        return W.np_fmix64(p.astype(np.uint64) ^ (q.astype(np.uint64) * np.uint64(GOLDEN)))
+
+
+def gpu_join(hj, Rk, Rp, Sk, Sp, bits=-1, mat=False, ctx=None):
+    c = ctx or hj.context(0, Rk.dtype.itemsize, Rp.dtype.itemsize)
+    res = c.join(dev(Rk), dev(Rp), dev(Sk), dev(Sp), radix_bits=bits,
+                 out_mode=hj.OUT_MATERIALIZE if mat else hj.OUT_COUNT_CHECKSUM)
+    torch.cuda.synchronize()
+    return res
+
+
+def to_np(t, width):
+    return t.cpu().numpy().view(np.uint32 if width == 4 else np.uint64)
+
+
+def check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=-1, mat=True, ctx=None):
+    m, c, r, s = oracle.hash_join(Rk, Rp, Sk, Sp, materialize=True)
+    res = gpu_join(hj, Rk, Rp, Sk, Sp, bits, mat=False, ctx=ctx)
+    assert (res.matches, res.checksum) == (m, c), f"count mode bits={bits}"
+    if mat:
+        res = gpu_join(hj, Rk, Rp, Sk, Sp, bits, mat=True, ctx=ctx)
+        assert (res.matches, res.checksum) == (m, c), f"materialize mode bits={bits}"
+        if m:
+            w = Rp.dtype.itemsize
+            got = oracle.pairs_sorted(to_np(res.r_pay, w), to_np(res.s_pay, w))
+            assert np.array_equal(got, oracle.pairs_sorted(r, s))
+    return res
+
+
+def adversarial(rng):
+    u32 = np.uint32
+    return {
+        "all_equal": (np.full(300, 5, u32), np.full(200, 5, u32)),
+        "disjoint": (np.arange(0, 5000, 2, dtype=u32), np.arange(1, 5001, 2, dtype=u32)),
+        "dups_both": (rng.integers(0, 40, 700).astype(u32), rng.integers(0, 40, 900).astype(u32)),
+        "extremes": (np.array([0, 0xFFFFFFFF, 1, 0xFFFFFFFE] * 3, u32), np.array([0xFFFFFFFF, 0, 0, 7], u32)),
+        "high_bits_only": ((np.arange(3000, dtype=u32) << u32(20)) | u32(3),
+                           (np.arange(0, 6000, dtype=u32) << u32(19)) | u32(3)),
+        "one_row": (np.array([42], u32), np.array([42, 42, 1], u32)),
+        "random_ragged": (rng.integers(0, 300000, 40961).astype(u32), rng.integers(0, 300000, 30011).astype(u32)),
+        "sparse_uniform": (rng.integers(0, 1 << 32, 100003, dtype=np.uint64).astype(u32),
+                           rng.integers(0, 1 << 32, 77777, dtype=np.uint64).astype(u32)),
+    }
+
+
+CASES = list(adversarial(np.random.default_rng(0)).keys())
+
+
+@pytest.mark.parametrize("name", CASES)
+@pytest.mark.parametrize("bits", [-1, 0, 1, 2, 5, 8, 13])
+def test_adversarial_vs_oracle(hj, name, bits):
+    rng = np.random.default_rng(99)
+    Rk, Sk = adversarial(rng)[name]
+    Rp = rng.integers(0, 1 << 32, len(Rk), dtype=np.uint64).astype(np.uint32)
+    Sp = rng.integers(0, 1 << 32, len(Sk), dtype=np.uint64).astype(np.uint32)
+    check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True)
+
+
+def test_empty_inputs(hj):
+    z = np.zeros(0, np.uint32)
+    a = np.arange(10, dtype=np.uint32)
+    for Rk, Sk in [(z, a), (a, z), (z, z)]:
+        res = gpu_join(hj, Rk, Rk.copy(), Sk, Sk.copy(), mat=True)
+        assert (res.matches, res.checksum) == (0, 0)
+
+
+@pytest.mark.parametrize("cap_r,chunk_s", [(7, 0), (100, 33), (0, 1), (513, 4097), (4096, 5)])
+def test_knob_invariance_block_nested_loops(hj, cap_r, chunk_s):
+    """Tiny C_R forces hash-based block nested loops; tiny C_S forces S splitting
+    (P:306-308). Results must not change."""
+    ctx = hj.Context(0, 4, 4)
+    ctx.set_option(hj.OPT_CAP_R, cap_r)
+    ctx.set_option(hj.OPT_CHUNK_S, chunk_s)
+    rng = np.random.default_rng(5)
+    Rk = rng.integers(0, 3000, 20000).astype(np.uint32)
+    Sk = rng.integers(0, 3000, 15000).astype(np.uint32)
+    Rp = np.arange(len(Rk), dtype=np.uint32)
+    Sp = np.arange(len(Sk), dtype=np.uint32)
+    for bits in (0, 4, 9):
+        check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True, ctx=ctx)
+    ctx.close()
+
+
+def test_materialize_overflow_regrows(hj):
+    """More matches than the initial capacity: grow and re-run the join phase (reading S11)."""
+    ctx = hj.Context(0, 4, 4)
+    ctx.set_option(hj.OPT_OUT_CAPACITY, 1000)
+    Rk = np.repeat(np.arange(50, dtype=np.uint32), 40)
+    Sk = np.repeat(np.arange(60, dtype=np.uint32), 30)
+    Rp = np.arange(len(Rk), dtype=np.uint32)
+    Sp = np.arange(len(Sk), dtype=np.uint32)
+    res = check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=3, mat=True, ctx=ctx)
+    assert res.matches == 50 * 40 * 30
+    ctx.close()
+
+
+@pytest.mark.parametrize("dist,keys,z", [("fk", "dense", 0), ("1to1", "sparse", 0), ("zipf", "dense", 1.5),
+                                         ("zipf", "sparse", 1.0), ("fk", "k8", 0), ("1to1", "k8", 0)])
+@pytest.mark.parametrize("nR,nS", [(1 << 16, 1 << 18), (40000, 70001)])
+def test_generated_vs_oracle(hj, dist, keys, z, nR, nS):
+    if dist == "1to1":
+        nS = nR
+    w = W.Workload("t", nR, nS, dist, keys=keys, z=z, seed=120)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=-1, mat=True)
+
+
+def test_8byte_adversarial(hj):
+    rng = np.random.default_rng(8)
+    Rk = rng.integers(0, 500, 30000, dtype=np.uint64) * np.uint64(0x100000001) + np.uint64(1 << 62)
+    Sk = rng.integers(0, 600, 20000, dtype=np.uint64) * np.uint64(0x100000001) + np.uint64(1 << 62)
+    Rp = rng.integers(0, 1 << 63, len(Rk), dtype=np.uint64)
+    Sp = rng.integers(0, 1 << 63, len(Sk), dtype=np.uint64)
+    for bits in (0, 3, 10):
+        check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True)
+
+
+@pytest.mark.parametrize("bits", [0, 1, 6, 11, 15])
+@pytest.mark.parametrize("width", [4, 8])
+def test_partition_vs_oracle(hj, bits, width):
+    """Steps a1-a4: every co-partition holds exactly the oracle's multiset of tuples."""
+    rng = np.random.default_rng(bits + width)
+    dt = np.uint32 if width == 4 else np.uint64
+    n = 300_001
+    keys = rng.integers(0, 1 << (8 * width - 1), n, dtype=np.uint64).astype(dt)
+    pays = np.arange(n, dtype=dt)
+    ok, op, offs = oracle.radix_partition(keys, pays, 0, bits)
+    ctx = hj.context(0, width, width)
+    t, start, count = ctx.partition(dev(keys), dev(pays), bits)
+    torch.cuda.synchronize()
+    assert np.array_equal(count, np.diff(offs.astype(np.int64)).astype(np.uint64))
+    tt = t.cpu().numpy()
+    if width == 4:
+        gk = (tt.view(np.uint64) & np.uint64(0xFFFFFFFF)).astype(np.uint32)
+        gp = (tt.view(np.uint64) >> np.uint64(32)).astype(np.uint32)
+    else:
+        gk = tt[:, 0].view(np.uint64)
+        gp = tt[:, 1].view(np.uint64)
+    # the partitions tile [0, n) and each equals the oracle's multiset
+    order = np.argsort(start, kind="stable")
+    assert start[order[0]] == 0
+    for p in range(1 << bits):
+        a, c = int(start[p]), int(count[p])
+        o0 = int(offs[p])
+        g = np.sort(gp[a:a + c])
+        e = np.sort(op[o0:o0 + c])
+        assert np.array_equal(g, e), f"partition {p}"
+        assert np.all((gk[a:a + c] & dt((1 << bits) - 1)) == p)
+    assert int(start.max() + count[np.argmax(start)]) <= n
+
+
+def test_join_host_matches_device(hj):
+    w = W.Workload("t", 1 << 15, 1 << 16, "fk", seed=121)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    m, c, r, s = oracle.hash_join(Rk, Rp, Sk, Sp, materialize=True)
+    res = hj.join_host(Rk, Rp, Sk, Sp, out_mode=hj.OUT_MATERIALIZE)
+    assert (res.matches, res.checksum) == (m, c)
+    assert np.array_equal(oracle.pairs_sorted(res.r_pay, res.s_pay), oracle.pairs_sorted(r, s))
+
+
+def test_c1_full_size_vs_oracle(hj):
+    """BASELINE config[0]: FK 1M ⋈ 1M, count + checksum, element by element vs the oracle."""
+    w = W.CONFIGS["c1"]
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=w.radix_bits, mat=True)
+
+
+def test_device_generator_matches_host(hj):
+    w = W.Workload("t", 1 << 18, 1 << 19, "zipf", z=1.5, seed=122)
+    a = W.np_generate(w)
+    b = W.torch_generate(w, device="cuda")
+    for x, y in zip(a, b):
+        assert np.array_equal(x, to_np(y, x.dtype.itemsize))
+
+
+@pytest.mark.slow
+@pytest.mark.parametrize("cfg", ["c2", "c3", "c4_z0.5", "c4_z1.0", "c4_z1.5"])
+def test_full_size_closed_form(hj, cfg):
+    """Full BASELINE sizes in the bench's launch configuration: matches == |S| and the checksum
+    equals sum_j sig(rho(j), j) computed on the host from the generator (closed form); for c3's
+    materialized output, the pairs sorted by s_pay are exactly (rho(j), j)."""
+    w = W.CONFIGS[cfg]
+    Rk, Rp, Sk, Sp = W.torch_generate(w, device="cuda")
+    ctx = hj.context(0, 4, 4)
+    res = ctx.join(Rk, Rp, Sk, Sp, radix_bits=w.radix_bits, out_mode=w.out_mode)
+    torch.cuda.synchronize()
+    del Rk, Rp, Sk, Sp
+    cdf = W.zipf_cdf(w.nR, w.z) if w.dist == "zipf" else None
+    j = np.arange(w.nS, dtype=np.uint64)
+    rho = W.np_rho_for(w, j, cdf)
+    assert res.matches == w.nS
+    assert res.checksum == int(np_sig(rho, j).sum(dtype=np.uint64))
+    if w.out_mode == 1:
+        s_pay = res.s_pay
+        order = torch.argsort(s_pay)
+        r_sorted = to_np(res.r_pay[order], 4).astype(np.uint64)
+        s_sorted = to_np(s_pay[order], 4).astype(np.uint64)
+        assert np.array_equal(s_sorted, j)
+        assert np.array_equal(r_sorted, rho)
