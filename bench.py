@@ -1,0 +1,294 @@
+#!/usr/bin/env python
+"""Benchmark of the B200 radix-partitioned hash join (DESIGN.md §6 states the contract).
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--config c3] [--impl hj|reference]
+
+One step = one hj_join call (all hot-path rows a1-a8) over the workload resident in HBM.
+Rank 0 prints ONE JSON line. Metric: (|R|+|S|) tuples/s (§V-A).
+Default workload: BASELINE.json config c3 (|R| = |S| = 2^27, 1:1 unique dense keys, 4 B keys
+and payloads, materialized output) -- the north star's roofline target.
+
+--impl reference times the CPU oracle (oracle/, the only other place bench.py executes it) on
+the box's host cores, on a bounded key-slice of the same workload (each step one slice).
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+import workloads as W  # noqa: E402
+
+METRIC = "join throughput (|R|+|S|) tuples/s"
+UNIT = "tuples/s"
+FALLBACK_HBM_GBS = 6650.0
+
+
+def parse():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=50)
+    ap.add_argument("--warmup", type=int, default=5)
+    ap.add_argument("--config", default="c3", choices=sorted(W.CONFIGS))
+    ap.add_argument("--impl", default="hj", choices=["hj", "reference"])
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--cpu-slice-bits", type=int, default=2, help="cpu_baseline sample = 1 of 2^bits key slices")
+    ap.add_argument("--e2e-steps", type=int, default=3)
+    return ap.parse_args()
+
+
+def peaks():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    if os.path.exists(p):
+        d = json.load(open(p))
+        return float(d["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs)"
+    return FALLBACK_HBM_GBS, "fallback (B200_PROFILING.md)"
+
+
+def workload_desc(w: W.Workload) -> str:
+    rel = {"fk": "FK uniform", "1to1": "1:1 (S a permutation of R's keys)", "zipf": f"FK Zipf z={w.z}"}[w.dist]
+    return (f"{w.name}: |R|={w.nR} |S|={w.nS} {rel}, {w.key_bytes} B keys ({w.keys}) + {w.key_bytes} B payloads, "
+            f"{'materialized' if w.out_mode else 'count+checksum'} output, seed {w.seed}")
+
+
+def alg_bytes(w: W.Workload, matches: int):
+    """Algorithmic HBM bytes per step: two partition passes read
+    and write every tuple (4w), the join reads every tuple once (w), materialization writes
+    2V per match; the histogram reads K per tuple (implementation bytes)."""
+    wb = 2 * w.key_bytes
+    n = w.n
+    out = 2 * w.key_bytes * matches if w.out_mode == 1 else 0
+    per_kernel = {"hist": w.key_bytes * n, "plan": 0, "pass1": 2 * wb * n, "pass2": 2 * wb * n, "join": wb * n + out}
+    path = 5 * wb * n + out
+    return per_kernel, path
+
+
+class ClockSampler:
+    """nvidia-smi-equivalent clock / throttle sampling (NVML) during the timed region."""
+
+    def __init__(self, index: int, period_s: float = 0.01):
+        self.samples, self.reasons, self.max_mhz = [], set(), None
+        self.period = period_s
+        self._stop = threading.Event()
+        try:
+            import pynvml
+
+            pynvml.nvmlInit()
+            self.nv = pynvml
+            self.h = pynvml.nvmlDeviceGetHandleByIndex(index)
+            self.max_mhz = pynvml.nvmlDeviceGetMaxClockInfo(self.h, pynvml.NVML_CLOCK_SM)
+        except Exception as e:  # pragma: no cover
+            self.nv = None
+            self.err = str(e)
+
+    def _run(self):
+        nv = self.nv
+        names = {
+            "hw_slowdown": getattr(nv, "nvmlClocksThrottleReasonHwSlowdown", 0x8),
+            "sw_thermal_slowdown": getattr(nv, "nvmlClocksThrottleReasonSwThermalSlowdown", 0x20),
+            "hw_thermal_slowdown": getattr(nv, "nvmlClocksThrottleReasonHwThermalSlowdown", 0x40),
+            "sw_power_cap": getattr(nv, "nvmlClocksThrottleReasonSwPowerCap", 0x4),
+            "hw_power_brake_slowdown": getattr(nv, "nvmlClocksThrottleReasonHwPowerBrakeSlowdown", 0x80),
+        }
+        while not self._stop.is_set():
+            try:
+                self.samples.append(nv.nvmlDeviceGetClockInfo(self.h, nv.NVML_CLOCK_SM))
+                r = nv.nvmlDeviceGetCurrentClocksThrottleReasons(self.h)
+                for k, bit in names.items():
+                    if r & bit:
+                        self.reasons.add(k)
+            except Exception:
+                pass
+            time.sleep(self.period)
+
+    def __enter__(self):
+        if self.nv:
+            self.t = threading.Thread(target=self._run, daemon=True)
+            self.t.start()
+        return self
+
+    def __exit__(self, *a):
+        if self.nv:
+            self._stop.set()
+            self.t.join()
+
+    def summary(self):
+        if not self.nv:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": [], "error": getattr(self, "err", "")}
+        med = float(np.median(self.samples)) if self.samples else None
+        return {"sm_mhz": med, "sm_max_mhz": self.max_mhz, "reasons": sorted(self.reasons), "samples": len(self.samples)}
+
+
+def dist_env():
+    ws = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    return ws, rank, local
+
+
+def cpu_oracle_sample(w: W.Workload, Rk, Rp, Sk, Sp, slice_bits: int):
+    """Time the oracle (as it stands, single thread) on key slice 0 of 2^slice_bits of the
+    workload; throughput extrapolated as (|R|+|S|) / (2^slice_bits * t_slice)."""
+    import oracle
+
+    t0 = time.perf_counter()
+    res = oracle.hash_join(Rk, Rp, Sk, Sp, materialize=bool(w.out_mode), slice_bits=slice_bits, slice_id=0)
+    dt = time.perf_counter() - t0
+    v = w.n / ((1 << slice_bits) * dt)
+    sample = (f"key slice 0 of {1 << slice_bits} (top {slice_bits} bits of fmix64(key)) of the full {w.name} input, "
+              f"oracle sliced mode incl. its filtering scans, {'materialized' if w.out_mode else 'count'}; "
+              f"{res[0]} matches in {dt:.2f} s; value = (|R|+|S|)/({1 << slice_bits}*t_slice)")
+    return {"value": v, "unit": UNIT, "cores": 1, "kind": "oracle", "sample": sample, "host_cpus": os.cpu_count()}
+
+
+def run_reference(args, w: W.Workload):
+    ws, rank, _ = dist_env()
+    if rank != 0:
+        return
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    bits = max(args.cpu_slice_bits, 4)
+    import oracle
+
+    oracle.build()
+    times = []
+    for i in range(args.warmup + args.steps):
+        t0 = time.perf_counter()
+        oracle.hash_join(Rk, Rp, Sk, Sp, materialize=bool(w.out_mode), slice_bits=bits, slice_id=i % (1 << bits))
+        if i >= args.warmup:
+            times.append(time.perf_counter() - t0)
+    t = float(np.mean(times))
+    v = w.n / ((1 << bits) * t)
+    cpu = {"value": v, "unit": UNIT, "cores": 1, "kind": "oracle", "host_cpus": os.cpu_count(),
+           "sample": f"each step one key slice (1 of {1 << bits}, fmix64 top bits) of the full {w.name} input; "
+                     f"value = (|R|+|S|)/({1 << bits}*mean t_slice)"}
+    print(json.dumps({"impl": "reference", "metric": METRIC, "value": v, "unit": UNIT, "n_gpus": ws,
+                      "steps": args.steps, "warmup": args.warmup, "ms_per_step": t * 1e3, "higher_is_better": True,
+                      "scaling": "weak", "vs_baseline": None, "dtype": "u32" if w.key_bytes == 4 else "u64",
+                      "data": "synthetic", "config": {"workload": workload_desc(w)}, "cpu_baseline": cpu,
+                      "e2e": {"value": v, "unit": UNIT, "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}),
+          flush=True)
+
+
+def main():
+    args = parse()
+    w = W.CONFIGS[args.config]
+    if args.impl == "reference":
+        return run_reference(args, w)
+
+    import torch
+
+    ws, rank, local = dist_env()
+    if ws > 1:
+        import torch.distributed as dist
+
+        torch.cuda.set_device(local)
+        dist.init_process_group("nccl")
+    dev = torch.device("cuda", local)
+    torch.cuda.set_device(dev)
+    import paper_conf_icde_sioulasckaa19_b200 as hj
+
+    ctx = hj.Context(local, w.key_bytes, w.key_bytes)
+    Rk, Rp, Sk, Sp = W.torch_generate(w, device=dev)
+    torch.cuda.synchronize()
+    stream = torch.cuda.current_stream(dev)
+
+    for _ in range(args.warmup):
+        res = ctx.join(Rk, Rp, Sk, Sp, radix_bits=w.radix_bits, out_mode=w.out_mode)
+    assert res.matches == w.nS, "closed form: FK / 1:1 joins produce |S| matches"
+
+    def barrier():
+        if ws > 1:
+            torch.distributed.barrier()
+        torch.cuda.synchronize()
+
+    per_k = np.zeros(5)
+    launches = 0
+    barrier()
+    with ClockSampler(local) as clk:
+        e0 = torch.cuda.Event(enable_timing=True)
+        e1 = torch.cuda.Event(enable_timing=True)
+        e0.record(stream)
+        for _ in range(args.steps):
+            res = ctx.join(Rk, Rp, Sk, Sp, radix_bits=w.radix_bits, out_mode=w.out_mode)
+            per_k += np.array(res.ms_kernel)
+            launches += res.kernels
+        e1.record(stream)
+        barrier()
+    ms = e0.elapsed_time(e1) / args.steps
+    if ws > 1:
+        t = torch.tensor([ms], device=dev)
+        torch.distributed.all_reduce(t, op=torch.distributed.ReduceOp.MAX)
+        ms = float(t.item())
+    per_k /= args.steps
+    value = ws * w.n / (ms * 1e-3)
+
+    if rank != 0:
+        if ws > 1:
+            torch.distributed.destroy_process_group()
+        return
+
+    peak, peak_src = peaks()
+    kb, path_bytes = alg_bytes(w, res.matches)
+    names = ["hist", "plan", "pass1", "pass2", "join"]
+    kms = dict(zip(names, per_k.tolist()))
+    dom = max(names, key=lambda k: kms[k])
+    traffic = None
+    tf = os.path.join(ROOT, "profiles", f"traffic_{w.name}.json")
+    if os.path.exists(tf):
+        traffic = json.load(open(tf)).get(dom)
+    ach = kb[dom] / (kms[dom] * 1e-3) / 1e9
+    roof = {"bound": "hbm", "kernel": dom, "achieved": ach, "peak": peak, "unit": "GB/s", "frac": ach / peak,
+            "traffic": traffic, "alg_bytes_per_launch": kb[dom], "ms_per_launch": kms[dom], "peak_source": peak_src}
+    path_ach = path_bytes / (ms * 1e-3) / 1e9
+    roof_path = {"bound": "hbm", "achieved": path_ach, "peak": peak, "unit": "GB/s", "frac": path_ach / peak,
+                 "alg_bytes_per_step": path_bytes,
+                 "kernel_fracs": {k: (kb[k] / (kms[k] * 1e-3) / 1e9 / peak if kms[k] > 0 else None) for k in names}}
+
+    out = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": ws, "steps": args.steps, "warmup": args.warmup,
+           "ms_per_step": ms, "higher_is_better": True, "scaling": "weak", "vs_baseline": None,
+           "dtype": "u32" if w.key_bytes == 4 else "u64", "data": "synthetic",
+           "config": {"workload": workload_desc(w), "radix_bits": res.radix_bits, "passes": res.passes,
+                      "join_items": res.n_items,
+                      "l2": "inputs larger than L2 (2 GiB in + 4 GiB partition buffers vs 126 MB L2); no flush",
+                      "parallelism": "1 GPU" if ws == 1 else f"{ws} independent replicas (exchange path: DESIGN.md §7)"},
+           "roofline": roof, "roofline_path": roof_path, "kernels_ms": kms, "clocks": clk.summary(),
+           "gpu_launches": launches}
+
+    if not args.no_e2e:
+        # end to end through the public API from pinned host memory: H2D of the inputs, the join,
+        # D2H of the result (matches/checksum, and the materialized pairs) every step
+        hcols = []
+        for t in (Rk, Rp, Sk, Sp):
+            h = torch.empty(t.shape, dtype=t.dtype, pin_memory=True)
+            h.copy_(t)
+            hcols.append(h.numpy())
+        ctx.join_host(*hcols, radix_bits=w.radix_bits, out_mode=w.out_mode)
+        t0 = time.perf_counter()
+        for _ in range(args.e2e_steps):
+            r2 = ctx.join_host(*hcols, radix_bits=w.radix_bits, out_mode=w.out_mode)
+        dt = (time.perf_counter() - t0) / args.e2e_steps
+        assert (r2.matches, r2.checksum) == (res.matches, res.checksum)
+        out["e2e"] = {"value": w.n / dt, "unit": UNIT, "h2d_bytes_per_step": int(sum(h.nbytes for h in hcols)),
+                      "d2h_bytes_per_step": 16 + (2 * w.key_bytes * r2.matches if w.out_mode else 0),
+                      "ms_per_step": dt * 1e3, "steps": args.e2e_steps, "api": "hj_join_host (pinned host columns)"}
+        del hcols
+
+    if not args.no_cpu_baseline and ws == 1:
+        host = [t.cpu().numpy().view(np.uint32 if w.key_bytes == 4 else np.uint64) for t in (Rk, Rp, Sk, Sp)]
+        out["cpu_baseline"] = cpu_oracle_sample(w, *host, slice_bits=args.cpu_slice_bits)
+    print(json.dumps(out), flush=True)
+    if ws > 1:
+        torch.distributed.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

@@ -78,6 +78,9 @@ typedef struct hj_result {
   float ms_total;        /* CUDA-event time of the whole call (first kernel -> result ready)     */
   float ms_partition;    /* histogram + scan + both passes                                      */
   float ms_join;         /* build + probe + output                                              */
+  float ms_kernel[5];    /* per step, CUDA events on the ctx stream: 0 histogram, 1 planner,
+                            2 pass 1, 3 pass 2, 4 join (HJ_OPT_TIMING = 1)                       */
+  uint32_t kernels;      /* kernels this call launched                                           */
 } hj_result;
 
 /* Create a context on CUDA device `device` for key/payload widths 4/4 or 8/8 bytes.

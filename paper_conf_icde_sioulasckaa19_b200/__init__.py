@@ -52,7 +52,7 @@ class _Result(ctypes.Structure):
     _fields_ = [("matches", ctypes.c_uint64), ("checksum", ctypes.c_uint64), ("r_pay_out", ctypes.c_void_p),
                 ("s_pay_out", ctypes.c_void_p), ("n_items", ctypes.c_uint64), ("radix_bits", ctypes.c_int),
                 ("passes", ctypes.c_int), ("ms_total", ctypes.c_float), ("ms_partition", ctypes.c_float),
-                ("ms_join", ctypes.c_float)]
+                ("ms_join", ctypes.c_float), ("ms_kernel", ctypes.c_float * 5), ("kernels", ctypes.c_uint32)]
 
 
 def _load_lib():
@@ -104,6 +104,8 @@ class JoinResult:
     ms_total: float = 0.0
     ms_partition: float = 0.0
     ms_join: float = 0.0
+    ms_kernel: tuple = ()
+    kernels: int = 0
 
 
 class Context:
@@ -204,7 +206,8 @@ class Context:
 def _result(res: _Result) -> JoinResult:
     return JoinResult(matches=int(res.matches), checksum=int(res.checksum), n_items=int(res.n_items),
                       radix_bits=res.radix_bits, passes=res.passes, ms_total=res.ms_total,
-                      ms_partition=res.ms_partition, ms_join=res.ms_join)
+                      ms_partition=res.ms_partition, ms_join=res.ms_join,
+                      ms_kernel=tuple(res.ms_kernel), kernels=int(res.kernels))
 
 
 def _as_device_col(t, width: int):

@@ -47,7 +47,8 @@ struct Ctx {
   void* h_out = nullptr;  // pinned host: materialized pairs (hj_join_host)
   size_t h_out_bytes = 0;
   DevBuf part_off_host_dummy;
-  cudaEvent_t ev[4] = {nullptr, nullptr, nullptr, nullptr};
+  cudaEvent_t ev[8] = {};
+  uint32_t launches = 0;
 };
 
 int fail(Ctx* c, int code, const char* fmt, ...) {
@@ -246,9 +247,14 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
 }
 
 // a1-a4 on the relations of P (both, or R only when nS == 0)
+void mark(Ctx* c, int i) {
+  if (c->opt_timing) cudaEventRecord(c->ev[i], c->stream);
+}
+
 template <typename K>
 int launch_partition(Ctx* c, const HostPlan& hp, const Plan& P) {
   cudaStream_t st = c->stream;
+  mark(c, 0);
   CUDA_TRY(c, cudaMemsetAsync(c->meta.p, 0, hp.zero_bytes, st));
   // a1 histogram
   {
@@ -262,9 +268,11 @@ int launch_partition(Ctx* c, const HostPlan& hp, const Plan& P) {
     else k_hist<K, false><<<grid, HIST_NT, 0, st>>>(P);
     CUDA_TRY(c, cudaGetLastError());
   }
+  mark(c, 1);
   // a2 + a5 planner
   k_plan<<<1, 1024, 0, st>>>(P);
   CUDA_TRY(c, cudaGetLastError());
+  mark(c, 2);
   // a3 pass 1
   {
     constexpr int IT = pass_items<K>();
@@ -274,6 +282,7 @@ int launch_partition(Ctx* c, const HostPlan& hp, const Plan& P) {
     k_pass<K, 1, PASS_NT, IT><<<g, PASS_NT, sm, st>>>(P, hp.b1);
     CUDA_TRY(c, cudaGetLastError());
   }
+  mark(c, 3);
   // a4 pass 2
   {
     constexpr int IT = pass_items<K>();
@@ -285,6 +294,8 @@ int launch_partition(Ctx* c, const HostPlan& hp, const Plan& P) {
     k_pass<K, 2, PASS_NT, IT><<<g, PASS_NT, sm, st>>>(P, hp.b2);
     CUDA_TRY(c, cudaGetLastError());
   }
+  mark(c, 4);
+  c->launches += 4;
   return HJ_OK;
 }
 
@@ -297,6 +308,8 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   if (mat) k_join<K, JOIN_NT, JOIN_SPT, true><<<g, JOIN_NT, hp.join_smem, st>>>(P, hp.ob_cap);
   else k_join<K, JOIN_NT, JOIN_SPT, false><<<g, JOIN_NT, hp.join_smem, st>>>(P, 0);
   CUDA_TRY(c, cudaGetLastError());
+  mark(c, 5);
+  c->launches += 1;
   return HJ_OK;
 }
 
@@ -329,18 +342,17 @@ int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, cons
   Plan P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
   cudaStream_t st = c->stream;
   const bool timing = c->opt_timing != 0;
-  if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[0], st));
+  c->launches = 0;
   if (c->key_bytes == 4) rc = launch_partition<uint32_t>(c, hp, P);
   else rc = launch_partition<uint64_t>(c, hp, P);
   if (rc) return rc;
-  if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[1], st));
   if (c->key_bytes == 4) rc = launch_join<uint32_t>(c, hp, P, mat);
   else rc = launch_join<uint64_t>(c, hp, P, mat);
   if (rc) return rc;
   unsigned long long* h = (unsigned long long*)c->h_res;
   CUDA_TRY(c, cudaMemcpyAsync(h, P.results, 4 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st));
   CUDA_TRY(c, cudaMemcpyAsync(h + 4, P.ist + (1ull << hp.B), sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
-  if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[2], st));
+  if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[6], st));
   CUDA_TRY(c, cudaStreamSynchronize(st));
   unsigned long long matches = h[RES_MATCHES];
   if (mat && matches > P.out_cap) {
@@ -356,7 +368,7 @@ int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, cons
     else rc = launch_join<uint64_t>(c, hp, P, mat);
     if (rc) return rc;
     CUDA_TRY(c, cudaMemcpyAsync(h, P.results, 4 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st));
-    if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[2], st));
+    if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[6], st));
     CUDA_TRY(c, cudaStreamSynchronize(st));
     matches = h[RES_MATCHES];
   }
@@ -370,10 +382,12 @@ int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, cons
     res->r_pay_out = c->out_r.p;
     res->s_pay_out = c->out_s.p;
   }
+  res->kernels = c->launches;
   if (timing) {
-    cudaEventElapsedTime(&res->ms_total, c->ev[0], c->ev[2]);
-    cudaEventElapsedTime(&res->ms_partition, c->ev[0], c->ev[1]);
-    cudaEventElapsedTime(&res->ms_join, c->ev[1], c->ev[2]);
+    cudaEventElapsedTime(&res->ms_total, c->ev[0], c->ev[6]);
+    cudaEventElapsedTime(&res->ms_partition, c->ev[0], c->ev[4]);
+    cudaEventElapsedTime(&res->ms_join, c->ev[4], c->ev[6]);
+    for (int k = 0; k < 5; ++k) cudaEventElapsedTime(&res->ms_kernel[k], c->ev[k], c->ev[k + 1]);
   }
   return HJ_OK;
 }
