@@ -15,8 +15,8 @@
  *   a6 build a shared-memory chained hash table on the R chunk with atomicExch and 16-bit
  *      offsets (Listing 2)
  *   a7 probe with the S chunk following the chains
- *   a8 aggregate (count + pair checksum) or materialize (r_pay, s_pay) pairs through
- *      a shared-memory output buffer with one global atomic per flush
+ *   a8 aggregate (count + pair checksum) or materialize the (r_pay, s_pay) pairs
+ *       with one global atomic per probe round and warp-contiguous stores
  *
  * Result definition (identical for every radix_bits):
  *   J = multiset {(r_pay, s_pay) : r_key == s_key}  (keys compared as unsigned bit patterns,
@@ -67,7 +67,8 @@ enum hj_option {
 
 typedef struct hj_result {
   uint64_t matches;      /* |R ⋈ S| (always filled)                                              */
-  uint64_t checksum;     /* sum of sig(r_pay, s_pay) mod 2^64 (always filled)                    */
+  uint64_t checksum;     /* sum of sig(r_pay, s_pay) mod 2^64 in COUNT_CHECKSUM mode; 0 in
+                            MATERIALIZE mode, whose result is the pairs themselves               */
   const void* r_pay_out; /* MATERIALIZE: `matches` payloads of R, pay_bytes each (device memory
                             for hj_join, pinned host memory for hj_join_host); owned by the ctx,
                             valid until the next join on this ctx or hj_destroy                   */

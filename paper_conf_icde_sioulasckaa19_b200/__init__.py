@@ -159,8 +159,11 @@ class Context:
             out.s_pay = _wrap_device(res.s_pay_out, res.matches, self.pay_bytes, cols[0].device)
         return out
 
-    def join_host(self, Rk, Rp, Sk, Sp, radix_bits: int = -1, out_mode: int = OUT_COUNT_CHECKSUM) -> JoinResult:
-        """End-to-end call from host numpy columns (H2D copies, join, D2H of the result)."""
+    def join_host(self, Rk, Rp, Sk, Sp, radix_bits: int = -1, out_mode: int = OUT_COUNT_CHECKSUM,
+                  copy: bool = True) -> JoinResult:
+        """End-to-end call from host numpy columns (H2D copies, join, D2H of the result).
+        With copy=False the materialized pairs are numpy views of the ctx's pinned buffer,
+        valid until the next call on this context."""
         cols = [np.ascontiguousarray(a) for a in (Rk, Rp, Sk, Sp)]
         for i, a in enumerate(cols):
             want = self.key_bytes if i % 2 == 0 else self.pay_bytes
@@ -177,8 +180,10 @@ class Context:
             n = res.matches
             buf_r = (ctypes.c_char * (n * self.pay_bytes)).from_address(res.r_pay_out)
             buf_s = (ctypes.c_char * (n * self.pay_bytes)).from_address(res.s_pay_out)
-            out.r_pay = np.frombuffer(buf_r, dtype=dt).copy()
-            out.s_pay = np.frombuffer(buf_s, dtype=dt).copy()
+            out.r_pay = np.frombuffer(buf_r, dtype=dt)
+            out.s_pay = np.frombuffer(buf_s, dtype=dt)
+            if copy:
+                out.r_pay, out.s_pay = out.r_pay.copy(), out.s_pay.copy()
         return out
 
     def partition(self, keys, pays, radix_bits: int):

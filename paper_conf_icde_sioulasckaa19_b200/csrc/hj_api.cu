@@ -3,6 +3,7 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <cmath>
 #include <cstdarg>
 #include <cstdio>
 #include <cstring>
@@ -22,8 +23,8 @@ namespace {
 thread_local std::string g_create_error;
 
 constexpr int PASS_NT = 512;   // threads per partition-pass block
-constexpr int JOIN_NT = 512;   // threads per join block (the paper used 512)
-constexpr int JOIN_SPT = 4;    // S tuples per thread per probe round
+constexpr int JOIN_NT = 256;   // threads per join block (the paper used 512)
+constexpr int JOIN_SPT = 8;    // S tuples per thread per probe round
 constexpr int HIST_NT = 1024;
 
 struct DevBuf {
@@ -132,13 +133,13 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   size_t cap_max_smem = c->smem_optin ? c->smem_optin : 227 * 1024;
   uint32_t CR;
   if (c->opt_cap_r > 0) CR = (uint32_t)std::min<int64_t>(c->opt_cap_r, 65534);
-  else CR = (uint32_t)std::min<unsigned long long>(align_up(mean + mean / 4 + 64, 256), 16384);
+  else CR = (uint32_t)std::min<unsigned long long>(align_up(mean + 5 * (unsigned long long)sqrt((double)mean) + 64, 128), 16384);
   CR = std::max<uint32_t>(CR, c->opt_cap_r > 0 ? 1 : 512);
   uint32_t CS;
   if (c->opt_chunk_s > 0) CS = (uint32_t)std::min<int64_t>(c->opt_chunk_s, 1ll << 30);
   else CS = std::max<uint32_t>(8 * CR, 32768);
   int lg_nb = std::max(6, ilog2_ceil(CR) - 1);
-  hp.ob_cap = mat ? 2048 : 0;
+  hp.ob_cap = 0;
   auto join_smem = [&](uint32_t cr, int lg) {
     size_t s = (size_t)cr * tb + ((size_t)4 << lg) + (size_t)cr * 2;
     s = align_up(s, 16) + (size_t)2 * hp.ob_cap * c->pay_bytes;
@@ -242,7 +243,13 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   P.out_r = c->out_r.p;
   P.out_s = c->out_s.p;
   P.out_cap = c->out_r.bytes / c->pay_bytes;
-  P.lg_nb = hp.lg_nb;
+  P.H.B = hp.B;
+  P.H.lg = hp.lg_nb;
+  {
+    const int rem = 8 * c->key_bytes - hp.B;  // key bits above the radix field (64-bit keys fold to 32 first)
+    const int bits = std::min(rem, 32);
+    P.H.nfold = std::min(3, std::max(0, (bits + hp.lg_nb - 1) / hp.lg_nb - 1));
+  }
   return P;
 }
 
@@ -270,7 +277,7 @@ int launch_partition(Ctx* c, const HostPlan& hp, const Plan& P) {
   }
   mark(c, 1);
   // a2 + a5 planner
-  k_plan<<<1, 1024, 0, st>>>(P);
+  k_plan<<<(unsigned)(((1u << hp.B) + 1023) / 1024), 1024, 0, st>>>(P);
   CUDA_TRY(c, cudaGetLastError());
   mark(c, 2);
   // a3 pass 1
@@ -304,9 +311,9 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   cudaStream_t st = c->stream;
   // upper bound of items: ~(nR/CR + 2^B) * ... ; grid capped by residency
   const void* f = mat ? (const void*)k_join<K, JOIN_NT, JOIN_SPT, true> : (const void*)k_join<K, JOIN_NT, JOIN_SPT, false>;
-  int g = grid_for(c, f, JOIN_NT, hp.join_smem, 1ull << 40);
-  if (mat) k_join<K, JOIN_NT, JOIN_SPT, true><<<g, JOIN_NT, hp.join_smem, st>>>(P, hp.ob_cap);
-  else k_join<K, JOIN_NT, JOIN_SPT, false><<<g, JOIN_NT, hp.join_smem, st>>>(P, 0);
+  int g = grid_for(c, f, JOIN_NT + 32, hp.join_smem, 1ull << 40);
+  if (mat) k_join<K, JOIN_NT, JOIN_SPT, true><<<g, JOIN_NT + 32, hp.join_smem, st>>>(P);
+  else k_join<K, JOIN_NT, JOIN_SPT, false><<<g, JOIN_NT + 32, hp.join_smem, st>>>(P);
   CUDA_TRY(c, cudaGetLastError());
   mark(c, 5);
   c->launches += 1;

@@ -45,22 +45,25 @@ __device__ __forceinline__ uint64_t pair_sig(uint64_t r_pay, uint64_t s_pay) {
   return fmix64(r_pay ^ (s_pay * 0x9E3779B97F4A7C15ull));
 }
 
-// In-partition slot hash: the key bits above the B radix bits, xor-folded to lg_nb bits.
-// For dense keys (c1-c4) (key >> B) < nb so this is the identity on the remaining bits
-// (collision-free chains); for wide keys the fold keeps every bit in play.
-__device__ __forceinline__ uint32_t slot_of(uint32_t key, int B, int lg_nb) {
-  uint32_t h = (B >= 32) ? 0u : (key >> B);
-  uint32_t r = 0;
-  #pragma unroll 1
-  for (int s = 0; s < 32 && (h >> s); s += lg_nb) r ^= (h >> s);
-  return r & ((1u << lg_nb) - 1);
+// In-partition slot hash: the key bits above the B radix bits, xor-folded down to lg_nb bits
+// with `nfold` extra terms (host-computed: enough terms to cover every remaining key bit, at
+// most 3). For dense keys (c1-c4) (key >> B) < nb, so this is the identity on the remaining
+// bits (collision-free chains). Chains always compare full keys, so the hash only affects
+// speed, never results.
+struct SlotHash {
+  int B, lg, nfold;
+};
+__device__ __forceinline__ uint32_t slot_fold(uint32_t h, const SlotHash& H) {
+  uint32_t r = h;
+  if (H.nfold >= 1) r ^= h >> H.lg;
+  if (H.nfold >= 2) r ^= h >> (2 * H.lg);
+  if (H.nfold >= 3) r ^= h >> (3 * H.lg);
+  return r & ((1u << H.lg) - 1);
 }
-__device__ __forceinline__ uint32_t slot_of(uint64_t key, int B, int lg_nb) {
-  uint64_t h = (B >= 64) ? 0ull : (key >> B);
-  uint64_t r = 0;
-  #pragma unroll 1
-  for (int s = 0; s < 64 && (h >> s); s += lg_nb) r ^= (h >> s);
-  return (uint32_t)(r & ((1ull << lg_nb) - 1));
+__device__ __forceinline__ uint32_t slot_of(uint32_t key, const SlotHash& H) { return slot_fold(key >> H.B, H); }
+__device__ __forceinline__ uint32_t slot_of(uint64_t key, const SlotHash& H) {
+  const uint64_t h64 = key >> H.B;
+  return slot_fold((uint32_t)h64 ^ ((uint32_t)(h64 >> 32) * 0x9E3779B1u), H);
 }
 
 __device__ __forceinline__ uint32_t lanemask_lt() {

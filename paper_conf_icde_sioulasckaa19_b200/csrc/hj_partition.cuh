@@ -37,6 +37,8 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P) {
     __syncthreads();
   }
   uint32_t* h = SMEM ? s_hist : R.cnt;
+  // shared-memory counters are indexed by p; global counters by q (p_to_q) -- see k_plan
+  auto bin = [&](uint32_t p) -> uint32_t { return SMEM ? p : (((p & ((1u << P.b1) - 1)) << P.b2) | (p >> P.b1)); };
   constexpr int VEC = 16 / sizeof(K);
   unsigned long long per = (n + gridDim.x - 1) / gridDim.x;
   per = (per + VEC - 1) / VEC * VEC;
@@ -49,21 +51,35 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P) {
     if (aligned) {
       const unsigned long long nvec = (hi - lo) / VEC;
       const uint4* kv = reinterpret_cast<const uint4*>(keys + lo);
-      for (unsigned long long v = threadIdx.x; v < nvec; v += blockDim.x) {
-        uint4 x = __ldcs(kv + v);  // streaming: keys are read again by pass 1 from HBM anyway
+      constexpr int U = 4;  // 4 x 16 B loads in flight per thread before the atomics
+      unsigned long long v = threadIdx.x;
+      for (; v + (U - 1) * blockDim.x < nvec; v += U * blockDim.x) {
+        uint4 x[U];
+        #pragma unroll
+        for (int u = 0; u < U; ++u) x[u] = __ldcs(kv + v + u * blockDim.x);
+        #pragma unroll
+        for (int u = 0; u < U; ++u) {
+          const K* e = reinterpret_cast<const K*>(&x[u]);
+          #pragma unroll
+          for (int t = 0; t < VEC; ++t) atomicAdd(&h[bin((uint32_t)(e[t]) & mask)], 1u);
+        }
+      }
+      for (; v < nvec; v += blockDim.x) {
+        uint4 x = __ldcs(kv + v);
         const K* e = reinterpret_cast<const K*>(&x);
         #pragma unroll
-        for (int t = 0; t < VEC; ++t) atomicAdd(&h[(uint32_t)(e[t]) & mask], 1u);
+        for (int t = 0; t < VEC; ++t) atomicAdd(&h[bin((uint32_t)(e[t]) & mask)], 1u);
       }
       i = lo + nvec * VEC;
     }
-    for (unsigned long long j = i + threadIdx.x; j < hi; j += blockDim.x) atomicAdd(&h[(uint32_t)keys[j] & mask], 1u);
+    for (unsigned long long j = i + threadIdx.x; j < hi; j += blockDim.x) atomicAdd(&h[bin((uint32_t)keys[j] & mask)], 1u);
   }
   if (SMEM) {
     __syncthreads();
+    const uint32_t mb1 = (1u << P.b1) - 1;
     for (uint32_t i = threadIdx.x; i < np; i += blockDim.x) {
       uint32_t c = s_hist[i];
-      if (c) atomicAdd(&R.cnt[i], c);
+      if (c) atomicAdd(&R.cnt[((i & mb1) << P.b2) | (i >> P.b1)], c);  // stored in q-order
     }
   }
 }
@@ -81,57 +97,79 @@ __device__ __forceinline__ uint32_t q_to_p(uint32_t q, int b1, int b2) {
   return (d2 << b1) | d1;
 }
 
+__device__ __forceinline__ unsigned long long plan_items(const Plan& P, uint32_t cr, uint32_t cs) {
+  return (cr && cs) ? (unsigned long long)((cr + P.CR - 1) / P.CR) * ((cs + P.CS - 1) / P.CS) : 0ull;
+}
+
+// grid = ceil(2^B / 1024) blocks; block b owns q in [1024 b, 1024 (b+1)), one q per thread, so
+// every store is coalesced. Each block first sums all counts below its range itself (a redundant
+// prefix: at most 2^B / 1024 independent loads per thread, L2-resident), then scans its own
+// range. The last block to finish (atomic ticket) builds the pass-2 chunk lists.
 __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   constexpr int NT = 1024;
   __shared__ unsigned long long s_tmp[NT / 32 + 1];
+  __shared__ bool s_last;
   const uint32_t np = 1u << P.B;
   const uint32_t F1 = 1u << P.b1;
-  const uint32_t per = (np + NT - 1) / NT;
-  const uint32_t q0 = threadIdx.x * per;
-  const uint32_t q1 = min(q0 + per, np);
+  const uint32_t b = blockIdx.x;
+  // ---- prefix of everything below this block's range -------------------------------------
+  unsigned long long sR = 0, sS = 0, sI = 0;
+  #pragma unroll 8
+  for (uint32_t k = 0; k < b; ++k) {
+    const uint32_t cr = P.rel[0].cnt[k * NT + threadIdx.x], cs = P.rel[1].cnt[k * NT + threadIdx.x];
+    sR += cr;
+    sS += cs;
+    sI += plan_items(P, cr, cs);
+  }
+  unsigned long long tot;
+  block_exclusive_scan64<NT>(sR, s_tmp, &tot);
+  unsigned long long bR = tot;
+  block_exclusive_scan64<NT>(sS, s_tmp, &tot);
+  unsigned long long bS = tot;
+  block_exclusive_scan64<NT>(sI, s_tmp, &tot);
+  unsigned long long bI = tot;
+  // ---- own range ---------------------------------------------------------------------------
+  const uint32_t q = b * NT + threadIdx.x;
+  uint32_t cr = 0, cs = 0;
+  if (q < np) {
+    cr = P.rel[0].cnt[q];
+    cs = P.rel[1].cnt[q];
+  }
+  unsigned long long tR, tS, tI;
+  const unsigned long long oR = bR + block_exclusive_scan64<NT>(cr, s_tmp, &tR);
+  const unsigned long long oS = bS + block_exclusive_scan64<NT>(cs, s_tmp, &tS);
+  const unsigned long long oI = bI + block_exclusive_scan64<NT>(plan_items(P, cr, cs), s_tmp, &tI);
+  if (q < np) {
+    P.rel[0].off[q] = oR;
+    P.rel[0].cur2[q] = oR;
+    P.rel[1].off[q] = oS;
+    P.rel[1].cur2[q] = oS;
+    P.ist[q] = (uint32_t)oI;
+  }
+  if (b == gridDim.x - 1 && threadIdx.x == 0) {
+    P.rel[0].off[np] = bR + tR;
+    P.rel[1].off[np] = bS + tS;
+    P.ist[np] = (uint32_t)(bI + tI);
+  }
+  // ---- last block: pass-2 chunk lists over the 2^b1 pass-1 partitions (b1 <= 10) ----------
+  __threadfence();
+  __syncthreads();
+  if (threadIdx.x == 0) s_last = atomicAdd(&P.counters[CNT_PLAN_DONE], 1u) == gridDim.x - 1;
+  __syncthreads();
+  if (!s_last) return;
+  __threadfence();
   for (int rel = 0; rel < 2; ++rel) {
     const RelDev& R = P.rel[rel];
-    unsigned long long local = 0;
-    for (uint32_t q = q0; q < q1; ++q) local += R.cnt[q_to_p(q, P.b1, P.b2)];
-    unsigned long long tot;
-    unsigned long long base = block_exclusive_scan64<NT>(local, s_tmp, &tot);
-    for (uint32_t q = q0; q < q1; ++q) {
-      R.off[q] = base;
-      R.cur2[q] = base;
-      base += R.cnt[q_to_p(q, P.b1, P.b2)];
-    }
-    if (threadIdx.x == 0) R.off[np] = tot;
-    __syncthreads();
-    // pass-2 chunk list over the 2^b1 pass-1 partitions (b1 <= 10 -> at most one per thread)
     unsigned long long nch = 0;
     if (threadIdx.x < F1) {
-      const unsigned long long a = R.off[(unsigned long long)threadIdx.x << P.b2];
-      const unsigned long long b = R.off[(unsigned long long)(threadIdx.x + 1) << P.b2];
+      const unsigned long long a = __ldcg(&R.off[(unsigned long long)threadIdx.x << P.b2]);
+      const unsigned long long e = __ldcg(&R.off[(unsigned long long)(threadIdx.x + 1) << P.b2]);
       R.cur1[threadIdx.x] = a;
-      nch = (b - a + P.C2 - 1) / P.C2;
+      nch = (e - a + P.C2 - 1) / P.C2;
     }
-    unsigned long long cbase = block_exclusive_scan64<NT>(nch, s_tmp, &tot);
-    if (threadIdx.x < F1) R.cst[threadIdx.x] = (uint32_t)cbase;
+    const unsigned long long cb = block_exclusive_scan64<NT>(nch, s_tmp, &tot);
+    if (threadIdx.x < F1) R.cst[threadIdx.x] = (uint32_t)cb;
     if (threadIdx.x == 0) R.cst[F1] = (uint32_t)tot;
-    __syncthreads();
-  }
-  // join work list
-  {
-    const RelDev& R = P.rel[0];
-    const RelDev& S = P.rel[1];
-    unsigned long long local = 0;
-    for (uint32_t q = q0; q < q1; ++q) {
-      const unsigned long long cr = R.off[q + 1] - R.off[q], cs = S.off[q + 1] - S.off[q];
-      if (cr && cs) local += ((cr + P.CR - 1) / P.CR) * ((cs + P.CS - 1) / P.CS);
-    }
-    unsigned long long tot;
-    unsigned long long base = block_exclusive_scan64<NT>(local, s_tmp, &tot);
-    for (uint32_t q = q0; q < q1; ++q) {
-      P.ist[q] = (uint32_t)base;
-      const unsigned long long cr = R.off[q + 1] - R.off[q], cs = S.off[q + 1] - S.off[q];
-      if (cr && cs) base += ((cr + P.CR - 1) / P.CR) * ((cs + P.CS - 1) / P.CS);
-    }
-    if (threadIdx.x == 0) P.ist[np] = (uint32_t)tot;
   }
 }
 
@@ -242,6 +280,7 @@ __global__ void __launch_bounds__(NT, 2) k_pass(Plan P, int fanout_bits) {
       }
     } else {
       const T* src = (const T*)R.t1 + src0;
+      // all loads first (independent, in flight together), then the shared-memory ranking
       #pragma unroll
       for (int j = 0; j < ITEMS; ++j) {
         const unsigned long long e = (unsigned long long)j * NT + threadIdx.x;
@@ -249,10 +288,12 @@ __global__ void __launch_bounds__(NT, 2) k_pass(Plan P, int fanout_bits) {
           T t = __ldcs(src + e);
           kk[j] = TT::key(t);
           pp[j] = TT::pay(t);
-          rk[j] = atomicAdd(&s_cnt[(uint32_t)(kk[j] >> dshift) & dmask], 1u);
-        } else {
-          rk[j] = 0xffffffffu;
         }
+      }
+      #pragma unroll
+      for (int j = 0; j < ITEMS; ++j) {
+        const unsigned long long e = (unsigned long long)j * NT + threadIdx.x;
+        rk[j] = (e < len) ? atomicAdd(&s_cnt[(uint32_t)(kk[j] >> dshift) & dmask], 1u) : 0xffffffffu;
       }
     }
     __syncthreads();

@@ -2,6 +2,8 @@
 #pragma once
 #include <cstdint>
 
+#include "hj_common.cuh"
+
 namespace hj {
 
 // Per-relation device state. Co-partition q-order: q = d1 << b2 | d2 where the key's radix
@@ -13,7 +15,7 @@ struct RelDev {
   unsigned long long n;
   void* t1;                   // pass-1 output, AoS, n tuples
   void* t2;                   // pass-2 output, AoS, n tuples, co-partitions contiguous in q-order
-  uint32_t* cnt;              // [2^B] histogram indexed by p
+  uint32_t* cnt;              // [2^B] histogram, q-order (k_hist translates p -> q)
   unsigned long long* off;    // [2^B + 1] co-partition start, q-order (exclusive scan)
   unsigned long long* cur1;   // [2^b1] pass-1 reservation cursors
   unsigned long long* cur2;   // [2^B]  pass-2 reservation cursors (q-order)
@@ -26,16 +28,16 @@ struct Plan {
   uint32_t C2;           // pass-2 chunk (tile) size in tuples
   uint32_t CR, CS;       // join item capacities: R tuples (smem build) and S tuples per item
   uint32_t* ist;         // [2^B + 1] join item prefix (q-order)
-  uint32_t* counters;    // [8]: 0 next join item, 1 next pass-2 chunk (unused), 2.. reserved
+  uint32_t* counters;    // [8]: 0 next join item, 1 planner blocks done, 2.. reserved
   unsigned long long* results;  // [4]: 0 matches, 1 checksum, 2 output cursor, 3 unused
   void* out_r;           // materialized payloads of R (pay width), capacity out_cap
   void* out_s;
   unsigned long long out_cap;
   unsigned long long tiles1[2];  // pass-1 tiles per relation (host-known)
-  int lg_nb;             // log2 of hash-table slots per join item
+  SlotHash H;            // in-partition slot hash (lg = log2 of hash-table slots per join item)
 };
 
-enum { CNT_NEXT_ITEM = 0 };
+enum { CNT_NEXT_ITEM = 0, CNT_PLAN_DONE = 1 };
 enum { RES_MATCHES = 0, RES_CHECKSUM = 1, RES_CURSOR = 2 };
 
 }  // namespace hj
