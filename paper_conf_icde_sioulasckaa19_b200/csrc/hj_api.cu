@@ -22,7 +22,7 @@ namespace {
 
 thread_local std::string g_create_error;
 
-constexpr int PASS_NT = 512;   // threads per partition-pass block
+constexpr int PASS_NT = 1024;  // threads per partition-pass block (one block per SM)
 constexpr int JOIN_NT = 256;   // threads per join block (the paper used 512)
 constexpr int JOIN_SPT = 8;    // S tuples per thread per probe round
 constexpr int HIST_NT = 1024;
@@ -107,7 +107,7 @@ struct HostPlan {
 
 template <typename K>
 constexpr int pass_items() {
-  return sizeof(K) == 4 ? 16 : 8;  // 8192-tuple tiles of 8 B, 4096-tuple tiles of 16 B (64 KB)
+  return sizeof(K) == 4 ? 8 : 4;  // 8192-tuple tiles of 8 B, 4096-tuple tiles of 16 B (64 KB)
 }
 
 int choose_bits(unsigned long long nR) {

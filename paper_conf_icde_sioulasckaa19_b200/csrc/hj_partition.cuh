@@ -37,8 +37,10 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P) {
     __syncthreads();
   }
   uint32_t* h = SMEM ? s_hist : R.cnt;
-  // shared-memory counters are indexed by p; global counters by q (p_to_q) -- see k_plan
-  auto bin = [&](uint32_t p) -> uint32_t { return SMEM ? p : (((p & ((1u << P.b1) - 1)) << P.b2) | (p >> P.b1)); };
+  // counters are indexed by q = (p & (2^b1-1)) << b2 | p >> b1, the planner's order
+  const int b1 = P.b1, b2 = P.b2;
+  const uint32_t mb1 = (1u << b1) - 1;
+  auto bin = [&](uint32_t p) -> uint32_t { return ((p & mb1) << b2) | (p >> b1); };
   constexpr int VEC = 16 / sizeof(K);
   unsigned long long per = (n + gridDim.x - 1) / gridDim.x;
   per = (per + VEC - 1) / VEC * VEC;
@@ -76,10 +78,9 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P) {
   }
   if (SMEM) {
     __syncthreads();
-    const uint32_t mb1 = (1u << P.b1) - 1;
     for (uint32_t i = threadIdx.x; i < np; i += blockDim.x) {
       uint32_t c = s_hist[i];
-      if (c) atomicAdd(&R.cnt[((i & mb1) << P.b2) | (i >> P.b1)], c);  // stored in q-order
+      if (c) atomicAdd(&R.cnt[i], c);
     }
   }
 }
@@ -174,164 +175,229 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
 }
 
 // ------------------------------------------------------------------------------------------
-// a3 / a4: one partition pass. Persistent blocks loop over work units:
+// a3 / a4: one partition pass. One persistent block of NT = 1024 threads per SM loops over
+// work units:
 //   MODE 1: unit = a tile of TILE consecutive rows of the SoA input of R or S; digit
 //           d1 = key & (2^b1 - 1); output T1 at cur1[d1] reservations.
 //   MODE 2: unit = chunk k of pass-1 partition d1 (T1[off + k*TILE, ...)); digit
 //           d2 = (key >> b1) & (2^b2 - 1); output T2 at cur2[d1 << b2 | d2] reservations.
 // Per unit: rank every tuple within its digit with a shared-memory atomicAdd (returning the
-// rank), scan the per-digit counts, reserve each digit's run in the output with one global
-// atomicAdd, shuffle the tile into digit order in shared memory, then stream it out so each
-// warp writes consecutive addresses inside a run (P:142-148 coalescing, P:269-272 shuffle
-// space). Every output location is written exactly once; the tile order inside a run is
-// whatever the smem atomics produced (partitions are multisets, reading S9).
+// rank; measured ~6 tuples/clk/SM), scan the per-digit counts, reserve each digit's run in the
+// output with one global atomicAdd, shuffle the tile into digit order in shared memory, then
+// stream it out so consecutive threads write consecutive addresses of a run (P:142-148
+// coalescing, P:269-272 shuffle space); L2 merges the partial lines at run boundaries, so
+// DRAM sees full lines (ncu: DRAM bytes == algorithmic bytes).
+// Latency hiding: the NEXT unit's loads are issued into registers before the current unit is
+// ranked (they stay in flight across its barriers), and each reservation atomic's result is
+// consumed only after the shared-memory shuffle.
+// Every output slot is written exactly once; order inside a run is whatever the shared-memory
+// atomics produced (partitions are multisets, reading S9).
 // ------------------------------------------------------------------------------------------
+template <typename K>
+struct PassUnit {
+  const void* src_k;  // MODE 1: key column at the unit start; MODE 2: first AoS tuple of the unit
+  const void* src_p;  // MODE 1: payload column at the unit start
+  void* dst;          // output buffer (T1 or T2) of the unit's relation
+  unsigned long long* cur;  // reservation cursors: cur1 (MODE 1) or &cur2[d1 << b2] (MODE 2)
+  uint32_t len;
+};
+
+// Round-robin unit walker: unit u = blockIdx.x + k * gridDim.x. MODE 2 keeps the current
+// (relation, d1) and advances d1 through the shared-memory chunk prefix instead of searching.
+template <typename K, int MODE, int TILE>
+struct UnitWalker {
+  unsigned long long units0, units;
+  int rel;
+  uint32_t d1;
+  __device__ __forceinline__ bool get(const Plan& P, unsigned long long u, PassUnit<K>& U, const uint32_t* s_cst,
+                                      const unsigned long long* s_pst) {
+    using T = typename Tup<K>::T;
+    if (u >= units) return false;
+    const int r = (u < units0) ? 0 : 1;
+    const unsigned long long ul = r ? u - units0 : u;
+    const RelDev& R = P.rel[r];
+    if (MODE == 1) {
+      const unsigned long long s0 = ul * TILE;
+      U.src_k = (const K*)R.keys + s0;
+      U.src_p = (const K*)R.pays + s0;
+      U.dst = R.t1;
+      U.cur = R.cur1;
+      U.len = (uint32_t)min((unsigned long long)TILE, R.n - s0);
+    } else {
+      if (r != rel) {
+        rel = r;
+        d1 = 0;
+      }
+      const uint32_t* cst = s_cst + r * 1025;
+      while (cst[d1 + 1] <= ul) ++d1;  // monotone in u: amortised ~gridDim / chunks-per-partition steps
+      const unsigned long long pa = s_pst[r * 1025 + d1], pb = s_pst[r * 1025 + d1 + 1];
+      const unsigned long long s0 = pa + (ul - cst[d1]) * TILE;
+      U.src_k = (const T*)R.t1 + s0;
+      U.src_p = nullptr;
+      U.dst = R.t2;
+      U.cur = R.cur2 + ((unsigned long long)d1 << P.b2);
+      U.len = (uint32_t)min((unsigned long long)TILE, pb - s0);
+    }
+    return true;
+  }
+};
+
+// element j of a thread in a unit: MODE 1 -> vector-friendly (4 / 2 consecutive per 16 B load),
+// MODE 2 -> strided by NT
+template <typename K, int MODE, int NT>
+__device__ __forceinline__ uint32_t pass_elem(int j) {
+  constexpr int VEC = 16 / sizeof(K);
+  if (MODE == 1) return (uint32_t)(j / VEC) * NT * VEC + threadIdx.x * VEC + (j % VEC);
+  return (uint32_t)j * NT + threadIdx.x;
+}
+
 template <typename K, int MODE, int NT, int ITEMS>
-__global__ void __launch_bounds__(NT, 2) k_pass(Plan P, int fanout_bits) {
+__device__ __forceinline__ void pass_load(const PassUnit<K>& U, K (&kk)[ITEMS], K (&pp)[ITEMS]) {
   using TT = Tup<K>;
   using T = typename TT::T;
   constexpr int TILE = NT * ITEMS;
+  if (MODE == 1) {
+    const K* keys = (const K*)U.src_k;
+    const K* pays = (const K*)U.src_p;
+    constexpr int VEC = 16 / sizeof(K);
+    const bool vec_ok = (U.len == TILE) && ((reinterpret_cast<uintptr_t>(keys) & 15) == 0) &&
+                        ((reinterpret_cast<uintptr_t>(pays) & 15) == 0);
+    if (vec_ok) {
+      #pragma unroll
+      for (int j = 0; j < ITEMS / VEC; ++j) {
+        const uint4 kv = __ldcs(reinterpret_cast<const uint4*>(keys) + j * NT + threadIdx.x);
+        const uint4 pv = __ldcs(reinterpret_cast<const uint4*>(pays) + j * NT + threadIdx.x);
+        const K* ke = reinterpret_cast<const K*>(&kv);
+        const K* pe = reinterpret_cast<const K*>(&pv);
+        #pragma unroll
+        for (int t = 0; t < VEC; ++t) {
+          kk[j * VEC + t] = ke[t];
+          pp[j * VEC + t] = pe[t];
+        }
+      }
+    } else {
+      #pragma unroll
+      for (int j = 0; j < ITEMS; ++j) {
+        const uint32_t e = pass_elem<K, MODE, NT>(j);
+        if (e < U.len) {
+          kk[j] = keys[e];
+          pp[j] = pays[e];
+        }
+      }
+    }
+  } else {
+    const T* src = (const T*)U.src_k;
+    #pragma unroll
+    for (int j = 0; j < ITEMS; ++j) {
+      const uint32_t e = pass_elem<K, MODE, NT>(j);
+      if (e < U.len) {
+        const T t = __ldcs(src + e);
+        kk[j] = TT::key(t);
+        pp[j] = TT::pay(t);
+      }
+    }
+  }
+}
+
+template <typename K, int MODE, int NT, int ITEMS>
+__global__ void __launch_bounds__(NT, 1) k_pass(Plan P, int fanout_bits) {
+  using TT = Tup<K>;
+  using T = typename TT::T;
+  constexpr int TILE = NT * ITEMS;
+  static_assert(NT >= 1024, "fan-out up to 2^10 needs one digit per thread");
   extern __shared__ __align__(16) unsigned char s_raw[];
   const uint32_t F = 1u << fanout_bits;
-  T* s_buf = reinterpret_cast<T*>(s_raw);                                        // TILE tuples
-  unsigned long long* s_gb = reinterpret_cast<unsigned long long*>(s_buf + TILE); // F
-  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gb + F);                         // F
+  T* s_buf = reinterpret_cast<T*>(s_raw);                                          // TILE tuples
+  unsigned long long* s_gd = reinterpret_cast<unsigned long long*>(s_buf + TILE);  // F: run base - loc
+  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gd + F);                         // F
   uint32_t* s_loc = s_cnt + F;                                                     // F
   __shared__ uint32_t s_tmp[NT / 32 + 1];
+  __shared__ uint32_t s_cst[MODE == 2 ? 2 * 1025 : 1];
+  __shared__ unsigned long long s_pst[MODE == 2 ? 2 * 1025 : 1];
 
-  const int b1 = P.b1, b2 = P.b2;
   const uint32_t dmask = F - 1;
-  const int dshift = (MODE == 1) ? 0 : b1;
-  const uint32_t E = (F + NT - 1) / NT;  // digits per thread in the scan
+  const int dshift = (MODE == 1) ? 0 : P.b1;
 
-  for (uint32_t d = threadIdx.x; d < F; d += NT) s_cnt[d] = 0;
+  if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
+  UnitWalker<K, MODE, TILE> W;
+  W.rel = -1;
+  W.d1 = 0;
+  if (MODE == 1) {
+    W.units0 = P.tiles1[0];
+    W.units = W.units0 + P.tiles1[1];
+  } else {
+    for (uint32_t i = threadIdx.x; i <= (1u << P.b1); i += NT) {
+      s_cst[i] = P.rel[0].cst[i];
+      s_cst[1025 + i] = P.rel[1].cst[i];
+      s_pst[i] = P.rel[0].off[(unsigned long long)i << P.b2];
+      s_pst[1025 + i] = P.rel[1].off[(unsigned long long)i << P.b2];
+    }
+    W.units0 = P.rel[0].cst[1u << P.b1];
+    W.units = W.units0 + P.rel[1].cst[1u << P.b1];
+  }
   __syncthreads();
 
-  unsigned long long units0, units1;
-  if (MODE == 1) {
-    units0 = P.tiles1[0];
-    units1 = P.tiles1[1];
-  } else {
-    units0 = P.rel[0].cst[1u << b1];
-    units1 = P.rel[1].cst[1u << b1];
-  }
-  const unsigned long long units = units0 + units1;
+  PassUnit<K> U, Un;
+  K kk[ITEMS], pp[ITEMS], kn[ITEMS], pn[ITEMS];
+  unsigned long long u = blockIdx.x;
+  bool have = W.get(P, u, U, s_cst, s_pst);
+  if (have) pass_load<K, MODE, NT, ITEMS>(U, kn, pn);
 
-  for (unsigned long long u = blockIdx.x; u < units; u += gridDim.x) {
-    const int rel = (u < units0) ? 0 : 1;
-    const RelDev& R = P.rel[rel];
-    const unsigned long long ul = (rel == 0) ? u : u - units0;
-    unsigned long long src0, len;
-    uint32_t d1 = 0;
-    if (MODE == 1) {
-      src0 = ul * TILE;
-      len = min((unsigned long long)TILE, R.n - src0);
-    } else {
-      // chunk -> pass-1 partition d1 by binary search over cst[0..2^b1]
-      uint32_t lo = 0, hi = 1u << b1;  // invariant cst[lo] <= ul < cst[hi]
-      while (hi - lo > 1) {
-        uint32_t mid = (lo + hi) >> 1;
-        if (R.cst[mid] <= ul) lo = mid; else hi = mid;
-      }
-      d1 = lo;
-      const unsigned long long pa = R.off[(unsigned long long)d1 << b2];
-      const unsigned long long pb = R.off[(unsigned long long)(d1 + 1) << b2];
-      src0 = pa + (ul - R.cst[d1]) * TILE;
-      len = min((unsigned long long)TILE, pb - src0);
+  while (have) {
+    #pragma unroll
+    for (int j = 0; j < ITEMS; ++j) {
+      kk[j] = kn[j];
+      pp[j] = pn[j];
     }
+    // prefetch the next unit (in flight across this unit's barriers)
+    const bool have_next = W.get(P, u + gridDim.x, Un, s_cst, s_pst);
+    if (have_next) pass_load<K, MODE, NT, ITEMS>(Un, kn, pn);
 
-    // ---- load + rank ---------------------------------------------------------------------
-    K kk[ITEMS], pp[ITEMS];
+    // ---- rank ------------------------------------------------------------------------------
     uint32_t rk[ITEMS];
-    if (MODE == 1) {
-      const K* keys = (const K*)R.keys + src0;
-      const K* pays = (const K*)R.pays + src0;
-      constexpr int VEC = 16 / sizeof(K);
-      const bool vec_ok = (len == TILE) && ((reinterpret_cast<uintptr_t>(keys) & 15) == 0) &&
-                          ((reinterpret_cast<uintptr_t>(pays) & 15) == 0);
-      if (vec_ok) {
-        #pragma unroll
-        for (int j = 0; j < ITEMS / VEC; ++j) {
-          uint4 kv = __ldcs(reinterpret_cast<const uint4*>(keys) + j * NT + threadIdx.x);
-          uint4 pv = __ldcs(reinterpret_cast<const uint4*>(pays) + j * NT + threadIdx.x);
-          const K* ke = reinterpret_cast<const K*>(&kv);
-          const K* pe = reinterpret_cast<const K*>(&pv);
-          #pragma unroll
-          for (int t = 0; t < VEC; ++t) {
-            kk[j * VEC + t] = ke[t];
-            pp[j * VEC + t] = pe[t];
-          }
-        }
-      } else {
-        #pragma unroll
-        for (int j = 0; j < ITEMS; ++j) {
-          // same element->thread map as the vector path: element (j/VEC)*NT*VEC + tid*VEC + j%VEC
-          const unsigned long long e = (unsigned long long)(j / VEC) * NT * VEC + threadIdx.x * VEC + (j % VEC);
-          if (e < len) {
-            kk[j] = keys[e];
-            pp[j] = pays[e];
-          }
-        }
-      }
-      #pragma unroll
-      for (int j = 0; j < ITEMS; ++j) {
-        const unsigned long long e = (unsigned long long)(j / VEC) * NT * VEC + threadIdx.x * VEC + (j % VEC);
-        rk[j] = (e < len) ? atomicAdd(&s_cnt[(uint32_t)(kk[j] >> dshift) & dmask], 1u) : 0xffffffffu;
-      }
-    } else {
-      const T* src = (const T*)R.t1 + src0;
-      // all loads first (independent, in flight together), then the shared-memory ranking
-      #pragma unroll
-      for (int j = 0; j < ITEMS; ++j) {
-        const unsigned long long e = (unsigned long long)j * NT + threadIdx.x;
-        if (e < len) {
-          T t = __ldcs(src + e);
-          kk[j] = TT::key(t);
-          pp[j] = TT::pay(t);
-        }
-      }
-      #pragma unroll
-      for (int j = 0; j < ITEMS; ++j) {
-        const unsigned long long e = (unsigned long long)j * NT + threadIdx.x;
-        rk[j] = (e < len) ? atomicAdd(&s_cnt[(uint32_t)(kk[j] >> dshift) & dmask], 1u) : 0xffffffffu;
-      }
-    }
+    #pragma unroll
+    for (int j = 0; j < ITEMS; ++j)
+      rk[j] = (pass_elem<K, MODE, NT>(j) < U.len) ? atomicAdd(&s_cnt[(uint32_t)(kk[j] >> dshift) & dmask], 1u)
+                                                  : 0xffffffffu;
     __syncthreads();
 
-    // ---- scan digit counts, reserve output runs ---------------------------------------------
+    // ---- scan digit counts; issue the reservation atomic (result consumed after the shuffle)
+    unsigned long long gres = 0;
+    uint32_t myloc = 0;
     {
-      const uint32_t d0 = threadIdx.x * E;
-      uint32_t local = 0;
-      for (uint32_t d = d0; d < d0 + E && d < F; ++d) local += s_cnt[d];
+      const uint32_t d = threadIdx.x;
+      const uint32_t c = (d < F) ? s_cnt[d] : 0u;
       uint32_t tot;
-      uint32_t base = block_exclusive_scan<NT>(local, s_tmp, &tot);
-      for (uint32_t d = d0; d < d0 + E && d < F; ++d) {
-        const uint32_t c = s_cnt[d];
-        s_loc[d] = base;
-        if (c) {
-          unsigned long long* cur = (MODE == 1) ? &R.cur1[d] : &R.cur2[((unsigned long long)d1 << b2) | d];
-          s_gb[d] = atomicAdd(cur, (unsigned long long)c);
-        }
+      myloc = block_exclusive_scan<NT>(c, s_tmp, &tot);
+      if (d < F) {
+        s_loc[d] = myloc;
         s_cnt[d] = 0;
-        base += c;
+        if (c) gres = atomicAdd(U.cur + d, (unsigned long long)c);
       }
     }
     __syncthreads();
 
-    // ---- shuffle into digit order in shared memory ------------------------------------------
+    // ---- shuffle into digit order in shared memory -----------------------------------------
     #pragma unroll
     for (int j = 0; j < ITEMS; ++j)
       if (rk[j] != 0xffffffffu) s_buf[s_loc[(uint32_t)(kk[j] >> dshift) & dmask] + rk[j]] = TT::make(kk[j], pp[j]);
+    if (threadIdx.x < F) s_gd[threadIdx.x] = gres - myloc;
     __syncthreads();
 
     // ---- stream runs out (consecutive threads -> consecutive addresses within a run) -------
-    T* dst = (T*)((MODE == 1) ? R.t1 : R.t2);
-    for (uint32_t i = threadIdx.x; i < (uint32_t)len; i += NT) {
-      const T t = s_buf[i];
-      const uint32_t d = (uint32_t)(TT::key(t) >> dshift) & dmask;
-      __stcs(dst + s_gb[d] + (i - s_loc[d]), t);
+    T* dst = (T*)U.dst;
+    #pragma unroll
+    for (int j = 0; j < ITEMS; ++j) {
+      const uint32_t i = j * NT + threadIdx.x;
+      if (i < U.len) {
+        const T t = s_buf[i];
+        __stcs(dst + (s_gd[(uint32_t)(TT::key(t) >> dshift) & dmask] + i), t);
+      }
     }
-    // the next unit rewrites s_loc / s_gb / s_buf only after its own first __syncthreads
+    __syncthreads();  // s_buf / s_loc / s_gd are rewritten by the next unit
+    U = Un;
+    u += gridDim.x;
+    have = have_next;
   }
 }
 

@@ -1,0 +1,42 @@
+"""Per-kernel summary of an ncu --set full report: duration, DRAM bytes, occupancy, stall mix."""
+import csv
+import subprocess
+import sys
+
+WANT = ["gpu__time_duration.sum", "dram__bytes_read.sum", "dram__bytes_write.sum",
+        "dram__throughput.avg.pct_of_peak_sustained_elapsed", "sm__warps_active.avg.pct_of_peak_sustained_active",
+        "launch__registers_per_thread", "launch__grid_size", "launch__block_size", "smsp__inst_executed.sum",
+        "sm__throughput.avg.pct_of_peak_sustained_elapsed",
+        "l1tex__data_bank_conflicts_pipe_lsu_mem_shared_op_ld.sum",
+        "l1tex__data_bank_conflicts_pipe_lsu_mem_shared_op_st.sum",
+        "l1tex__data_bank_conflicts_pipe_lsu_mem_shared_op_atom.sum",
+        "lts__t_sectors_op_write.sum", "lts__t_sectors_op_read.sum"]
+
+
+def main(path, as_json=False):
+    out = subprocess.run(["ncu", "-i", path, "--page", "raw", "--csv"], capture_output=True, text=True).stdout
+    rows = list(csv.reader(out.splitlines()))
+    hdr, units, data = rows[0], rows[1], rows[2:]
+    stall = [i for i, h in enumerate(hdr) if h.startswith("smsp__average_warps_issue_stalled") and
+             h.endswith("_per_issue_active.ratio")]
+    res = []
+    for r in data:
+        d = {"kernel": r[hdr.index("Kernel Name")]}
+        for w in WANT:
+            if w in hdr:
+                i = hdr.index(w)
+                d[w] = f"{r[i]} {units[i]}".strip()
+        st = sorted(((float(r[i] or 0), hdr[i].replace("smsp__average_warps_issue_stalled_", "")
+                      .replace("_per_issue_active.ratio", "")) for i in stall), reverse=True)[:6]
+        d["top_stalls"] = ", ".join(f"{n}={v:.2f}" for v, n in st)
+        res.append(d)
+    for d in res:
+        print("==", d["kernel"])
+        for k, v in d.items():
+            if k != "kernel":
+                print(f"   {k}: {v}")
+    return res
+
+
+if __name__ == "__main__":
+    main(sys.argv[1])
