@@ -135,6 +135,31 @@ int hj_join_host(hj_ctx* ctx,
 int hj_partition(hj_ctx* ctx, const void* keys, const void* pays, uint64_t n, int radix_bits,
                  const void** tuples_out, uint64_t* part_start, uint64_t* part_count);
 
+/* ---- multi-GPU exchange; the caller runs the collectives in between ------
+ * Co-partitions are independent, so G = 2^gpu_bits ranks each own the co-partitions
+ * whose radix field is extended by gpu_bits on top: rank j = (key >> local_bits) & (G - 1).
+ *
+ * hj_exchange_pack: rows a1-a3 on this rank's `n` SoA tuples of relation `rel` (0 = R, 1 = S),
+ * with the pass-1 digit widened by the rank bits, so the send buffer is grouped by destination
+ * rank and, inside each rank's segment, by the local pass-1 digit d1.
+ *   *send_out:   device, n AoS tuples (layout as hj_partition), ctx-owned until the next pack of
+ *                the same rel; rank j's segment starts at sum_{i<j} dest_counts[i].
+ *   *counts_out: device, [G][2^local_bits] uint32 per-co-partition counts (q-order, see the
+ *                implementation notes in DESIGN.md §7); row j goes to rank j. ctx-owned.
+ *   dest_counts: HOST array of G uint64 (caller-allocated): tuples destined to each rank.
+ * Requires gpu_bits + ceil(local_bits / 2) <= 10. */
+int hj_exchange_pack(hj_ctx* ctx, int rel, const void* keys, const void* pays, uint64_t n, int gpu_bits,
+                     int local_bits, const void** send_out, const uint32_t** counts_out, uint64_t* dest_counts);
+
+/* hj_join_received: rows a4-a8 on what this rank received: R_recv / S_recv are device AoS tuples
+ * concatenated in source-rank order (each source's segment grouped by d1, as packed), and
+ * R_counts / S_counts are device [nsrc][2^local_bits] uint32 count rows (row s = what source s
+ * sent, i.e. source s's counts_out row for this rank). Results are this rank's share of the join
+ * (sum matches / checksums over ranks mod 2^64; the union of the materialized pairs). */
+int hj_join_received(hj_ctx* ctx, const void* R_recv, uint64_t nR, const uint32_t* R_counts,
+                     const void* S_recv, uint64_t nS, const uint32_t* S_counts, int nsrc, int local_bits,
+                     int out_mode, hj_result* res);
+
 /* Library build string (compile flags, arch). */
 const char* hj_version(void);
 

@@ -39,7 +39,7 @@ _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4:
 
 # every symbol include/hj.h declares (checked by tests/test_abi.py)
 EXPORTS = ("hj_create", "hj_destroy", "hj_last_error", "hj_set_stream", "hj_set_option", "hj_join",
-           "hj_join_host", "hj_partition", "hj_version")
+           "hj_join_host", "hj_partition", "hj_exchange_pack", "hj_join_received", "hj_version")
 
 
 class HJError(RuntimeError):
@@ -76,6 +76,11 @@ def _load_lib():
         f.restype = i32
     lib.hj_partition.argtypes = [vp, vp, vp, u64, i32, ctypes.POINTER(vp), ctypes.POINTER(u64), ctypes.POINTER(u64)]
     lib.hj_partition.restype = i32
+    lib.hj_exchange_pack.argtypes = [vp, i32, vp, vp, u64, i32, i32, ctypes.POINTER(vp), ctypes.POINTER(vp),
+                                     ctypes.POINTER(u64)]
+    lib.hj_exchange_pack.restype = i32
+    lib.hj_join_received.argtypes = [vp, vp, u64, vp, vp, u64, vp, i32, i32, i32, ctypes.POINTER(_Result)]
+    lib.hj_join_received.restype = i32
     lib.hj_version.argtypes = []
     lib.hj_version.restype = ctypes.c_char_p
     return lib
@@ -206,6 +211,49 @@ class Context:
         if self.key_bytes == 8:
             t = t.view(n, 2)
         return t, np.frombuffer(start, dtype=np.uint64).copy(), np.frombuffer(count, dtype=np.uint64).copy()
+
+
+    # ---- multi-GPU exchange (used by paper_conf_icde_sioulasckaa19_b200.dist) -------------------
+    def exchange_pack(self, rel: int, keys, pays, gpu_bits: int, local_bits: int):
+        """Rows a1-a3 with the pass-1 digit widened by `gpu_bits` rank bits (hj_exchange_pack).
+        Returns (send, counts, dest): send = int64 tensor view of the AoS send buffer (one word per
+        4/4 tuple, two per 8/8 tuple), counts = int32 tensor [G, 2^local_bits] (row j goes to rank
+        j), dest = numpy uint64 [G] tuples per destination. Views are ctx-owned (valid until the
+        next pack of the same relation)."""
+        import torch
+
+        k = _as_device_col(keys, self.key_bytes)
+        p = _as_device_col(pays, self.pay_bytes)
+        self.set_stream(torch.cuda.current_stream(k.device).cuda_stream)
+        G = 1 << gpu_bits
+        send, cnt = ctypes.c_void_p(), ctypes.c_void_p()
+        dest = (ctypes.c_uint64 * G)()
+        self._check(_lib.hj_exchange_pack(self._h, rel, _ptr(k), _ptr(p), k.numel(), gpu_bits, local_bits,
+                                          ctypes.byref(send), ctypes.byref(cnt), dest))
+        words = k.numel() * (self.key_bytes + self.pay_bytes) // 8
+        send_t = (_wrap_device(send.value, words, 8, k.device) if words
+                  else torch.zeros(0, dtype=torch.int64, device=k.device))
+        cnt_t = _wrap_device(cnt.value, G << local_bits, 4, k.device).view(G, 1 << local_bits)
+        return send_t, cnt_t, np.frombuffer(dest, dtype=np.uint64).copy()
+
+    def join_received(self, R_recv, nR: int, R_counts, S_recv, nS: int, S_counts, nsrc: int, local_bits: int,
+                      out_mode: int = OUT_COUNT_CHECKSUM) -> JoinResult:
+        """Rows a4-a8 on received tuples (hj_join_received): this rank's share of the join."""
+        import torch
+
+        dev_ = R_counts.device
+        self.set_stream(torch.cuda.current_stream(dev_).cuda_stream)
+        for t in (R_recv, S_recv, R_counts, S_counts):
+            if not t.is_cuda or not t.is_contiguous():
+                raise ValueError("join_received takes contiguous CUDA tensors")
+        res = _Result()
+        self._check(_lib.hj_join_received(self._h, _ptr(R_recv), nR, _ptr(R_counts), _ptr(S_recv), nS,
+                                          _ptr(S_counts), nsrc, local_bits, out_mode, ctypes.byref(res)))
+        out = _result(res)
+        if out_mode == OUT_MATERIALIZE and res.matches:
+            out.r_pay = _wrap_device(res.r_pay_out, res.matches, self.pay_bytes, dev_)
+            out.s_pay = _wrap_device(res.s_pay_out, res.matches, self.pay_bytes, dev_)
+        return out
 
 
 def _result(res: _Result) -> JoinResult:

@@ -43,7 +43,7 @@ struct Ctx {
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0;
   // workspace
-  DevBuf t1[2], t2[2], meta, out_r, out_s, in[4];
+  DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2];
   void* h_res = nullptr;  // pinned host: results readback
   void* h_out = nullptr;  // pinned host: materialized pairs (hj_join_host)
   size_t h_out_bytes = 0;
@@ -93,16 +93,18 @@ int ilog2_ceil(unsigned long long x) {
 // Host-side plan of one call: radix bits, capacities, launch shapes, metadata layout.
 struct HostPlan {
   int B = 0, b1 = 0, b2 = 0;
+  int g = 0, nsrc = 1, mode = PLAN_FULL;
   uint32_t CR = 0, CS = 0, C2 = 0;
   int lg_nb = 6;
   size_t join_smem = 0;
-  uint32_t ob_cap = 0;
-  size_t pass_smem = 0;
   int tile = 0;
   // metadata offsets (bytes) inside ctx->meta
-  size_t o_cnt[2], o_off[2], o_cur1[2], o_cur2[2], o_cst[2], o_ist, o_counters, o_results;
+  size_t o_cnt[2], o_off[2], o_cur1[2], o_cur2[2], o_pst[2], o_cst[2], o_ist, o_counters, o_results;
   size_t zero_bytes = 0;  // [0, zero_bytes) is memset to 0 per call
   size_t meta_bytes = 0;
+  int pb() const { return g + b1; }
+  int qbits() const { return g + B; }
+  uint32_t npieces() const { return (uint32_t)nsrc << pb(); }
 };
 
 template <typename K>
@@ -117,16 +119,22 @@ int choose_bits(unsigned long long nR) {
   return std::min(B, 20);
 }
 
-int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat) {
+// mode PLAN_FULL: one GPU; PLAN_SEND: exchange sender (g rank bits); PLAN_RECV: exchange
+// receiver (nsrc count rows). nR / nS are the tuples this GPU partitions / joins.
+int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat, int g = 0,
+              int nsrc = 1, int mode = PLAN_FULL) {
   const size_t tb = (size_t)c->key_bytes + c->pay_bytes;  // AoS tuple bytes
   hp.B = radix_bits < 0 ? choose_bits(nR) : radix_bits;
   if (hp.B > 20) return fail(c, HJ_ERR_UNSUPPORTED, "radix_bits %d > 20", hp.B);
   hp.b1 = (hp.B + 1) / 2;
   hp.b2 = hp.B / 2;
+  hp.g = g;
+  hp.nsrc = nsrc;
+  hp.mode = mode;
+  if (hp.pb() > 10 || hp.b2 > 10 || hp.npieces() > 1024)
+    return fail(c, HJ_ERR_UNSUPPORTED, "pass fan-out too large (g=%d b1=%d b2=%d sources=%d)", g, hp.b1, hp.b2, nsrc);
   hp.tile = PASS_NT * (c->key_bytes == 4 ? pass_items<uint32_t>() : pass_items<uint64_t>());
   hp.C2 = (uint32_t)hp.tile;
-  const uint32_t F = 1u << std::max(hp.b1, hp.b2);
-  hp.pass_smem = (size_t)hp.tile * tb + (size_t)F * (8 + 4 + 4);
 
   // join capacities
   const unsigned long long mean = (nR + (1ull << hp.B) - 1) >> hp.B;
@@ -139,11 +147,8 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   if (c->opt_chunk_s > 0) CS = (uint32_t)std::min<int64_t>(c->opt_chunk_s, 1ll << 30);
   else CS = std::max<uint32_t>(8 * CR, 32768);
   int lg_nb = std::max(6, ilog2_ceil(CR) - 1);
-  hp.ob_cap = 0;
-  auto join_smem = [&](uint32_t cr, int lg) {
-    size_t s = (size_t)cr * tb + ((size_t)4 << lg) + (size_t)cr * 2;
-    s = align_up(s, 16) + (size_t)2 * hp.ob_cap * c->pay_bytes;
-    return s;
+  auto join_smem = [&](uint32_t cr, int lg) {  // 2 R tile buffers (TMA double buffer) + heads + next
+    return (size_t)2 * ((cr + 3) & ~1u) * tb + ((size_t)4 << lg) + (size_t)cr * 2;
   };
   while (join_smem(CR, lg_nb) > cap_max_smem - 8 * 1024 && CR > 256) {
     CR /= 2;
@@ -155,7 +160,7 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   hp.join_smem = join_smem(CR, lg_nb);
 
   // metadata layout
-  const size_t np = (size_t)1 << hp.B, F1 = (size_t)1 << hp.b1;
+  const size_t nq = (size_t)1 << hp.qbits(), F1 = (size_t)1 << hp.pb(), npc = hp.npieces();
   size_t o = 0;
   auto take = [&](size_t bytes) {
     size_t r = o;
@@ -165,16 +170,16 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   // zeroed region first
   hp.o_counters = take(64);
   hp.o_results = take(64);
-  hp.o_cnt[0] = take(np * 4);
-  hp.o_cnt[1] = take(np * 4);
+  for (int r = 0; r < 2; ++r) hp.o_cnt[r] = take(mode == PLAN_RECV ? 0 : nq * 4);
   hp.zero_bytes = o;
   for (int r = 0; r < 2; ++r) {
-    hp.o_off[r] = take((np + 1) * 8);
+    hp.o_off[r] = take((nq + 1) * 8);
     hp.o_cur1[r] = take(F1 * 8);
-    hp.o_cur2[r] = take(np * 8);
-    hp.o_cst[r] = take((F1 + 1) * 4);
+    hp.o_cur2[r] = take(nq * 8);
+    hp.o_pst[r] = take((npc + 1) * 8);
+    hp.o_cst[r] = take((npc + 1) * 4);
   }
-  hp.o_ist = take((np + 1) * 4);
+  hp.o_ist = take((((size_t)1 << hp.B) + 1) * 4);
   hp.meta_bytes = o;
   (void)nS;
   return HJ_OK;
@@ -190,9 +195,11 @@ int set_kernel_attrs(Ctx* c) {
                              (int)(c->smem_optin - fa.sharedSizeBytes)) != cudaSuccess)
       rc = -1;
   };
-  attr((const void*)k_hist<K, true>);
-  attr((const void*)k_pass<K, 1, PASS_NT, pass_items<K>()>);
-  attr((const void*)k_pass<K, 2, PASS_NT, pass_items<K>()>);
+  attr((const void*)k_hist<K, true, false>);
+  attr((const void*)k_hist<K, true, true>);
+  attr((const void*)k_pass<K, 1, PASS_NT, pass_items<K>(), false>);
+  attr((const void*)k_pass<K, 1, PASS_NT, pass_items<K>(), true>);
+  attr((const void*)k_pass<K, 2, PASS_NT, pass_items<K>(), false>);
   attr((const void*)k_join<K, JOIN_NT, JOIN_SPT, false>);
   attr((const void*)k_join<K, JOIN_NT, JOIN_SPT, true>);
   return rc;
@@ -208,7 +215,7 @@ int grid_for(Ctx* c, const void* f, int nt, size_t smem, unsigned long long unit
   return (int)std::max<unsigned long long>(g, 1);
 }
 
-// Fill the device Plan for one call; rel 1 may be empty (hj_partition).
+// Fill the device Plan for one call; rel 1 may be empty (hj_partition, hj_exchange_pack).
 Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk,
                  const void* Sp, unsigned long long nS) {
   Plan P;
@@ -228,12 +235,16 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
     d.off = (unsigned long long*)(m + hp.o_off[r]);
     d.cur1 = (unsigned long long*)(m + hp.o_cur1[r]);
     d.cur2 = (unsigned long long*)(m + hp.o_cur2[r]);
+    d.pst = (unsigned long long*)(m + hp.o_pst[r]);
     d.cst = (uint32_t*)(m + hp.o_cst[r]);
     P.tiles1[r] = (ns[r] + hp.tile - 1) / hp.tile;
   }
   P.B = hp.B;
   P.b1 = hp.b1;
   P.b2 = hp.b2;
+  P.g = hp.g;
+  P.nsrc = hp.nsrc;
+  P.mode = hp.mode;
   P.C2 = hp.C2;
   P.CR = hp.CR;
   P.CS = hp.CS;
@@ -253,63 +264,71 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   return P;
 }
 
-// a1-a4 on the relations of P (both, or R only when nS == 0)
 void mark(Ctx* c, int i) {
   if (c->opt_timing) cudaEventRecord(c->ev[i], c->stream);
 }
 
+// a1 (histogram), a2/a5 (planner), a3 (pass 1). PLAN_RECV skips a1 and a3 (counts and the
+// pass-1 layout arrive through the exchange). Events 0..3.
 template <typename K>
-int launch_partition(Ctx* c, const HostPlan& hp, const Plan& P) {
+int launch_front(Ctx* c, const HostPlan& hp, const Plan& P) {
   cudaStream_t st = c->stream;
+  const bool gd = hp.g > 0;
   mark(c, 0);
   CUDA_TRY(c, cudaMemsetAsync(c->meta.p, 0, hp.zero_bytes, st));
-  // a1 histogram
-  {
-    const bool smem = hp.B <= 15;
-    const size_t sm = smem ? ((size_t)4 << hp.B) : 0;
+  if (hp.mode != PLAN_RECV) {
+    const bool smem = hp.qbits() <= 15;
+    const size_t sm = smem ? ((size_t)4 << hp.qbits()) : 0;
     const unsigned long long nmax = std::max(P.rel[0].n, P.rel[1].n);
-    const void* f = smem ? (const void*)k_hist<K, true> : (const void*)k_hist<K, false>;
+    const void* f = smem ? (gd ? (const void*)k_hist<K, true, true> : (const void*)k_hist<K, true, false>)
+                         : (const void*)k_hist<K, false, false>;
     int g = grid_for(c, f, HIST_NT, sm, (nmax + 4095) / 4096);
     dim3 grid((unsigned)std::max(1, g / 2), 2);
-    if (smem) k_hist<K, true><<<grid, HIST_NT, sm, st>>>(P);
-    else k_hist<K, false><<<grid, HIST_NT, 0, st>>>(P);
+    if (smem && gd) k_hist<K, true, true><<<grid, HIST_NT, sm, st>>>(P);
+    else if (smem) k_hist<K, true, false><<<grid, HIST_NT, sm, st>>>(P);
+    else if (gd) k_hist<K, false, true><<<grid, HIST_NT, 0, st>>>(P);
+    else k_hist<K, false, false><<<grid, HIST_NT, 0, st>>>(P);
     CUDA_TRY(c, cudaGetLastError());
+    c->launches += 1;
   }
   mark(c, 1);
-  // a2 + a5 planner
-  k_plan<<<(unsigned)(((1u << hp.B) + 1023) / 1024), 1024, 0, st>>>(P);
+  k_plan<<<(unsigned)((((size_t)1 << hp.qbits()) + 1023) / 1024), 1024, 0, st>>>(P);
   CUDA_TRY(c, cudaGetLastError());
+  c->launches += 1;
   mark(c, 2);
-  // a3 pass 1
-  {
+  if (hp.mode != PLAN_RECV) {
     constexpr int IT = pass_items<K>();
-    const void* f = (const void*)k_pass<K, 1, PASS_NT, IT>;
-    const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.b1) * 16;
+    const void* f = gd ? (const void*)k_pass<K, 1, PASS_NT, IT, true> : (const void*)k_pass<K, 1, PASS_NT, IT, false>;
+    const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.pb()) * 16;
     int g = grid_for(c, f, PASS_NT, sm, P.tiles1[0] + P.tiles1[1]);
-    k_pass<K, 1, PASS_NT, IT><<<g, PASS_NT, sm, st>>>(P, hp.b1);
+    if (gd) k_pass<K, 1, PASS_NT, IT, true><<<g, PASS_NT, sm, st>>>(P, hp.pb());
+    else k_pass<K, 1, PASS_NT, IT, false><<<g, PASS_NT, sm, st>>>(P, hp.pb());
     CUDA_TRY(c, cudaGetLastError());
+    c->launches += 1;
   }
   mark(c, 3);
-  // a4 pass 2
-  {
-    constexpr int IT = pass_items<K>();
-    const void* f = (const void*)k_pass<K, 2, PASS_NT, IT>;
-    const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.b2) * 16;
-    // chunks: at most tiles1 + 2^b1 per relation
-    unsigned long long units = P.tiles1[0] + P.tiles1[1] + 2 * (1ull << hp.b1);
-    int g = grid_for(c, f, PASS_NT, sm, units);
-    k_pass<K, 2, PASS_NT, IT><<<g, PASS_NT, sm, st>>>(P, hp.b2);
-    CUDA_TRY(c, cudaGetLastError());
-  }
+  return HJ_OK;
+}
+
+// a4: pass 2 over the pass-1 pieces. Event 4.
+template <typename K>
+int launch_pass2(Ctx* c, const HostPlan& hp, const Plan& P) {
+  constexpr int IT = pass_items<K>();
+  const void* f = (const void*)k_pass<K, 2, PASS_NT, IT, false>;
+  const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.b2) * 16;
+  // chunks: at most n / C2 + npieces per relation
+  unsigned long long units = (P.rel[0].n + P.rel[1].n) / hp.C2 + 2ull * hp.npieces() + 2;
+  int g = grid_for(c, f, PASS_NT, sm, units);
+  k_pass<K, 2, PASS_NT, IT, false><<<g, PASS_NT, sm, c->stream>>>(P, hp.b2);
+  CUDA_TRY(c, cudaGetLastError());
+  c->launches += 1;
   mark(c, 4);
-  c->launches += 4;
   return HJ_OK;
 }
 
 template <typename K>
 int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   cudaStream_t st = c->stream;
-  // upper bound of items: ~(nR/CR + 2^B) * ... ; grid capped by residency
   const void* f = mat ? (const void*)k_join<K, JOIN_NT, JOIN_SPT, true> : (const void*)k_join<K, JOIN_NT, JOIN_SPT, false>;
   int g = grid_for(c, f, JOIN_NT + 32, hp.join_smem, 1ull << 40);
   if (mat) k_join<K, JOIN_NT, JOIN_SPT, true><<<g, JOIN_NT + 32, hp.join_smem, st>>>(P);
@@ -320,14 +339,15 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   return HJ_OK;
 }
 
-int prepare(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat) {
-  int rc = make_plan(c, hp, nR, nS, radix_bits, mat);
+int prepare(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat, int g = 0,
+            int nsrc = 1, int mode = PLAN_FULL) {
+  int rc = make_plan(c, hp, nR, nS, radix_bits, mat, g, nsrc, mode);
   if (rc) return rc;
   const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
   const unsigned long long ns[2] = {nR, nS};
   for (int r = 0; r < 2; ++r) {
-    if ((rc = ensure(c, c->t1[r], ns[r] * tb))) return rc;
-    if ((rc = ensure(c, c->t2[r], ns[r] * tb))) return rc;
+    if (mode == PLAN_FULL && (rc = ensure(c, c->t1[r], ns[r] * tb))) return rc;
+    if (mode != PLAN_SEND && (rc = ensure(c, c->t2[r], ns[r] * tb + 64))) return rc;  // +64: aligned bulk-copy tail
   }
   if ((rc = ensure(c, c->meta, hp.meta_bytes))) return rc;
   if (mat) {
@@ -340,21 +360,11 @@ int prepare(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, 
   return HJ_OK;
 }
 
-int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk, const void* Sp,
-             unsigned long long nS, int radix_bits, int out_mode, hj_result* res) {
-  const bool mat = out_mode == HJ_OUT_MATERIALIZE;
-  HostPlan hp;
-  int rc = prepare(c, hp, nR, nS, radix_bits, mat);
-  if (rc) return rc;
-  Plan P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
+// Join phase + result readback shared by hj_join and hj_join_received.
+int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res) {
   cudaStream_t st = c->stream;
   const bool timing = c->opt_timing != 0;
-  c->launches = 0;
-  if (c->key_bytes == 4) rc = launch_partition<uint32_t>(c, hp, P);
-  else rc = launch_partition<uint64_t>(c, hp, P);
-  if (rc) return rc;
-  if (c->key_bytes == 4) rc = launch_join<uint32_t>(c, hp, P, mat);
-  else rc = launch_join<uint64_t>(c, hp, P, mat);
+  int rc = c->key_bytes == 4 ? launch_join<uint32_t>(c, hp, P, mat) : launch_join<uint64_t>(c, hp, P, mat);
   if (rc) return rc;
   unsigned long long* h = (unsigned long long*)c->h_res;
   CUDA_TRY(c, cudaMemcpyAsync(h, P.results, 4 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st));
@@ -371,8 +381,7 @@ int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, cons
     P.out_cap = matches;
     CUDA_TRY(c, cudaMemsetAsync(P.results, 0, 4 * sizeof(unsigned long long), st));
     CUDA_TRY(c, cudaMemsetAsync(P.counters, 0, 8 * sizeof(uint32_t), st));
-    if (c->key_bytes == 4) rc = launch_join<uint32_t>(c, hp, P, mat);
-    else rc = launch_join<uint64_t>(c, hp, P, mat);
+    rc = c->key_bytes == 4 ? launch_join<uint32_t>(c, hp, P, mat) : launch_join<uint64_t>(c, hp, P, mat);
     if (rc) return rc;
     CUDA_TRY(c, cudaMemcpyAsync(h, P.results, 4 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st));
     if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[6], st));
@@ -397,6 +406,19 @@ int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, cons
     for (int k = 0; k < 5; ++k) cudaEventElapsedTime(&res->ms_kernel[k], c->ev[k], c->ev[k + 1]);
   }
   return HJ_OK;
+}
+
+int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk, const void* Sp,
+             unsigned long long nS, int radix_bits, int out_mode, hj_result* res) {
+  const bool mat = out_mode == HJ_OUT_MATERIALIZE;
+  HostPlan hp;
+  int rc = prepare(c, hp, nR, nS, radix_bits, mat);
+  if (rc) return rc;
+  Plan P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
+  c->launches = 0;
+  if ((rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P))) return rc;
+  if ((rc = c->key_bytes == 4 ? launch_pass2<uint32_t>(c, hp, P) : launch_pass2<uint64_t>(c, hp, P))) return rc;
+  return finish_join(c, hp, P, mat, res);
 }
 
 int check_args(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk, const void* Sp,
@@ -457,7 +479,7 @@ int hj_create(hj_ctx** out, int device, int key_bytes, int pay_bytes, void* cuda
     return fail(nullptr, HJ_ERR_CUDA, "kernel attribute setup failed: %s", cudaGetErrorString(e));
   }
   if (cudaStreamCreateWithFlags(&c->own_stream, cudaStreamNonBlocking) != cudaSuccess ||
-      cudaMallocHost(&c->h_res, 64) != cudaSuccess) {
+      cudaMallocHost(&c->h_res, 8 * 1025 + 64) != cudaSuccess) {
     cudaSetDevice(prev);
     delete h;
     return fail(nullptr, HJ_ERR_CUDA, "stream / pinned allocation failed");
@@ -476,8 +498,9 @@ void hj_destroy(hj_ctx* h) {
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
   if (c->stream) cudaStreamSynchronize(c->stream);
-  DevBuf* bufs[] = {&c->t1[0], &c->t1[1], &c->t2[0], &c->t2[1], &c->meta, &c->out_r, &c->out_s,
-                    &c->in[0], &c->in[1], &c->in[2], &c->in[3]};
+  DevBuf* bufs[] = {&c->t1[0], &c->t1[1], &c->t2[0], &c->t2[1], &c->meta,    &c->out_r,    &c->out_s,
+                    &c->in[0], &c->in[1], &c->in[2], &c->in[3], &c->xsend[0], &c->xsend[1], &c->xcnt[0],
+                    &c->xcnt[1]};
   for (DevBuf* b : bufs)
     if (b->p) cudaFree(b->p);
   if (c->h_res) cudaFreeHost(c->h_res);
@@ -590,7 +613,9 @@ int hj_partition(hj_ctx* h, const void* keys, const void* pays, uint64_t n, int 
   int rc = prepare(c, hp, n, 0, radix_bits, false);
   if (rc == HJ_OK) {
     Plan P = device_plan(c, hp, keys, pays, n, nullptr, nullptr, 0);
-    rc = c->key_bytes == 4 ? launch_partition<uint32_t>(c, hp, P) : launch_partition<uint64_t>(c, hp, P);
+    c->launches = 0;
+    rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P);
+    if (rc == HJ_OK) rc = c->key_bytes == 4 ? launch_pass2<uint32_t>(c, hp, P) : launch_pass2<uint64_t>(c, hp, P);
     if (rc == HJ_OK) {
       const size_t np = (size_t)1 << hp.B;
       unsigned long long* off = new unsigned long long[np + 1];
@@ -608,6 +633,83 @@ int hj_partition(hj_ctx* h, const void* keys, const void* pays, uint64_t n, int 
       }
       delete[] off;
     }
+  }
+  cudaSetDevice(prev);
+  return rc;
+}
+
+int hj_exchange_pack(hj_ctx* h, int rel, const void* keys, const void* pays, uint64_t n, int gpu_bits, int local_bits,
+                     const void** send_out, const uint32_t** counts_out, uint64_t* dest_counts) {
+  if (!h || !send_out || !counts_out || !dest_counts) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  if (rel != 0 && rel != 1) return fail(c, HJ_ERR_INVALID, "rel must be 0 (R) or 1 (S)");
+  if (gpu_bits < 0 || gpu_bits > 10 || local_bits < 0 || local_bits > 20)
+    return fail(c, HJ_ERR_INVALID, "gpu_bits 0..10, local_bits 0..20");
+  if (n && (!keys || !pays)) return fail(c, HJ_ERR_INVALID, "null column with n > 0");
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  HostPlan hp;
+  int rc = prepare(c, hp, n, 0, local_bits, false, gpu_bits, 1, PLAN_SEND);
+  const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
+  const size_t nq = (size_t)1 << hp.qbits();
+  if (rc == HJ_OK) rc = ensure(c, c->xsend[rel], n * tb + 16);
+  if (rc == HJ_OK) rc = ensure(c, c->xcnt[rel], nq * 4);
+  if (rc == HJ_OK) {
+    Plan P = device_plan(c, hp, keys, pays, n, nullptr, nullptr, 0);
+    P.rel[0].t1 = c->xsend[rel].p;
+    P.rel[0].cnt = (uint32_t*)c->xcnt[rel].p;
+    c->launches = 0;
+    cudaError_t e = cudaMemsetAsync(c->xcnt[rel].p, 0, nq * 4, c->stream);
+    if (e != cudaSuccess) rc = fail(c, HJ_ERR_CUDA, "memset: %s", cudaGetErrorString(e));
+    if (rc == HJ_OK) rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P);
+    if (rc == HJ_OK) {
+      const uint32_t F1 = 1u << hp.pb();
+      unsigned long long* pst = (unsigned long long*)c->h_res;  // >= F1 + 1 entries (pinned, 8 KB + 64)
+      e = cudaMemcpyAsync(pst, P.rel[0].pst, (F1 + 1) * 8, cudaMemcpyDeviceToHost, c->stream);
+      if (e == cudaSuccess) e = cudaStreamSynchronize(c->stream);
+      if (e != cudaSuccess) rc = fail(c, HJ_ERR_CUDA, "exchange pack: %s", cudaGetErrorString(e));
+      else {
+        const int G = 1 << gpu_bits;
+        for (int j = 0; j < G; ++j) dest_counts[j] = pst[(size_t)(j + 1) << hp.b1] - pst[(size_t)j << hp.b1];
+        *send_out = c->xsend[rel].p;
+        *counts_out = (const uint32_t*)c->xcnt[rel].p;
+      }
+    }
+  }
+  cudaSetDevice(prev);
+  return rc;
+}
+
+int hj_join_received(hj_ctx* h, const void* R_recv, uint64_t nR, const uint32_t* R_counts, const void* S_recv, uint64_t nS,
+                     const uint32_t* S_counts, int nsrc, int local_bits, int out_mode, hj_result* res) {
+  if (!h || !res) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  if (out_mode != HJ_OUT_COUNT_CHECKSUM && out_mode != HJ_OUT_MATERIALIZE)
+    return fail(c, HJ_ERR_INVALID, "bad out_mode %d", out_mode);
+  if (nsrc < 1 || nsrc > 1024 || local_bits < 0 || local_bits > 20)
+    return fail(c, HJ_ERR_INVALID, "nsrc 1..1024, local_bits 0..20");
+  if (!R_counts || !S_counts || (nR && !R_recv) || (nS && !S_recv)) return fail(c, HJ_ERR_INVALID, "null argument");
+  memset(res, 0, sizeof *res);
+  if (nR == 0 || nS == 0) return HJ_OK;
+  const bool mat = out_mode == HJ_OUT_MATERIALIZE;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  HostPlan hp;
+  int rc = prepare(c, hp, nR, nS, local_bits, mat, 0, nsrc, PLAN_RECV);
+  if (rc == HJ_OK) {
+    Plan P = device_plan(c, hp, nullptr, nullptr, nR, nullptr, nullptr, nS);
+    P.rel[0].t1 = const_cast<void*>(R_recv);
+    P.rel[1].t1 = const_cast<void*>(S_recv);
+    P.rel[0].cnt = const_cast<uint32_t*>(R_counts);
+    P.rel[1].cnt = const_cast<uint32_t*>(S_counts);
+    c->launches = 0;
+    rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P);
+    if (rc == HJ_OK) rc = c->key_bytes == 4 ? launch_pass2<uint32_t>(c, hp, P) : launch_pass2<uint64_t>(c, hp, P);
+    if (rc == HJ_OK) rc = finish_join(c, hp, P, mat, res);
   }
   cudaSetDevice(prev);
   return rc;

@@ -53,17 +53,47 @@ __device__ __forceinline__ uint64_t pair_sig(uint64_t r_pay, uint64_t s_pay) {
 struct SlotHash {
   int B, lg, nfold;
 };
+// h ^ (h >> lg) ^ (h >> 2lg) ^ (h >> 3lg), shifts clamped at 32 (funnel shift, no branches)
 __device__ __forceinline__ uint32_t slot_fold(uint32_t h, const SlotHash& H) {
-  uint32_t r = h;
-  if (H.nfold >= 1) r ^= h >> H.lg;
-  if (H.nfold >= 2) r ^= h >> (2 * H.lg);
-  if (H.nfold >= 3) r ^= h >> (3 * H.lg);
+  const uint32_t r = h ^ __funnelshift_rc(h, 0u, H.lg) ^ __funnelshift_rc(h, 0u, 2 * H.lg) ^
+                     __funnelshift_rc(h, 0u, 3 * H.lg);
   return r & ((1u << H.lg) - 1);
 }
 __device__ __forceinline__ uint32_t slot_of(uint32_t key, const SlotHash& H) { return slot_fold(key >> H.B, H); }
 __device__ __forceinline__ uint32_t slot_of(uint64_t key, const SlotHash& H) {
   const uint64_t h64 = key >> H.B;
   return slot_fold((uint32_t)h64 ^ ((uint32_t)(h64 >> 32) * 0x9E3779B1u), H);
+}
+
+// ---- TMA 1-D bulk copies + mbarriers (sm_90+/sm_100a PTX) ---------------------------------
+__device__ __forceinline__ uint32_t smem_u32(const void* p) { return (uint32_t)__cvta_generic_to_shared(p); }
+__device__ __forceinline__ void mbar_init(unsigned long long* bar, uint32_t count) {
+  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count) : "memory");
+}
+__device__ __forceinline__ void fence_mbar_init() { asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory"); }
+__device__ __forceinline__ void fence_proxy_async() { asm volatile("fence.proxy.async.shared::cta;" ::: "memory"); }
+__device__ __forceinline__ void mbar_arrive_expect_tx(unsigned long long* bar, uint32_t bytes) {
+  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes) : "memory");
+}
+// global -> shared bulk copy; dst, src 16-byte aligned, bytes a multiple of 16
+__device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, unsigned long long* bar) {
+  asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+                   smem_u32(dst)),
+               "l"(src), "r"(bytes), "r"(smem_u32(bar))
+               : "memory");
+}
+__device__ __forceinline__ bool mbar_try_wait(unsigned long long* bar, uint32_t parity) {
+  uint32_t ok;
+  asm volatile(
+      "{\n\t.reg .pred p;\n\tmbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n\tselp.u32 %0, 1, 0, p;\n\t}"
+      : "=r"(ok)
+      : "r"(smem_u32(bar)), "r"(parity)
+      : "memory");
+  return ok != 0;
+}
+__device__ __forceinline__ void mbar_wait(unsigned long long* bar, uint32_t parity) {
+  while (!mbar_try_wait(bar, parity)) {
+  }
 }
 
 __device__ __forceinline__ uint32_t lanemask_lt() {

@@ -21,7 +21,7 @@ namespace hj {
 constexpr uint32_t NIL16 = 0xffffu;
 
 struct JoinJob {
-  uint32_t item, nr;
+  uint32_t item, nr, shift;  // shift: tuples between the 16-byte aligned copy start and rb
   unsigned long long rb, sb, se;
 };
 
@@ -30,7 +30,7 @@ struct JoinJob {
 __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items) {
   JoinJob j;
   j.item = atomicAdd(&P.counters[CNT_NEXT_ITEM], 1u);
-  j.nr = 0;
+  j.nr = j.shift = 0;
   j.rb = j.sb = j.se = 0;
   if (j.item < total_items) {
     const uint32_t np = 1u << P.B;
@@ -53,33 +53,47 @@ __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items
   return j;
 }
 
+// TMA bulk copy of a job's R chunk (the 16-byte aligned superset) into an smem tile buffer.
+template <typename T>
+__device__ __forceinline__ void issue_r_copy(const Plan& P, JoinJob& j, T* buf, unsigned long long* bar) {
+  const uintptr_t a = reinterpret_cast<uintptr_t>((const T*)P.rel[0].t2 + j.rb);
+  const uintptr_t a0 = a & ~(uintptr_t)15;
+  const uint32_t bytes = (uint32_t)(((a + (uintptr_t)j.nr * sizeof(T) - a0) + 15) & ~(uintptr_t)15);
+  j.shift = (uint32_t)((a - a0) / sizeof(T));
+  fence_proxy_async();  // prior generic-proxy reads of buf (the item before last) are ordered before
+  mbar_arrive_expect_tx(bar, bytes);
+  bulk_g2s(buf, reinterpret_cast<const void*>(a0), bytes, bar);
+}
+
 __device__ __forceinline__ void bar_compute(int nthreads) {  // named barrier 1: compute warps only
   asm volatile("bar.sync 1, %0;" ::"r"(nthreads) : "memory");
 }
 
 // Block = NT compute threads + one scheduler warp. The scheduler warp claims and decodes item
-// k+1 while the compute warps join item k (it only joins the end-of-item barrier), so the
-// dependent global loads of the item lookup never stall the join.
+// k+1 and starts its R chunk's TMA bulk copy into the other half of a double-buffered smem tile
+// while the compute warps join item k; it only joins the end-of-item barrier. So neither the
+// dependent global loads of the item lookup nor the R-chunk load sit on the join's critical path.
 //
 // Output of the materialized mode: per probe round every thread knows the match count of each
 // of its S tuples (first chain walk, which also keeps the first match's payload); the compute
-// warps reserve the round's total with ONE global atomicAdd, then each warp carves its range
-// per tuple slot with a shared-memory atomic and lanes write their pairs at warp-contiguous
-// positions (coalesced stores). This replaces the paper's per-warp buffer + global atomic per
-// flush. Chains are re-walked only for S tuples with more than one match.
+// warps reserve the round's total with ONE global atomicAdd, each warp's base comes from a scan
+// of the warp totals, and lanes write their pairs at warp-contiguous positions (coalesced
+// stores). This replaces the paper's per-warp buffer + global atomic per flush.
+// Chains are re-walked only for S tuples with more than one match.
 template <typename K, int NT, int SPT, bool MAT>
-__global__ void __launch_bounds__(NT + 32, 3) k_join(Plan P) {
+__global__ void __launch_bounds__(NT + 32, 2) k_join(Plan P) {
   using TT = Tup<K>;
   using T = typename TT::T;
   extern __shared__ __align__(16) unsigned char s_raw[];
   const SlotHash H = P.H;
   const uint32_t nb = 1u << H.lg;
-  T* s_rt = reinterpret_cast<T*>(s_raw);                        // CR tuples
-  uint32_t* s_head = reinterpret_cast<uint32_t*>(s_rt + P.CR);  // nb
-  uint16_t* s_next = reinterpret_cast<uint16_t*>(s_head + nb);  // CR
+  const uint32_t cap = (P.CR + 3) & ~1u;  // tile buffer in tuples: +2 for the aligned superset, even -> 16 B aligned
+  T* s_rtb = reinterpret_cast<T*>(s_raw);                            // 2 x cap tuples
+  uint32_t* s_head = reinterpret_cast<uint32_t*>(s_rtb + 2 * cap);   // nb
+  uint16_t* s_next = reinterpret_cast<uint16_t*>(s_head + nb);       // CR
   __shared__ JoinJob s_jobs[2];
+  __shared__ __align__(8) unsigned long long s_bar[2];
   __shared__ unsigned long long s_base;
-  __shared__ uint32_t s_wcur;
   __shared__ uint32_t s_wsum[NT / 32];
   __shared__ unsigned long long s_red[2][NT / 32 + 1];
 
@@ -91,19 +105,30 @@ __global__ void __launch_bounds__(NT + 32, 3) k_join(Plan P) {
   const T* ssrc = (const T*)P.rel[1].t2;
   unsigned long long my_cnt = 0, my_chk = 0;
 
-  if (sched && lane == 0) s_jobs[0] = claim_job(P, total_items);
+  if (threadIdx.x == NT) {
+    mbar_init(&s_bar[0], 1);
+    mbar_init(&s_bar[1], 1);
+    fence_mbar_init();
+    JoinJob j = claim_job(P, total_items);
+    if (j.item < total_items) issue_r_copy<T>(P, j, s_rtb, &s_bar[0]);
+    s_jobs[0] = j;
+  }
   __syncthreads();
 
   for (uint32_t it = 0;; ++it) {
     const JoinJob job = s_jobs[it & 1];
     if (job.item >= total_items) break;
     if (sched) {
-      if (lane == 0) s_jobs[(it + 1) & 1] = claim_job(P, total_items);
+      if (lane == 0) {
+        JoinJob j = claim_job(P, total_items);
+        if (j.item < total_items) issue_r_copy<T>(P, j, s_rtb + ((it + 1) & 1) * cap, &s_bar[(it + 1) & 1]);
+        s_jobs[(it + 1) & 1] = j;
+      }
       __syncthreads();  // end-of-item barrier (matches the compute warps' one below)
       continue;
     }
 
-    // ---- issue the first probe round's S loads, then the R chunk (all in flight together) ----
+    // ---- first probe round's S loads (in flight during the build) --------------------------
     K sk[SPT], sp[SPT];
     auto load_s = [&](unsigned long long base) {
       #pragma unroll
@@ -117,20 +142,9 @@ __global__ void __launch_bounds__(NT + 32, 3) k_join(Plan P) {
       }
     };
     load_s(job.sb);
-    {
-      const T* rsrc = (const T*)P.rel[0].t2 + job.rb;
-      for (uint32_t i = threadIdx.x; i < nb; i += NT) s_head[i] = NIL16;
-      constexpr int U = 4;
-      for (uint32_t i = threadIdx.x; i < job.nr; i += U * NT) {
-        T v[U];
-        #pragma unroll
-        for (int u = 0; u < U; ++u)
-          if (i + u * NT < job.nr) v[u] = __ldcs(rsrc + i + u * NT);
-        #pragma unroll
-        for (int u = 0; u < U; ++u)
-          if (i + u * NT < job.nr) s_rt[i + u * NT] = v[u];
-      }
-    }
+    for (uint32_t i = threadIdx.x; i < nb; i += NT) s_head[i] = NIL16;
+    const T* s_rt = s_rtb + (it & 1) * cap + job.shift;
+    mbar_wait(&s_bar[it & 1], (it >> 1) & 1);  // R chunk landed (TMA)
     bar_compute(NT);
     // ---- build (a6): wait-free push-front insert (Listing 2) ----------------------
     for (uint32_t i = threadIdx.x; i < job.nr; i += NT)
@@ -180,12 +194,15 @@ __global__ void __launch_bounds__(NT + 32, 3) k_join(Plan P) {
         if (threadIdx.x == 0) {
           uint32_t tot = 0;
           #pragma unroll
-          for (int w = 0; w < NT / 32; ++w) tot += s_wsum[w];
+          for (int w = 0; w < NT / 32; ++w) {
+            const uint32_t c = s_wsum[w];
+            s_wsum[w] = tot;  // exclusive warp base
+            tot += c;
+          }
           s_base = tot ? atomicAdd(&P.results[RES_CURSOR], (unsigned long long)tot) : 0ull;
-          s_wcur = 0;
         }
         bar_compute(NT);
-        const unsigned long long gbase = s_base;
+        unsigned long long pos0 = s_base + s_wsum[warp];
         #pragma unroll
         for (int j = 0; j < SPT; ++j) {
           // warp-exclusive scan of m[j]; the common case (every m <= 1) is one ballot
@@ -204,11 +221,8 @@ __global__ void __launch_bounds__(NT + 32, 3) k_join(Plan P) {
             excl = x - m[j];
             wtot = __shfl_sync(0xffffffffu, x, 31);
           }
-          if (wtot == 0) continue;
-          uint32_t wb = 0;
-          if (lane == 0) wb = atomicAdd(&s_wcur, wtot);
-          wb = __shfl_sync(0xffffffffu, wb, 0);
-          unsigned long long pos = gbase + wb + excl;
+          unsigned long long pos = pos0 + excl;
+          pos0 += wtot;
           if (m[j] == 1) {
             if (pos < P.out_cap) {
               out_r[pos] = rfirst[j];
@@ -227,10 +241,10 @@ __global__ void __launch_bounds__(NT + 32, 3) k_join(Plan P) {
             }
           }
         }
-        bar_compute(NT);  // s_base / s_wcur are reused by the next round
+        bar_compute(NT);  // s_base / s_wsum are reused by the next round
       }
     }
-    __syncthreads();  // end of item: s_rt / s_head are rewritten, s_jobs[it+1] is ready
+    __syncthreads();  // end of item: the tile buffer and s_head are reused, s_jobs[it+1] is ready
   }
 
   // ---- aggregate: warp shuffle reduce, then one 64-bit atomic per block --------

@@ -19,28 +19,23 @@ namespace hj {
 
 // ------------------------------------------------------------------------------------------
 // a1: histogram. grid = (blocks_per_rel, 2). Each block counts a contiguous, 16-byte aligned
-// range of one relation's keys in 2^B shared-memory counters (smem atomics measured at ~6
-// tuples/clk/SM on B200, tools/microbench/mb_rank.cu), then merges non-zero counters with
-// one global RED each. For B > 15 (more than 128 KB of counters) SMEM = false counts with
-// global atomics directly (correct, slower; not used by the benchmark configs).
+// range of one relation's keys in 2^qbits shared-memory counters indexed by the planner's
+// q-order bin (smem atomics measured at ~6 tuples/clk/SM on B200, tools/microbench/mb_rank.cu),
+// then merges non-zero counters with one global RED each (coalesced). For qbits > 15 (more than
+// 128 KB of counters) SMEM = false counts with global atomics directly (correct, slower).
 // ------------------------------------------------------------------------------------------
-template <typename K, bool SMEM>
+template <typename K, bool SMEM, bool GD>
 __global__ void __launch_bounds__(1024) k_hist(Plan P) {
   extern __shared__ uint32_t s_hist[];
   const int rel = blockIdx.y;
   const RelDev& R = P.rel[rel];
   const unsigned long long n = R.n;
-  const uint32_t np = 1u << P.B;
-  const uint32_t mask = np - 1;
+  const uint32_t np = 1u << P.qbits();
   if (SMEM) {
     for (uint32_t i = threadIdx.x; i < np; i += blockDim.x) s_hist[i] = 0;
     __syncthreads();
   }
   uint32_t* h = SMEM ? s_hist : R.cnt;
-  // counters are indexed by q = (p & (2^b1-1)) << b2 | p >> b1, the planner's order
-  const int b1 = P.b1, b2 = P.b2;
-  const uint32_t mb1 = (1u << b1) - 1;
-  auto bin = [&](uint32_t p) -> uint32_t { return ((p & mb1) << b2) | (p >> b1); };
   constexpr int VEC = 16 / sizeof(K);
   unsigned long long per = (n + gridDim.x - 1) / gridDim.x;
   per = (per + VEC - 1) / VEC * VEC;
@@ -63,18 +58,18 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P) {
         for (int u = 0; u < U; ++u) {
           const K* e = reinterpret_cast<const K*>(&x[u]);
           #pragma unroll
-          for (int t = 0; t < VEC; ++t) atomicAdd(&h[bin((uint32_t)(e[t]) & mask)], 1u);
+          for (int t = 0; t < VEC; ++t) atomicAdd(&h[qbin<GD>(e[t], P)], 1u);
         }
       }
       for (; v < nvec; v += blockDim.x) {
         uint4 x = __ldcs(kv + v);
         const K* e = reinterpret_cast<const K*>(&x);
         #pragma unroll
-        for (int t = 0; t < VEC; ++t) atomicAdd(&h[bin((uint32_t)(e[t]) & mask)], 1u);
+        for (int t = 0; t < VEC; ++t) atomicAdd(&h[qbin<GD>(e[t], P)], 1u);
       }
       i = lo + nvec * VEC;
     }
-    for (unsigned long long j = i + threadIdx.x; j < hi; j += blockDim.x) atomicAdd(&h[bin((uint32_t)keys[j] & mask)], 1u);
+    for (unsigned long long j = i + threadIdx.x; j < hi; j += blockDim.x) atomicAdd(&h[qbin<GD>(keys[j], P)], 1u);
   }
   if (SMEM) {
     __syncthreads();
@@ -86,73 +81,97 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P) {
 }
 
 // ------------------------------------------------------------------------------------------
-// a2 + a5: the planner. One block of 1024 threads; 2^B <= 2^20 entries per relation.
-//   off[q]  = exclusive scan of cnt[p(q)] in q-order          (co-partition starts, T2)
-//   cur1[d1] = off[d1 << b2], cur2[q] = off[q]                (pass reservation cursors)
-//   cst[d1]  = exclusive scan of ceil(|partition d1| / C2)    (pass-2 chunk list)
-//   ist[q]   = exclusive scan of items(q),  items(q) = ceil(|R_q|/CR) * ceil(|S_q|/CS) if both
-//              non-empty else 0                                (join work list)
+// a2 + a5: the planner. grid = ceil(2^qbits / 1024) blocks of 1024 threads.
+//   off[q]  = exclusive scan over q of sum_s cnt[s][q]             (co-partition starts in T2)
+//   cur2[q] = off[q]                                               (pass-2 reservation cursors)
+//   pst[i]  = exclusive scan of piece sizes, i = (s, D)            (pass-2 input pieces in T1)
+//   cur1[D] = pst[D] (one source)                                  (pass-1 reservation cursors)
+//   cst[i]  = exclusive scan of ceil(|piece i| / C2)               (pass-2 chunk list)
+//   ist[q]  = exclusive scan of items(q), items(q) = ceil(|R_q|/CR) * ceil(|S_q|/CS) if both
+//             non-empty else 0                                     (join work list)
+// Block b owns q in [1024 b, 1024 (b+1)), one q per thread, so every store is coalesced. Each
+// block first sums all counts below its range itself (a redundant prefix: at most 2^qbits/1024
+// independent loads per thread, L2-resident), then scans its own range. With several sources
+// the blocks also sum piece sizes (a warp per piece). The last block (atomic ticket) scans the
+// pieces.
 // ------------------------------------------------------------------------------------------
-__device__ __forceinline__ uint32_t q_to_p(uint32_t q, int b1, int b2) {
-  const uint32_t d1 = q >> b2, d2 = q & ((1u << b2) - 1);
-  return (d2 << b1) | d1;
+__device__ __forceinline__ unsigned long long plan_items(const Plan& P, unsigned long long cr, unsigned long long cs) {
+  return (cr && cs) ? ((cr + P.CR - 1) / P.CR) * ((cs + P.CS - 1) / P.CS) : 0ull;
 }
 
-__device__ __forceinline__ unsigned long long plan_items(const Plan& P, uint32_t cr, uint32_t cs) {
-  return (cr && cs) ? (unsigned long long)((cr + P.CR - 1) / P.CR) * ((cs + P.CS - 1) / P.CS) : 0ull;
+__device__ __forceinline__ unsigned long long plan_count(const RelDev& R, int nsrc, uint32_t np, uint32_t q) {
+  unsigned long long c = 0;
+  for (int s = 0; s < nsrc; ++s) c += R.cnt[(size_t)s * np + q];
+  return c;
 }
 
-// grid = ceil(2^B / 1024) blocks; block b owns q in [1024 b, 1024 (b+1)), one q per thread, so
-// every store is coalesced. Each block first sums all counts below its range itself (a redundant
-// prefix: at most 2^B / 1024 independent loads per thread, L2-resident), then scans its own
-// range. The last block to finish (atomic ticket) builds the pass-2 chunk lists.
 __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   constexpr int NT = 1024;
   __shared__ unsigned long long s_tmp[NT / 32 + 1];
   __shared__ bool s_last;
-  const uint32_t np = 1u << P.B;
-  const uint32_t F1 = 1u << P.b1;
+  const uint32_t np = 1u << P.qbits();
   const uint32_t b = blockIdx.x;
+  const int nsrc = P.nsrc;
+  const bool items = P.mode != PLAN_SEND;
   // ---- prefix of everything below this block's range -------------------------------------
   unsigned long long sR = 0, sS = 0, sI = 0;
-  #pragma unroll 8
+  #pragma unroll 4
   for (uint32_t k = 0; k < b; ++k) {
-    const uint32_t cr = P.rel[0].cnt[k * NT + threadIdx.x], cs = P.rel[1].cnt[k * NT + threadIdx.x];
+    const unsigned long long cr = plan_count(P.rel[0], nsrc, np, k * NT + threadIdx.x);
+    const unsigned long long cs = plan_count(P.rel[1], nsrc, np, k * NT + threadIdx.x);
     sR += cr;
     sS += cs;
-    sI += plan_items(P, cr, cs);
+    if (items) sI += plan_items(P, cr, cs);
   }
   unsigned long long tot;
   block_exclusive_scan64<NT>(sR, s_tmp, &tot);
-  unsigned long long bR = tot;
+  const unsigned long long bR = tot;
   block_exclusive_scan64<NT>(sS, s_tmp, &tot);
-  unsigned long long bS = tot;
+  const unsigned long long bS = tot;
   block_exclusive_scan64<NT>(sI, s_tmp, &tot);
-  unsigned long long bI = tot;
+  const unsigned long long bI = tot;
   // ---- own range ---------------------------------------------------------------------------
   const uint32_t q = b * NT + threadIdx.x;
-  uint32_t cr = 0, cs = 0;
+  unsigned long long cr = 0, cs = 0;
   if (q < np) {
-    cr = P.rel[0].cnt[q];
-    cs = P.rel[1].cnt[q];
+    cr = plan_count(P.rel[0], nsrc, np, q);
+    cs = plan_count(P.rel[1], nsrc, np, q);
   }
   unsigned long long tR, tS, tI;
   const unsigned long long oR = bR + block_exclusive_scan64<NT>(cr, s_tmp, &tR);
   const unsigned long long oS = bS + block_exclusive_scan64<NT>(cs, s_tmp, &tS);
-  const unsigned long long oI = bI + block_exclusive_scan64<NT>(plan_items(P, cr, cs), s_tmp, &tI);
+  const unsigned long long oI = bI + block_exclusive_scan64<NT>(items ? plan_items(P, cr, cs) : 0ull, s_tmp, &tI);
   if (q < np) {
     P.rel[0].off[q] = oR;
     P.rel[0].cur2[q] = oR;
     P.rel[1].off[q] = oS;
     P.rel[1].cur2[q] = oS;
-    P.ist[q] = (uint32_t)oI;
+    if (items) P.ist[q] = (uint32_t)oI;
   }
   if (b == gridDim.x - 1 && threadIdx.x == 0) {
     P.rel[0].off[np] = bR + tR;
     P.rel[1].off[np] = bS + tS;
-    P.ist[np] = (uint32_t)(bI + tI);
+    if (items) P.ist[np] = (uint32_t)(bI + tI);
   }
-  // ---- last block: pass-2 chunk lists over the 2^b1 pass-1 partitions (b1 <= 10) ----------
+  // ---- several sources: piece sizes, a warp per piece (stored in pst[i + 1]) --------------
+  const uint32_t npieces = P.npieces();
+  const int pb = P.pb(), b2 = P.b2;
+  if (nsrc > 1) {
+    const uint32_t lane = threadIdx.x & 31, gw = b * (NT / 32) + (threadIdx.x >> 5), nw = gridDim.x * (NT / 32);
+    for (int rel = 0; rel < 2; ++rel) {
+      const RelDev& R = P.rel[rel];
+      for (uint32_t i = gw; i < npieces; i += nw) {
+        const uint32_t src = i >> pb, D = i & ((1u << pb) - 1);
+        const uint32_t* row = R.cnt + (size_t)src * np + ((size_t)D << b2);
+        unsigned long long c = 0;
+        for (uint32_t t = lane; t < (1u << b2); t += 32) c += row[t];
+        #pragma unroll
+        for (int o = 16; o; o >>= 1) c += __shfl_xor_sync(0xffffffffu, c, o);
+        if (lane == 0) R.pst[i + 1] = c;
+      }
+    }
+  }
+  // ---- last block: piece starts, pass-1 cursors, pass-2 chunk lists (npieces <= 1024) ------
   __threadfence();
   __syncthreads();
   if (threadIdx.x == 0) s_last = atomicAdd(&P.counters[CNT_PLAN_DONE], 1u) == gridDim.x - 1;
@@ -161,16 +180,28 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   __threadfence();
   for (int rel = 0; rel < 2; ++rel) {
     const RelDev& R = P.rel[rel];
-    unsigned long long nch = 0;
-    if (threadIdx.x < F1) {
-      const unsigned long long a = __ldcg(&R.off[(unsigned long long)threadIdx.x << P.b2]);
-      const unsigned long long e = __ldcg(&R.off[(unsigned long long)(threadIdx.x + 1) << P.b2]);
-      R.cur1[threadIdx.x] = a;
-      nch = (e - a + P.C2 - 1) / P.C2;
+    const uint32_t i = threadIdx.x;
+    unsigned long long sz = 0;
+    if (i < npieces) {
+      if (nsrc == 1)
+        sz = __ldcg(&R.off[(unsigned long long)(i + 1) << b2]) - __ldcg(&R.off[(unsigned long long)i << b2]);
+      else
+        sz = __ldcg(&R.pst[i + 1]);
     }
-    const unsigned long long cb = block_exclusive_scan64<NT>(nch, s_tmp, &tot);
-    if (threadIdx.x < F1) R.cst[threadIdx.x] = (uint32_t)cb;
-    if (threadIdx.x == 0) R.cst[F1] = (uint32_t)tot;
+    unsigned long long ptot;
+    const unsigned long long ps = block_exclusive_scan64<NT>(sz, s_tmp, &ptot);
+    const unsigned long long nch = (sz + P.C2 - 1) / P.C2;
+    unsigned long long ctot;
+    const unsigned long long cb = block_exclusive_scan64<NT>(nch, s_tmp, &ctot);
+    if (i < npieces) {
+      R.pst[i] = ps;
+      R.cst[i] = (uint32_t)cb;
+      if (nsrc == 1) R.cur1[i] = ps;
+    }
+    if (i == 0) {
+      R.pst[npieces] = ptot;
+      R.cst[npieces] = (uint32_t)ctot;
+    }
   }
 }
 
@@ -203,12 +234,13 @@ struct PassUnit {
 };
 
 // Round-robin unit walker: unit u = blockIdx.x + k * gridDim.x. MODE 2 keeps the current
-// (relation, d1) and advances d1 through the shared-memory chunk prefix instead of searching.
+// (relation, piece) and advances the piece through the shared-memory chunk prefix instead of
+// searching (units are visited in increasing order).
 template <typename K, int MODE, int TILE>
 struct UnitWalker {
   unsigned long long units0, units;
   int rel;
-  uint32_t d1;
+  uint32_t piece;
   __device__ __forceinline__ bool get(const Plan& P, unsigned long long u, PassUnit<K>& U, const uint32_t* s_cst,
                                       const unsigned long long* s_pst) {
     using T = typename Tup<K>::T;
@@ -226,16 +258,17 @@ struct UnitWalker {
     } else {
       if (r != rel) {
         rel = r;
-        d1 = 0;
+        piece = 0;
       }
       const uint32_t* cst = s_cst + r * 1025;
-      while (cst[d1 + 1] <= ul) ++d1;  // monotone in u: amortised ~gridDim / chunks-per-partition steps
-      const unsigned long long pa = s_pst[r * 1025 + d1], pb = s_pst[r * 1025 + d1 + 1];
-      const unsigned long long s0 = pa + (ul - cst[d1]) * TILE;
+      while (cst[piece + 1] <= ul) ++piece;  // monotone in u: amortised ~gridDim / chunks-per-piece steps
+      const unsigned long long pa = s_pst[r * 1025 + piece], pb = s_pst[r * 1025 + piece + 1];
+      const unsigned long long s0 = pa + (ul - cst[piece]) * TILE;
+      const uint32_t D = piece & ((1u << P.pb()) - 1);  // pass-1 digit of the piece
       U.src_k = (const T*)R.t1 + s0;
       U.src_p = nullptr;
       U.dst = R.t2;
-      U.cur = R.cur2 + ((unsigned long long)d1 << P.b2);
+      U.cur = R.cur2 + ((unsigned long long)D << P.b2);
       U.len = (uint32_t)min((unsigned long long)TILE, pb - s0);
     }
     return true;
@@ -299,7 +332,7 @@ __device__ __forceinline__ void pass_load(const PassUnit<K>& U, K (&kk)[ITEMS], 
   }
 }
 
-template <typename K, int MODE, int NT, int ITEMS>
+template <typename K, int MODE, int NT, int ITEMS, bool GD>
 __global__ void __launch_bounds__(NT, 1) k_pass(Plan P, int fanout_bits) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -315,25 +348,26 @@ __global__ void __launch_bounds__(NT, 1) k_pass(Plan P, int fanout_bits) {
   __shared__ uint32_t s_cst[MODE == 2 ? 2 * 1025 : 1];
   __shared__ unsigned long long s_pst[MODE == 2 ? 2 * 1025 : 1];
 
-  const uint32_t dmask = F - 1;
-  const int dshift = (MODE == 1) ? 0 : P.b1;
+  // digit of a key in this pass: D (pass 1, possibly widened by rank bits) or d2 (pass 2)
+  auto digit = [&](K key) -> uint32_t { return MODE == 1 ? dig1<GD>(key, P) : dig2(key, P); };
 
   if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
   UnitWalker<K, MODE, TILE> W;
   W.rel = -1;
-  W.d1 = 0;
+  W.piece = 0;
   if (MODE == 1) {
     W.units0 = P.tiles1[0];
     W.units = W.units0 + P.tiles1[1];
   } else {
-    for (uint32_t i = threadIdx.x; i <= (1u << P.b1); i += NT) {
+    const uint32_t npc = P.npieces();  // <= 1024
+    for (uint32_t i = threadIdx.x; i <= npc; i += NT) {
       s_cst[i] = P.rel[0].cst[i];
       s_cst[1025 + i] = P.rel[1].cst[i];
-      s_pst[i] = P.rel[0].off[(unsigned long long)i << P.b2];
-      s_pst[1025 + i] = P.rel[1].off[(unsigned long long)i << P.b2];
+      s_pst[i] = P.rel[0].pst[i];
+      s_pst[1025 + i] = P.rel[1].pst[i];
     }
-    W.units0 = P.rel[0].cst[1u << P.b1];
-    W.units = W.units0 + P.rel[1].cst[1u << P.b1];
+    W.units0 = P.rel[0].cst[npc];
+    W.units = W.units0 + P.rel[1].cst[npc];
   }
   __syncthreads();
 
@@ -357,8 +391,7 @@ __global__ void __launch_bounds__(NT, 1) k_pass(Plan P, int fanout_bits) {
     uint32_t rk[ITEMS];
     #pragma unroll
     for (int j = 0; j < ITEMS; ++j)
-      rk[j] = (pass_elem<K, MODE, NT>(j) < U.len) ? atomicAdd(&s_cnt[(uint32_t)(kk[j] >> dshift) & dmask], 1u)
-                                                  : 0xffffffffu;
+      rk[j] = (pass_elem<K, MODE, NT>(j) < U.len) ? atomicAdd(&s_cnt[digit(kk[j])], 1u) : 0xffffffffu;
     __syncthreads();
 
     // ---- scan digit counts; issue the reservation atomic (result consumed after the shuffle)
@@ -380,7 +413,7 @@ __global__ void __launch_bounds__(NT, 1) k_pass(Plan P, int fanout_bits) {
     // ---- shuffle into digit order in shared memory -----------------------------------------
     #pragma unroll
     for (int j = 0; j < ITEMS; ++j)
-      if (rk[j] != 0xffffffffu) s_buf[s_loc[(uint32_t)(kk[j] >> dshift) & dmask] + rk[j]] = TT::make(kk[j], pp[j]);
+      if (rk[j] != 0xffffffffu) s_buf[s_loc[digit(kk[j])] + rk[j]] = TT::make(kk[j], pp[j]);
     if (threadIdx.x < F) s_gd[threadIdx.x] = gres - myloc;
     __syncthreads();
 
@@ -391,7 +424,7 @@ __global__ void __launch_bounds__(NT, 1) k_pass(Plan P, int fanout_bits) {
       const uint32_t i = j * NT + threadIdx.x;
       if (i < U.len) {
         const T t = s_buf[i];
-        __stcs(dst + (s_gd[(uint32_t)(TT::key(t) >> dshift) & dmask] + i), t);
+        __stcs(dst + (s_gd[digit(TT::key(t))] + i), t);
       }
     }
     __syncthreads();  // s_buf / s_loc / s_gd are rewritten by the next unit

@@ -6,25 +6,37 @@
 
 namespace hj {
 
-// Per-relation device state. Co-partition q-order: q = d1 << b2 | d2 where the key's radix
-// field p = key & (2^B - 1) splits into d1 = p & (2^b1 - 1) (pass 1) and d2 = p >> b1 (pass 2).
-// Partition d1 of pass 1 is then the contiguous q range [d1 << b2, (d1 + 1) << b2).
+// Radix field and co-partition order. The local radix field p = key & (2^B - 1) splits into
+// d1 = p & (2^b1 - 1) (pass 1) and d2 = p >> b1 (pass 2). On the multi-GPU exchange sender the
+// pass-1 digit is widened by g rank bits taken from just above the local field:
+//   D = ((key >> B) & (2^g - 1)) << b1 | d1        (pb = g + b1 bits)
+// Counts, offsets and cursors use q-order q = D << b2 | d2 over a q-space of qbits = pb + b2
+// bits, so pass-1 partition D is the contiguous q range [D << b2, (D + 1) << b2) and, on the
+// sender, rank j's co-partitions are the contiguous range [j << B, (j + 1) << B).
+// Pass 2 reads "pieces": piece i = (source s, D) = (i >> pb, i & (2^pb - 1)); on one GPU the
+// pieces are the pass-1 partitions, on the exchange receiver the d1-segments sent by each rank.
+enum { PLAN_FULL = 0, PLAN_SEND = 1, PLAN_RECV = 2 };
+
 struct RelDev {
   const void* keys;  // SoA input (caller-owned)
   const void* pays;
   unsigned long long n;
-  void* t1;                   // pass-1 output, AoS, n tuples
-  void* t2;                   // pass-2 output, AoS, n tuples, co-partitions contiguous in q-order
-  uint32_t* cnt;              // [2^B] histogram, q-order (k_hist translates p -> q)
-  unsigned long long* off;    // [2^B + 1] co-partition start, q-order (exclusive scan)
-  unsigned long long* cur1;   // [2^b1] pass-1 reservation cursors
-  unsigned long long* cur2;   // [2^B]  pass-2 reservation cursors (q-order)
-  uint32_t* cst;              // [2^b1 + 1] pass-2 chunk prefix (chunks of C2 tuples per d1)
+  void* t1;                   // pass-1 output / pass-2 input, AoS (the receive buffer on PLAN_RECV)
+  void* t2;                   // pass-2 output, AoS, co-partitions contiguous in q-order
+  uint32_t* cnt;              // nsrc rows of [2^qbits] counts, q-order (k_hist writes row 0)
+  unsigned long long* off;    // [2^qbits + 1] co-partition start (counts summed over rows)
+  unsigned long long* cur1;   // [2^pb] pass-1 reservation cursors
+  unsigned long long* cur2;   // [2^qbits] pass-2 reservation cursors
+  unsigned long long* pst;    // [npieces + 1] pass-2 input piece starts in t1
+  uint32_t* cst;              // [npieces + 1] pass-2 chunk prefix (chunks of C2 tuples per piece)
 };
 
 struct Plan {
   RelDev rel[2];  // 0 = R (build), 1 = S (probe)
-  int B, b1, b2;
+  int B, b1, b2;  // local radix field
+  int g;          // rank bits in the pass-1 digit (PLAN_SEND), else 0
+  int nsrc;       // count rows / piece sources (PLAN_RECV: ranks), else 1
+  int mode;       // PLAN_FULL, PLAN_SEND, PLAN_RECV
   uint32_t C2;           // pass-2 chunk (tile) size in tuples
   uint32_t CR, CS;       // join item capacities: R tuples (smem build) and S tuples per item
   uint32_t* ist;         // [2^B + 1] join item prefix (q-order)
@@ -35,7 +47,26 @@ struct Plan {
   unsigned long long out_cap;
   unsigned long long tiles1[2];  // pass-1 tiles per relation (host-known)
   SlotHash H;            // in-partition slot hash (lg = log2 of hash-table slots per join item)
+  __host__ __device__ int pb() const { return g + b1; }
+  __host__ __device__ int qbits() const { return g + B; }
+  __host__ __device__ uint32_t npieces() const { return (uint32_t)nsrc << (g + b1); }
 };
+
+// pass-1 digit D, pass-2 digit d2 and the q-order histogram bin of a key
+template <bool GD, typename K>
+__device__ __forceinline__ uint32_t dig1(K key, const Plan& P) {
+  uint32_t d = (uint32_t)key & ((1u << P.b1) - 1);
+  if (GD) d |= ((uint32_t)(key >> P.B) & ((1u << P.g) - 1)) << P.b1;
+  return d;
+}
+template <typename K>
+__device__ __forceinline__ uint32_t dig2(K key, const Plan& P) {
+  return (uint32_t)(key >> P.b1) & ((1u << P.b2) - 1);
+}
+template <bool GD, typename K>
+__device__ __forceinline__ uint32_t qbin(K key, const Plan& P) {
+  return (dig1<GD>(key, P) << P.b2) | dig2(key, P);
+}
 
 enum { CNT_NEXT_ITEM = 0, CNT_PLAN_DONE = 1 };
 enum { RES_MATCHES = 0, RES_CHECKSUM = 1, RES_CURSOR = 2 };

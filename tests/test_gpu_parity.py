@@ -221,20 +221,28 @@ def test_full_size_closed_form(hj, cfg):
     materialized output, the pairs sorted by s_pay are exactly (rho(j), j)."""
     w = W.CONFIGS[cfg]
     Rk, Rp, Sk, Sp = W.torch_generate(w, device="cuda")
+    cdf = W.zipf_cdf(w.nR, w.z) if w.dist == "zipf" else None
+    # the device-generated inputs equal the host generator on a sample of rows
+    rows = np.random.default_rng(0).integers(0, w.nS, 1 << 16).astype(np.uint64)
+    rho_s = W.np_rho_for(w, rows, cdf)
+    Rk_h = W.np_generate(w, s_rows=slice(0, 0))[0]  # R keys only
+    assert np.array_equal(to_np(Sk[torch.from_numpy(rows.astype(np.int64)).cuda()], 4), Rk_h[rho_s.astype(np.int64)]), \
+        "device generator differs from the host generator"
     ctx = hj.context(0, 4, 4)
     res = ctx.join(Rk, Rp, Sk, Sp, radix_bits=w.radix_bits, out_mode=w.out_mode)
     torch.cuda.synchronize()
     del Rk, Rp, Sk, Sp
-    cdf = W.zipf_cdf(w.nR, w.z) if w.dist == "zipf" else None
     j = np.arange(w.nS, dtype=np.uint64)
     rho = W.np_rho_for(w, j, cdf)
-    assert res.matches == w.nS
+    assert res.matches == w.nS, f"matches {res.matches} != |S| {w.nS} (items {res.n_items})"
     if w.out_mode == 0:
-        assert res.checksum == int(np_sig(rho, j).sum(dtype=np.uint64))
+        exp = int(np_sig(rho, j).sum(dtype=np.uint64))
+        assert res.checksum == exp, f"checksum {res.checksum:#x} != closed form {exp:#x} (items {res.n_items})"
     if w.out_mode == 1:
         s_pay = res.s_pay
         order = torch.argsort(s_pay)
         r_sorted = to_np(res.r_pay[order], 4).astype(np.uint64)
         s_sorted = to_np(s_pay[order], 4).astype(np.uint64)
-        assert np.array_equal(s_sorted, j)
-        assert np.array_equal(r_sorted, rho)
+        assert np.array_equal(s_sorted, j), "materialized s_pay is not a permutation of S's rows"
+        bad = np.nonzero(r_sorted != rho)[0]
+        assert len(bad) == 0, f"{len(bad)} materialized pairs differ, first at s_pay {bad[:5]}"
