@@ -299,7 +299,7 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P) {
   if (hp.mode != PLAN_RECV) {
     constexpr int IT = pass_items<K>();
     const void* f = gd ? (const void*)k_pass<K, 1, PASS_NT, IT, true> : (const void*)k_pass<K, 1, PASS_NT, IT, false>;
-    const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.pb()) * 16;
+    const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.pb()) * 24 + 16;
     int g = grid_for(c, f, PASS_NT, sm, P.tiles1[0] + P.tiles1[1]);
     if (gd) k_pass<K, 1, PASS_NT, IT, true><<<g, PASS_NT, sm, st>>>(P, hp.pb());
     else k_pass<K, 1, PASS_NT, IT, false><<<g, PASS_NT, sm, st>>>(P, hp.pb());
@@ -315,7 +315,7 @@ template <typename K>
 int launch_pass2(Ctx* c, const HostPlan& hp, const Plan& P) {
   constexpr int IT = pass_items<K>();
   const void* f = (const void*)k_pass<K, 2, PASS_NT, IT, false>;
-  const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.b2) * 16;
+  const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.b2) * 24 + 16;
   // chunks: at most n / C2 + npieces per relation
   unsigned long long units = (P.rel[0].n + P.rel[1].n) / hp.C2 + 2ull * hp.npieces() + 2;
   int g = grid_for(c, f, PASS_NT, sm, units);

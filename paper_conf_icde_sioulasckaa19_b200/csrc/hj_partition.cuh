@@ -100,6 +100,7 @@ __device__ __forceinline__ unsigned long long plan_items(const Plan& P, unsigned
 }
 
 __device__ __forceinline__ unsigned long long plan_count(const RelDev& R, int nsrc, uint32_t np, uint32_t q) {
+  if (nsrc == 1) return R.cnt[q];
   unsigned long long c = 0;
   for (int s = 0; s < nsrc; ++s) c += R.cnt[(size_t)s * np + q];
   return c;
@@ -115,7 +116,7 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   const bool items = P.mode != PLAN_SEND;
   // ---- prefix of everything below this block's range -------------------------------------
   unsigned long long sR = 0, sS = 0, sI = 0;
-  #pragma unroll 4
+  #pragma unroll 8
   for (uint32_t k = 0; k < b; ++k) {
     const unsigned long long cr = plan_count(P.rel[0], nsrc, np, k * NT + threadIdx.x);
     const unsigned long long cs = plan_count(P.rel[1], nsrc, np, k * NT + threadIdx.x);
@@ -225,26 +226,26 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
 // atomics produced (partitions are multisets, reading S9).
 // ------------------------------------------------------------------------------------------
 template <typename K>
-struct PassUnit {
+struct __align__(16) PassUnit {
   const void* src_k;  // MODE 1: key column at the unit start; MODE 2: first AoS tuple of the unit
   const void* src_p;  // MODE 1: payload column at the unit start
   void* dst;          // output buffer (T1 or T2) of the unit's relation
   unsigned long long* cur;  // reservation cursors: cur1 (MODE 1) or &cur2[d1 << b2] (MODE 2)
   uint32_t len;
+  uint32_t valid;
 };
 
-// Round-robin unit walker: unit u = blockIdx.x + k * gridDim.x. MODE 2 keeps the current
-// (relation, piece) and advances the piece through the shared-memory chunk prefix instead of
-// searching (units are visited in increasing order).
+// Unit u (round-robin: u = blockIdx.x + k * gridDim.x) -> its descriptor. MODE 2 maps the chunk
+// to its piece by binary search in the shared-memory chunk prefix (stateless: no registers live
+// across the unit loop).
 template <typename K, int MODE, int TILE>
 struct UnitWalker {
   unsigned long long units0, units;
-  int rel;
-  uint32_t piece;
   __device__ __forceinline__ bool get(const Plan& P, unsigned long long u, PassUnit<K>& U, const uint32_t* s_cst,
-                                      const unsigned long long* s_pst) {
+                                      const unsigned long long* s_pst) const {
     using T = typename Tup<K>::T;
-    if (u >= units) return false;
+    U.valid = u < units;
+    if (!U.valid) return false;
     const int r = (u < units0) ? 0 : 1;
     const unsigned long long ul = r ? u - units0 : u;
     const RelDev& R = P.rel[r];
@@ -256,15 +257,16 @@ struct UnitWalker {
       U.cur = R.cur1;
       U.len = (uint32_t)min((unsigned long long)TILE, R.n - s0);
     } else {
-      if (r != rel) {
-        rel = r;
-        piece = 0;
-      }
       const uint32_t* cst = s_cst + r * 1025;
-      while (cst[piece + 1] <= ul) ++piece;  // monotone in u: amortised ~gridDim / chunks-per-piece steps
-      const unsigned long long pa = s_pst[r * 1025 + piece], pb = s_pst[r * 1025 + piece + 1];
-      const unsigned long long s0 = pa + (ul - cst[piece]) * TILE;
-      const uint32_t D = piece & ((1u << P.pb()) - 1);  // pass-1 digit of the piece
+      const uint32_t uc = (uint32_t)ul;
+      uint32_t lo = 0, hi = P.npieces();  // largest piece with cst[piece] <= uc
+      while (hi - lo > 1) {
+        const uint32_t mid = (lo + hi) >> 1;
+        if (cst[mid] <= uc) lo = mid; else hi = mid;
+      }
+      const unsigned long long pa = s_pst[r * 1025 + lo], pb = s_pst[r * 1025 + lo + 1];
+      const unsigned long long s0 = pa + (unsigned long long)(uc - cst[lo]) * TILE;
+      const uint32_t D = lo & ((1u << P.pb()) - 1);  // pass-1 digit of the piece
       U.src_k = (const T*)R.t1 + s0;
       U.src_p = nullptr;
       U.dst = R.t2;
@@ -332,29 +334,45 @@ __device__ __forceinline__ void pass_load(const PassUnit<K>& U, K (&kk)[ITEMS], 
   }
 }
 
+// Two-barrier software pipeline per unit i (one block of NT threads):
+//   phase 1  rank unit i (smem atomics)                                            | barrier
+//   phase 2  all threads: write unit i-1 out of s_buf (its run bases in s_gd[(i-1)&1]);
+//            threads d < F additionally scan unit i's digit counts (named barrier among them),
+//            reserve each run with one global atomic and store base - loc in s_gd[i&1]  | barrier
+//   phase 3  shuffle unit i into digit order in s_buf
+// so each reservation atomic's latency overlaps the previous unit's write-out.
 template <typename K, int MODE, int NT, int ITEMS, bool GD>
 __global__ void __launch_bounds__(NT, 1) k_pass(Plan P, int fanout_bits) {
   using TT = Tup<K>;
   using T = typename TT::T;
   constexpr int TILE = NT * ITEMS;
   static_assert(NT >= 1024, "fan-out up to 2^10 needs one digit per thread");
+  static_assert(TILE <= 65536 && ITEMS % 2 == 0, "16-bit packed ranks");
   extern __shared__ __align__(16) unsigned char s_raw[];
   const uint32_t F = 1u << fanout_bits;
   T* s_buf = reinterpret_cast<T*>(s_raw);                                          // TILE tuples
-  unsigned long long* s_gd = reinterpret_cast<unsigned long long*>(s_buf + TILE);  // F: run base - loc
-  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gd + F);                         // F
-  uint32_t* s_loc = s_cnt + F;                                                     // F
-  __shared__ uint32_t s_tmp[NT / 32 + 1];
+  unsigned long long* s_gd = reinterpret_cast<unsigned long long*>(s_buf + TILE);  // 2 x F: run base - loc
+  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gd + 2 * F);                     // F + 1 (spare)
+  uint32_t* s_loc = s_cnt + F + 4;                                                 // F
+  __shared__ uint32_t s_wt[NT / 32];
   __shared__ uint32_t s_cst[MODE == 2 ? 2 * 1025 : 1];
   __shared__ unsigned long long s_pst[MODE == 2 ? 2 * 1025 : 1];
 
-  // digit of a key in this pass: D (pass 1, possibly widened by rank bits) or d2 (pass 2)
-  auto digit = [&](K key) -> uint32_t { return MODE == 1 ? dig1<GD>(key, P) : dig2(key, P); };
+  // digit of a key in this pass: D (pass 1, possibly widened by rank bits) or d2 (pass 2);
+  // shifts and masks live in registers (not re-read from the parameter struct per tuple)
+  const uint32_t dsh = MODE == 1 ? 0u : (uint32_t)P.b1;
+  const uint32_t dmask = MODE == 1 ? ((1u << P.b1) - 1) : ((1u << P.b2) - 1);
+  const uint32_t gsh = (uint32_t)P.B, gmask = (1u << P.g) - 1, gup = (uint32_t)P.b1;
+  auto digit = [=](K key) -> uint32_t {
+    uint32_t d = (uint32_t)(key >> dsh) & dmask;
+    if (MODE == 1 && GD) d |= ((uint32_t)(key >> gsh) & gmask) << gup;
+    return d;
+  };
+  const uint32_t nscan = F < 32 ? 32u : F;  // threads in the digit scan (whole warps)
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
 
   if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
   UnitWalker<K, MODE, TILE> W;
-  W.rel = -1;
-  W.piece = 0;
   if (MODE == 1) {
     W.units0 = P.tiles1[0];
     W.units = W.units0 + P.tiles1[1];
@@ -371,67 +389,107 @@ __global__ void __launch_bounds__(NT, 1) k_pass(Plan P, int fanout_bits) {
   }
   __syncthreads();
 
-  PassUnit<K> U, Un;
+  // unit descriptors live in a 3-slot shared ring: one thread computes unit i+2 during unit i's
+  // phase 2 (slot (i+2) % 3 held unit i-1, whose fields were copied to registers already)
+  __shared__ PassUnit<K> s_desc[3];
+  const unsigned long long G = gridDim.x;
+  if (threadIdx.x == NT - 1) {
+    W.get(P, blockIdx.x, s_desc[0], s_cst, s_pst);
+    W.get(P, blockIdx.x + G, s_desc[1], s_cst, s_pst);
+  }
+  __syncthreads();
+  T* prev_dst = nullptr;  // unit i-1 awaiting write-out
+  uint32_t prev_len = 0;
   K kk[ITEMS], pp[ITEMS], kn[ITEMS], pn[ITEMS];
   unsigned long long u = blockIdx.x;
-  bool have = W.get(P, u, U, s_cst, s_pst);
-  if (have) pass_load<K, MODE, NT, ITEMS>(U, kn, pn);
+  if (s_desc[0].valid) pass_load<K, MODE, NT, ITEMS>(s_desc[0], kn, pn);
+  uint32_t it = 0, slot = 0;
 
-  while (have) {
+  auto write_out = [&](const unsigned long long* gd) {
+    if (prev_len == TILE) {
+      #pragma unroll
+      for (int j = 0; j < ITEMS; ++j) {
+        const uint32_t i = j * NT + threadIdx.x;
+        const T t = s_buf[i];
+        __stcs(prev_dst + (gd[digit(TT::key(t))] + i), t);
+      }
+    } else {
+      #pragma unroll
+      for (int j = 0; j < ITEMS; ++j) {
+        const uint32_t i = j * NT + threadIdx.x;
+        if (i < prev_len) {
+          const T t = s_buf[i];
+          __stcs(prev_dst + (gd[digit(TT::key(t))] + i), t);
+        }
+      }
+    }
+  };
+
+  while (s_desc[slot].valid) {
+    const uint32_t nslot = slot == 2 ? 0 : slot + 1;
     #pragma unroll
     for (int j = 0; j < ITEMS; ++j) {
       kk[j] = kn[j];
       pp[j] = pn[j];
     }
     // prefetch the next unit (in flight across this unit's barriers)
-    const bool have_next = W.get(P, u + gridDim.x, Un, s_cst, s_pst);
-    if (have_next) pass_load<K, MODE, NT, ITEMS>(Un, kn, pn);
+    if (s_desc[nslot].valid) pass_load<K, MODE, NT, ITEMS>(s_desc[nslot], kn, pn);
 
-    // ---- rank ------------------------------------------------------------------------------
-    uint32_t rk[ITEMS];
-    #pragma unroll
-    for (int j = 0; j < ITEMS; ++j)
-      rk[j] = (pass_elem<K, MODE, NT>(j) < U.len) ? atomicAdd(&s_cnt[digit(kk[j])], 1u) : 0xffffffffu;
-    __syncthreads();
-
-    // ---- scan digit counts; issue the reservation atomic (result consumed after the shuffle)
-    unsigned long long gres = 0;
-    uint32_t myloc = 0;
-    {
-      const uint32_t d = threadIdx.x;
-      const uint32_t c = (d < F) ? s_cnt[d] : 0u;
-      uint32_t tot;
-      myloc = block_exclusive_scan<NT>(c, s_tmp, &tot);
-      if (d < F) {
-        s_loc[d] = myloc;
-        s_cnt[d] = 0;
-        if (c) gres = atomicAdd(U.cur + d, (unsigned long long)c);
-      }
-    }
-    __syncthreads();
-
-    // ---- shuffle into digit order in shared memory -----------------------------------------
-    #pragma unroll
-    for (int j = 0; j < ITEMS; ++j)
-      if (rk[j] != 0xffffffffu) s_buf[s_loc[digit(kk[j])] + rk[j]] = TT::make(kk[j], pp[j]);
-    if (threadIdx.x < F) s_gd[threadIdx.x] = gres - myloc;
-    __syncthreads();
-
-    // ---- stream runs out (consecutive threads -> consecutive addresses within a run) -------
-    T* dst = (T*)U.dst;
+    // ---- phase 1: rank ------------------------------------------------------------------------
+    // elements past the unit's end count into the spare counter s_cnt[F] (no branches)
+    uint32_t rk[ITEMS / 2];  // ranks < TILE <= 2^16, two per register
+    const uint32_t ulen = s_desc[slot].len;
+    const bool full = ulen == TILE;
     #pragma unroll
     for (int j = 0; j < ITEMS; ++j) {
-      const uint32_t i = j * NT + threadIdx.x;
-      if (i < U.len) {
-        const T t = s_buf[i];
-        __stcs(dst + (s_gd[digit(TT::key(t))] + i), t);
+      const uint32_t d = (full || pass_elem<K, MODE, NT>(j) < ulen) ? digit(kk[j]) : F;
+      const uint32_t r = atomicAdd(&s_cnt[d], 1u);
+      if (j & 1) rk[j / 2] |= r << 16; else rk[j / 2] = r & 0xffffu;
+    }
+    __syncthreads();
+
+    // ---- phase 2: scan + reserve unit i (threads < F) | write unit i-1 out (all) ---------------
+    unsigned long long* gd = s_gd + (it & 1) * F;
+    if (threadIdx.x < nscan) {
+      const uint32_t d = threadIdx.x;
+      const uint32_t c = d < F ? s_cnt[d] : 0u;
+      uint32_t x = c;
+      #pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+        if (lane >= o) x += y;
+      }
+      if (lane == 31) s_wt[warp] = x;
+      asm volatile("bar.sync 1, %0;" ::"r"(nscan) : "memory");
+      uint32_t base = 0;
+      for (int w = 0; w < warp; ++w) base += s_wt[w];
+      const uint32_t loc = base + x - c;
+      if (d < F) {
+        s_loc[d] = loc;
+        s_cnt[d] = 0;
+        if (c) gd[d] = atomicAdd(s_desc[slot].cur + d, (unsigned long long)c) - loc;
       }
     }
-    __syncthreads();  // s_buf / s_loc / s_gd are rewritten by the next unit
-    U = Un;
-    u += gridDim.x;
-    have = have_next;
+    if (threadIdx.x == NT - 1)  // publish unit i+2
+      W.get(P, u + 2 * G, s_desc[nslot == 2 ? 0 : nslot + 1], s_cst, s_pst);
+    write_out(s_gd + ((it + 1) & 1) * F);
+    __syncthreads();
+
+    // ---- phase 3: shuffle unit i into digit order in shared memory -----------------------------
+    #pragma unroll
+    for (int j = 0; j < ITEMS; ++j)
+      if (full || pass_elem<K, MODE, NT>(j) < ulen)
+        s_buf[s_loc[digit(kk[j])] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = TT::make(kk[j], pp[j]);
+    // (no barrier: the next unit's phase 1 touches only s_cnt; its phase 2 reads s_buf / s_gd
+    //  after the next phase-1 barrier)
+    prev_dst = (T*)s_desc[slot].dst;
+    prev_len = ulen;
+    u += G;
+    slot = nslot;
+    ++it;
   }
+  __syncthreads();
+  write_out(s_gd + ((it + 1) & 1) * F);  // the last unit (it was incremented past it)
 }
 
 }  // namespace hj
