@@ -23,8 +23,13 @@ namespace {
 thread_local std::string g_create_error;
 
 constexpr int PASS_NT = 1024;  // threads per partition-pass block (one block per SM)
-constexpr int JOIN_NT = 256;   // threads per join block (the paper used 512)
-constexpr int JOIN_SPT = 8;    // S tuples per thread per probe round
+// Join kernel shapes selectable with HJ_OPT_JOIN_VARIANT (tuning; results never change).
+//   variant: compute threads, S tuples / thread / round, min blocks / SM, R tile buffers
+struct JoinShape {
+  int nt, spt, minb, rbuf;
+};
+constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1}, {256, 8, 2, 2}, {224, 8, 3, 1}, {256, 12, 3, 1}, {192, 8, 3, 1}};
+constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
 
 struct DevBuf {
@@ -41,7 +46,7 @@ struct Ctx {
   size_t smem_optin = 0;
   std::string err;
   // options
-  int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0;
+  int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = 0;
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2];
   void* h_res = nullptr;  // pinned host: results readback
@@ -147,8 +152,9 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   if (c->opt_chunk_s > 0) CS = (uint32_t)std::min<int64_t>(c->opt_chunk_s, 1ll << 30);
   else CS = std::max<uint32_t>(8 * CR, 32768);
   int lg_nb = std::max(6, ilog2_ceil(CR) - 1);
-  auto join_smem = [&](uint32_t cr, int lg) {  // 2 R tile buffers (TMA double buffer) + heads + next
-    return (size_t)2 * ((cr + 3) & ~1u) * tb + ((size_t)4 << lg) + (size_t)cr * 2;
+  const int rbuf = JOIN_SHAPES[c->opt_join_variant].rbuf;
+  auto join_smem = [&](uint32_t cr, int lg) {  // R tile buffer(s) (TMA) + heads + next
+    return (size_t)rbuf * ((cr + 3) & ~1u) * tb + ((size_t)4 << lg) + (size_t)cr * 2;
   };
   while (join_smem(CR, lg_nb) > cap_max_smem - 8 * 1024 && CR > 256) {
     CR /= 2;
@@ -185,6 +191,13 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   return HJ_OK;
 }
 
+template <typename K, int V, typename F>
+void attr_join(F&& attr) {
+  constexpr JoinShape S = JOIN_SHAPES[V];
+  attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf>);
+  attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf>);
+}
+
 template <typename K>
 int set_kernel_attrs(Ctx* c) {
   int rc = 0;
@@ -200,8 +213,11 @@ int set_kernel_attrs(Ctx* c) {
   attr((const void*)k_pass<K, 1, PASS_NT, pass_items<K>(), false>);
   attr((const void*)k_pass<K, 1, PASS_NT, pass_items<K>(), true>);
   attr((const void*)k_pass<K, 2, PASS_NT, pass_items<K>(), false>);
-  attr((const void*)k_join<K, JOIN_NT, JOIN_SPT, false>);
-  attr((const void*)k_join<K, JOIN_NT, JOIN_SPT, true>);
+  attr_join<K, 0>(attr);
+  attr_join<K, 1>(attr);
+  attr_join<K, 2>(attr);
+  attr_join<K, 3>(attr);
+  attr_join<K, 4>(attr);
   return rc;
 }
 
@@ -279,15 +295,17 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P) {
   if (hp.mode != PLAN_RECV) {
     const bool smem = hp.qbits() <= 15;
     const size_t sm = smem ? ((size_t)4 << hp.qbits()) : 0;
-    const unsigned long long nmax = std::max(P.rel[0].n, P.rel[1].n);
+    const unsigned long long nR = P.rel[0].n, nS = P.rel[1].n;
     const void* f = smem ? (gd ? (const void*)k_hist<K, true, true> : (const void*)k_hist<K, true, false>)
                          : (const void*)k_hist<K, false, false>;
-    int g = grid_for(c, f, HIST_NT, sm, (nmax + 4095) / 4096);
-    dim3 grid((unsigned)std::max(1, g / 2), 2);
-    if (smem && gd) k_hist<K, true, true><<<grid, HIST_NT, sm, st>>>(P);
-    else if (smem) k_hist<K, true, false><<<grid, HIST_NT, sm, st>>>(P);
-    else if (gd) k_hist<K, false, true><<<grid, HIST_NT, 0, st>>>(P);
-    else k_hist<K, false, false><<<grid, HIST_NT, 0, st>>>(P);
+    const int g = std::max(2, grid_for(c, f, HIST_NT, sm, (nR + nS + 4095) / 4096 + 2));
+    // blocks split proportionally to the relation sizes (at least one each)
+    uint32_t gr = (uint32_t)((double)g * (double)nR / (double)std::max<unsigned long long>(nR + nS, 1) + 0.5);
+    gr = std::min<uint32_t>(std::max<uint32_t>(gr, 1), (uint32_t)g - 1);
+    if (smem && gd) k_hist<K, true, true><<<g, HIST_NT, sm, st>>>(P, gr);
+    else if (smem) k_hist<K, true, false><<<g, HIST_NT, sm, st>>>(P, gr);
+    else if (gd) k_hist<K, false, true><<<g, HIST_NT, 0, st>>>(P, gr);
+    else k_hist<K, false, false><<<g, HIST_NT, 0, st>>>(P, gr);
     CUDA_TRY(c, cudaGetLastError());
     c->launches += 1;
   }
@@ -326,14 +344,30 @@ int launch_pass2(Ctx* c, const HostPlan& hp, const Plan& P) {
   return HJ_OK;
 }
 
+template <typename K, int V>
+int launch_join_v(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
+  constexpr JoinShape S = JOIN_SHAPES[V];
+  cudaStream_t st = c->stream;
+  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf>
+                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf>;
+  int g = grid_for(c, f, S.nt + 32, hp.join_smem, 1ull << 40);
+  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  CUDA_TRY(c, cudaGetLastError());
+  return HJ_OK;
+}
+
 template <typename K>
 int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
-  cudaStream_t st = c->stream;
-  const void* f = mat ? (const void*)k_join<K, JOIN_NT, JOIN_SPT, true> : (const void*)k_join<K, JOIN_NT, JOIN_SPT, false>;
-  int g = grid_for(c, f, JOIN_NT + 32, hp.join_smem, 1ull << 40);
-  if (mat) k_join<K, JOIN_NT, JOIN_SPT, true><<<g, JOIN_NT + 32, hp.join_smem, st>>>(P);
-  else k_join<K, JOIN_NT, JOIN_SPT, false><<<g, JOIN_NT + 32, hp.join_smem, st>>>(P);
-  CUDA_TRY(c, cudaGetLastError());
+  int rc;
+  switch (c->opt_join_variant) {
+    case 1: rc = launch_join_v<K, 1>(c, hp, P, mat); break;
+    case 2: rc = launch_join_v<K, 2>(c, hp, P, mat); break;
+    case 3: rc = launch_join_v<K, 3>(c, hp, P, mat); break;
+    case 4: rc = launch_join_v<K, 4>(c, hp, P, mat); break;
+    default: rc = launch_join_v<K, 0>(c, hp, P, mat); break;
+  }
+  if (rc) return rc;
   mark(c, 5);
   c->launches += 1;
   return HJ_OK;
@@ -530,6 +564,10 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_OUT_CAPACITY: c->opt_out_cap = v; break;
     case HJ_OPT_TIMING: c->opt_timing = v; break;
     case HJ_OPT_BLOCKS_PER_SM: c->opt_bps = v; break;
+    case HJ_OPT_JOIN_VARIANT:
+      if (v >= JOIN_NVARIANTS) return fail(c, HJ_ERR_INVALID, "join variant %lld >= %d", (long long)v, JOIN_NVARIANTS);
+      c->opt_join_variant = v;
+      break;
     default: return fail(c, HJ_ERR_INVALID, "unknown option %d", opt);
   }
   return HJ_OK;

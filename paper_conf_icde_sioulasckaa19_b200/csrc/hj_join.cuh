@@ -27,6 +27,7 @@ struct JoinJob {
 
 // Claim the next work item and decode it (item -> co-partition q by binary search over the
 // planner's item prefix; then the R chunk and S chunk of q it covers). One lane.
+template <typename T>
 __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items) {
   JoinJob j;
   j.item = atomicAdd(&P.counters[CNT_NEXT_ITEM], 1u);
@@ -49,17 +50,18 @@ __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items
     j.nr = (uint32_t)min((unsigned long long)P.CR, rn - rc * P.CR);
     j.sb = s0 + sc * P.CS;
     j.se = j.sb + min((unsigned long long)P.CS, sn - sc * P.CS);
+    const uintptr_t a = reinterpret_cast<uintptr_t>((const T*)P.rel[0].t2 + j.rb);
+    j.shift = (uint32_t)((a & 15) / sizeof(T));  // tuples between the 16 B aligned copy start and rb
   }
   return j;
 }
 
 // TMA bulk copy of a job's R chunk (the 16-byte aligned superset) into an smem tile buffer.
 template <typename T>
-__device__ __forceinline__ void issue_r_copy(const Plan& P, JoinJob& j, T* buf, unsigned long long* bar) {
+__device__ __forceinline__ void issue_r_copy(const Plan& P, const JoinJob& j, T* buf, unsigned long long* bar) {
   const uintptr_t a = reinterpret_cast<uintptr_t>((const T*)P.rel[0].t2 + j.rb);
   const uintptr_t a0 = a & ~(uintptr_t)15;
   const uint32_t bytes = (uint32_t)(((a + (uintptr_t)j.nr * sizeof(T) - a0) + 15) & ~(uintptr_t)15);
-  j.shift = (uint32_t)((a - a0) / sizeof(T));
   fence_proxy_async();  // prior generic-proxy reads of buf (the item before last) are ordered before
   mbar_arrive_expect_tx(bar, bytes);
   bulk_g2s(buf, reinterpret_cast<const void*>(a0), bytes, bar);
@@ -80,16 +82,18 @@ __device__ __forceinline__ void bar_compute(int nthreads) {  // named barrier 1:
 // of the warp totals, and lanes write their pairs at warp-contiguous positions (coalesced
 // stores). This replaces the paper's per-warp buffer + global atomic per flush.
 // Chains are re-walked only for S tuples with more than one match.
-template <typename K, int NT, int SPT, bool MAT>
-__global__ void __launch_bounds__(NT + 32, 2) k_join(Plan P) {
+// RBUF = 2: the next item's R chunk is copied while the current item is joined (double buffer);
+// RBUF = 1: it is copied right after the end-of-item barrier (less smem -> more blocks per SM).
+template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF>
+__global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
   using TT = Tup<K>;
   using T = typename TT::T;
   extern __shared__ __align__(16) unsigned char s_raw[];
   const SlotHash H = P.H;
   const uint32_t nb = 1u << H.lg;
   const uint32_t cap = (P.CR + 3) & ~1u;  // tile buffer in tuples: +2 for the aligned superset, even -> 16 B aligned
-  T* s_rtb = reinterpret_cast<T*>(s_raw);                            // 2 x cap tuples
-  uint32_t* s_head = reinterpret_cast<uint32_t*>(s_rtb + 2 * cap);   // nb
+  T* s_rtb = reinterpret_cast<T*>(s_raw);                             // RBUF x cap tuples
+  uint32_t* s_head = reinterpret_cast<uint32_t*>(s_rtb + RBUF * cap);  // nb
   uint16_t* s_next = reinterpret_cast<uint16_t*>(s_head + nb);       // CR
   __shared__ JoinJob s_jobs[2];
   __shared__ __align__(8) unsigned long long s_bar[2];
@@ -109,7 +113,7 @@ __global__ void __launch_bounds__(NT + 32, 2) k_join(Plan P) {
     mbar_init(&s_bar[0], 1);
     mbar_init(&s_bar[1], 1);
     fence_mbar_init();
-    JoinJob j = claim_job(P, total_items);
+    JoinJob j = claim_job<T>(P, total_items);
     if (j.item < total_items) issue_r_copy<T>(P, j, s_rtb, &s_bar[0]);
     s_jobs[0] = j;
   }
@@ -119,12 +123,14 @@ __global__ void __launch_bounds__(NT + 32, 2) k_join(Plan P) {
     const JoinJob job = s_jobs[it & 1];
     if (job.item >= total_items) break;
     if (sched) {
+      JoinJob j;
       if (lane == 0) {
-        JoinJob j = claim_job(P, total_items);
-        if (j.item < total_items) issue_r_copy<T>(P, j, s_rtb + ((it + 1) & 1) * cap, &s_bar[(it + 1) & 1]);
+        j = claim_job<T>(P, total_items);
+        if (RBUF == 2 && j.item < total_items) issue_r_copy<T>(P, j, s_rtb + ((it + 1) & 1) * cap, &s_bar[(it + 1) & 1]);
         s_jobs[(it + 1) & 1] = j;
       }
       __syncthreads();  // end-of-item barrier (matches the compute warps' one below)
+      if (RBUF == 1 && lane == 0 && j.item < total_items) issue_r_copy<T>(P, j, s_rtb, &s_bar[(it + 1) & 1]);
       continue;
     }
 
@@ -143,7 +149,7 @@ __global__ void __launch_bounds__(NT + 32, 2) k_join(Plan P) {
     };
     load_s(job.sb);
     for (uint32_t i = threadIdx.x; i < nb; i += NT) s_head[i] = NIL16;
-    const T* s_rt = s_rtb + (it & 1) * cap + job.shift;
+    const T* s_rt = s_rtb + (RBUF == 2 ? (it & 1) * cap : 0) + job.shift;
     mbar_wait(&s_bar[it & 1], (it >> 1) & 1);  // R chunk landed (TMA)
     bar_compute(NT);
     // ---- build (a6): wait-free push-front insert (Listing 2) ----------------------

@@ -25,11 +25,14 @@ namespace hj {
 // 128 KB of counters) SMEM = false counts with global atomics directly (correct, slower).
 // ------------------------------------------------------------------------------------------
 template <typename K, bool SMEM, bool GD>
-__global__ void __launch_bounds__(1024) k_hist(Plan P) {
+__global__ void __launch_bounds__(1024) k_hist(Plan P, uint32_t blocks_r) {
   extern __shared__ uint32_t s_hist[];
-  const int rel = blockIdx.y;
+  // blocks [0, blocks_r) count R, the rest count S (split proportionally to |R| : |S|)
+  const int rel = blockIdx.x < blocks_r ? 0 : 1;
   const RelDev& R = P.rel[rel];
   const unsigned long long n = R.n;
+  const uint32_t nblk = rel ? gridDim.x - blocks_r : blocks_r;
+  const uint32_t bid = rel ? blockIdx.x - blocks_r : blockIdx.x;
   const uint32_t np = 1u << P.qbits();
   if (SMEM) {
     for (uint32_t i = threadIdx.x; i < np; i += blockDim.x) s_hist[i] = 0;
@@ -37,9 +40,9 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P) {
   }
   uint32_t* h = SMEM ? s_hist : R.cnt;
   constexpr int VEC = 16 / sizeof(K);
-  unsigned long long per = (n + gridDim.x - 1) / gridDim.x;
+  unsigned long long per = (n + nblk - 1) / nblk;
   per = (per + VEC - 1) / VEC * VEC;
-  const unsigned long long lo = (unsigned long long)blockIdx.x * per;
+  const unsigned long long lo = (unsigned long long)bid * per;
   const unsigned long long hi = lo + per < n ? lo + per : n;
   const K* keys = (const K*)R.keys;
   if (lo < hi) {
