@@ -35,6 +35,7 @@ OPT_OUT_CAPACITY = 3
 OPT_TIMING = 4
 OPT_BLOCKS_PER_SM = 5
 OPT_JOIN_VARIANT = 6
+OPT_PASS_THREADS = 7
 
 _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4: "HJ_ERR_CUDA", -5: "HJ_ERR_COMM"}
 

@@ -22,7 +22,6 @@ namespace {
 
 thread_local std::string g_create_error;
 
-constexpr int PASS_NT = 1024;  // threads per partition-pass block (one block per SM)
 // Join kernel shapes selectable with HJ_OPT_JOIN_VARIANT (tuning; results never change).
 //   variant: compute threads, S tuples / thread / round, min blocks / SM, R tile buffers
 struct JoinShape {
@@ -46,7 +45,8 @@ struct Ctx {
   size_t smem_optin = 0;
   std::string err;
   // options
-  int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = 0;
+  int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = 0,
+          opt_pass_nt = 0;
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2];
   void* h_res = nullptr;  // pinned host: results readback
@@ -117,6 +117,11 @@ constexpr int pass_items() {
   return sizeof(K) == 4 ? 8 : 4;  // 8192-tuple tiles of 8 B, 4096-tuple tiles of 16 B (64 KB)
 }
 
+int pass_threads(const Ctx* c, int fanout_bits, int items) {
+  if (c->opt_pass_nt) return (int)c->opt_pass_nt == 512 && (1 << fanout_bits) <= 512 ? 512 : 1024;
+  return (512 * items) >> fanout_bits >= 32 ? 512 : 1024;
+}
+
 int choose_bits(unsigned long long nR) {
   // mean R co-partition ~4096 tuples: the paper's shared-memory reservation
   if (nR <= 4096) return 0;
@@ -138,8 +143,12 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   hp.mode = mode;
   if (hp.pb() > 10 || hp.b2 > 10 || hp.npieces() > 1024)
     return fail(c, HJ_ERR_UNSUPPORTED, "pass fan-out too large (g=%d b1=%d b2=%d sources=%d)", g, hp.b1, hp.b2, nsrc);
-  hp.tile = PASS_NT * (c->key_bytes == 4 ? pass_items<uint32_t>() : pass_items<uint64_t>());
-  hp.C2 = (uint32_t)hp.tile;
+  const int items = c->key_bytes == 4 ? pass_items<uint32_t>() : pass_items<uint64_t>();
+  // pass tiles: two 512-thread blocks per SM when a 512-thread tile still averages >= 32 tuples
+  // per digit run (measured: shorter runs cost more than the extra block's overlap), else one
+  // 1024-thread block. The pass-2 chunk is that kernel's tile.
+  hp.tile = pass_threads(c, hp.pb(), items) * items;
+  hp.C2 = (uint32_t)(pass_threads(c, hp.b2, items) * items);
 
   // join capacities
   const unsigned long long mean = (nR + (1ull << hp.B) - 1) >> hp.B;
@@ -210,9 +219,12 @@ int set_kernel_attrs(Ctx* c) {
   };
   attr((const void*)k_hist<K, true, false>);
   attr((const void*)k_hist<K, true, true>);
-  attr((const void*)k_pass<K, 1, PASS_NT, pass_items<K>(), false>);
-  attr((const void*)k_pass<K, 1, PASS_NT, pass_items<K>(), true>);
-  attr((const void*)k_pass<K, 2, PASS_NT, pass_items<K>(), false>);
+  attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), false>);
+  attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), true>);
+  attr((const void*)k_pass<K, 2, 1024, pass_items<K>(), false>);
+  attr((const void*)k_pass<K, 1, 512, pass_items<K>(), false>);
+  attr((const void*)k_pass<K, 1, 512, pass_items<K>(), true>);
+  attr((const void*)k_pass<K, 2, 512, pass_items<K>(), false>);
   attr_join<K, 0>(attr);
   attr_join<K, 1>(attr);
   attr_join<K, 2>(attr);
@@ -286,6 +298,9 @@ void mark(Ctx* c, int i) {
 
 // a1 (histogram), a2/a5 (planner), a3 (pass 1). PLAN_RECV skips a1 and a3 (counts and the
 // pass-1 layout arrive through the exchange). Events 0..3.
+template <typename K, int MODE, int NT, bool GD>
+int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits);
+
 template <typename K>
 int launch_front(Ctx* c, const HostPlan& hp, const Plan& P) {
   cudaStream_t st = c->stream;
@@ -315,31 +330,45 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P) {
   c->launches += 1;
   mark(c, 2);
   if (hp.mode != PLAN_RECV) {
-    constexpr int IT = pass_items<K>();
-    const void* f = gd ? (const void*)k_pass<K, 1, PASS_NT, IT, true> : (const void*)k_pass<K, 1, PASS_NT, IT, false>;
-    const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.pb()) * 24 + 16;
-    int g = grid_for(c, f, PASS_NT, sm, P.tiles1[0] + P.tiles1[1]);
-    if (gd) k_pass<K, 1, PASS_NT, IT, true><<<g, PASS_NT, sm, st>>>(P, hp.pb());
-    else k_pass<K, 1, PASS_NT, IT, false><<<g, PASS_NT, sm, st>>>(P, hp.pb());
-    CUDA_TRY(c, cudaGetLastError());
-    c->launches += 1;
+    int rc = hp.tile == 512 * pass_items<K>()
+                 ? (gd ? launch_pass<K, 1, 512, true>(c, hp, P, hp.pb()) : launch_pass<K, 1, 512, false>(c, hp, P, hp.pb()))
+                 : (gd ? launch_pass<K, 1, 1024, true>(c, hp, P, hp.pb()) : launch_pass<K, 1, 1024, false>(c, hp, P, hp.pb()));
+    if (rc) return rc;
   }
   mark(c, 3);
   return HJ_OK;
 }
 
 // a4: pass 2 over the pass-1 pieces. Event 4.
-template <typename K>
-int launch_pass2(Ctx* c, const HostPlan& hp, const Plan& P) {
+// a4: pass 2 over the pass-1 pieces. Event 4.
+template <typename K, int MODE, int NT, bool GD>
+int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
   constexpr int IT = pass_items<K>();
-  const void* f = (const void*)k_pass<K, 2, PASS_NT, IT, false>;
-  const size_t sm = (size_t)PASS_NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << hp.b2) * 24 + 16;
-  // chunks: at most n / C2 + npieces per relation
-  unsigned long long units = (P.rel[0].n + P.rel[1].n) / hp.C2 + 2ull * hp.npieces() + 2;
-  int g = grid_for(c, f, PASS_NT, sm, units);
-  k_pass<K, 2, PASS_NT, IT, false><<<g, PASS_NT, sm, c->stream>>>(P, hp.b2);
+  const void* f = (const void*)k_pass<K, MODE, NT, IT, GD>;
+  const size_t sm = (size_t)NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << fanout_bits) * 24 + 16;
+  const unsigned long long tile = (unsigned long long)NT * IT;
+  // units: pass 1 = tiles; pass 2 = at most n / tile + pieces per relation
+  Plan Q = P;
+  Q.C2 = (uint32_t)tile;
+  unsigned long long units = MODE == 1 ? (P.rel[0].n + tile - 1) / tile + (P.rel[1].n + tile - 1) / tile
+                                       : (P.rel[0].n + P.rel[1].n) / tile + 2ull * hp.npieces() + 2;
+  if (MODE == 1) {
+    Q.tiles1[0] = (P.rel[0].n + tile - 1) / tile;
+    Q.tiles1[1] = (P.rel[1].n + tile - 1) / tile;
+  }
+  int g = grid_for(c, f, NT, sm, units);
+  k_pass<K, MODE, NT, IT, GD><<<g, NT, sm, c->stream>>>(Q, fanout_bits);
   CUDA_TRY(c, cudaGetLastError());
   c->launches += 1;
+  return HJ_OK;
+}
+
+// a4: pass 2 over the pass-1 pieces. Event 4.
+template <typename K>
+int launch_pass2(Ctx* c, const HostPlan& hp, const Plan& P) {
+  int rc = hp.C2 == (uint32_t)(512 * pass_items<K>()) ? launch_pass<K, 2, 512, false>(c, hp, P, hp.b2)
+                                                       : launch_pass<K, 2, 1024, false>(c, hp, P, hp.b2);
+  if (rc) return rc;
   mark(c, 4);
   return HJ_OK;
 }
@@ -564,6 +593,10 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_OUT_CAPACITY: c->opt_out_cap = v; break;
     case HJ_OPT_TIMING: c->opt_timing = v; break;
     case HJ_OPT_BLOCKS_PER_SM: c->opt_bps = v; break;
+    case HJ_OPT_PASS_THREADS:
+      if (v != 0 && v != 512 && v != 1024) return fail(c, HJ_ERR_INVALID, "pass threads must be 0, 512 or 1024");
+      c->opt_pass_nt = v;
+      break;
     case HJ_OPT_JOIN_VARIANT:
       if (v >= JOIN_NVARIANTS) return fail(c, HJ_ERR_INVALID, "join variant %lld >= %d", (long long)v, JOIN_NVARIANTS);
       c->opt_join_variant = v;

@@ -345,11 +345,11 @@ __device__ __forceinline__ void pass_load(const PassUnit<K>& U, K (&kk)[ITEMS], 
 //   phase 3  shuffle unit i into digit order in s_buf
 // so each reservation atomic's latency overlaps the previous unit's write-out.
 template <typename K, int MODE, int NT, int ITEMS, bool GD>
-__global__ void __launch_bounds__(NT, 1) k_pass(Plan P, int fanout_bits) {
+__global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits) {
   using TT = Tup<K>;
   using T = typename TT::T;
   constexpr int TILE = NT * ITEMS;
-  static_assert(NT >= 1024, "fan-out up to 2^10 needs one digit per thread");
+  static_assert(NT == 512 || NT == 1024, "block size");  // the launcher guarantees fan-out <= NT
   static_assert(TILE <= 65536 && ITEMS % 2 == 0, "16-bit packed ranks");
   extern __shared__ __align__(16) unsigned char s_raw[];
   const uint32_t F = 1u << fanout_bits;

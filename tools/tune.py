@@ -14,7 +14,7 @@ import paper_conf_icde_sioulasckaa19_b200 as hj  # noqa: E402
 import workloads as W  # noqa: E402
 
 OPTS = {"join_variant": hj.OPT_JOIN_VARIANT, "cap_r": hj.OPT_CAP_R, "chunk_s": hj.OPT_CHUNK_S,
-        "blocks_per_sm": hj.OPT_BLOCKS_PER_SM}
+        "blocks_per_sm": hj.OPT_BLOCKS_PER_SM, "pass_threads": hj.OPT_PASS_THREADS}
 
 
 def main():
