@@ -27,7 +27,8 @@ thread_local std::string g_create_error;
 struct JoinShape {
   int nt, spt, minb, rbuf;
 };
-constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1}, {256, 8, 2, 2}, {224, 8, 3, 1}, {256, 12, 3, 1}, {192, 8, 3, 1}};
+constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1}, {256, 8, 2, 2}, {224, 8, 3, 1}, {256, 12, 3, 1}, {192, 8, 3, 1},
+                                     {256, 4, 2, 1}, {512, 4, 1, 1}, {256, 8, 2, 1}, {384, 4, 1, 2}};
 constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
 
@@ -45,7 +46,7 @@ struct Ctx {
   size_t smem_optin = 0;
   std::string err;
   // options
-  int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = 0,
+  int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
           opt_pass_nt = 0;
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2];
@@ -117,6 +118,12 @@ constexpr int pass_items() {
   return sizeof(K) == 4 ? 8 : 4;  // 8192-tuple tiles of 8 B, 4096-tuple tiles of 16 B (64 KB)
 }
 
+// default join shape per key width (measured with tools/tune.py): 4 B -> shape 0, 8 B -> shape 5
+int join_variant(const Ctx* c) {
+  if (c->opt_join_variant >= 0) return (int)c->opt_join_variant;
+  return c->key_bytes == 4 ? 0 : 5;
+}
+
 int pass_threads(const Ctx* c, int fanout_bits, int items) {
   if (c->opt_pass_nt) return (int)c->opt_pass_nt == 512 && (1 << fanout_bits) <= 512 ? 512 : 1024;
   return (512 * items) >> fanout_bits >= 32 ? 512 : 1024;
@@ -161,7 +168,7 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   if (c->opt_chunk_s > 0) CS = (uint32_t)std::min<int64_t>(c->opt_chunk_s, 1ll << 30);
   else CS = std::max<uint32_t>(8 * CR, 32768);
   int lg_nb = std::max(6, ilog2_ceil(CR) - 1);
-  const int rbuf = JOIN_SHAPES[c->opt_join_variant].rbuf;
+  const int rbuf = JOIN_SHAPES[join_variant(c)].rbuf;
   auto join_smem = [&](uint32_t cr, int lg) {  // R tile buffer(s) (TMA) + heads + next
     return (size_t)rbuf * ((cr + 3) & ~1u) * tb + ((size_t)4 << lg) + (size_t)cr * 2;
   };
@@ -217,8 +224,10 @@ int set_kernel_attrs(Ctx* c) {
                              (int)(c->smem_optin - fa.sharedSizeBytes)) != cudaSuccess)
       rc = -1;
   };
-  attr((const void*)k_hist<K, true, false>);
-  attr((const void*)k_hist<K, true, true>);
+  attr((const void*)k_hist<K, true, false, true>);
+  attr((const void*)k_hist<K, true, true, true>);
+  attr((const void*)k_hist<K, true, false, false>);
+  attr((const void*)k_hist<K, true, true, false>);
   attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), false>);
   attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), true>);
   attr((const void*)k_pass<K, 2, 1024, pass_items<K>(), false>);
@@ -230,6 +239,10 @@ int set_kernel_attrs(Ctx* c) {
   attr_join<K, 2>(attr);
   attr_join<K, 3>(attr);
   attr_join<K, 4>(attr);
+  attr_join<K, 5>(attr);
+  attr_join<K, 6>(attr);
+  attr_join<K, 7>(attr);
+  attr_join<K, 8>(attr);
   return rc;
 }
 
@@ -308,8 +321,9 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P) {
   mark(c, 0);
   CUDA_TRY(c, cudaMemsetAsync(c->meta.p, 0, hp.zero_bytes, st));
   if (hp.mode != PLAN_RECV) {
-    const bool smem = hp.qbits() <= 15;
-    const size_t sm = smem ? ((size_t)4 << hp.qbits()) : 0;
+    const bool smem = hp.qbits() <= 16;
+    const bool c32 = hp.qbits() <= 15;  // 16 bins: packed 16-bit counters (128 KB)
+    const size_t sm = smem ? (c32 ? ((size_t)4 << hp.qbits()) : ((size_t)2 << hp.qbits())) : 0;
     const unsigned long long nR = P.rel[0].n, nS = P.rel[1].n;
     const void* f = smem ? (gd ? (const void*)k_hist<K, true, true> : (const void*)k_hist<K, true, false>)
                          : (const void*)k_hist<K, false, false>;
@@ -317,8 +331,10 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P) {
     // blocks split proportionally to the relation sizes (at least one each)
     uint32_t gr = (uint32_t)((double)g * (double)nR / (double)std::max<unsigned long long>(nR + nS, 1) + 0.5);
     gr = std::min<uint32_t>(std::max<uint32_t>(gr, 1), (uint32_t)g - 1);
-    if (smem && gd) k_hist<K, true, true><<<g, HIST_NT, sm, st>>>(P, gr);
-    else if (smem) k_hist<K, true, false><<<g, HIST_NT, sm, st>>>(P, gr);
+    if (smem && c32 && gd) k_hist<K, true, true, true><<<g, HIST_NT, sm, st>>>(P, gr);
+    else if (smem && c32) k_hist<K, true, false, true><<<g, HIST_NT, sm, st>>>(P, gr);
+    else if (smem && gd) k_hist<K, true, true, false><<<g, HIST_NT, sm, st>>>(P, gr);
+    else if (smem) k_hist<K, true, false, false><<<g, HIST_NT, sm, st>>>(P, gr);
     else if (gd) k_hist<K, false, true><<<g, HIST_NT, 0, st>>>(P, gr);
     else k_hist<K, false, false><<<g, HIST_NT, 0, st>>>(P, gr);
     CUDA_TRY(c, cudaGetLastError());
@@ -389,7 +405,11 @@ int launch_join_v(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
 template <typename K>
 int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   int rc;
-  switch (c->opt_join_variant) {
+  switch (join_variant(c)) {
+    case 5: rc = launch_join_v<K, 5>(c, hp, P, mat); break;
+    case 6: rc = launch_join_v<K, 6>(c, hp, P, mat); break;
+    case 7: rc = launch_join_v<K, 7>(c, hp, P, mat); break;
+    case 8: rc = launch_join_v<K, 8>(c, hp, P, mat); break;
     case 1: rc = launch_join_v<K, 1>(c, hp, P, mat); break;
     case 2: rc = launch_join_v<K, 2>(c, hp, P, mat); break;
     case 3: rc = launch_join_v<K, 3>(c, hp, P, mat); break;
@@ -598,8 +618,8 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
       c->opt_pass_nt = v;
       break;
     case HJ_OPT_JOIN_VARIANT:
-      if (v >= JOIN_NVARIANTS) return fail(c, HJ_ERR_INVALID, "join variant %lld >= %d", (long long)v, JOIN_NVARIANTS);
-      c->opt_join_variant = v;
+      if (v > JOIN_NVARIANTS) return fail(c, HJ_ERR_INVALID, "join variant %lld >= %d", (long long)v, JOIN_NVARIANTS);
+      c->opt_join_variant = v == 0 ? -1 : v - 1;  // 0 = auto, k = shape k - 1
       break;
     default: return fail(c, HJ_ERR_INVALID, "unknown option %d", opt);
   }

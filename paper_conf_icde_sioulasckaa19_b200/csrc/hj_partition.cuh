@@ -24,7 +24,26 @@ namespace hj {
 // then merges non-zero counters with one global RED each (coalesced). For qbits > 15 (more than
 // 128 KB of counters) SMEM = false counts with global atomics directly (correct, slower).
 // ------------------------------------------------------------------------------------------
-template <typename K, bool SMEM, bool GD>
+// Shared-memory counters, one 32-bit atomicAdd per key:
+//   C32 = true : 2^qbits u32 counters (qbits <= 15, <= 128 KB)
+//   C32 = false: 2^qbits u16 counters packed in pairs (qbits == 16, 128 KB). A wrap of a 16-bit
+//                half (old value 0xFFFF) is detected from the atomic's return value: the carry
+//                into the upper half is undone and 65536 is added to the global counter.
+template <bool C32>
+__device__ __forceinline__ void hist_add(uint32_t* h, uint32_t bin, uint32_t* gcnt) {
+  if (C32) {
+    atomicAdd(&h[bin], 1u);
+  } else {
+    const uint32_t sh = (bin & 1) << 4;
+    const uint32_t old = atomicAdd(&h[bin >> 1], 1u << sh);
+    if (((old >> sh) & 0xffffu) == 0xffffu) {
+      if (sh == 0) atomicSub(&h[bin >> 1], 1u << 16);
+      atomicAdd(&gcnt[bin], 65536u);
+    }
+  }
+}
+
+template <typename K, bool SMEM, bool GD, bool C32 = true>
 __global__ void __launch_bounds__(1024) k_hist(Plan P, uint32_t blocks_r) {
   extern __shared__ uint32_t s_hist[];
   // blocks [0, blocks_r) count R, the rest count S (split proportionally to |R| : |S|)
@@ -34,11 +53,16 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P, uint32_t blocks_r) {
   const uint32_t nblk = rel ? gridDim.x - blocks_r : blocks_r;
   const uint32_t bid = rel ? blockIdx.x - blocks_r : blockIdx.x;
   const uint32_t np = 1u << P.qbits();
+  const uint32_t nwords = C32 ? np : np / 2;
   if (SMEM) {
-    for (uint32_t i = threadIdx.x; i < np; i += blockDim.x) s_hist[i] = 0;
+    for (uint32_t i = threadIdx.x; i < nwords; i += blockDim.x) s_hist[i] = 0;
     __syncthreads();
   }
-  uint32_t* h = SMEM ? s_hist : R.cnt;
+  auto add = [&](K key) {
+    const uint32_t b = qbin<GD>(key, P);
+    if (SMEM) hist_add<C32>(s_hist, b, R.cnt);
+    else atomicAdd(&R.cnt[b], 1u);
+  };
   constexpr int VEC = 16 / sizeof(K);
   unsigned long long per = (n + nblk - 1) / nblk;
   per = (per + VEC - 1) / VEC * VEC;
@@ -61,23 +85,23 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P, uint32_t blocks_r) {
         for (int u = 0; u < U; ++u) {
           const K* e = reinterpret_cast<const K*>(&x[u]);
           #pragma unroll
-          for (int t = 0; t < VEC; ++t) atomicAdd(&h[qbin<GD>(e[t], P)], 1u);
+          for (int t = 0; t < VEC; ++t) add(e[t]);
         }
       }
       for (; v < nvec; v += blockDim.x) {
         uint4 x = __ldcs(kv + v);
         const K* e = reinterpret_cast<const K*>(&x);
         #pragma unroll
-        for (int t = 0; t < VEC; ++t) atomicAdd(&h[qbin<GD>(e[t], P)], 1u);
+        for (int t = 0; t < VEC; ++t) add(e[t]);
       }
       i = lo + nvec * VEC;
     }
-    for (unsigned long long j = i + threadIdx.x; j < hi; j += blockDim.x) atomicAdd(&h[qbin<GD>(keys[j], P)], 1u);
+    for (unsigned long long j = i + threadIdx.x; j < hi; j += blockDim.x) add(keys[j]);
   }
   if (SMEM) {
     __syncthreads();
     for (uint32_t i = threadIdx.x; i < np; i += blockDim.x) {
-      uint32_t c = s_hist[i];
+      const uint32_t c = C32 ? s_hist[i] : ((s_hist[i >> 1] >> ((i & 1) << 4)) & 0xffffu);
       if (c) atomicAdd(&R.cnt[i], c);
     }
   }

@@ -246,3 +246,29 @@ def test_full_size_closed_form(hj, cfg):
         assert np.array_equal(s_sorted, j), "materialized s_pay is not a permutation of S's rows"
         bad = np.nonzero(r_sorted != rho)[0]
         assert len(bad) == 0, f"{len(bad)} materialized pairs differ, first at s_pay {bad[:5]}"
+
+
+@pytest.mark.parametrize("width", [4, 8])
+def test_partition_16bit_counters_wrap(hj, width):
+    """2^16 co-partitions use packed 16-bit shared-memory counters; > 65535 equal keys in one
+    block exercise the wrap/carry correction."""
+    rng = np.random.default_rng(16)
+    dt = np.uint32 if width == 4 else np.uint64
+    n = 400_000
+    keys = rng.integers(0, 1 << (8 * width - 1), n, dtype=np.uint64).astype(dt)
+    keys[: 3 * n // 4] = dt(0x12345)  # 300K copies of one key
+    rng.shuffle(keys)
+    pays = np.arange(n, dtype=dt)
+    _, _, offs = oracle.radix_partition(keys, pays, 0, 16)
+    t, start, count = hj.context(0, width, width).partition(dev(keys), dev(pays), 16)
+    torch.cuda.synchronize()
+    assert np.array_equal(count, np.diff(offs.astype(np.int64)).astype(np.uint64))
+
+
+def test_join_16bit_counters(hj):
+    rng = np.random.default_rng(17)
+    Rk = rng.integers(0, 1 << 20, 150_000).astype(np.uint32)
+    Sk = np.concatenate([rng.integers(0, 1 << 20, 100_000), np.full(90_000, Rk[7])]).astype(np.uint32)
+    Rp = np.arange(len(Rk), dtype=np.uint32)
+    Sp = np.arange(len(Sk), dtype=np.uint32)
+    check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=16, mat=True)

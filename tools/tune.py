@@ -27,7 +27,7 @@ def main():
     w = W.CONFIGS[a.config]
     cols = W.torch_generate(w, device="cuda")
     ref = None
-    for v in a.values:
+    for v in a.values:  # join_variant: 0 = auto, k = shape k-1
         ctx = hj.Context(0, w.key_bytes, w.key_bytes)
         ctx.set_option(OPTS[a.opt], v)
         for _ in range(3):

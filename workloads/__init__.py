@@ -313,7 +313,9 @@ CONFIGS = {
     "c4_z0.5": Workload("c4_z0.5", 16 * M, 256 * M, "zipf", z=0.5, seed=4, out_mode=0, radix_bits=12),
     "c4_z1.0": Workload("c4_z1.0", 16 * M, 256 * M, "zipf", z=1.0, seed=5, out_mode=0, radix_bits=12),
     "c4_z1.5": Workload("c4_z1.5", 16 * M, 256 * M, "zipf", z=1.5, seed=6, out_mode=0, radix_bits=12),
-    "c5": Workload("c5", 2048 * M, 2048 * M, "1to1", keys="k8", seed=7, out_mode=0, radix_bits=15),
+    "c5": Workload("c5", 2048 * M, 2048 * M, "1to1", keys="k8", seed=7, out_mode=0, radix_bits=19),
+    # one GPU's share of c5 at 8 GPUs (2^28 x 2^28, 8 B keys / payloads), for single-GPU runs
+    "c5_gpu": Workload("c5_gpu", 256 * M, 256 * M, "1to1", keys="k8", seed=7, out_mode=0, radix_bits=16),
 }
 
 
