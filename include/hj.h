@@ -64,7 +64,9 @@ enum hj_option {
   HJ_OPT_TIMING = 4,       /* 1 = record per-phase CUDA events into hj_result (default 1)     */
   HJ_OPT_BLOCKS_PER_SM = 5, /* persistent-grid residency override for the passes (0 = auto)   */
   HJ_OPT_JOIN_VARIANT = 6,  /* join kernel shape (tuning; 0 = auto, k = shape k-1 of hj_api.cu)  */
-  HJ_OPT_PASS_THREADS = 7   /* partition-pass block size 512 / 1024 (0 = auto)                   */
+  HJ_OPT_PASS_THREADS = 7,  /* partition-pass block size 512 / 1024 (0 = auto)                   */
+  HJ_OPT_STREAM_CHUNK = 8   /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
+                               least 2^22; >= |S| = copy everything, then join)                   */
 };
 
 typedef struct hj_result {
@@ -116,9 +118,13 @@ int hj_join(hj_ctx* ctx,
             const void* S_keys, const void* S_pay, uint64_t nS,
             int radix_bits, int out_mode, hj_result* res);
 
-/* Same join from HOST columns (pageable or pinned): copies the inputs host->device on the ctx
- * stream, runs hj_join's pipeline, and copies the result back (matches/checksum, and for
- * MATERIALIZE the pairs into ctx-owned pinned host memory returned in res->*_pay_out). */
+/* Same join from HOST columns (pinned for full overlap; pageable works): the streaming probe
+ * of the paper's out-of-GPU strategy (NEXT-3). R is copied and
+ * partitioned once; S is copied in chunks (HJ_OPT_STREAM_CHUNK) on a copy stream into two
+ * device buffers while the compute stream partitions and joins the previous chunk with the
+ * resident R; MATERIALIZE pairs are drained to ctx-owned pinned host memory on a third stream
+ * as chunks finish (res->r_pay_out / s_pay_out, valid until the next call on ctx). If the result
+ * outgrows the device output buffer the call redoes the join with everything copied first. */
 int hj_join_host(hj_ctx* ctx,
                  const void* R_keys, const void* R_pay, uint64_t nR,
                  const void* S_keys, const void* S_pay, uint64_t nS,

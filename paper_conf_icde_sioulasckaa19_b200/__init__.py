@@ -36,6 +36,7 @@ OPT_TIMING = 4
 OPT_BLOCKS_PER_SM = 5
 OPT_JOIN_VARIANT = 6
 OPT_PASS_THREADS = 7
+OPT_STREAM_CHUNK = 8
 
 _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4: "HJ_ERR_CUDA", -5: "HJ_ERR_COMM"}
 

@@ -42,12 +42,16 @@ struct Ctx {
   int key_bytes = 4, pay_bytes = 4;
   cudaStream_t stream = nullptr;
   cudaStream_t own_stream = nullptr;
+  cudaStream_t h2d_stream = nullptr, d2h_stream = nullptr;  // streaming hj_join_host (NEXT-3)
+  cudaEvent_t sev[12] = {};                                  // streaming events
+  DevBuf sin[2][2];                                          // S chunk double buffers [buf][keys/pays]
+  void* h_cur = nullptr;                                     // pinned: output cursor per chunk
   int num_sms = 148;
   size_t smem_optin = 0;
   std::string err;
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
-          opt_pass_nt = 0;
+          opt_pass_nt = 0, opt_stream_chunk = 0;
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2];
   void* h_res = nullptr;  // pinned host: results readback
@@ -315,11 +319,16 @@ template <typename K, int MODE, int NT, bool GD>
 int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits);
 
 template <typename K>
-int launch_front(Ctx* c, const HostPlan& hp, const Plan& P) {
+int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false) {
   cudaStream_t st = c->stream;
   const bool gd = hp.g > 0;
   mark(c, 0);
-  CUDA_TRY(c, cudaMemsetAsync(c->meta.p, 0, hp.zero_bytes, st));
+  if (!chunk) {
+    CUDA_TRY(c, cudaMemsetAsync(c->meta.p, 0, hp.zero_bytes, st));
+  } else {  // streaming S chunk: keep R's counts and the accumulated results
+    CUDA_TRY(c, cudaMemsetAsync((char*)c->meta.p + hp.o_counters, 0, 64, st));
+    CUDA_TRY(c, cudaMemsetAsync((char*)c->meta.p + hp.o_cnt[1], 0, (size_t)4 << hp.qbits(), st));
+  }
   if (hp.mode != PLAN_RECV) {
     const bool smem = hp.qbits() <= 16;
     const bool c32 = hp.qbits() <= 15;  // 16 bins: packed 16-bit counters (128 KB)
@@ -331,6 +340,7 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P) {
     // blocks split proportionally to the relation sizes (at least one each)
     uint32_t gr = (uint32_t)((double)g * (double)nR / (double)std::max<unsigned long long>(nR + nS, 1) + 0.5);
     gr = std::min<uint32_t>(std::max<uint32_t>(gr, 1), (uint32_t)g - 1);
+    if (nR == 0) gr = 0;  // streaming S chunk: every block counts S
     if (smem && c32 && gd) k_hist<K, true, true, true><<<g, HIST_NT, sm, st>>>(P, gr);
     else if (smem && c32) k_hist<K, true, false, true><<<g, HIST_NT, sm, st>>>(P, gr);
     else if (smem && gd) k_hist<K, true, true, false><<<g, HIST_NT, sm, st>>>(P, gr);
@@ -515,6 +525,157 @@ int check_args(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, co
   return HJ_OK;
 }
 
+
+// ---- NEXT-3: streaming join from host memory (§IV-A, §IV-C) ---------
+// R is copied and partitioned once; S is copied in chunks on a copy stream into two device
+// buffers (one being copied, one being processed) while the compute stream
+// partitions each chunk and joins it with the resident R (the union of the chunk joins is the
+// join); materialized pairs are drained to pinned host memory on a third stream as
+// each chunk finishes. Falls back to the serial path if the result outgrows the
+// device output buffer.
+int join_host_serial(Ctx* c, const void* Rk, const void* Rp, uint64_t nR, const void* Sk, const void* Sp, uint64_t nS,
+                     int radix_bits, int out_mode, hj_result* res);
+
+int ensure_host(Ctx* c, size_t need) {
+  if (c->h_out_bytes >= need) return HJ_OK;
+  if (c->h_out) cudaFreeHost(c->h_out);
+  c->h_out = nullptr;
+  c->h_out_bytes = 0;
+  if (cudaMallocHost(&c->h_out, need) != cudaSuccess) return fail(c, HJ_ERR_OOM, "pinned host alloc of %zu B", need);
+  c->h_out_bytes = need;
+  return HJ_OK;
+}
+
+template <typename K>
+int join_host_stream(Ctx* c, const void* Rk, const void* Rp, uint64_t nR, const void* Sk, const void* Sp, uint64_t nS,
+                     int radix_bits, int out_mode, uint64_t chunk, hj_result* res) {
+  const bool mat = out_mode == HJ_OUT_MATERIALIZE;
+  const size_t kb = c->key_bytes, pb = c->pay_bytes;
+  cudaStream_t e = c->stream, t = c->h2d_stream, d = c->d2h_stream;
+  cudaEvent_t ev_start = c->sev[0], ev_r = c->sev[1], ev_s[2] = {c->sev[2], c->sev[3]},
+              ev_free[2] = {c->sev[4], c->sev[5]}, ev_j[2] = {c->sev[6], c->sev[7]}, ev_d = c->sev[8],
+              ev_end = c->sev[9];
+  HostPlan hp;
+  int rc = prepare(c, hp, nR, chunk, radix_bits, mat);
+  if (rc) return rc;
+  const unsigned long long cap = c->opt_out_cap > 0 ? (unsigned long long)c->opt_out_cap : std::max<unsigned long long>(nS, 1 << 20);
+  if (mat) {
+    if ((rc = ensure(c, c->out_r, cap * pb)) || (rc = ensure(c, c->out_s, cap * pb))) return rc;
+    if ((rc = ensure_host(c, 2 * cap * pb))) return rc;
+  }
+  if ((rc = ensure(c, c->in[0], nR * kb)) || (rc = ensure(c, c->in[1], nR * pb))) return rc;
+  for (int b = 0; b < 2; ++b)
+    if ((rc = ensure(c, c->sin[b][0], chunk * kb)) || (rc = ensure(c, c->sin[b][1], chunk * pb))) return rc;
+  c->launches = 0;
+  CUDA_TRY(c, cudaEventRecord(ev_start, t));
+  // R: copy, then partition (rows a1-a4 with S empty)
+  CUDA_TRY(c, cudaMemcpyAsync(c->in[0].p, Rk, nR * kb, cudaMemcpyHostToDevice, t));
+  CUDA_TRY(c, cudaMemcpyAsync(c->in[1].p, Rp, nR * pb, cudaMemcpyHostToDevice, t));
+  CUDA_TRY(c, cudaEventRecord(ev_r, t));
+  CUDA_TRY(c, cudaStreamWaitEvent(e, ev_r, 0));
+  Plan P = device_plan(c, hp, c->in[0].p, c->in[1].p, nR, nullptr, nullptr, 0);
+  if ((rc = launch_front<K>(c, hp, P))) return rc;
+  if ((rc = launch_pass2<K>(c, hp, P))) return rc;
+  char* ho = (char*)c->h_out;
+  unsigned long long* hcur = (unsigned long long*)c->h_cur;
+  unsigned long long drained = 0;
+  bool overflow = false;
+  const uint64_t nch = (nS + chunk - 1) / chunk;
+  auto drain = [&](int slot) -> int {  // host: chunk in `slot` finished -> copy its new pairs out
+    CUDA_TRY(c, cudaEventSynchronize(ev_j[slot]));
+    const unsigned long long cur = hcur[slot];
+    if (cur > cap) overflow = true;
+    if (overflow || cur <= drained) return HJ_OK;
+    CUDA_TRY(c, cudaStreamWaitEvent(d, ev_j[slot], 0));
+    CUDA_TRY(c, cudaMemcpyAsync(ho + drained * pb, (char*)c->out_r.p + drained * pb, (cur - drained) * pb,
+                                cudaMemcpyDeviceToHost, d));
+    CUDA_TRY(c, cudaMemcpyAsync(ho + (cap + drained) * pb, (char*)c->out_s.p + drained * pb, (cur - drained) * pb,
+                                cudaMemcpyDeviceToHost, d));
+    drained = cur;
+    return HJ_OK;
+  };
+  for (uint64_t k = 0; k < nch; ++k) {
+    const int b = (int)(k & 1);
+    const uint64_t s0 = k * chunk, len = std::min<uint64_t>(chunk, nS - s0);
+    // copy stream: S chunk k into buffer b once chunk k-2 has left it
+    if (k >= 2) CUDA_TRY(c, cudaStreamWaitEvent(t, ev_free[b], 0));
+    CUDA_TRY(c, cudaMemcpyAsync(c->sin[b][0].p, (const char*)Sk + s0 * kb, len * kb, cudaMemcpyHostToDevice, t));
+    CUDA_TRY(c, cudaMemcpyAsync(c->sin[b][1].p, (const char*)Sp + s0 * pb, len * pb, cudaMemcpyHostToDevice, t));
+    CUDA_TRY(c, cudaEventRecord(ev_s[b], t));
+    // compute stream: partition the chunk (R skipped) and join it with R
+    CUDA_TRY(c, cudaStreamWaitEvent(e, ev_s[b], 0));
+    Plan Q = device_plan(c, hp, nullptr, nullptr, 0, c->sin[b][0].p, c->sin[b][1].p, len);
+    Q.skip_r = 1;
+    if ((rc = launch_front<K>(c, hp, Q, true))) return rc;
+    CUDA_TRY(c, cudaEventRecord(ev_free[b], e));  // pass 1 consumed buffer b
+    if ((rc = launch_pass2<K>(c, hp, Q))) return rc;
+    if ((rc = launch_join<K>(c, hp, Q, mat))) return rc;
+    if (mat) {
+      CUDA_TRY(c, cudaMemcpyAsync(hcur + b, Q.results + RES_CURSOR, 8, cudaMemcpyDeviceToHost, e));
+      CUDA_TRY(c, cudaEventRecord(ev_j[b], e));
+      if (k >= 1 && (rc = drain(1 - b))) return rc;  // chunk k-1 is done by now or soon
+    }
+  }
+  if (mat && (rc = drain((int)((nch - 1) & 1)))) return rc;
+  unsigned long long* h = (unsigned long long*)c->h_res;
+  Plan F = device_plan(c, hp, nullptr, nullptr, 0, nullptr, nullptr, 0);
+  CUDA_TRY(c, cudaMemcpyAsync(h, F.results, 4 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, e));
+  CUDA_TRY(c, cudaEventRecord(ev_d, d));
+  CUDA_TRY(c, cudaStreamWaitEvent(e, ev_d, 0));
+  CUDA_TRY(c, cudaEventRecord(ev_end, e));
+  CUDA_TRY(c, cudaStreamSynchronize(e));
+  if (overflow || h[RES_MATCHES] > cap) return join_host_serial(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
+  memset(res, 0, sizeof *res);
+  res->matches = h[RES_MATCHES];
+  res->checksum = h[RES_CHECKSUM];
+  res->radix_bits = hp.B;
+  res->passes = hp.B >= 2 ? 2 : (hp.B == 1 ? 1 : 0);
+  res->kernels = c->launches;
+  if (mat) {
+    res->r_pay_out = ho;
+    res->s_pay_out = ho + cap * pb;
+  }
+  cudaEventElapsedTime(&res->ms_total, ev_start, ev_end);
+  return HJ_OK;
+}
+
+int join_host_serial(Ctx* c, const void* Rk, const void* Rp, uint64_t nR, const void* Sk, const void* Sp, uint64_t nS,
+                     int radix_bits, int out_mode, hj_result* res) {
+  int rc = HJ_OK;
+  const size_t kb = c->key_bytes, pb = c->pay_bytes;
+  cudaStream_t st = c->stream;
+  const void* src[4] = {Rk, Rp, Sk, Sp};
+  const size_t bytes[4] = {nR * kb, nR * pb, nS * kb, nS * pb};
+  for (int i = 0; i < 4 && rc == HJ_OK; ++i) {
+    rc = ensure(c, c->in[i], bytes[i]);
+    if (rc == HJ_OK && cudaMemcpyAsync(c->in[i].p, src[i], bytes[i], cudaMemcpyHostToDevice, st) != cudaSuccess)
+      rc = fail(c, HJ_ERR_CUDA, "H2D copy failed");
+  }
+  if (rc == HJ_OK)
+    rc = run_join(c, c->in[0].p, c->in[1].p, nR, c->in[2].p, c->in[3].p, nS, radix_bits, out_mode, res);
+  if (rc == HJ_OK && out_mode == HJ_OUT_MATERIALIZE && res->matches) {
+    const size_t need = 2 * res->matches * pb;
+    if (c->h_out_bytes < need) {
+      if (c->h_out) cudaFreeHost(c->h_out);
+      c->h_out = nullptr;
+      c->h_out_bytes = 0;
+      if (cudaMallocHost(&c->h_out, need) != cudaSuccess) rc = fail(c, HJ_ERR_OOM, "pinned host alloc of %zu B", need);
+      else c->h_out_bytes = need;
+    }
+    if (rc == HJ_OK) {
+      char* ho = (char*)c->h_out;
+      if (cudaMemcpyAsync(ho, res->r_pay_out, res->matches * pb, cudaMemcpyDeviceToHost, st) != cudaSuccess ||
+          cudaMemcpyAsync(ho + res->matches * pb, res->s_pay_out, res->matches * pb, cudaMemcpyDeviceToHost, st) !=
+              cudaSuccess ||
+          cudaStreamSynchronize(st) != cudaSuccess)
+        rc = fail(c, HJ_ERR_CUDA, "D2H copy of pairs failed");
+      res->r_pay_out = ho;
+      res->s_pay_out = ho + res->matches * pb;
+    }
+  }
+  return rc;
+}
+
 }  // namespace
 
 struct hj_ctx {
@@ -569,6 +730,10 @@ int hj_create(hj_ctx** out, int device, int key_bytes, int pay_bytes, void* cuda
   }
   c->stream = cuda_stream ? (cudaStream_t)cuda_stream : c->own_stream;
   for (auto& ev : c->ev) cudaEventCreate(&ev);
+  for (auto& ev : c->sev) cudaEventCreate(&ev);
+  cudaStreamCreateWithFlags(&c->h2d_stream, cudaStreamNonBlocking);
+  cudaStreamCreateWithFlags(&c->d2h_stream, cudaStreamNonBlocking);
+  cudaMallocHost(&c->h_cur, 64);
   cudaSetDevice(prev);
   *out = h;
   return HJ_OK;
@@ -590,6 +755,14 @@ void hj_destroy(hj_ctx* h) {
   if (c->h_out) cudaFreeHost(c->h_out);
   for (auto& ev : c->ev)
     if (ev) cudaEventDestroy(ev);
+  for (auto& ev : c->sev)
+    if (ev) cudaEventDestroy(ev);
+  for (auto& b : c->sin)
+    for (auto& x : b)
+      if (x.p) cudaFree(x.p);
+  if (c->h_cur) cudaFreeHost(c->h_cur);
+  if (c->h2d_stream) cudaStreamDestroy(c->h2d_stream);
+  if (c->d2h_stream) cudaStreamDestroy(c->d2h_stream);
   if (c->own_stream) cudaStreamDestroy(c->own_stream);
   cudaSetDevice(prev);
   delete h;
@@ -613,6 +786,7 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_OUT_CAPACITY: c->opt_out_cap = v; break;
     case HJ_OPT_TIMING: c->opt_timing = v; break;
     case HJ_OPT_BLOCKS_PER_SM: c->opt_bps = v; break;
+    case HJ_OPT_STREAM_CHUNK: c->opt_stream_chunk = v; break;
     case HJ_OPT_PASS_THREADS:
       if (v != 0 && v != 512 && v != 1024) return fail(c, HJ_ERR_INVALID, "pass threads must be 0, 512 or 1024");
       c->opt_pass_nt = v;
@@ -655,37 +829,12 @@ int hj_join_host(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const v
   int prev = 0;
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
-  const size_t kb = c->key_bytes, pb = c->pay_bytes;
-  cudaStream_t st = c->stream;
-  const void* src[4] = {Rk, Rp, Sk, Sp};
-  const size_t bytes[4] = {nR * kb, nR * pb, nS * kb, nS * pb};
-  for (int i = 0; i < 4 && rc == HJ_OK; ++i) {
-    rc = ensure(c, c->in[i], bytes[i]);
-    if (rc == HJ_OK && cudaMemcpyAsync(c->in[i].p, src[i], bytes[i], cudaMemcpyHostToDevice, st) != cudaSuccess)
-      rc = fail(c, HJ_ERR_CUDA, "H2D copy failed");
-  }
-  if (rc == HJ_OK)
-    rc = run_join(c, c->in[0].p, c->in[1].p, nR, c->in[2].p, c->in[3].p, nS, radix_bits, out_mode, res);
-  if (rc == HJ_OK && out_mode == HJ_OUT_MATERIALIZE && res->matches) {
-    const size_t need = 2 * res->matches * pb;
-    if (c->h_out_bytes < need) {
-      if (c->h_out) cudaFreeHost(c->h_out);
-      c->h_out = nullptr;
-      c->h_out_bytes = 0;
-      if (cudaMallocHost(&c->h_out, need) != cudaSuccess) rc = fail(c, HJ_ERR_OOM, "pinned host alloc of %zu B", need);
-      else c->h_out_bytes = need;
-    }
-    if (rc == HJ_OK) {
-      char* ho = (char*)c->h_out;
-      if (cudaMemcpyAsync(ho, res->r_pay_out, res->matches * pb, cudaMemcpyDeviceToHost, st) != cudaSuccess ||
-          cudaMemcpyAsync(ho + res->matches * pb, res->s_pay_out, res->matches * pb, cudaMemcpyDeviceToHost, st) !=
-              cudaSuccess ||
-          cudaStreamSynchronize(st) != cudaSuccess)
-        rc = fail(c, HJ_ERR_CUDA, "D2H copy of pairs failed");
-      res->r_pay_out = ho;
-      res->s_pay_out = ho + res->matches * pb;
-    }
-  }
+  // chunk: HJ_OPT_STREAM_CHUNK, else auto (|S| / 8, at least 2^22 tuples)
+  const uint64_t chunk = c->opt_stream_chunk > 0 ? (uint64_t)c->opt_stream_chunk
+                                                 : std::max<uint64_t>((nS + 7) / 8, 1ull << 22);
+  if (chunk >= nS) rc = join_host_serial(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
+  else if (c->key_bytes == 4) rc = join_host_stream<uint32_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, chunk, res);
+  else rc = join_host_stream<uint64_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, chunk, res);
   cudaSetDevice(prev);
   return rc;
 }

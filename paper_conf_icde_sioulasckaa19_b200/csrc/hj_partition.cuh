@@ -411,7 +411,7 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
       s_pst[i] = P.rel[0].pst[i];
       s_pst[1025 + i] = P.rel[1].pst[i];
     }
-    W.units0 = P.rel[0].cst[npc];
+    W.units0 = P.skip_r ? 0ull : P.rel[0].cst[npc];
     W.units = W.units0 + P.rel[1].cst[npc];
   }
   __syncthreads();

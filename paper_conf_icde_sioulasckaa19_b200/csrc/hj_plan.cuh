@@ -37,6 +37,7 @@ struct Plan {
   int g;          // rank bits in the pass-1 digit (PLAN_SEND), else 0
   int nsrc;       // count rows / piece sources (PLAN_RECV: ranks), else 1
   int mode;       // PLAN_FULL, PLAN_SEND, PLAN_RECV
+  int skip_r;     // streaming S chunks: R is already partitioned (its pass-2 units are skipped)
   uint32_t C2;           // pass-2 chunk (tile) size in tuples
   uint32_t CR, CS;       // join item capacities: R tuples (smem build) and S tuples per item
   uint32_t* ist;         // [2^B + 1] join item prefix (q-order)

@@ -272,3 +272,50 @@ def test_join_16bit_counters(hj):
     Rp = np.arange(len(Rk), dtype=np.uint32)
     Sp = np.arange(len(Sk), dtype=np.uint32)
     check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=16, mat=True)
+
+
+@pytest.mark.parametrize("chunk", [1000, 4097, 65536])
+@pytest.mark.parametrize("dist_", ["fk", "zipf"])
+def test_join_host_streaming_vs_oracle(hj, chunk, dist_):
+    """NEXT-3 streaming probe (P:412-446): S copied and joined in chunks against the resident R;
+    the union of the chunk joins is the join."""
+    w = W.Workload("t", 30_000, 200_003, dist_, keys="sparse", z=1.0, seed=150)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    m, c, r, s = oracle.hash_join(Rk, Rp, Sk, Sp, materialize=True)
+    ctx = hj.Context(0, 4, 4)
+    ctx.set_option(hj.OPT_STREAM_CHUNK, chunk)
+    res = ctx.join_host(Rk, Rp, Sk, Sp)
+    assert (res.matches, res.checksum) == (m, c)
+    res = ctx.join_host(Rk, Rp, Sk, Sp, out_mode=hj.OUT_MATERIALIZE)
+    assert res.matches == m
+    assert np.array_equal(oracle.pairs_sorted(res.r_pay, res.s_pay), oracle.pairs_sorted(r, s))
+    ctx.close()
+
+
+def test_join_host_streaming_duplicates_and_overflow(hj):
+    """Duplicate keys on both sides; the result outgrows the initial output capacity, so the
+    streamed call falls back to the copy-everything path and regrows (reading S11)."""
+    rng = np.random.default_rng(151)
+    Rk = rng.integers(0, 300, 5000).astype(np.uint32)
+    Sk = rng.integers(0, 300, 20000).astype(np.uint32)
+    Rp = np.arange(len(Rk), dtype=np.uint32)
+    Sp = np.arange(len(Sk), dtype=np.uint32)
+    m, c, r, s = oracle.hash_join(Rk, Rp, Sk, Sp, materialize=True)
+    ctx = hj.Context(0, 4, 4)
+    ctx.set_option(hj.OPT_STREAM_CHUNK, 3000)
+    ctx.set_option(hj.OPT_OUT_CAPACITY, 50_000)
+    res = ctx.join_host(Rk, Rp, Sk, Sp, out_mode=hj.OUT_MATERIALIZE)
+    assert res.matches == m > 50_000
+    assert np.array_equal(oracle.pairs_sorted(res.r_pay, res.s_pay), oracle.pairs_sorted(r, s))
+    assert ctx.join_host(Rk, Rp, Sk, Sp).checksum == c
+    ctx.close()
+
+
+def test_join_host_streaming_8byte(hj):
+    w = W.Workload("t", 1 << 14, 1 << 17, "fk", keys="k8", seed=152)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    m, c = oracle.hash_join(Rk, Rp, Sk, Sp)
+    ctx = hj.Context(0, 8, 8)
+    ctx.set_option(hj.OPT_STREAM_CHUNK, 10_000)
+    assert (lambda r: (r.matches, r.checksum))(ctx.join_host(Rk, Rp, Sk, Sp)) == (m, c)
+    ctx.close()
