@@ -829,9 +829,9 @@ int hj_join_host(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const v
   int prev = 0;
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
-  // chunk: HJ_OPT_STREAM_CHUNK, else auto (|S| / 8, at least 2^22 tuples)
+  // chunk: HJ_OPT_STREAM_CHUNK, else auto (|S| / 16, at least 2^22 tuples; measured on c3)
   const uint64_t chunk = c->opt_stream_chunk > 0 ? (uint64_t)c->opt_stream_chunk
-                                                 : std::max<uint64_t>((nS + 7) / 8, 1ull << 22);
+                                                 : std::max<uint64_t>((nS + 15) / 16, 1ull << 22);
   if (chunk >= nS) rc = join_host_serial(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
   else if (c->key_bytes == 4) rc = join_host_stream<uint32_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, chunk, res);
   else rc = join_host_stream<uint64_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, chunk, res);
