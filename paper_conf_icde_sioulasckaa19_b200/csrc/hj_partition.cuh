@@ -382,6 +382,7 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
   uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gd + 2 * F);                     // F + 1 (spare)
   uint32_t* s_loc = s_cnt + F + 4;                                                 // F
   __shared__ uint32_t s_wt[NT / 32];
+  __shared__ uint32_t s_hot, s_hot_next;
   __shared__ uint32_t s_cst[MODE == 2 ? 2 * 1025 : 1];
   __shared__ unsigned long long s_pst[MODE == 2 ? 2 * 1025 : 1];
 
@@ -399,6 +400,7 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
 
   if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
+  if (threadIdx.x == 0) s_hot = s_hot_next = 0xffffffffu;
   UnitWalker<K, MODE, TILE> W;
   if (MODE == 1) {
     W.units0 = P.tiles1[0];
@@ -467,11 +469,33 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
     uint32_t rk[ITEMS / 2];  // ranks < TILE <= 2^16, two per register
     const uint32_t ulen = s_desc[slot].len;
     const bool full = ulen == TILE;
-    #pragma unroll
-    for (int j = 0; j < ITEMS; ++j) {
-      const uint32_t d = (full || pass_elem<K, MODE, NT>(j) < ulen) ? digit(kk[j]) : F;
-      const uint32_t r = atomicAdd(&s_cnt[d], 1u);
-      if (j & 1) rk[j / 2] |= r << 16; else rk[j / 2] = r & 0xffffu;
+    const uint32_t hot = s_hot;  // digit holding > 1/4 of the previous unit, or none (> F)
+    if (hot > F) {
+      #pragma unroll
+      for (int j = 0; j < ITEMS; ++j) {
+        const uint32_t d = (full || pass_elem<K, MODE, NT>(j) < ulen) ? digit(kk[j]) : F;
+        const uint32_t r = atomicAdd(&s_cnt[d], 1u);
+        if (j & 1) rk[j / 2] |= r << 16; else rk[j / 2] = r & 0xffffu;
+      }
+    } else {
+      // skew: lanes on the hot digit are ranked with one ballot + one atomic per warp instead
+      // of serialising on the same shared counter (Zipf probe sides)
+      #pragma unroll
+      for (int j = 0; j < ITEMS; ++j) {
+        const uint32_t d = (full || pass_elem<K, MODE, NT>(j) < ulen) ? digit(kk[j]) : F;
+        const uint32_t hm = __ballot_sync(0xffffffffu, d == hot);
+        uint32_t r;
+        if (hm) {
+          const int leader = __ffs(hm) - 1;
+          uint32_t base = 0;
+          if (lane == leader) base = atomicAdd(&s_cnt[hot], (uint32_t)__popc(hm));
+          base = __shfl_sync(0xffffffffu, base, leader);
+          r = (d == hot) ? base + __popc(hm & lanemask_lt()) : atomicAdd(&s_cnt[d], 1u);
+        } else {
+          r = atomicAdd(&s_cnt[d], 1u);
+        }
+        if (j & 1) rk[j / 2] |= r << 16; else rk[j / 2] = r & 0xffffu;
+      }
     }
     __syncthreads();
 
@@ -495,6 +519,7 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
         s_loc[d] = loc;
         s_cnt[d] = 0;
         if (c) gd[d] = atomicAdd(s_desc[slot].cur + d, (unsigned long long)c) - loc;
+        if (c > TILE / 4) s_hot_next = d;  // predicts the next unit's hot digit
       }
     }
     if (threadIdx.x == NT - 1)  // publish unit i+2
@@ -503,6 +528,10 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
     __syncthreads();
 
     // ---- phase 3: shuffle unit i into digit order in shared memory -----------------------------
+    if (threadIdx.x == 0) {  // read by the next unit's phase 1 (after this thread's own reads)
+      s_hot = s_hot_next;
+      s_hot_next = 0xffffffffu;
+    }
     #pragma unroll
     for (int j = 0; j < ITEMS; ++j)
       if (full || pass_elem<K, MODE, NT>(j) < ulen)
