@@ -65,6 +65,9 @@ enum hj_option {
   HJ_OPT_BLOCKS_PER_SM = 5, /* persistent-grid residency override for the passes (0 = auto)   */
   HJ_OPT_JOIN_VARIANT = 6,  /* join kernel shape (tuning; 0 = auto, k = shape k-1 of hj_api.cu)  */
   HJ_OPT_PASS_THREADS = 7,  /* partition-pass block size 512 / 1024 (0 = auto)                   */
+  HJ_OPT_JOIN_ALGO = 9,     /* 0 = radix-partitioned + smem hash table (default); 1 = radix-
+                               partitioned + ballot nested loops (Listing 1); 2 = non-
+                               partitioned hash join on a device-memory table (Fig. 8) */
   HJ_OPT_STREAM_CHUNK = 8   /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
                                least 2^22; >= |S| = copy everything, then join)                   */
 };

@@ -12,6 +12,7 @@
 #include "../../include/hj.h"
 #include "hj_join.cuh"
 #include "hj_partition.cuh"
+#include "hj_variants.cuh"
 
 using namespace hj;
 
@@ -51,9 +52,9 @@ struct Ctx {
   std::string err;
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
-          opt_pass_nt = 0, opt_stream_chunk = 0;
+          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0;
   // workspace
-  DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2];
+  DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2], np_heads, np_next;
   void* h_res = nullptr;  // pinned host: results readback
   void* h_out = nullptr;  // pinned host: materialized pairs (hj_join_host)
   size_t h_out_bytes = 0;
@@ -228,6 +229,8 @@ int set_kernel_attrs(Ctx* c) {
                              (int)(c->smem_optin - fa.sharedSizeBytes)) != cudaSuccess)
       rc = -1;
   };
+  attr((const void*)k_join_nlj<K, 256, false>);
+  attr((const void*)k_join_nlj<K, 256, true>);
   attr((const void*)k_hist<K, true, false, true>);
   attr((const void*)k_hist<K, true, true, true>);
   attr((const void*)k_hist<K, true, false, false>);
@@ -415,6 +418,17 @@ int launch_join_v(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
 template <typename K>
 int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   int rc;
+  if (c->opt_join_algo == 1) {  // ballot nested-loop co-partition join (Listing 1)
+    const size_t sm = (size_t)hp.CR * 2 * sizeof(K);
+    const void* f = mat ? (const void*)k_join_nlj<K, 256, true> : (const void*)k_join_nlj<K, 256, false>;
+    const int g = grid_for(c, f, 256, sm, 1ull << 40);
+    if (mat) k_join_nlj<K, 256, true><<<g, 256, sm, c->stream>>>(P);
+    else k_join_nlj<K, 256, false><<<g, 256, sm, c->stream>>>(P);
+    CUDA_TRY(c, cudaGetLastError());
+    mark(c, 5);
+    c->launches += 1;
+    return HJ_OK;
+  }
   switch (join_variant(c)) {
     case 5: rc = launch_join_v<K, 5>(c, hp, P, mat); break;
     case 6: rc = launch_join_v<K, 6>(c, hp, P, mat); break;
@@ -501,9 +515,78 @@ int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res) {
   return HJ_OK;
 }
 
+// HJ_OPT_JOIN_ALGO = 2: the non-partitioned GPU hash join (device-memory chained table; the
+// paper's Fig. 8 baseline). No histogram, no passes: build R, probe S.
+template <typename K>
+int run_join_np(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk, const void* Sp,
+                unsigned long long nS, bool mat, hj_result* res) {
+  HostPlan hp;
+  int rc = make_plan(c, hp, nR, nS, 0, mat);
+  if (rc) return rc;
+  const int lg = std::max(1, ilog2_ceil(nR));
+  if ((rc = ensure(c, c->meta, hp.meta_bytes)) || (rc = ensure(c, c->np_heads, (size_t)4 << lg)) ||
+      (rc = ensure(c, c->np_next, nR * 4)))
+    return rc;
+  unsigned long long cap = c->opt_out_cap > 0 ? (unsigned long long)c->opt_out_cap : std::max<unsigned long long>(nS, 1 << 20);
+  if (mat && c->out_r.bytes < cap * c->pay_bytes &&
+      ((rc = ensure(c, c->out_r, cap * c->pay_bytes)) || (rc = ensure(c, c->out_s, cap * c->pay_bytes))))
+    return rc;
+  Plan P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
+  cudaStream_t st = c->stream;
+  c->launches = 0;
+  for (int attempt = 0; attempt < 2; ++attempt) {
+    mark(c, 0);
+    CUDA_TRY(c, cudaMemsetAsync(c->meta.p, 0, hp.zero_bytes, st));
+    CUDA_TRY(c, cudaMemsetAsync(c->np_heads.p, 0xff, (size_t)4 << lg, st));
+    for (int k = 1; k <= 4; ++k) mark(c, k);
+    const int g = 4 * c->num_sms;
+    k_np_build<K><<<g, 512, 0, st>>>((const K*)Rk, nR, (uint32_t*)c->np_heads.p, (uint32_t*)c->np_next.p, lg);
+    if (mat)
+      k_np_probe<K, true><<<g, 512, 0, st>>>(P, (const K*)Rk, (const K*)Rp, (const K*)Sk, (const K*)Sp, nS,
+                                              (const uint32_t*)c->np_heads.p, (const uint32_t*)c->np_next.p, lg);
+    else
+      k_np_probe<K, false><<<g, 512, 0, st>>>(P, (const K*)Rk, (const K*)Rp, (const K*)Sk, (const K*)Sp, nS,
+                                               (const uint32_t*)c->np_heads.p, (const uint32_t*)c->np_next.p, lg);
+    CUDA_TRY(c, cudaGetLastError());
+    c->launches += 2;
+    mark(c, 5);
+    unsigned long long* h = (unsigned long long*)c->h_res;
+    CUDA_TRY(c, cudaMemcpyAsync(h, P.results, 4 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st));
+    mark(c, 6);
+    CUDA_TRY(c, cudaStreamSynchronize(st));
+    if (mat && h[RES_MATCHES] > P.out_cap && attempt == 0) {  // grow and re-run (reading S11)
+      if ((rc = ensure(c, c->out_r, h[RES_MATCHES] * c->pay_bytes)) ||
+          (rc = ensure(c, c->out_s, h[RES_MATCHES] * c->pay_bytes)))
+        return rc;
+      P.out_r = c->out_r.p;
+      P.out_s = c->out_s.p;
+      P.out_cap = h[RES_MATCHES];
+      continue;
+    }
+    memset(res, 0, sizeof *res);
+    res->matches = h[RES_MATCHES];
+    res->checksum = h[RES_CHECKSUM];
+    res->kernels = c->launches;
+    if (mat) {
+      res->r_pay_out = c->out_r.p;
+      res->s_pay_out = c->out_s.p;
+    }
+    if (c->opt_timing) {
+      cudaEventElapsedTime(&res->ms_total, c->ev[0], c->ev[6]);
+      cudaEventElapsedTime(&res->ms_join, c->ev[4], c->ev[6]);
+      for (int k = 0; k < 5; ++k) cudaEventElapsedTime(&res->ms_kernel[k], c->ev[k], c->ev[k + 1]);
+    }
+    return HJ_OK;
+  }
+  return HJ_OK;
+}
+
 int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk, const void* Sp,
              unsigned long long nS, int radix_bits, int out_mode, hj_result* res) {
   const bool mat = out_mode == HJ_OUT_MATERIALIZE;
+  if (c->opt_join_algo == 2)
+    return c->key_bytes == 4 ? run_join_np<uint32_t>(c, Rk, Rp, nR, Sk, Sp, nS, mat, res)
+                             : run_join_np<uint64_t>(c, Rk, Rp, nR, Sk, Sp, nS, mat, res);
   HostPlan hp;
   int rc = prepare(c, hp, nR, nS, radix_bits, mat);
   if (rc) return rc;
@@ -748,7 +831,7 @@ void hj_destroy(hj_ctx* h) {
   if (c->stream) cudaStreamSynchronize(c->stream);
   DevBuf* bufs[] = {&c->t1[0], &c->t1[1], &c->t2[0], &c->t2[1], &c->meta,    &c->out_r,    &c->out_s,
                     &c->in[0], &c->in[1], &c->in[2], &c->in[3], &c->xsend[0], &c->xsend[1], &c->xcnt[0],
-                    &c->xcnt[1]};
+                    &c->xcnt[1], &c->np_heads, &c->np_next};
   for (DevBuf* b : bufs)
     if (b->p) cudaFree(b->p);
   if (c->h_res) cudaFreeHost(c->h_res);
@@ -787,6 +870,10 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_TIMING: c->opt_timing = v; break;
     case HJ_OPT_BLOCKS_PER_SM: c->opt_bps = v; break;
     case HJ_OPT_STREAM_CHUNK: c->opt_stream_chunk = v; break;
+    case HJ_OPT_JOIN_ALGO:
+      if (v > 2) return fail(c, HJ_ERR_INVALID, "join algorithm must be 0, 1 or 2");
+      c->opt_join_algo = v;
+      break;
     case HJ_OPT_PASS_THREADS:
       if (v != 0 && v != 512 && v != 1024) return fail(c, HJ_ERR_INVALID, "pass threads must be 0, 512 or 1024");
       c->opt_pass_nt = v;
@@ -832,7 +919,7 @@ int hj_join_host(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const v
   // chunk: HJ_OPT_STREAM_CHUNK, else auto (|S| / 16, at least 2^22 tuples; measured on c3)
   const uint64_t chunk = c->opt_stream_chunk > 0 ? (uint64_t)c->opt_stream_chunk
                                                  : std::max<uint64_t>((nS + 15) / 16, 1ull << 22);
-  if (chunk >= nS) rc = join_host_serial(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
+  if (chunk >= nS || c->opt_join_algo == 2) rc = join_host_serial(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
   else if (c->key_bytes == 4) rc = join_host_stream<uint32_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, chunk, res);
   else rc = join_host_stream<uint64_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, chunk, res);
   cudaSetDevice(prev);

@@ -319,3 +319,40 @@ def test_join_host_streaming_8byte(hj):
     ctx.set_option(hj.OPT_STREAM_CHUNK, 10_000)
     assert (lambda r: (r.matches, r.checksum))(ctx.join_host(Rk, Rp, Sk, Sp)) == (m, c)
     ctx.close()
+
+
+@pytest.mark.parametrize("algo", [1, 2])
+@pytest.mark.parametrize("name", ["all_equal", "dups_both", "extremes", "random_ragged", "sparse_uniform", "one_row"])
+def test_comparator_algorithms_vs_oracle(hj, algo, name):
+    """NEXT-4: the ballot nested-loop co-partition join (Listing 1) and the non-partitioned
+    device-memory hash join (Fig. 8 baseline) return exactly the oracle's result."""
+    rng = np.random.default_rng(99)
+    Rk, Sk = adversarial(rng)[name]
+    Rp = rng.integers(0, 1 << 32, len(Rk), dtype=np.uint64).astype(np.uint32)
+    Sp = rng.integers(0, 1 << 32, len(Sk), dtype=np.uint64).astype(np.uint32)
+    ctx = hj.Context(0, 4, 4)
+    ctx.set_option(hj.OPT_JOIN_ALGO, algo)
+    for bits in (-1, 0, 6):
+        check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True, ctx=ctx)
+    ctx.close()
+
+
+@pytest.mark.parametrize("algo", [1, 2])
+@pytest.mark.parametrize("dist,keys", [("fk", "dense"), ("zipf", "sparse"), ("1to1", "k8")])
+def test_comparator_algorithms_generated(hj, algo, dist, keys):
+    w = W.Workload("t", 1 << 14, 1 << 14, dist, keys=keys, z=1.2, seed=160)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    ctx = hj.Context(0, w.key_bytes, w.key_bytes)
+    ctx.set_option(hj.OPT_JOIN_ALGO, algo)
+    check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=-1, mat=True, ctx=ctx)
+    ctx.close()
+
+
+@pytest.mark.parametrize("dist,z,rep", [("zipf_build", 0.5, 1), ("zipf_build", 1.0, 1), ("zipf_both", 0.5, 1),
+                                        ("zipf_both", 1.0, 1), ("replicas", 0, 2), ("replicas", 0, 4)])
+def test_next2_skew_and_replicas_vs_oracle(hj, dist, z, rep):
+    """NEXT-2: build-side skew (R co-partitions beyond shared memory -> hash-based block nested
+    loops), identical skew (output explosion -> exact growth), replicas."""
+    w = W.Workload("t", 1 << 15, 1 << 15, dist, keys="sparse", z=z, rep=rep, seed=170)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=-1, mat=True)

@@ -219,3 +219,21 @@ def test_copartition_property():
         tm += m
         tc = (tc + c) & M64
     assert (tm, tc) == full
+
+
+@pytest.mark.parametrize("dist,z,rep", [("zipf_build", 1.0, 1), ("zipf_both", 0.75, 1), ("replicas", 0, 2),
+                                        ("replicas", 0, 4)])
+def test_oracle_next2_vs_sort_merge(dist, z, rep):
+    """NEXT-2 workloads (Fig. 17 build-side / identical skew, Fig. 19 replicas): the oracle's count
+    equals sum_k cR(k) * cS(k) and the closed form where one exists."""
+    w = W.Workload("t", 1 << 13, 1 << 13, dist, z=z, rep=rep, seed=112)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    ur, cr = np.unique(Rk, return_counts=True)
+    us, cs = np.unique(Sk, return_counts=True)
+    _, ir, is_ = np.intersect1d(ur, us, return_indices=True)
+    expected = int((cr[ir].astype(np.int64) * cs[is_].astype(np.int64)).sum())
+    m, _ = oracle.hash_join(Rk, Rp, Sk, Sp)
+    assert m == expected
+    cf = W.expected_matches_closed_form(w)
+    if cf is not None:
+        assert m == cf

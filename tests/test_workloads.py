@@ -95,3 +95,27 @@ def test_torch_generator_int32_layout():
     w = W.Workload("t", 1 << 10, 1 << 10, "1to1", seed=108)
     Rk, Rp, Sk, Sp = W.torch_generate(w, device="cpu")
     assert Rk.dtype == torch.int32 and Rk.is_contiguous()
+
+
+@pytest.mark.parametrize("dist", ["zipf_build", "zipf_both", "replicas"])
+@pytest.mark.parametrize("keys", ["dense", "k8"])
+def test_next2_generators_agree(dist, keys):
+    w = W.Workload("t", 1 << 12, 1 << 13, dist, keys=keys, z=1.0, seed=109, rep=4)
+    a = W.np_generate(w)
+    b = W.torch_generate(w, device="cpu")
+    for x, y in zip(a, b):
+        assert np.array_equal(x, y.numpy().view(x.dtype))
+
+
+def test_next2_shapes():
+    # build skew: R has duplicates, S is a permutation of the domain
+    w = W.Workload("t", 1 << 14, 1 << 14, "zipf_build", z=1.0, seed=110)
+    Rk, _, Sk, _ = W.np_generate(w)
+    assert len(np.unique(Sk)) == len(Sk) and np.isin(Rk, Sk).all()
+    _, c = np.unique(Rk, return_counts=True)
+    assert c.max() > 100  # the top build-side value repeats
+    # replicas: every key exactly rep times on each side
+    w = W.Workload("t", 1 << 12, 1 << 12, "replicas", rep=4, seed=111)
+    Rk, _, Sk, _ = W.np_generate(w)
+    assert set(np.unique(Rk, return_counts=True)[1]) == {4}
+    assert set(np.unique(Sk, return_counts=True)[1]) == {4}

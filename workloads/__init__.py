@@ -27,6 +27,10 @@ Definitions (all arithmetic mod 2^64 unless stated):
   key maps             dense4: x + 1;  sparse4: fmix32(x + 1);  k8: fmix64((x + 1) ^ seed_k)
   R                    R_key[i] = K(perm_n(seed_R, nR, i)), R_pay[i] = i
   S                    S_key[j] = R_key[rho(j)], S_pay[j] = j
+  NEXT-2 skew / duplicate workloads (Fig. 17 build-side and identical skew, Fig. 19 replicas):
+    'zipf_build': R_key[i] = K(perm_n(seed_Z, nS, zrank(seed,'B',i; nS))), S_key[j] = K(perm_n(seed_S, nS, j))
+    'zipf_both' : R_key[i] = K(perm_n(seed_Z, nR, zrank(seed,'B',i; nR))), S_key[j] = K(perm_n(seed_Z, nR, zrank(seed,'Z',j; nR)))
+    'replicas'  : R_key[i] = K(perm_n(seed_R, nR, i) mod D), S_key[j] = K(perm_n(seed_S, nS, j) mod D), D = nR / rep
   rho                  'fk'   : mulhi32(rng(seed,'U',j) >> 32, nR)  (== rng >> (64-log2 nR) for 2^k)
                        '1to1' : perm_n(seed_S, nS, j)  (nS == nR)
                        'zipf' : perm_n(seed_Z, nR, rank_j), rank_j = first k with CDF[k] >= u_j*CDF[-1]
@@ -48,6 +52,7 @@ TAG_S = 0x53  # 'S'
 TAG_Z = 0x5A  # 'Z'
 TAG_U = 0x55  # 'U'
 TAG_K = 0x4B  # 'K'
+TAG_B = 0x42  # 'B'
 
 
 # ----------------------------------------------------------------------------------------------
@@ -153,6 +158,13 @@ def zipf_cdf(n: int, z: float) -> np.ndarray:
     return np.cumsum(w)
 
 
+def np_zrank(seed: int, tag: int, idx: np.ndarray, cdf: np.ndarray) -> np.ndarray:
+    """Zipf rank of row idx: first k with CDF[k] >= u * CDF[-1], u = (rng >> 11) * 2^-53."""
+    u = (np_rng(seed, tag, idx) >> np.uint64(11)).astype(np.float64) * (2.0 ** -53)
+    rank = np.searchsorted(cdf, u * cdf[-1], side="left")
+    return np.minimum(rank, len(cdf) - 1).astype(np.uint64)
+
+
 def np_rho(dist: str, seed: int, nR: int, nS: int, j: np.ndarray, z: float = 0.0, cdf=None) -> np.ndarray:
     j = j.astype(np.uint64)
     if dist == "fk":
@@ -256,6 +268,14 @@ def torch_keymap(kind: str, x, seed: int):
     raise ValueError(kind)
 
 
+def torch_zrank(seed: int, tag: int, idx, cdf):
+    import torch
+
+    cdf_t = torch.from_numpy(cdf).to(idx.device)
+    u = _srl(torch_rng(seed, tag, idx), 11).to(torch.float64) * (2.0 ** -53)
+    return torch.searchsorted(cdf_t, u * cdf_t[-1], side="left").clamp_(max=len(cdf) - 1)
+
+
 def torch_rho(dist: str, seed: int, nR: int, nS: int, j, z: float = 0.0, cdf=None):
     import torch
 
@@ -291,6 +311,7 @@ class Workload:
     seed: int = 1
     out_mode: int = 0  # 0 count+checksum, 1 materialize
     radix_bits: int = -1
+    rep: int = 1  # 'replicas': copies of every key on each side
 
     @property
     def key_bytes(self) -> int:
@@ -319,6 +340,9 @@ CONFIGS = {
 }
 
 
+SKEW_DISTS = ("zipf_build", "zipf_both", "replicas")
+
+
 def np_generate(w: Workload, s_rows: slice | None = None, cdf=None):
     """Return (R_key, R_pay, S_key, S_pay) as numpy arrays (host).
 
@@ -326,16 +350,36 @@ def np_generate(w: Workload, s_rows: slice | None = None, cdf=None):
     any row range independently computable)."""
     pay_dt = np.uint64 if w.keys == "k8" else np.uint32
     i = np.arange(w.nR, dtype=np.uint64)
+    lo, hi = (0, w.nS) if s_rows is None else (s_rows.start, s_rows.stop)
+    j = np.arange(lo, hi, dtype=np.uint64)
+    if w.dist in SKEW_DISTS:
+        xR, xS = np_skew_x(w, i, j)
+        return (np_keymap(w.keys, xR, w.seed), i.astype(pay_dt), np_keymap(w.keys, xS, w.seed), j.astype(pay_dt))
     xR = np_perm_n(sub_seed(w.seed, TAG_R), w.nR, i)
     Rk = np_keymap(w.keys, xR, w.seed)
     Rp = i.astype(pay_dt)
     del xR
-    lo, hi = (0, w.nS) if s_rows is None else (s_rows.start, s_rows.stop)
-    j = np.arange(lo, hi, dtype=np.uint64)
     rho = np_rho(w.dist, w.seed, w.nR, w.nS, j, w.z, cdf)
     Sk = Rk[rho.astype(np.int64)]
     Sp = j.astype(pay_dt)
     return Rk, Rp, Sk, Sp
+
+
+def np_skew_x(w: Workload, i: np.ndarray, j: np.ndarray):
+    """Domain indices of the NEXT-2 workloads (see the module docstring)."""
+    if w.dist == "zipf_build":
+        cdf = zipf_cdf(w.nS, w.z)
+        xR = np_perm_n(sub_seed(w.seed, TAG_Z), w.nS, np_zrank(w.seed, TAG_B, i, cdf))
+        xS = np_perm_n(sub_seed(w.seed, TAG_S), w.nS, j)
+    elif w.dist == "zipf_both":
+        cdf = zipf_cdf(w.nR, w.z)
+        xR = np_perm_n(sub_seed(w.seed, TAG_Z), w.nR, np_zrank(w.seed, TAG_B, i, cdf))
+        xS = np_perm_n(sub_seed(w.seed, TAG_Z), w.nR, np_zrank(w.seed, TAG_Z, j, cdf))
+    else:  # replicas
+        D = np.uint64(max(1, w.nR // w.rep))
+        xR = np_perm_n(sub_seed(w.seed, TAG_R), w.nR, i) % D
+        xS = np_perm_n(sub_seed(w.seed, TAG_S), w.nS, j) % D
+    return xR, xS
 
 
 def np_rho_for(w: Workload, j: np.ndarray, cdf=None) -> np.ndarray:
@@ -350,13 +394,29 @@ def torch_generate(w: Workload, device="cuda", cdf=None):
     import torch
 
     i = torch.arange(w.nR, dtype=torch.int64, device=device)
-    xR = torch_perm_n(sub_seed(w.seed, TAG_R), w.nR, i)
-    Rk64 = torch_keymap(w.keys, xR, w.seed)
-    del xR
     j = torch.arange(w.nS, dtype=torch.int64, device=device)
-    rho = torch_rho(w.dist, w.seed, w.nR, w.nS, j, w.z, cdf)
-    Sk64 = Rk64[rho]
-    del rho
+    if w.dist in SKEW_DISTS:
+        if w.dist == "zipf_build":
+            c = zipf_cdf(w.nS, w.z)
+            xR = torch_perm_n(sub_seed(w.seed, TAG_Z), w.nS, torch_zrank(w.seed, TAG_B, i, c))
+            xS = torch_perm_n(sub_seed(w.seed, TAG_S), w.nS, j)
+        elif w.dist == "zipf_both":
+            c = zipf_cdf(w.nR, w.z)
+            xR = torch_perm_n(sub_seed(w.seed, TAG_Z), w.nR, torch_zrank(w.seed, TAG_B, i, c))
+            xS = torch_perm_n(sub_seed(w.seed, TAG_Z), w.nR, torch_zrank(w.seed, TAG_Z, j, c))
+        else:
+            D = max(1, w.nR // w.rep)
+            xR = torch_perm_n(sub_seed(w.seed, TAG_R), w.nR, i) % D
+            xS = torch_perm_n(sub_seed(w.seed, TAG_S), w.nS, j) % D
+        Rk64, Sk64 = torch_keymap(w.keys, xR, w.seed), torch_keymap(w.keys, xS, w.seed)
+        del xR, xS
+    else:
+        xR = torch_perm_n(sub_seed(w.seed, TAG_R), w.nR, i)
+        Rk64 = torch_keymap(w.keys, xR, w.seed)
+        del xR
+        rho = torch_rho(w.dist, w.seed, w.nR, w.nS, j, w.z, cdf)
+        Sk64 = Rk64[rho]
+        del rho
     if w.keys == "k8":
         return Rk64, i, Sk64, j
     return (_as_u32_bits(Rk64), _as_u32_bits(i), _as_u32_bits(Sk64), _as_u32_bits(j))
@@ -371,8 +431,13 @@ def _as_u32_bits(t):
 
 
 def expected_matches_closed_form(w: Workload) -> int | None:
-    """FK and 1:1 joins over unique R keys produce exactly one match per S row
-    (every S key is some R key and R keys are unique)."""
+    """FK and 1:1 joins over unique R keys produce exactly one match per S row (every S key is
+    some R key and R keys are unique); a build-skewed R over a domain S covers exactly once
+    produces one match per R row; replicas produce rep matches per R row when rep | nR, nS."""
     if w.dist in ("fk", "1to1", "zipf"):
         return w.nS
+    if w.dist == "zipf_build":
+        return w.nR
+    if w.dist == "replicas" and w.nR % w.rep == 0 and w.nS % (w.nR // w.rep) == 0:
+        return w.nR * (w.nS // (w.nR // w.rep))
     return None
