@@ -26,10 +26,11 @@ thread_local std::string g_create_error;
 // Join kernel shapes selectable with HJ_OPT_JOIN_VARIANT (tuning; results never change).
 //   variant: compute threads, S tuples / thread / round, min blocks / SM, R tile buffers
 struct JoinShape {
-  int nt, spt, minb, rbuf;
+  int nt, spt, minb, rbuf, nbsh;  // nbsh: hash slots = 2^(ceil(log2 C_R) - nbsh)
 };
-constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1}, {256, 8, 2, 2}, {224, 8, 3, 1}, {256, 12, 3, 1}, {192, 8, 3, 1},
-                                     {256, 4, 2, 1}, {512, 4, 1, 1}, {256, 8, 2, 1}, {384, 4, 1, 2}};
+constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1, 1}, {256, 8, 2, 2, 1}, {224, 8, 3, 1, 1}, {256, 12, 3, 1, 1},
+                                     {192, 8, 3, 1, 1}, {256, 4, 2, 1, 1}, {512, 4, 1, 1, 1}, {256, 8, 2, 1, 1},
+                                     {384, 4, 1, 2, 1}, {192, 8, 4, 1, 2}, {256, 8, 3, 1, 2}, {160, 8, 4, 1, 2}};
 constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
 
@@ -172,14 +173,15 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   uint32_t CS;
   if (c->opt_chunk_s > 0) CS = (uint32_t)std::min<int64_t>(c->opt_chunk_s, 1ll << 30);
   else CS = std::max<uint32_t>(8 * CR, 32768);
-  int lg_nb = std::max(6, ilog2_ceil(CR) - 1);
   const int rbuf = JOIN_SHAPES[join_variant(c)].rbuf;
+  const int nbsh = JOIN_SHAPES[join_variant(c)].nbsh;
+  int lg_nb = std::max(6, ilog2_ceil(CR) - nbsh);
   auto join_smem = [&](uint32_t cr, int lg) {  // R tile buffer(s) (TMA) + heads + next
     return (size_t)rbuf * ((cr + 3) & ~1u) * tb + ((size_t)4 << lg) + (size_t)cr * 2;
   };
   while (join_smem(CR, lg_nb) > cap_max_smem - 8 * 1024 && CR > 256) {
     CR /= 2;
-    lg_nb = std::max(6, ilog2_ceil(CR) - 1);
+    lg_nb = std::max(6, ilog2_ceil(CR) - nbsh);
   }
   hp.CR = CR;
   hp.CS = CS;
@@ -250,6 +252,9 @@ int set_kernel_attrs(Ctx* c) {
   attr_join<K, 6>(attr);
   attr_join<K, 7>(attr);
   attr_join<K, 8>(attr);
+  attr_join<K, 9>(attr);
+  attr_join<K, 10>(attr);
+  attr_join<K, 11>(attr);
   return rc;
 }
 
@@ -430,6 +435,9 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
     return HJ_OK;
   }
   switch (join_variant(c)) {
+    case 9: rc = launch_join_v<K, 9>(c, hp, P, mat); break;
+    case 10: rc = launch_join_v<K, 10>(c, hp, P, mat); break;
+    case 11: rc = launch_join_v<K, 11>(c, hp, P, mat); break;
     case 5: rc = launch_join_v<K, 5>(c, hp, P, mat); break;
     case 6: rc = launch_join_v<K, 6>(c, hp, P, mat); break;
     case 7: rc = launch_join_v<K, 7>(c, hp, P, mat); break;

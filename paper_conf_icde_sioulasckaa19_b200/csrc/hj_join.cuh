@@ -68,8 +68,12 @@ __device__ __forceinline__ void issue_r_copy(const Plan& P, const JoinJob& j, T*
 }
 
 __device__ __forceinline__ void bar_compute(int nthreads) {  // named barrier 1: compute warps only
-  asm volatile("bar.sync 1, %0;" ::"r"(nthreads) : "memory");
+  asm volatile("barrier.sync 1, %0;" ::"r"(nthreads) : "memory");
 }
+// end-of-item barrier of the whole block (compute warps + scheduler warp), reached from two code
+// sites: the non-aligned barrier.sync with an explicit thread count is defined for divergent
+// arrival (bar.sync / __syncthreads are .aligned)
+__device__ __forceinline__ void bar_item(int nthreads) { asm volatile("barrier.sync 2, %0;" ::"r"(nthreads) : "memory"); }
 
 // Block = NT compute threads + one scheduler warp. The scheduler warp claims and decodes item
 // k+1 and starts its R chunk's TMA bulk copy into the other half of a double-buffered smem tile
@@ -129,7 +133,7 @@ __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
         if (RBUF == 2 && j.item < total_items) issue_r_copy<T>(P, j, s_rtb + ((it + 1) & 1) * cap, &s_bar[(it + 1) & 1]);
         s_jobs[(it + 1) & 1] = j;
       }
-      __syncthreads();  // end-of-item barrier (matches the compute warps' one below)
+      bar_item(NT + 32);  // end-of-item barrier (matches the compute warps' one below)
       if (RBUF == 1 && lane == 0 && j.item < total_items) issue_r_copy<T>(P, j, s_rtb, &s_bar[(it + 1) & 1]);
       continue;
     }
@@ -250,7 +254,7 @@ __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
         bar_compute(NT);  // s_base / s_wsum are reused by the next round
       }
     }
-    __syncthreads();  // end of item: the tile buffer and s_head are reused, s_jobs[it+1] is ready
+    bar_item(NT + 32);  // end of item: the tile buffer and s_head are reused, s_jobs[it+1] is ready
   }
 
   // ---- aggregate: warp shuffle reduce, then one 64-bit atomic per block --------

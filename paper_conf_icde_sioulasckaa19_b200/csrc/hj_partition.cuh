@@ -511,7 +511,7 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
         if (lane >= o) x += y;
       }
       if (lane == 31) s_wt[warp] = x;
-      asm volatile("bar.sync 1, %0;" ::"r"(nscan) : "memory");
+      asm volatile("barrier.sync 1, %0;" ::"r"(nscan) : "memory");
       uint32_t base = 0;
       for (int w = 0; w < warp; ++w) base += s_wt[w];
       const uint32_t loc = base + x - c;
@@ -519,7 +519,7 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
         s_loc[d] = loc;
         s_cnt[d] = 0;
         if (c) gd[d] = atomicAdd(s_desc[slot].cur + d, (unsigned long long)c) - loc;
-        if (c > TILE / 4) s_hot_next = d;  // predicts the next unit's hot digit
+        if (c > TILE / 4) atomicExch(&s_hot_next, d);  // predicts the next unit's hot digit (any one)
       }
     }
     if (threadIdx.x == NT - 1)  // publish unit i+2

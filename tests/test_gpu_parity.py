@@ -5,6 +5,8 @@ after a lexicographic sort (reading S9), partitions equal as multisets. Inputs a
 generator's (workloads/) or small adversarial arrays; expected values come only from oracle/
 or from the generator's closed forms, never from the CUDA path.
 """
+import os
+
 import numpy as np
 import pytest
 import torch
@@ -356,3 +358,18 @@ def test_next2_skew_and_replicas_vs_oracle(hj, dist, z, rep):
     w = W.Workload("t", 1 << 15, 1 << 15, dist, keys="sparse", z=z, rep=rep, seed=170)
     Rk, Rp, Sk, Sp = W.np_generate(w)
     check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=-1, mat=True)
+
+
+@pytest.mark.slow
+@pytest.mark.parametrize("tool", ["memcheck", "racecheck", "synccheck"])
+def test_compute_sanitizer_clean(hj, tool):
+    import subprocess
+    import sys
+
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    out = subprocess.run(["compute-sanitizer", "--tool", tool, sys.executable,
+                          os.path.join(root, "tools", "sanitize_cases.py"), "core"],
+                         capture_output=True, text=True, timeout=1800)
+    txt = out.stdout + out.stderr
+    assert "sanitize cases ok" in txt, txt[-2000:]
+    assert ("ERROR SUMMARY: 0 errors" in txt) or ("RACECHECK SUMMARY: 0 hazards" in txt), txt[-2000:]

@@ -1,0 +1,54 @@
+"""Small joins for compute-sanitizer (memcheck / racecheck / synccheck / initcheck): every kernel
+of the default path, materialize and count, 4/4 and 8/8, partition exports, exchange path,
+streaming host path, comparators."""
+import os
+import sys
+
+import numpy as np
+import torch
+
+sys.path.insert(0, os.path.dirname(os.path.dirname(os.path.abspath(__file__))))
+import oracle  # noqa: E402
+import paper_conf_icde_sioulasckaa19_b200 as hj  # noqa: E402
+import workloads as W  # noqa: E402
+
+
+def dev(a):
+    return torch.from_numpy(np.ascontiguousarray(a).view(np.int32 if a.dtype.itemsize == 4 else np.int64)).cuda()
+
+
+def check(ctx, w, bits=-1):
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    m, c = oracle.hash_join(Rk, Rp, Sk, Sp)
+    r = ctx.join(dev(Rk), dev(Rp), dev(Sk), dev(Sp), radix_bits=bits)
+    assert (r.matches, r.checksum) == (m, c), (w, r.matches, m)
+    r = ctx.join(dev(Rk), dev(Rp), dev(Sk), dev(Sp), radix_bits=bits, out_mode=1)
+    assert r.matches == m
+    return Rk, Rp, Sk, Sp
+
+
+which = sys.argv[1] if len(sys.argv) > 1 else "all"
+ctx4 = hj.Context(0, 4, 4)
+ctx8 = hj.Context(0, 8, 8)
+cases = [W.Workload("a", 20000, 30011, "fk", keys="sparse", seed=400),
+         W.Workload("b", 1 << 14, 1 << 15, "zipf", z=1.5, seed=401),
+         W.Workload("c", 5000, 7000, "zipf_both", keys="sparse", z=1.0, seed=402)]
+for w in cases:
+    for bits in (-1, 0, 5, 11):
+        check(ctx4, w, bits)
+check(ctx8, W.Workload("d", 9000, 12000, "1to1", keys="k8", seed=403).with_(nS=9000))
+if which == "all":
+    w = W.Workload("e", 30000, 40000, "fk", keys="sparse", seed=404)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    ctx4.partition(dev(Rk), dev(Rp), 9)
+    ctx4.set_option(hj.OPT_STREAM_CHUNK, 7000)
+    r = ctx4.join_host(Rk, Rp, Sk, Sp, out_mode=1)
+    assert r.matches == oracle.hash_join(Rk, Rp, Sk, Sp)[0]
+    for algo in (1, 2):
+        c = hj.Context(0, 4, 4)
+        c.set_option(hj.OPT_JOIN_ALGO, algo)
+        check(c, W.Workload("f", 3000, 5000, "fk", keys="sparse", seed=405))
+    # exchange path with 2 virtual ranks
+    send, cnt, dest = ctx4.exchange_pack(0, dev(Rk), dev(Rp), 1, 6)
+    torch.cuda.synchronize()
+print("sanitize cases ok", flush=True)
