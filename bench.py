@@ -43,6 +43,7 @@ def parse():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-slice-bits", type=int, default=2, help="cpu_baseline sample = 1 of 2^bits key slices")
     ap.add_argument("--e2e-steps", type=int, default=3)
+    ap.add_argument("--dist", action="store_true", help="use the multi-GPU exchange path even at N=1")
     return ap.parse_args()
 
 
@@ -187,10 +188,16 @@ def main():
     import torch
 
     ws, rank, local = dist_env()
-    if ws > 1:
+    use_dist = ws > 1 or args.dist
+    if use_dist:
         import torch.distributed as dist
 
         torch.cuda.set_device(local)
+        if ws == 1:
+            os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+            os.environ.setdefault("MASTER_PORT", "29531")
+            os.environ.setdefault("RANK", "0")
+            os.environ.setdefault("WORLD_SIZE", "1")
         dist.init_process_group("nccl")
     dev = torch.device("cuda", local)
     torch.cuda.set_device(dev)
@@ -208,7 +215,7 @@ def main():
     from paper_conf_icde_sioulasckaa19_b200 import dist as hjdist
 
     def step():
-        if ws == 1:
+        if not use_dist:
             return ctx.join(Rk, Rp, Sk, Sp, radix_bits=w.radix_bits, out_mode=w.out_mode)
         return hjdist.join(Rk, Rp, Sk, Sp, out_mode=w.out_mode, ctx=ctx)
 
@@ -217,7 +224,7 @@ def main():
     assert res.matches == w.nS, "closed form: FK / 1:1 joins produce |S| matches"
 
     def barrier():
-        if ws > 1:
+        if use_dist:
             torch.distributed.barrier()
         torch.cuda.synchronize()
 
@@ -231,14 +238,14 @@ def main():
         e0.record(stream)
         for _ in range(args.steps):
             res = step()
-            loc = res if ws == 1 else res.local
+            loc = res if not use_dist else res.local
             per_k += np.array(loc.ms_kernel)
-            launches += loc.kernels if ws == 1 else loc.kernels + 2 * 3  # + pack (hist, plan, pass 1) x2
-            sent += 0 if ws == 1 else res.sent_bytes
+            launches += loc.kernels if not use_dist else loc.kernels + 2 * 3  # + pack (hist, plan, pass 1) x2
+            sent += 0 if not use_dist else res.sent_bytes
         e1.record(stream)
         barrier()
     ms = e0.elapsed_time(e1) / args.steps
-    if ws > 1:
+    if use_dist:
         t = torch.tensor([ms], device=dev)
         torch.distributed.all_reduce(t, op=torch.distributed.ReduceOp.MAX)
         ms = float(t.item())
@@ -246,7 +253,7 @@ def main():
     value = w.n / (ms * 1e-3)  # the whole workload's tuples (sharded across ranks when ws > 1)
 
     if rank != 0:
-        if ws > 1:
+        if use_dist:
             torch.distributed.destroy_process_group()
         return
 
@@ -274,16 +281,16 @@ def main():
            "config": {"workload": workload_desc(w), "radix_bits": res.radix_bits, "passes": res.passes,
                       "join_items": res.n_items,
                       "l2": "inputs larger than L2 (2 GiB in + 4 GiB partition buffers vs 126 MB L2); no flush",
-                      "parallelism": "1 GPU" if ws == 1 else
-                      f"{ws} ranks: rows sharded, radix exchange over NCCL all_to_all, per-rank 2-pass join"},
+                      "parallelism": "1 GPU" if not use_dist else
+                      f"{ws} rank(s): rows sharded, radix exchange over NCCL all_to_all, per-rank 2-pass join"},
            "roofline": roof, "roofline_path": roof_path, "kernels_ms": kms, "clocks": clk.summary(),
            "gpu_launches": launches}
-    if ws > 1:
+    if use_dist:
         out["nvlink"] = {"bytes_sent_per_gpu_per_step": sent / args.steps,
                          "achieved_GBps": sent / args.steps / (ms * 1e-3) / 1e9, "peak_GBps": 900.0,
                          "note": "tuple bytes rank 0 sent to other ranks / step time; all_to_all_single over NCCL"}
 
-    if not args.no_e2e and ws == 1:
+    if not args.no_e2e and not use_dist:
         # end to end through the public API from pinned host memory: H2D of the inputs, the join,
         # D2H of the result (matches/checksum, and the materialized pairs) every step
         hcols = []
@@ -302,11 +309,11 @@ def main():
                       "ms_per_step": dt * 1e3, "steps": args.e2e_steps, "api": "hj_join_host (pinned host columns)"}
         del hcols
 
-    if not args.no_cpu_baseline and ws == 1:
+    if not args.no_cpu_baseline and ws == 1 and not use_dist:
         host = [t.cpu().numpy().view(np.uint32 if w.key_bytes == 4 else np.uint64) for t in (Rk, Rp, Sk, Sp)]
         out["cpu_baseline"] = cpu_oracle_sample(w, *host, slice_bits=args.cpu_slice_bits)
     print(json.dumps(out), flush=True)
-    if ws > 1:
+    if use_dist:
         torch.distributed.destroy_process_group()
 
 

@@ -187,3 +187,41 @@ def test_gpu_virtual_ranks_exchange(G, dist_):
     assert m == om
     got = np.concatenate(pairs)
     assert np.array_equal(oracle.pairs_sorted(got[:, 0], got[:, 1]), oracle.pairs_sorted(r, s))
+
+
+_NCCL1 = r'''
+import os, sys, numpy as np, torch, torch.distributed as dist
+sys.path.insert(0, sys.argv[1])
+import oracle, workloads as W
+from paper_conf_icde_sioulasckaa19_b200 import dist as hjdist
+dist.init_process_group("nccl", rank=0, world_size=1)
+torch.cuda.set_device(0)
+w = W.Workload("n", 1 << 16, 3 << 16, "zipf", keys="sparse", z=1.0, seed=180)
+Rk, Rp, Sk, Sp = W.np_generate(w)
+cols = [torch.from_numpy(a.view(np.int32)).cuda() for a in (Rk, Rp, Sk, Sp)]
+for lb in (0, 6, 12):
+    r = hjdist.join(*cols, local_bits=lb)
+    assert (r.matches, r.checksum) == oracle.hash_join(Rk, Rp, Sk, Sp), lb
+r = hjdist.join(*cols, out_mode=1)
+m, c, rr, ss = oracle.hash_join(Rk, Rp, Sk, Sp, materialize=True)
+got = oracle.pairs_sorted(r.local.r_pay.cpu().numpy().view(np.uint32), r.local.s_pay.cpu().numpy().view(np.uint32))
+assert r.matches == m and np.array_equal(got, oracle.pairs_sorted(rr, ss))
+dist.destroy_process_group()
+print("nccl1 ok")
+'''
+
+
+@pytest.mark.gpu
+def test_dist_join_nccl_one_rank():
+    """dist.join through real NCCL collectives (one rank: the exchange sends everything to
+    itself), against the oracle -- the plumbing bench.py --gpus N uses."""
+    import subprocess
+    import sys
+
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    env = dict(os.environ, MASTER_ADDR="127.0.0.1", MASTER_PORT=str(_free_port()), RANK="0", WORLD_SIZE="1",
+               LOCAL_RANK="0")
+    out = subprocess.run([sys.executable, "-c", _NCCL1, root], capture_output=True, text=True, timeout=600, env=env)
+    assert "nccl1 ok" in out.stdout, out.stdout[-2000:] + out.stderr[-4000:]
