@@ -258,7 +258,7 @@ def main():
         return
 
     peak, peak_src = peaks()
-    kb, path_bytes = alg_bytes(w, res.matches)
+    kb, path_bytes = alg_bytes(w, res.matches)  # res.matches: the whole join's (all ranks)
     names = ["hist", "plan", "pass1", "pass2", "join"]
     kms = dict(zip(names, per_k.tolist()))
     dom = max(names, key=lambda k: kms[k])
@@ -272,14 +272,15 @@ def main():
     path_ach = path_bytes / (ms * 1e-3) / 1e9
     roof_path = {"bound": "hbm", "achieved": path_ach, "peak": peak, "unit": "GB/s", "frac": path_ach / peak,
                  "alg_bytes_per_step": path_bytes,
-                 "kernel_fracs": {k: (kb[k] / (kms[k] * 1e-3) / 1e9 / peak if kms[k] > 0 else None) for k in names}}
+                 "kernel_fracs": {k: (kb[k] / (kms[k] * 1e-3) / 1e9 / peak if kms[k] > 0.01 and kb[k] else None)
+                                  for k in names}}
 
     out = {"metric": METRIC, "value": value, "unit": UNIT, "n_gpus": ws, "steps": args.steps, "warmup": args.warmup,
            "ms_per_step": ms, "higher_is_better": True, "scaling": "weak" if ws == 1 else "strong",
            "vs_baseline": None,
            "dtype": "u32" if w.key_bytes == 4 else "u64", "data": "synthetic",
-           "config": {"workload": workload_desc(w), "radix_bits": res.radix_bits, "passes": res.passes,
-                      "join_items": res.n_items,
+           "config": {"workload": workload_desc(w), "radix_bits": loc.radix_bits, "passes": loc.passes,
+                      "join_items": loc.n_items,
                       "l2": "inputs larger than L2 (2 GiB in + 4 GiB partition buffers vs 126 MB L2); no flush",
                       "parallelism": "1 GPU" if not use_dist else
                       f"{ws} rank(s): rows sharded, radix exchange over NCCL all_to_all, per-rank 2-pass join"},
