@@ -68,6 +68,9 @@ enum hj_option {
   HJ_OPT_JOIN_ALGO = 9,     /* 0 = radix-partitioned + smem hash table (default); 1 = radix-
                                partitioned + ballot nested loops (Listing 1); 2 = non-
                                partitioned hash join on a device-memory table (Fig. 8) */
+  HJ_OPT_PASS1_BASES = 10,  /* 1 = pass 1 uses per-block bases computed by the histogram kernel and
+                               TMA bulk-store write-out instead of atomic run reservation (opt-in;
+                               measured slower on B200, kept for comparison)                      */
   HJ_OPT_STREAM_CHUNK = 8   /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
                                least 2^22; >= |S| = copy everything, then join)                   */
 };

@@ -38,6 +38,7 @@ OPT_JOIN_VARIANT = 6
 OPT_PASS_THREADS = 7
 OPT_STREAM_CHUNK = 8
 OPT_JOIN_ALGO = 9
+OPT_PASS1_BASES = 10
 ALGO_HASH, ALGO_NLJ, ALGO_NONPARTITIONED = 0, 1, 2
 
 _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4: "HJ_ERR_CUDA", -5: "HJ_ERR_COMM"}

@@ -53,7 +53,7 @@ struct Ctx {
   std::string err;
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
-          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0;
+          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0;
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2], np_heads, np_next;
   void* h_res = nullptr;  // pinned host: results readback
@@ -112,6 +112,9 @@ struct HostPlan {
   int tile = 0;
   // metadata offsets (bytes) inside ctx->meta
   size_t o_cnt[2], o_off[2], o_cur1[2], o_cur2[2], o_pst[2], o_cst[2], o_ist, o_counters, o_results;
+  size_t o_cntb = 0, o_relb = 0;  // pass-1 per-block digit counts / bases
+  bool bases = false;             // pass 1 = k_pass1b (per-block bases, TMA bulk write-out)
+  uint32_t g1max = 0;
   size_t zero_bytes = 0;  // [0, zero_bytes) is memset to 0 per call
   size_t meta_bytes = 0;
   int pb() const { return g + b1; }
@@ -209,6 +212,15 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
     hp.o_cst[r] = take((npc + 1) * 4);
   }
   hp.o_ist = take((((size_t)1 << hp.B) + 1) * 4);
+  // pass 1 with precomputed per-block bases and TMA bulk-store write-out (opt-in: measured
+  // slower than the atomic-reservation pass on c2/c3/c4); needs the exact
+  // shared histogram (<= 2^15 u32 bins)
+  hp.bases = mode != PLAN_RECV && hp.qbits() <= 15 && c->opt_pass1_bases;
+  if (hp.bases) {
+    hp.g1max = 2 * (uint32_t)c->num_sms;
+    hp.o_cntb = take((size_t)2 * hp.g1max * F1 * 4);
+    hp.o_relb = take((size_t)2 * hp.g1max * F1 * 8);
+  }
   hp.meta_bytes = o;
   (void)nS;
   return HJ_OK;
@@ -240,6 +252,10 @@ int set_kernel_attrs(Ctx* c) {
   attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), false>);
   attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), true>);
   attr((const void*)k_pass<K, 2, 1024, pass_items<K>(), false>);
+  attr((const void*)k_pass1b<K, 1024, pass_items<K>(), false>);
+  attr((const void*)k_pass1b<K, 1024, pass_items<K>(), true>);
+  attr((const void*)k_pass1b<K, 512, pass_items<K>(), false>);
+  attr((const void*)k_pass1b<K, 512, pass_items<K>(), true>);
   attr((const void*)k_pass<K, 1, 512, pass_items<K>(), false>);
   attr((const void*)k_pass<K, 1, 512, pass_items<K>(), true>);
   attr((const void*)k_pass<K, 2, 512, pass_items<K>(), false>);
@@ -302,6 +318,10 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   P.CR = hp.CR;
   P.CS = hp.CS;
   P.ist = (uint32_t*)(m + hp.o_ist);
+  if (hp.bases) {
+    P.cntb = (uint32_t*)(m + hp.o_cntb);
+    P.relb = (unsigned long long*)(m + hp.o_relb);
+  }
   P.counters = (uint32_t*)(m + hp.o_counters);
   P.results = (unsigned long long*)(m + hp.o_results);
   P.out_r = c->out_r.p;
@@ -327,6 +347,12 @@ template <typename K, int MODE, int NT, bool GD>
 int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits);
 
 template <typename K>
+size_t pass1b_smem(const HostPlan& hp, int nt) {
+  const size_t F = (size_t)1 << hp.pb(), tb = sizeof(typename Tup<K>::T);
+  return ((size_t)nt * pass_items<K>() + 2 * F) * tb + 16 * F + 4 * (F + 4) + 8 * F;
+}
+
+template <typename K>
 int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false) {
   cudaStream_t st = c->stream;
   const bool gd = hp.g > 0;
@@ -337,6 +363,19 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false) 
     CUDA_TRY(c, cudaMemsetAsync((char*)c->meta.p + hp.o_counters, 0, 64, st));
     CUDA_TRY(c, cudaMemsetAsync((char*)c->meta.p + hp.o_cnt[1], 0, (size_t)4 << hp.qbits(), st));
   }
+  Plan Pb = P;  // P with the pass-1 grid / tile when pass 1 uses per-block bases
+  if (hp.mode != PLAN_RECV && hp.bases) {
+    const int nt = hp.tile == 512 * pass_items<K>() ? 512 : 1024;
+    const size_t sm = pass1b_smem<K>(hp, nt);
+    const void* f = nt == 512 ? (gd ? (const void*)k_pass1b<K, 512, pass_items<K>(), true>
+                                    : (const void*)k_pass1b<K, 512, pass_items<K>(), false>)
+                              : (gd ? (const void*)k_pass1b<K, 1024, pass_items<K>(), true>
+                                    : (const void*)k_pass1b<K, 1024, pass_items<K>(), false>);
+    Pb.tile1 = (uint32_t)hp.tile;
+    Pb.tiles1[0] = (P.rel[0].n + hp.tile - 1) / hp.tile;
+    Pb.tiles1[1] = (P.rel[1].n + hp.tile - 1) / hp.tile;
+    Pb.g1 = (uint32_t)std::min<unsigned long long>(grid_for(c, f, nt, sm, Pb.tiles1[0] + Pb.tiles1[1]), hp.g1max);
+  }
   if (hp.mode != PLAN_RECV) {
     const bool smem = hp.qbits() <= 16;
     const bool c32 = hp.qbits() <= 15;  // 16 bins: packed 16-bit counters (128 KB)
@@ -344,26 +383,36 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false) 
     const unsigned long long nR = P.rel[0].n, nS = P.rel[1].n;
     const void* f = smem ? (gd ? (const void*)k_hist<K, true, true> : (const void*)k_hist<K, true, false>)
                          : (const void*)k_hist<K, false, false>;
-    const int g = std::max(2, grid_for(c, f, HIST_NT, sm, (nR + nS + 4095) / 4096 + 2));
+    int g = std::max(2, grid_for(c, f, HIST_NT, sm, (nR + nS + 4095) / 4096 + 2));
     // blocks split proportionally to the relation sizes (at least one each)
     uint32_t gr = (uint32_t)((double)g * (double)nR / (double)std::max<unsigned long long>(nR + nS, 1) + 0.5);
     gr = std::min<uint32_t>(std::max<uint32_t>(gr, 1), (uint32_t)g - 1);
     if (nR == 0) gr = 0;  // streaming S chunk: every block counts S
-    if (smem && c32 && gd) k_hist<K, true, true, true><<<g, HIST_NT, sm, st>>>(P, gr);
-    else if (smem && c32) k_hist<K, true, false, true><<<g, HIST_NT, sm, st>>>(P, gr);
-    else if (smem && gd) k_hist<K, true, true, false><<<g, HIST_NT, sm, st>>>(P, gr);
-    else if (smem) k_hist<K, true, false, false><<<g, HIST_NT, sm, st>>>(P, gr);
-    else if (gd) k_hist<K, false, true><<<g, HIST_NT, 0, st>>>(P, gr);
-    else k_hist<K, false, false><<<g, HIST_NT, 0, st>>>(P, gr);
+    if (Pb.g1) g = (int)Pb.g1;  // bases: the histogram walks exactly pass 1's tiles per block
+    if (smem && c32 && gd) k_hist<K, true, true, true><<<g, HIST_NT, sm, st>>>(Pb, gr);
+    else if (smem && c32) k_hist<K, true, false, true><<<g, HIST_NT, sm, st>>>(Pb, gr);
+    else if (smem && gd) k_hist<K, true, true, false><<<g, HIST_NT, sm, st>>>(Pb, gr);
+    else if (smem) k_hist<K, true, false, false><<<g, HIST_NT, sm, st>>>(Pb, gr);
+    else if (gd) k_hist<K, false, true><<<g, HIST_NT, 0, st>>>(Pb, gr);
+    else k_hist<K, false, false><<<g, HIST_NT, 0, st>>>(Pb, gr);
     CUDA_TRY(c, cudaGetLastError());
     c->launches += 1;
   }
   mark(c, 1);
-  k_plan<<<(unsigned)((((size_t)1 << hp.qbits()) + 1023) / 1024), 1024, 0, st>>>(P);
+  k_plan<<<(unsigned)((((size_t)1 << hp.qbits()) + 1023) / 1024), 1024, 0, st>>>(Pb);
   CUDA_TRY(c, cudaGetLastError());
   c->launches += 1;
   mark(c, 2);
-  if (hp.mode != PLAN_RECV) {
+  if (hp.mode != PLAN_RECV && Pb.g1) {
+    const int nt = hp.tile == 512 * pass_items<K>() ? 512 : 1024;
+    const size_t sm = pass1b_smem<K>(hp, nt);
+    if (nt == 512 && gd) k_pass1b<K, 512, pass_items<K>(), true><<<Pb.g1, 512, sm, st>>>(Pb, hp.pb());
+    else if (nt == 512) k_pass1b<K, 512, pass_items<K>(), false><<<Pb.g1, 512, sm, st>>>(Pb, hp.pb());
+    else if (gd) k_pass1b<K, 1024, pass_items<K>(), true><<<Pb.g1, 1024, sm, st>>>(Pb, hp.pb());
+    else k_pass1b<K, 1024, pass_items<K>(), false><<<Pb.g1, 1024, sm, st>>>(Pb, hp.pb());
+    CUDA_TRY(c, cudaGetLastError());
+    c->launches += 1;
+  } else if (hp.mode != PLAN_RECV) {
     int rc = hp.tile == 512 * pass_items<K>()
                  ? (gd ? launch_pass<K, 1, 512, true>(c, hp, P, hp.pb()) : launch_pass<K, 1, 512, false>(c, hp, P, hp.pb()))
                  : (gd ? launch_pass<K, 1, 1024, true>(c, hp, P, hp.pb()) : launch_pass<K, 1, 1024, false>(c, hp, P, hp.pb()));
@@ -878,6 +927,7 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_TIMING: c->opt_timing = v; break;
     case HJ_OPT_BLOCKS_PER_SM: c->opt_bps = v; break;
     case HJ_OPT_STREAM_CHUNK: c->opt_stream_chunk = v; break;
+    case HJ_OPT_PASS1_BASES: c->opt_pass1_bases = v; break;
     case HJ_OPT_JOIN_ALGO:
       if (v > 2) return fail(c, HJ_ERR_INVALID, "join algorithm must be 0, 1 or 2");
       c->opt_join_algo = v;

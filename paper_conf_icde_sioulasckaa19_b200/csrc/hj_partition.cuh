@@ -46,31 +46,45 @@ __device__ __forceinline__ void hist_add(uint32_t* h, uint32_t bin, uint32_t* gc
 template <typename K, bool SMEM, bool GD, bool C32 = true>
 __global__ void __launch_bounds__(1024) k_hist(Plan P, uint32_t blocks_r) {
   extern __shared__ uint32_t s_hist[];
-  // blocks [0, blocks_r) count R, the rest count S (split proportionally to |R| : |S|)
-  const int rel = blockIdx.x < blocks_r ? 0 : 1;
-  const RelDev& R = P.rel[rel];
-  const unsigned long long n = R.n;
-  const uint32_t nblk = rel ? gridDim.x - blocks_r : blocks_r;
-  const uint32_t bid = rel ? blockIdx.x - blocks_r : blockIdx.x;
+  __shared__ uint32_t s_blk[2][1024];  // BLK mode: this block's pass-1 digit counts per relation
   const uint32_t np = 1u << P.qbits();
   const uint32_t nwords = C32 ? np : np / 2;
+  const bool blk = P.g1 != 0;
   if (SMEM) {
     for (uint32_t i = threadIdx.x; i < nwords; i += blockDim.x) s_hist[i] = 0;
-    __syncthreads();
   }
+  const uint32_t F1 = 1u << P.pb();
+  if (blk)
+    for (uint32_t i = threadIdx.x; i < 2 * 1024; i += blockDim.x) (&s_blk[0][0])[i] = 0;
+  __syncthreads();
+  constexpr int VEC = 16 / sizeof(K);
+  int rel = 0;
   auto add = [&](K key) {
     const uint32_t b = qbin<GD>(key, P);
-    if (SMEM) hist_add<C32>(s_hist, b, R.cnt);
-    else atomicAdd(&R.cnt[b], 1u);
+    if (SMEM) hist_add<C32>(s_hist, b, P.rel[rel].cnt);
+    else atomicAdd(&P.rel[rel].cnt[b], 1u);
   };
-  constexpr int VEC = 16 / sizeof(K);
-  unsigned long long per = (n + nblk - 1) / nblk;
-  per = (per + VEC - 1) / VEC * VEC;
-  const unsigned long long lo = (unsigned long long)bid * per;
-  const unsigned long long hi = lo + per < n ? lo + per : n;
-  const K* keys = (const K*)R.keys;
-  if (lo < hi) {
-    const bool aligned = ((reinterpret_cast<uintptr_t>(keys) & 15) == 0);
+  // merge the shared q-histogram of relation r into the global one and clear it
+  auto flush_q = [&](int r) {
+    __syncthreads();
+    if (blk)  // this block's pass-1 digit counts: D = q >> b2 sums 2^b2 consecutive bins
+      for (uint32_t d = threadIdx.x; d < F1; d += blockDim.x) {
+        uint32_t t = 0;
+        for (uint32_t j = d << P.b2; j < (d + 1) << P.b2; ++j)
+          t += C32 ? s_hist[j] : ((s_hist[j >> 1] >> ((j & 1) << 4)) & 0xffffu);
+        s_blk[r][d] = t;
+      }
+    for (uint32_t i = threadIdx.x; i < np; i += blockDim.x) {
+      const uint32_t c = C32 ? s_hist[i] : ((s_hist[i >> 1] >> ((i & 1) << 4)) & 0xffffu);
+      if (c) atomicAdd(&P.rel[r].cnt[i], c);
+    }
+    __syncthreads();
+    for (uint32_t i = threadIdx.x; i < nwords; i += blockDim.x) s_hist[i] = 0;
+    __syncthreads();
+  };
+  auto count_range = [&](const K* keys, unsigned long long lo, unsigned long long hi) {
+    if (lo >= hi) return;
+    const bool aligned = ((reinterpret_cast<uintptr_t>(keys + lo) & 15) == 0);
     unsigned long long i = lo;
     if (aligned) {
       const unsigned long long nvec = (hi - lo) / VEC;
@@ -97,13 +111,35 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P, uint32_t blocks_r) {
       i = lo + nvec * VEC;
     }
     for (unsigned long long j = i + threadIdx.x; j < hi; j += blockDim.x) add(keys[j]);
-  }
-  if (SMEM) {
-    __syncthreads();
-    for (uint32_t i = threadIdx.x; i < np; i += blockDim.x) {
-      const uint32_t c = C32 ? s_hist[i] : ((s_hist[i >> 1] >> ((i & 1) << 4)) & 0xffffu);
-      if (c) atomicAdd(&R.cnt[i], c);
+  };
+  if (!blk) {
+    // blocks [0, blocks_r) count R, the rest count S (split proportionally to |R| : |S|)
+    rel = blockIdx.x < blocks_r ? 0 : 1;
+    const unsigned long long n = P.rel[rel].n;
+    const uint32_t nblk = rel ? gridDim.x - blocks_r : blocks_r;
+    const uint32_t bid = rel ? blockIdx.x - blocks_r : blockIdx.x;
+    unsigned long long per = (n + nblk - 1) / nblk;
+    per = (per + VEC - 1) / VEC * VEC;
+    const unsigned long long lo = (unsigned long long)bid * per;
+    count_range((const K*)P.rel[rel].keys, lo, lo + per < n ? lo + per : n);
+  } else {
+    // exactly the tiles pass 1 block blockIdx.x will process: u = blockIdx.x + k * g1
+    const unsigned long long units0 = P.tiles1[0], units = units0 + P.tiles1[1];
+    for (unsigned long long u = blockIdx.x; u < units; u += gridDim.x) {
+      const int r = u < units0 ? 0 : 1;
+      if (SMEM && r != rel) flush_q(rel);  // R's tiles come first; flush R before counting S
+      rel = r;
+      const unsigned long long s0 = (rel ? u - units0 : u) * P.tile1;
+      const unsigned long long n = P.rel[rel].n;
+      count_range((const K*)P.rel[rel].keys, s0, s0 + P.tile1 < n ? s0 + P.tile1 : n);
     }
+  }
+  if (SMEM) flush_q(rel);
+  if (blk) {
+    __syncthreads();
+    for (int r = 0; r < 2; ++r)
+      for (uint32_t d = threadIdx.x; d < F1; d += blockDim.x)
+        P.cntb[((size_t)r * gridDim.x + blockIdx.x) * F1 + d] = s_blk[r][d];
   }
 }
 
@@ -196,6 +232,27 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
         #pragma unroll
         for (int o = 16; o; o >>= 1) c += __shfl_xor_sync(0xffffffffu, c, o);
         if (lane == 0) R.pst[i + 1] = c;
+      }
+    }
+  }
+  // ---- pass-1 bases: exclusive prefix over pass-1 blocks of each (relation, digit) column ----
+  if (P.g1) {
+    const uint32_t F1 = 1u << pb, g1 = P.g1;
+    const uint32_t lane = threadIdx.x & 31, gw = b * (NT / 32) + (threadIdx.x >> 5), nw = gridDim.x * (NT / 32);
+    for (uint32_t col = gw; col < 2 * F1; col += nw) {
+      const size_t r0 = (size_t)(col / F1) * g1, D = col % F1;
+      unsigned long long run = 0;
+      for (uint32_t b0 = 0; b0 < g1; b0 += 32) {
+        const bool ok = b0 + lane < g1;
+        const unsigned long long v = ok ? P.cntb[(r0 + b0 + lane) * F1 + D] : 0ull;
+        unsigned long long x = v;
+        #pragma unroll
+        for (int o = 1; o < 32; o <<= 1) {
+          const unsigned long long y = __shfl_up_sync(0xffffffffu, x, o);
+          if (lane >= o) x += y;
+        }
+        if (ok) P.relb[(r0 + b0 + lane) * F1 + D] = run + x - v;
+        run += __shfl_sync(0xffffffffu, x, 31);
       }
     }
   }
@@ -546,6 +603,224 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
   }
   __syncthreads();
   write_out(s_gd + ((it + 1) & 1) * F);  // the last unit (it was incremented past it)
+}
+
+// ------------------------------------------------------------------------------------------
+// a3 with precomputed per-block bases (default pass 1 when 2^qbits <= 2^15): block b's run of
+// digit d in its k-th tile starts at pst[d] + relb[b][d] + (its earlier tiles' counts of d) --
+// no atomics, and every run's global start is known BEFORE the shuffle. Each run is placed in
+// shared memory at the same 16-byte phase as its destination (one spare slot per digit), so the
+// write-out is one TMA bulk store (cp.async.bulk shared -> global) per run plus at most one
+// scalar tuple at each end, issued by one thread per digit and completed asynchronously.
+// Per tile: rank | scan + wait for the previous tile's bulk reads | shuffle + proxy fence |
+// issue bulk stores (overlapping the next tile's rank).
+// ------------------------------------------------------------------------------------------
+__device__ __forceinline__ void bulk_s2g(void* dst, const void* src, uint32_t bytes) {
+  asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;" ::"l"(dst), "r"(smem_u32(src)), "r"(bytes)
+               : "memory");
+}
+__device__ __forceinline__ void bulk_commit() { asm volatile("cp.async.bulk.commit_group;" ::: "memory"); }
+__device__ __forceinline__ void bulk_wait_read() { asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory"); }
+__device__ __forceinline__ void bulk_wait_all() { asm volatile("cp.async.bulk.wait_group 0;" ::: "memory"); }
+
+template <typename K, int NT, int ITEMS, bool GD>
+__global__ void __launch_bounds__(NT, 1024 / NT) k_pass1b(Plan P, int fanout_bits) {
+  using TT = Tup<K>;
+  using T = typename TT::T;
+  constexpr int TILE = NT * ITEMS;
+  constexpr int TPS = 16 / sizeof(T);  // tuples per 16-byte segment (2 for 8 B tuples, 1 for 16 B)
+  static_assert(NT == 512 || NT == 1024, "block size");
+  static_assert(TILE <= 65536 && ITEMS % 2 == 0, "16-bit packed ranks");
+  extern __shared__ __align__(16) unsigned char s_raw[];
+  const uint32_t F = 1u << fanout_bits;
+  T* s_buf = reinterpret_cast<T*>(s_raw);                                                  // TILE + 2F tuples
+  unsigned long long* s_cur = reinterpret_cast<unsigned long long*>(s_buf + TILE + 2 * F);  // F: next global slot
+  unsigned long long* s_gst = s_cur + F;                                                   // F: run start (global)
+  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gst + F);                                // F + 1 (spare)
+  uint32_t* s_loc = s_cnt + F + 4;                                                         // F: run start (smem)
+  uint32_t* s_len = s_loc + F;                                                             // F: run length
+  __shared__ uint32_t s_wt[NT / 32];
+  __shared__ uint32_t s_hot, s_hot_next;
+
+  const uint32_t dmask = (1u << P.b1) - 1;
+  const uint32_t gsh = (uint32_t)P.B, gmask = (1u << P.g) - 1, gup = (uint32_t)P.b1;
+  auto digit = [=](K key) -> uint32_t {
+    uint32_t d = (uint32_t)key & dmask;
+    if (GD) d |= ((uint32_t)(key >> gsh) & gmask) << gup;
+    return d;
+  };
+  const uint32_t nscan = F < 32 ? 32u : F;
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const unsigned long long G = gridDim.x;
+  const unsigned long long units0 = P.tiles1[0], units = units0 + P.tiles1[1];
+
+  if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
+  if (threadIdx.x == 0) s_hot = s_hot_next = 0xffffffffu;
+  int cur_rel = -1;
+  auto load_bases = [&](int r) {  // cursors of this block for relation r
+    if (threadIdx.x < F)
+      s_cur[threadIdx.x] = P.rel[r].pst[threadIdx.x] + P.relb[((size_t)r * G + blockIdx.x) * F + threadIdx.x];
+  };
+  auto unit = [&](unsigned long long u, const K*& kp, const K*& pp_, uint32_t& len, int& r) {
+    r = u < units0 ? 0 : 1;
+    const unsigned long long s0 = (r ? u - units0 : u) * TILE;
+    kp = (const K*)P.rel[r].keys + s0;
+    pp_ = (const K*)P.rel[r].pays + s0;
+    len = (uint32_t)min((unsigned long long)TILE, P.rel[r].n - s0);
+  };
+  K kk[ITEMS], pp[ITEMS], kn[ITEMS], pn[ITEMS];
+  auto load = [&](const K* keys, const K* pays, uint32_t len) {
+    constexpr int VEC = 16 / sizeof(K);
+    const bool vec_ok = (len == TILE) && ((reinterpret_cast<uintptr_t>(keys) & 15) == 0) &&
+                        ((reinterpret_cast<uintptr_t>(pays) & 15) == 0);
+    if (vec_ok) {
+      #pragma unroll
+      for (int j = 0; j < ITEMS / VEC; ++j) {
+        const uint4 kv = __ldcs(reinterpret_cast<const uint4*>(keys) + j * NT + threadIdx.x);
+        const uint4 pv = __ldcs(reinterpret_cast<const uint4*>(pays) + j * NT + threadIdx.x);
+        const K* ke = reinterpret_cast<const K*>(&kv);
+        const K* pe = reinterpret_cast<const K*>(&pv);
+        #pragma unroll
+        for (int t = 0; t < VEC; ++t) {
+          kn[j * VEC + t] = ke[t];
+          pn[j * VEC + t] = pe[t];
+        }
+      }
+    } else {
+      #pragma unroll
+      for (int j = 0; j < ITEMS; ++j) {
+        const uint32_t e = pass_elem<K, 1, NT>(j);
+        if (e < len) {
+          kn[j] = keys[e];
+          pn[j] = pays[e];
+        }
+      }
+    }
+  };
+
+  unsigned long long u = blockIdx.x;
+  const K *ck, *cp;
+  uint32_t clen = 0;
+  int crel = 0;
+  if (u < units) {
+    unit(u, ck, cp, clen, crel);
+    load(ck, cp, clen);
+  }
+  __syncthreads();
+  bool pending = false;  // this thread issued bulk stores not yet known to be read
+  T* dst = nullptr;
+  while (u < units) {
+    const uint32_t ulen = clen;
+    const int urel = crel;
+    #pragma unroll
+    for (int j = 0; j < ITEMS; ++j) {
+      kk[j] = kn[j];
+      pp[j] = pn[j];
+    }
+    const unsigned long long un = u + G;
+    if (un < units) {
+      unit(un, ck, cp, clen, crel);
+      load(ck, cp, clen);
+    }
+    if (urel != cur_rel) {  // block-uniform; the previous relation's stores were waited for below
+      load_bases(urel);
+      cur_rel = urel;
+      dst = (T*)P.rel[urel].t1;
+    }
+    // ---- phase 1: rank (hot-digit aggregation as in k_pass) ---------------------------------
+    uint32_t rk[ITEMS / 2];
+    const bool full = ulen == TILE;
+    const uint32_t hot = s_hot;
+    #pragma unroll
+    for (int j = 0; j < ITEMS; ++j) {
+      const uint32_t d = (full || pass_elem<K, 1, NT>(j) < ulen) ? digit(kk[j]) : F;
+      uint32_t r;
+      if (hot > F) {
+        r = atomicAdd(&s_cnt[d], 1u);
+      } else {
+        const uint32_t hm = __ballot_sync(0xffffffffu, d == hot);
+        if (hm) {
+          const int leader = __ffs(hm) - 1;
+          uint32_t base = 0;
+          if (lane == leader) base = atomicAdd(&s_cnt[hot], (uint32_t)__popc(hm));
+          base = __shfl_sync(0xffffffffu, base, leader);
+          r = (d == hot) ? base + __popc(hm & lanemask_lt()) : atomicAdd(&s_cnt[d], 1u);
+        } else {
+          r = atomicAdd(&s_cnt[d], 1u);
+        }
+      }
+      if (j & 1) rk[j / 2] |= r << 16; else rk[j / 2] = r & 0xffffu;
+    }
+    __syncthreads();
+    // ---- phase 2: scan -> smem run starts aligned to the destination's 16 B phase ------------
+    if (threadIdx.x < nscan) {
+      const uint32_t d = threadIdx.x;
+      const uint32_t c = d < F ? s_cnt[d] : 0u;
+      uint32_t x = c;
+      #pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+        if (lane >= o) x += y;
+      }
+      if (lane == 31) s_wt[warp] = x;
+      asm volatile("barrier.sync 1, %0;" ::"r"(nscan) : "memory");
+      uint32_t base = 0;
+      for (int w = 0; w < warp; ++w) base += s_wt[w];
+      if (pending) {  // the previous tile's bulk stores must have read s_buf before the shuffle
+        bulk_wait_read();
+        pending = false;
+      }
+      if (d < F) {
+        const uint32_t loc = base + x - c;
+        const unsigned long long g0 = s_cur[d];
+        // digit d owns smem slots [loc + TPS*d, loc + TPS*d + c + TPS - 1]: shift by 0..TPS-1 to
+        // match the destination's phase within a 16-byte segment
+        const uint32_t s0 = loc + (uint32_t)TPS * d;
+        const uint32_t sh = (uint32_t)((g0 + TPS - (s0 % TPS)) % TPS);
+        s_loc[d] = s0 + sh;
+        s_gst[d] = g0;
+        s_len[d] = c;
+        s_cur[d] = g0 + c;
+        s_cnt[d] = 0;
+        if (c > TILE / 4) atomicExch(&s_hot_next, d);
+      }
+    }
+    __syncthreads();
+    // ---- phase 3: shuffle into the aligned run slots; make the writes visible to the TMA -----
+    if (threadIdx.x == 0) {
+      s_hot = s_hot_next;
+      s_hot_next = 0xffffffffu;
+    }
+    #pragma unroll
+    for (int j = 0; j < ITEMS; ++j)
+      if (full || pass_elem<K, 1, NT>(j) < ulen)
+        s_buf[s_loc[digit(kk[j])] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = TT::make(kk[j], pp[j]);
+    fence_proxy_async();
+    __syncthreads();
+    // ---- phase 4: one bulk store per run (+ ragged ends), completed asynchronously -------------
+    if (threadIdx.x < F) {
+      const uint32_t d = threadIdx.x, c = s_len[d];
+      if (c) {
+        const uint32_t sl = s_loc[d];
+        const unsigned long long g0 = s_gst[d];
+        const uint32_t head = (uint32_t)min((unsigned long long)c, (TPS - g0 % TPS) % TPS);
+        for (uint32_t t = 0; t < head; ++t) dst[g0 + t] = s_buf[sl + t];
+        const uint32_t body = (c - head) / TPS * TPS;
+        if (body) {
+          bulk_s2g(dst + g0 + head, s_buf + sl + head, body * (uint32_t)sizeof(T));
+          bulk_commit();
+          pending = true;
+        }
+        for (uint32_t t = head + body; t < c; ++t) dst[g0 + t] = s_buf[sl + t];
+      }
+    }
+    u = un;
+    if (u < units && (u < units0 ? 0 : 1) != cur_rel && pending) {  // before the cursors switch
+      bulk_wait_read();
+      pending = false;
+    }
+  }
+  bulk_wait_all();  // the bulk stores' global writes complete before the kernel (and pass 2) ends
 }
 
 }  // namespace hj

@@ -38,6 +38,12 @@ struct Plan {
   int nsrc;       // count rows / piece sources (PLAN_RECV: ranks), else 1
   int mode;       // PLAN_FULL, PLAN_SEND, PLAN_RECV
   int skip_r;     // streaming S chunks: R is already partitioned (its pass-2 units are skipped)
+  // pass 1 with precomputed per-block bases (k_pass1b): the histogram kernel runs with the same
+  // grid and tile -> block assignment as pass 1 and also counts each block's pass-1 digits
+  uint32_t g1;                  // pass-1 grid (0 = bases not used)
+  uint32_t tile1;               // pass-1 tile (tuples)
+  uint32_t* cntb;               // [2][g1][2^pb] per-block pass-1 digit counts (k_hist)
+  unsigned long long* relb;     // [2][g1][2^pb] exclusive prefix over blocks (k_plan)
   uint32_t C2;           // pass-2 chunk (tile) size in tuples
   uint32_t CR, CS;       // join item capacities: R tuples (smem build) and S tuples per item
   uint32_t* ist;         // [2^B + 1] join item prefix (q-order)

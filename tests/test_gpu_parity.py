@@ -373,3 +373,20 @@ def test_compute_sanitizer_clean(hj, tool):
     txt = out.stdout + out.stderr
     assert "sanitize cases ok" in txt, txt[-2000:]
     assert ("ERROR SUMMARY: 0 errors" in txt) or ("RACECHECK SUMMARY: 0 hazards" in txt), txt[-2000:]
+
+
+@pytest.mark.parametrize("name", ["dups_both", "random_ragged", "sparse_uniform"])
+@pytest.mark.parametrize("width", [4, 8])
+def test_pass1_bases_variant_vs_oracle(hj, name, width):
+    """HJ_OPT_PASS1_BASES: per-block bases from the histogram + TMA bulk-store write-out."""
+    rng = np.random.default_rng(77)
+    Rk, Sk = adversarial(rng)[name]
+    dt = np.uint32 if width == 4 else np.uint64
+    Rk, Sk = Rk.astype(dt) * dt(0x10001), Sk.astype(dt) * dt(0x10001)
+    Rp = np.arange(len(Rk), dtype=dt)
+    Sp = np.arange(len(Sk), dtype=dt)
+    ctx = hj.Context(0, width, width)
+    ctx.set_option(hj.OPT_PASS1_BASES, 1)
+    for bits in (-1, 3, 12):
+        check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True, ctx=ctx)
+    ctx.close()
