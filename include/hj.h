@@ -71,6 +71,9 @@ enum hj_option {
   HJ_OPT_PASS1_BASES = 10,  /* 1 = pass 1 uses per-block bases computed by the histogram kernel and
                                TMA bulk-store write-out instead of atomic run reservation (opt-in;
                                measured slower on B200, kept for comparison)                      */
+  HJ_OPT_GRAPH = 11,        /* 1 = hj_join captures its launch sequence in a CUDA graph and replays
+                               it while the call signature is unchanged (launch-bound small joins;
+                               per-kernel ms_kernel are not reported in this mode)               */
   HJ_OPT_STREAM_CHUNK = 8   /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
                                least 2^22; >= |S| = copy everything, then join)                   */
 };

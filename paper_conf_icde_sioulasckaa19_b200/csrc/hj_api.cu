@@ -53,7 +53,7 @@ struct Ctx {
   std::string err;
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
-          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0;
+          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0, opt_graph = 0;
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2], np_heads, np_next;
   void* h_res = nullptr;  // pinned host: results readback
@@ -62,6 +62,11 @@ struct Ctx {
   DevBuf part_off_host_dummy;
   cudaEvent_t ev[8] = {};
   uint32_t launches = 0;
+  // HJ_OPT_GRAPH: the launch sequence of the last hj_join, captured once and replayed while the
+  // call signature (columns, sizes, radix bits, mode, workspace) is unchanged
+  cudaGraphExec_t graph = nullptr;
+  unsigned long long graph_key[12] = {};
+  uint32_t graph_launches = 0;
 };
 
 int fail(Ctx* c, int code, const char* fmt, ...) {
@@ -638,6 +643,86 @@ int run_join_np(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, c
   return HJ_OK;
 }
 
+// One-shot graph path (HJ_OPT_GRAPH): kernels + result readback captured from the ctx stream;
+// timing events are recorded around the replay only (ms_kernel stays 0).
+int run_join_graph_on(Ctx* c, HostPlan& hp, Plan& P, bool mat, const unsigned long long* key, hj_result* res);
+
+// The capture and replays run on the ctx-owned stream (the caller's may be the legacy default
+// stream, which cannot be captured), ordered after the caller's stream by an event; the call is
+// synchronous, so later work on the caller's stream sees the results.
+int run_join_graph(Ctx* c, HostPlan& hp, Plan& P, bool mat, const unsigned long long* key, hj_result* res) {
+  cudaStream_t caller = c->stream;
+  if (caller != c->own_stream) {
+    CUDA_TRY(c, cudaEventRecord(c->ev[7], caller));
+    CUDA_TRY(c, cudaStreamWaitEvent(c->own_stream, c->ev[7], 0));
+  }
+  c->stream = c->own_stream;
+  const int rc = run_join_graph_on(c, hp, P, mat, key, res);
+  c->stream = caller;
+  return rc;
+}
+
+int run_join_graph_on(Ctx* c, HostPlan& hp, Plan& P, bool mat, const unsigned long long* key, hj_result* res) {
+  cudaStream_t st = c->stream;
+  unsigned long long* h = (unsigned long long*)c->h_res;
+  if (!c->graph || memcmp(key, c->graph_key, sizeof c->graph_key) != 0) {
+    if (c->graph) cudaGraphExecDestroy(c->graph);
+    c->graph = nullptr;
+    const int64_t timing = c->opt_timing;
+    c->opt_timing = 0;  // no event records inside the capture
+    c->launches = 0;
+    CUDA_TRY(c, cudaStreamBeginCapture(st, cudaStreamCaptureModeThreadLocal));
+    int rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P);
+    if (!rc) rc = c->key_bytes == 4 ? launch_pass2<uint32_t>(c, hp, P) : launch_pass2<uint64_t>(c, hp, P);
+    if (!rc) rc = c->key_bytes == 4 ? launch_join<uint32_t>(c, hp, P, mat) : launch_join<uint64_t>(c, hp, P, mat);
+    if (!rc && cudaMemcpyAsync(h, P.results, 4 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st) != cudaSuccess)
+      rc = fail(c, HJ_ERR_CUDA, "capture: results copy");
+    if (!rc && cudaMemcpyAsync(h + 4, P.ist + (1ull << hp.B), sizeof(uint32_t), cudaMemcpyDeviceToHost, st) != cudaSuccess)
+      rc = fail(c, HJ_ERR_CUDA, "capture: items copy");
+    cudaGraph_t g = nullptr;
+    cudaError_t e = cudaStreamEndCapture(st, &g);
+    c->opt_timing = timing;
+    if (rc) {
+      if (g) cudaGraphDestroy(g);
+      return rc;
+    }
+    if (e != cudaSuccess) return fail(c, HJ_ERR_CUDA, "graph capture: %s", cudaGetErrorString(e));
+    e = cudaGraphInstantiate(&c->graph, g, 0);
+    cudaGraphDestroy(g);
+    if (e != cudaSuccess) {
+      c->graph = nullptr;
+      return fail(c, HJ_ERR_CUDA, "graph instantiate: %s", cudaGetErrorString(e));
+    }
+    memcpy(c->graph_key, key, sizeof c->graph_key);
+    c->graph_launches = c->launches;
+  }
+  if (c->opt_timing) CUDA_TRY(c, cudaEventRecord(c->ev[0], st));
+  CUDA_TRY(c, cudaGraphLaunch(c->graph, st));
+  if (c->opt_timing) CUDA_TRY(c, cudaEventRecord(c->ev[6], st));
+  CUDA_TRY(c, cudaStreamSynchronize(st));
+  if (mat && h[RES_MATCHES] > P.out_cap) {  // overflow: drop the graph, redo on the normal path
+    cudaGraphExecDestroy(c->graph);
+    c->graph = nullptr;
+    c->launches = 0;
+    int rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P);
+    if (!rc) rc = c->key_bytes == 4 ? launch_pass2<uint32_t>(c, hp, P) : launch_pass2<uint64_t>(c, hp, P);
+    return rc ? rc : finish_join(c, hp, P, mat, res);
+  }
+  memset(res, 0, sizeof *res);
+  res->matches = h[RES_MATCHES];
+  res->checksum = h[RES_CHECKSUM];
+  res->n_items = (uint32_t)h[4];
+  res->radix_bits = hp.B;
+  res->passes = hp.B >= 2 ? 2 : (hp.B == 1 ? 1 : 0);
+  res->kernels = c->graph_launches;
+  if (mat) {
+    res->r_pay_out = c->out_r.p;
+    res->s_pay_out = c->out_s.p;
+  }
+  if (c->opt_timing) cudaEventElapsedTime(&res->ms_total, c->ev[0], c->ev[6]);
+  return HJ_OK;
+}
+
 int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk, const void* Sp,
              unsigned long long nS, int radix_bits, int out_mode, hj_result* res) {
   const bool mat = out_mode == HJ_OUT_MATERIALIZE;
@@ -648,6 +733,14 @@ int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, cons
   int rc = prepare(c, hp, nR, nS, radix_bits, mat);
   if (rc) return rc;
   Plan P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
+  if (c->opt_graph) {
+    const unsigned long long key[12] = {(unsigned long long)Rk, (unsigned long long)Rp, nR, (unsigned long long)Sk,
+                                        (unsigned long long)Sp, nS, (unsigned long long)hp.B * 2 + mat,
+                                        (unsigned long long)c->meta.p, (unsigned long long)c->out_r.p,
+                                        (unsigned long long)c->t1[1].p, (unsigned long long)c->t2[1].p,
+                                        (unsigned long long)c->opt_join_algo};
+    return run_join_graph(c, hp, P, mat, key, res);
+  }
   c->launches = 0;
   if ((rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P))) return rc;
   if ((rc = c->key_bytes == 4 ? launch_pass2<uint32_t>(c, hp, P) : launch_pass2<uint64_t>(c, hp, P))) return rc;
@@ -891,6 +984,7 @@ void hj_destroy(hj_ctx* h) {
                     &c->xcnt[1], &c->np_heads, &c->np_next};
   for (DevBuf* b : bufs)
     if (b->p) cudaFree(b->p);
+  if (c->graph) cudaGraphExecDestroy(c->graph);
   if (c->h_res) cudaFreeHost(c->h_res);
   if (c->h_out) cudaFreeHost(c->h_out);
   for (auto& ev : c->ev)
@@ -928,6 +1022,13 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_BLOCKS_PER_SM: c->opt_bps = v; break;
     case HJ_OPT_STREAM_CHUNK: c->opt_stream_chunk = v; break;
     case HJ_OPT_PASS1_BASES: c->opt_pass1_bases = v; break;
+    case HJ_OPT_GRAPH:
+      c->opt_graph = v;
+      if (!v && c->graph) {
+        cudaGraphExecDestroy(c->graph);
+        c->graph = nullptr;
+      }
+      break;
     case HJ_OPT_JOIN_ALGO:
       if (v > 2) return fail(c, HJ_ERR_INVALID, "join algorithm must be 0, 1 or 2");
       c->opt_join_algo = v;

@@ -390,3 +390,29 @@ def test_pass1_bases_variant_vs_oracle(hj, name, width):
     for bits in (-1, 3, 12):
         check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True, ctx=ctx)
     ctx.close()
+
+
+def test_graph_replay_matches_oracle(hj):
+    """HJ_OPT_GRAPH: the captured launch sequence replays with identical results; a new call
+    signature recaptures; materialize overflow falls back to the normal path."""
+    ctx = hj.Context(0, 4, 4)
+    ctx.set_option(hj.OPT_GRAPH, 1)
+    for seed in (190, 191):
+        w = W.Workload("g", 1 << 14, 1 << 15, "zipf", keys="sparse", z=1.0, seed=seed)
+        Rk, Rp, Sk, Sp = W.np_generate(w)
+        m, c, r, s = oracle.hash_join(Rk, Rp, Sk, Sp, materialize=True)
+        cols = [dev(a) for a in (Rk, Rp, Sk, Sp)]
+        for _ in range(3):
+            res = ctx.join(*cols)
+            assert (res.matches, res.checksum) == (m, c)
+        for _ in range(2):
+            res = ctx.join(*cols, out_mode=hj.OUT_MATERIALIZE)
+            assert res.matches == m
+            assert np.array_equal(oracle.pairs_sorted(to_np(res.r_pay, 4), to_np(res.s_pay, 4)), oracle.pairs_sorted(r, s))
+    ctx.set_option(hj.OPT_OUT_CAPACITY, 1000)
+    Rk = np.repeat(np.arange(50, dtype=np.uint32), 40)
+    Sk = np.repeat(np.arange(60, dtype=np.uint32), 30)
+    res = check_against_oracle(hj, Rk, np.arange(len(Rk), dtype=np.uint32), Sk, np.arange(len(Sk), dtype=np.uint32),
+                               bits=3, mat=True, ctx=ctx)
+    assert res.matches == 50 * 40 * 30
+    ctx.close()
