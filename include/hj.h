@@ -74,6 +74,13 @@ enum hj_option {
   HJ_OPT_GRAPH = 11,        /* 1 = hj_join captures its launch sequence in a CUDA graph and replays
                                it while the call signature is unchanged (launch-bound small joins;
                                per-kernel ms_kernel are not reported in this mode)               */
+  HJ_OPT_PARTITIONER = 12,  /* hj_join only: 0 = histogram + prefix sum + exact placement (north
+                               star, default); 1 = the paper's histogram-free bucket chains
+                               (NEXT-1): no histogram pass, partitions are chains of
+                               buckets from a pool, pass 2 takes one bucket at a time. Needs more
+                               device memory (bucket slack); ms_kernel[0..1] are 0 and
+                               ms_kernel[2..3] include each pass's bucket bookkeeping. Ignored by
+                               hj_join_host / hj_partition / the exchange calls and by graph mode */
   HJ_OPT_STREAM_CHUNK = 8   /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
                                least 2^22; >= |S| = copy everything, then join)                   */
 };

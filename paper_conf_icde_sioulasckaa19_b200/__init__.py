@@ -40,6 +40,7 @@ OPT_STREAM_CHUNK = 8
 OPT_JOIN_ALGO = 9
 OPT_PASS1_BASES = 10
 OPT_GRAPH = 11
+OPT_PARTITIONER = 12  # 0 = histogram (default), 1 = bucket chains (NEXT-1)
 ALGO_HASH, ALGO_NLJ, ALGO_NONPARTITIONED = 0, 1, 2
 
 _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4: "HJ_ERR_CUDA", -5: "HJ_ERR_COMM"}

@@ -27,10 +27,12 @@ thread_local std::string g_create_error;
 //   variant: compute threads, S tuples / thread / round, min blocks / SM, R tile buffers
 struct JoinShape {
   int nt, spt, minb, rbuf, nbsh;  // nbsh: hash slots = 2^(ceil(log2 C_R) - nbsh)
+  bool h16;                       // 16-bit chain heads
 };
 constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1, 1}, {256, 8, 2, 2, 1}, {224, 8, 3, 1, 1}, {256, 12, 3, 1, 1},
                                      {192, 8, 3, 1, 1}, {256, 4, 2, 1, 1}, {512, 4, 1, 1, 1}, {256, 8, 2, 1, 1},
-                                     {384, 4, 1, 2, 1}, {192, 8, 4, 1, 2}, {256, 8, 3, 1, 2}, {160, 8, 4, 1, 2}};
+                                     {384, 4, 1, 2, 1}, {192, 8, 4, 1, 2}, {256, 8, 3, 1, 2}, {160, 8, 4, 1, 2},
+                                     {224, 8, 4, 1, 1, true}, {192, 8, 4, 1, 1, true}, {256, 8, 3, 1, 1, true}};
 constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
 
@@ -53,7 +55,9 @@ struct Ctx {
   std::string err;
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
-          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0, opt_graph = 0;
+          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0, opt_graph = 0,
+          opt_partitioner = 0;
+  DevBuf bc_pool1[2], bc_pool2[2], bc_meta;  // HJ_OPT_PARTITIONER = 1 (NEXT-1 bucket chains)
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2], np_heads, np_next;
   void* h_res = nullptr;  // pinned host: results readback
@@ -183,9 +187,10 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   else CS = std::max<uint32_t>(8 * CR, 32768);
   const int rbuf = JOIN_SHAPES[join_variant(c)].rbuf;
   const int nbsh = JOIN_SHAPES[join_variant(c)].nbsh;
+  const size_t head_bytes = JOIN_SHAPES[join_variant(c)].h16 ? 2 : 4;
   int lg_nb = std::max(6, ilog2_ceil(CR) - nbsh);
   auto join_smem = [&](uint32_t cr, int lg) {  // R tile buffer(s) (TMA) + heads + next
-    return (size_t)rbuf * ((cr + 3) & ~1u) * tb + ((size_t)4 << lg) + (size_t)cr * 2;
+    return (size_t)rbuf * ((cr + 3) & ~1u) * tb + (head_bytes << lg) + (size_t)cr * 2;
   };
   while (join_smem(CR, lg_nb) > cap_max_smem - 8 * 1024 && CR > 256) {
     CR /= 2;
@@ -234,8 +239,8 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
 template <typename K, int V, typename F>
 void attr_join(F&& attr) {
   constexpr JoinShape S = JOIN_SHAPES[V];
-  attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf>);
-  attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf>);
+  attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16>);
+  attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16>);
 }
 
 template <typename K>
@@ -264,6 +269,10 @@ int set_kernel_attrs(Ctx* c) {
   attr((const void*)k_pass<K, 1, 512, pass_items<K>(), false>);
   attr((const void*)k_pass<K, 1, 512, pass_items<K>(), true>);
   attr((const void*)k_pass<K, 2, 512, pass_items<K>(), false>);
+  attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), false, true>);
+  attr((const void*)k_pass<K, 1, 512, pass_items<K>(), false, true>);
+  attr((const void*)k_pass<K, 2, 1024, pass_items<K>(), false, true>);
+  attr((const void*)k_pass<K, 2, 512, pass_items<K>(), false, true>);
   attr_join<K, 0>(attr);
   attr_join<K, 1>(attr);
   attr_join<K, 2>(attr);
@@ -276,6 +285,9 @@ int set_kernel_attrs(Ctx* c) {
   attr_join<K, 9>(attr);
   attr_join<K, 10>(attr);
   attr_join<K, 11>(attr);
+  attr_join<K, 12>(attr);
+  attr_join<K, 13>(attr);
+  attr_join<K, 14>(attr);
   return rc;
 }
 
@@ -348,7 +360,7 @@ void mark(Ctx* c, int i) {
 
 // a1 (histogram), a2/a5 (planner), a3 (pass 1). PLAN_RECV skips a1 and a3 (counts and the
 // pass-1 layout arrive through the exchange). Events 0..3.
-template <typename K, int MODE, int NT, bool GD>
+template <typename K, int MODE, int NT, bool GD, bool BC = false>
 int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits);
 
 template <typename K>
@@ -429,10 +441,10 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false) 
 
 // a4: pass 2 over the pass-1 pieces. Event 4.
 // a4: pass 2 over the pass-1 pieces. Event 4.
-template <typename K, int MODE, int NT, bool GD>
+template <typename K, int MODE, int NT, bool GD, bool BC>
 int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
   constexpr int IT = pass_items<K>();
-  const void* f = (const void*)k_pass<K, MODE, NT, IT, GD>;
+  const void* f = (const void*)k_pass<K, MODE, NT, IT, GD, BC>;
   const size_t sm = (size_t)NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << fanout_bits) * 24 + 16;
   const unsigned long long tile = (unsigned long long)NT * IT;
   // units: pass 1 = tiles; pass 2 = at most n / tile + pieces per relation
@@ -440,12 +452,13 @@ int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
   Q.C2 = (uint32_t)tile;
   unsigned long long units = MODE == 1 ? (P.rel[0].n + tile - 1) / tile + (P.rel[1].n + tile - 1) / tile
                                        : (P.rel[0].n + P.rel[1].n) / tile + 2ull * hp.npieces() + 2;
+  if (BC && MODE == 2) units = (P.rel[0].n + P.rel[1].n) / tile + P.bc_rel[0].nbmax1 + P.bc_rel[1].nbmax1 + 2;
   if (MODE == 1) {
     Q.tiles1[0] = (P.rel[0].n + tile - 1) / tile;
     Q.tiles1[1] = (P.rel[1].n + tile - 1) / tile;
   }
   int g = grid_for(c, f, NT, sm, units);
-  k_pass<K, MODE, NT, IT, GD><<<g, NT, sm, c->stream>>>(Q, fanout_bits);
+  k_pass<K, MODE, NT, IT, GD, BC><<<g, NT, sm, c->stream>>>(Q, fanout_bits);
   CUDA_TRY(c, cudaGetLastError());
   c->launches += 1;
   return HJ_OK;
@@ -465,11 +478,11 @@ template <typename K, int V>
 int launch_join_v(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   constexpr JoinShape S = JOIN_SHAPES[V];
   cudaStream_t st = c->stream;
-  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf>
-                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf>;
+  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16>
+                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16>;
   int g = grid_for(c, f, S.nt + 32, hp.join_smem, 1ull << 40);
-  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
-  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16><<<g, S.nt + 32, hp.join_smem, st>>>(P);
   CUDA_TRY(c, cudaGetLastError());
   return HJ_OK;
 }
@@ -489,6 +502,9 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
     return HJ_OK;
   }
   switch (join_variant(c)) {
+    case 12: rc = launch_join_v<K, 12>(c, hp, P, mat); break;
+    case 13: rc = launch_join_v<K, 13>(c, hp, P, mat); break;
+    case 14: rc = launch_join_v<K, 14>(c, hp, P, mat); break;
     case 9: rc = launch_join_v<K, 9>(c, hp, P, mat); break;
     case 10: rc = launch_join_v<K, 10>(c, hp, P, mat); break;
     case 11: rc = launch_join_v<K, 11>(c, hp, P, mat); break;
@@ -540,6 +556,7 @@ int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res) {
   CUDA_TRY(c, cudaMemcpyAsync(h + 4, P.ist + (1ull << hp.B), sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
   if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[6], st));
   CUDA_TRY(c, cudaStreamSynchronize(st));
+  if (P.bc && h[RES_BC_OVERFLOW]) return fail(c, HJ_ERR_CUDA, "bucket pool overflow (pool bound violated)");
   unsigned long long matches = h[RES_MATCHES];
   if (mat && matches > P.out_cap) {
     // materialization overflow (reading S11): grow to the exact size and re-run only the join
@@ -723,12 +740,121 @@ int run_join_graph_on(Ctx* c, HostPlan& hp, Plan& P, bool mat, const unsigned lo
   return HJ_OK;
 }
 
+// HJ_OPT_PARTITIONER = 1: the paper's histogram-free bucket-chain partitioner (NEXT-1,
+// hj_bucket.cuh). Pool sizes are the proven bounds of hj_bucket.cuh: a closed bucket holds >= cap
+// tuples, so n / cap + min(partitions, n) buckets suffice per relation and pass.
+template <typename K>
+int run_join_bc(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk, const void* Sp,
+                unsigned long long nS, int radix_bits, bool mat, hj_result* res) {
+  HostPlan hp;
+  int rc = make_plan(c, hp, nR, nS, radix_bits, mat);
+  if (rc) return rc;
+  if ((rc = ensure(c, c->meta, hp.meta_bytes))) return rc;
+  if (mat) {
+    unsigned long long cap = c->opt_out_cap > 0 ? (unsigned long long)c->opt_out_cap : std::max<unsigned long long>(nS, 1 << 20);
+    if (c->out_r.bytes < cap * c->pay_bytes &&
+        ((rc = ensure(c, c->out_r, cap * c->pay_bytes)) || (rc = ensure(c, c->out_s, cap * c->pay_bytes))))
+      return rc;
+  }
+  Plan P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
+  P.bc = 1;
+  const size_t tb = sizeof(typename Tup<K>::T);
+  const unsigned long long ns[2] = {nR, nS}, F1 = 1ull << hp.b1, np = 1ull << hp.B;
+  const uint32_t tile1 = (uint32_t)hp.tile, C2 = hp.C2;
+  // metadata layout: zeroed part first (states, pass-2 fills, slice counts)
+  size_t o = 0, o_st1[2], o_st2[2], o_fill2[2], o_nsl[2], o_fill1[2], o_part1[2], o_part2[2], o_sl[2],
+         o_sst[2], o_scur[2];
+  auto take = [&](size_t bytes) {
+    size_t r = o;
+    o = align_up(o + bytes, 256);
+    return r;
+  };
+  // capacities: 2x the mean partition (uniform inputs never close a bucket; a skewed partition
+  // closes one per cap tuples), at least 4 tiles in pass 1; stride = cap + tile (closing run)
+  auto cap_for = [](unsigned long long mean, uint32_t tile, unsigned long long min_tiles) {
+    const unsigned long long t = std::max<unsigned long long>(min_tiles, (2 * mean + tile - 1) / tile);
+    return (uint32_t)std::min<unsigned long long>(t * tile, 1ull << 30);
+  };
+  for (int r = 0; r < 2; ++r) {
+    BcRel& B = P.bc_rel[r];
+    B.cap1 = cap_for((ns[r] + F1 - 1) / F1, tile1, 4);
+    B.bsz1 = (unsigned long long)B.cap1 + tile1;
+    B.cap2 = cap_for((ns[r] + np - 1) / np, C2, 1);
+    B.bsz2 = (unsigned long long)B.cap2 + C2;
+    B.np1 = (uint32_t)F1;
+    B.np2 = (uint32_t)np;
+    B.nbmax1 = (uint32_t)(ns[r] / B.cap1 + F1 + 1);
+    if (B.nbmax1 + 5 > BC_MAX_NB1) return fail(c, HJ_ERR_INVALID, "bucket chains: %u pass-1 buckets", B.nbmax1);
+    B.nbmax2 = (uint32_t)(ns[r] / B.cap2 + np + 1);
+    B.csl = r == 0 ? hp.CR : hp.CS;
+    o_st1[r] = take(F1 * 8);
+    o_st2[r] = take(np * 8);
+    o_nsl[r] = take(np * 4);
+  }
+  const size_t zero_bytes = o;
+  for (int r = 0; r < 2; ++r) {
+    const BcRel& B = P.bc_rel[r];
+    o_fill1[r] = take((size_t)B.nbmax1 * 4);
+    o_part1[r] = take((size_t)B.nbmax1 * 4);
+    o_part2[r] = take((size_t)B.nbmax2 * 4);
+    o_fill2[r] = take((size_t)B.nbmax2 * 4);
+    o_sl[r] = take((ns[r] / B.csl + B.nbmax2 + 1) * 16);
+    o_sst[r] = take((np + 1) * 4);
+    o_scur[r] = take(np * 4);
+  }
+  if ((rc = ensure(c, c->bc_meta, o))) return rc;
+  for (int r = 0; r < 2; ++r) {
+    BcRel& B = P.bc_rel[r];
+    if ((rc = ensure(c, c->bc_pool1[r], (size_t)B.nbmax1 * B.bsz1 * tb))) return rc;
+    if ((rc = ensure(c, c->bc_pool2[r], (size_t)B.nbmax2 * B.bsz2 * tb))) return rc;
+    char* m = (char*)c->bc_meta.p;
+    B.pool1 = c->bc_pool1[r].p;
+    B.pool2 = c->bc_pool2[r].p;
+    B.st1 = (unsigned long long*)(m + o_st1[r]);
+    B.st2 = (unsigned long long*)(m + o_st2[r]);
+    B.fill1 = (uint32_t*)(m + o_fill1[r]);
+    B.part1 = (uint32_t*)(m + o_part1[r]);
+    B.fill2 = (uint32_t*)(m + o_fill2[r]);
+    B.part2 = (uint32_t*)(m + o_part2[r]);
+    B.sl = (uint4*)(m + o_sl[r]);
+    B.nsl = (uint32_t*)(m + o_nsl[r]);
+    B.sst = (uint32_t*)(m + o_sst[r]);
+    B.scur = (uint32_t*)(m + o_scur[r]);
+    P.rel[r].t2 = B.pool2;  // the join reads slices of the pass-2 pool
+  }
+  cudaStream_t st = c->stream;
+  c->launches = 0;
+  mark(c, 0);
+  CUDA_TRY(c, cudaMemsetAsync(c->meta.p, 0, hp.zero_bytes, st));
+  CUDA_TRY(c, cudaMemsetAsync(c->bc_meta.p, 0, zero_bytes, st));
+  mark(c, 1);  // no histogram
+  mark(c, 2);  // no planner before the passes
+  rc = hp.tile == 512 * pass_items<K>() ? launch_pass<K, 1, 512, false, true>(c, hp, P, hp.b1)
+                                        : launch_pass<K, 1, 1024, false, true>(c, hp, P, hp.b1);
+  if (rc) return rc;
+  mark(c, 3);
+  rc = C2 == (uint32_t)(512 * pass_items<K>()) ? launch_pass<K, 2, 512, false, true>(c, hp, P, hp.b2)
+                                               : launch_pass<K, 2, 1024, false, true>(c, hp, P, hp.b2);
+  if (rc) return rc;
+  const unsigned long long idx = np + std::max(P.bc_rel[0].nbmax2, P.bc_rel[1].nbmax2);
+  const int gc = (int)std::min<unsigned long long>((idx + 255) / 256, 4ull * c->num_sms);
+  k_bc_plan<<<(unsigned)((np + 1023) / 1024), 1024, 0, st>>>(P);
+  k_bc_slices<<<gc, 256, 0, st>>>(P);
+  CUDA_TRY(c, cudaGetLastError());
+  c->launches += 2;
+  mark(c, 4);
+  return finish_join(c, hp, P, mat, res);
+}
+
 int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk, const void* Sp,
              unsigned long long nS, int radix_bits, int out_mode, hj_result* res) {
   const bool mat = out_mode == HJ_OUT_MATERIALIZE;
   if (c->opt_join_algo == 2)
     return c->key_bytes == 4 ? run_join_np<uint32_t>(c, Rk, Rp, nR, Sk, Sp, nS, mat, res)
                              : run_join_np<uint64_t>(c, Rk, Rp, nR, Sk, Sp, nS, mat, res);
+  if (c->opt_partitioner == 1)
+    return c->key_bytes == 4 ? run_join_bc<uint32_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, mat, res)
+                             : run_join_bc<uint64_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, mat, res);
   HostPlan hp;
   int rc = prepare(c, hp, nR, nS, radix_bits, mat);
   if (rc) return rc;
@@ -1022,6 +1148,10 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_BLOCKS_PER_SM: c->opt_bps = v; break;
     case HJ_OPT_STREAM_CHUNK: c->opt_stream_chunk = v; break;
     case HJ_OPT_PASS1_BASES: c->opt_pass1_bases = v; break;
+    case HJ_OPT_PARTITIONER:
+      if (v > 1) return fail(c, HJ_ERR_INVALID, "partitioner must be 0 (histogram) or 1 (bucket chains)");
+      c->opt_partitioner = v;
+      break;
     case HJ_OPT_GRAPH:
       c->opt_graph = v;
       if (!v && c->graph) {

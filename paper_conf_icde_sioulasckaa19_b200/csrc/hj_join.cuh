@@ -16,6 +16,8 @@
 #include "hj_common.cuh"
 #include "hj_plan.cuh"
 
+#include <type_traits>
+
 namespace hj {
 
 constexpr uint32_t NIL16 = 0xffffu;
@@ -41,6 +43,18 @@ __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items
       if (P.ist[mid] <= j.item) lo = mid; else hi = mid;
     }
     const uint32_t q = lo;
+    if (P.bc) {  // bucket chains (NEXT-1): item = (R slice, S slice) of q, slices from k_bc_slices
+      const uint32_t loc = j.item - P.ist[q], nsch = P.bc_rel[1].sst[q + 1] - P.bc_rel[1].sst[q];
+      const uint4 rs = P.bc_rel[0].sl[P.bc_rel[0].sst[q] + loc / nsch];
+      const uint4 ss = P.bc_rel[1].sl[P.bc_rel[1].sst[q] + loc % nsch];
+      j.rb = ((unsigned long long)rs.y << 32) | rs.x;
+      j.nr = rs.z;
+      j.sb = ((unsigned long long)ss.y << 32) | ss.x;
+      j.se = j.sb + ss.z;
+      const uintptr_t a = reinterpret_cast<uintptr_t>((const T*)P.rel[0].t2 + j.rb);
+      j.shift = (uint32_t)((a & 15) / sizeof(T));
+      return j;
+    }
     const unsigned long long r0 = P.rel[0].off[q], rn = P.rel[0].off[q + 1] - r0;
     const unsigned long long s0 = P.rel[1].off[q], sn = P.rel[1].off[q + 1] - s0;
     const unsigned long long nsch = (sn + P.CS - 1) / P.CS;
@@ -88,7 +102,19 @@ __device__ __forceinline__ void bar_item(int nthreads) { asm volatile("barrier.s
 // Chains are re-walked only for S tuples with more than one match.
 // RBUF = 2: the next item's R chunk is copied while the current item is joined (double buffer);
 // RBUF = 1: it is copied right after the end-of-item barrier (less smem -> more blocks per SM).
-template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF>
+// 16-bit wait-free push-front for H16 heads: a 16-bit CAS loop (retries only when two R tuples
+// of the same slot insert at the same time)
+__device__ __forceinline__ uint32_t exch16(unsigned short* a, uint32_t v) {
+  unsigned short old = *a, assumed;
+  do {
+    assumed = old;
+    old = atomicCAS(a, assumed, (unsigned short)v);
+  } while (old != assumed);
+  return old;
+}
+
+// H16: 16-bit chain heads (half the head array -> one more block per SM fits in shared memory)
+template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false>
 __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -97,7 +123,8 @@ __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
   const uint32_t nb = 1u << H.lg;
   const uint32_t cap = (P.CR + 3) & ~1u;  // tile buffer in tuples: +2 for the aligned superset, even -> 16 B aligned
   T* s_rtb = reinterpret_cast<T*>(s_raw);                             // RBUF x cap tuples
-  uint32_t* s_head = reinterpret_cast<uint32_t*>(s_rtb + RBUF * cap);  // nb
+  using HT = typename std::conditional<H16, unsigned short, uint32_t>::type;
+  HT* s_head = reinterpret_cast<HT*>(s_rtb + RBUF * cap);             // nb
   uint16_t* s_next = reinterpret_cast<uint16_t*>(s_head + nb);       // CR
   __shared__ JoinJob s_jobs[2];
   __shared__ __align__(8) unsigned long long s_bar[2];
@@ -158,7 +185,8 @@ __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
     bar_compute(NT);
     // ---- build (a6): wait-free push-front insert (Listing 2) ----------------------
     for (uint32_t i = threadIdx.x; i < job.nr; i += NT)
-      s_next[i] = (uint16_t)atomicExch(&s_head[slot_of(TT::key(s_rt[i]), H)], i);
+      s_next[i] = H16 ? (uint16_t)exch16(reinterpret_cast<unsigned short*>(&s_head[slot_of(TT::key(s_rt[i]), H)]), i)
+                      : (uint16_t)atomicExch(reinterpret_cast<uint32_t*>(&s_head[slot_of(TT::key(s_rt[i]), H)]), i);
     bar_compute(NT);
 
     // ---- probe (a7) + output (a8), SPT tuples per thread per round --------------------------

@@ -12,6 +12,7 @@
 // range reserved with one global atomic per (tile, digit) -- the histogram-derived cursors
 // replace the paper's bucket chains (reading D2 in DESIGN.md).
 #pragma once
+#include "hj_bucket.cuh"
 #include "hj_common.cuh"
 #include "hj_plan.cuh"
 
@@ -317,22 +318,58 @@ struct __align__(16) PassUnit {
   unsigned long long* cur;  // reservation cursors: cur1 (MODE 1) or &cur2[d1 << b2] (MODE 2)
   uint32_t len;
   uint32_t valid;
+  uint32_t rel;    // bucket chains (BC): relation and first partition index of the unit's digits
+  uint32_t pbase;
 };
 
 // Unit u (round-robin: u = blockIdx.x + k * gridDim.x) -> its descriptor. MODE 2 maps the chunk
 // to its piece by binary search in the shared-memory chunk prefix (stateless: no registers live
 // across the unit loop).
-template <typename K, int MODE, int TILE>
+template <typename K, int MODE, int TILE, bool BC = false>
 struct UnitWalker {
   unsigned long long units0, units;
   __device__ __forceinline__ bool get(const Plan& P, unsigned long long u, PassUnit<K>& U, const uint32_t* s_cst,
-                                      const unsigned long long* s_pst) const {
+                                      const unsigned long long* s_pst, const uint32_t* s_bfill = nullptr,
+                                      const uint16_t* s_bd = nullptr) const {
     using T = typename Tup<K>::T;
-    U.valid = u < units;
+    // bucket-chain pass 2 keeps its unit counts in shared memory (spare top slots of s_cst):
+    // no registers live across k_pass's tile loop
+    const unsigned long long n0 = (BC && MODE == 2) ? s_cst[2 * BC_MAX_NB1 - 3] : units0;
+    const unsigned long long nn = (BC && MODE == 2) ? s_cst[2 * BC_MAX_NB1 - 4] : units;
+    U.valid = u < nn;
     if (!U.valid) return false;
-    const int r = (u < units0) ? 0 : 1;
-    const unsigned long long ul = r ? u - units0 : u;
+    const int r = (u < n0) ? 0 : 1;
+    const unsigned long long ul = r ? u - n0 : u;
     const RelDev& R = P.rel[r];
+    U.rel = r;
+    U.pbase = 0;
+    if (BC) {  // bucket chains: pass 1 as below into the pass-1 pool; pass 2 = one bucket unit
+      const BcRel& Bc = P.bc_rel[r];
+      if (MODE == 1) {
+        const unsigned long long s0 = ul * TILE;
+        U.src_k = (const K*)R.keys + s0;
+        U.src_p = (const K*)R.pays + s0;
+        U.dst = Bc.pool1;
+        U.cur = Bc.st1;
+        U.len = (uint32_t)min((unsigned long long)TILE, R.n - s0);
+      } else {  // unit -> (pass-1 bucket, tile) by binary search over the shared unit prefix
+        const uint32_t* cst = s_cst + r * BC_MAX_NB1;
+        const uint32_t uc = (uint32_t)ul;
+        uint32_t lo = 0, hi = s_cst[2 * BC_MAX_NB1 - 1 - r];  // buckets of r; largest with cst[b] <= uc
+        while (hi - lo > 1) {
+          const uint32_t mid = (lo + hi) >> 1;
+          if (cst[mid] <= uc) lo = mid; else hi = mid;
+        }
+        const uint32_t k = uc - cst[lo];
+        U.src_k = (const T*)Bc.pool1 + (unsigned long long)lo * Bc.bsz1 + (unsigned long long)k * TILE;
+        U.src_p = nullptr;
+        U.dst = Bc.pool2;
+        U.pbase = (uint32_t)s_bd[r * BC_MAX_NB1 + lo] << P.b2;
+        U.cur = Bc.st2 + U.pbase;
+        U.len = min((uint32_t)TILE, s_bfill[r * BC_MAX_NB1 + lo] - k * TILE);
+      }
+      return true;
+    }
     if (MODE == 1) {
       const unsigned long long s0 = ul * TILE;
       U.src_k = (const K*)R.keys + s0;
@@ -425,7 +462,46 @@ __device__ __forceinline__ void pass_load(const PassUnit<K>& U, K (&kk)[ITEMS], 
 //            reserve each run with one global atomic and store base - loc in s_gd[i&1]  | barrier
 //   phase 3  shuffle unit i into digit order in s_buf
 // so each reservation atomic's latency overlaps the previous unit's write-out.
-template <typename K, int MODE, int NT, int ITEMS, bool GD>
+// Bucket chains, pass 2 prologue: pass-1 buckets -> shared unit prefix (the bucket-at-a-time
+// unit list). Each bucket's fill (its partition's state if it is the current bucket,
+// else recorded by its closer), partition and pass-2 tiles, scanned over the buckets (<= 1.5 x
+// 2^b1 + 1 per relation). Not inlined: keeps its temporaries out of k_pass's register budget.
+template <int NT, int TILE>
+__device__ __noinline__ void bc_pass2_units(const BcRel* s_bc, const uint32_t* counters, uint32_t F1, uint32_t* s_cst,
+                                            uint32_t* s_bfill, uint16_t* s_bd) {
+  __shared__ unsigned long long s_scan[NT / 32 + 1];
+  unsigned long long tot[2];
+  for (int r = 0; r < 2; ++r) {
+    const BcRel& Bc = s_bc[r];
+    const uint32_t nb = min(F1 + counters[CNT_BC_NB1 + r], Bc.nbmax1);
+    const uint32_t per = (nb + NT - 1) / NT, b0 = threadIdx.x * per, b1 = min(b0 + per, nb);
+    unsigned long long mine = 0;
+    for (uint32_t b = b0; b < b1; ++b) {
+      const uint32_t p = b < F1 ? b : Bc.part1[b];
+      const unsigned long long st = Bc.st1[p];
+      const uint32_t j = (uint32_t)(st >> 32);
+      const uint32_t f = (j ? F1 + j - 1 : p) == b ? (uint32_t)st : Bc.fill1[b];
+      s_bfill[r * BC_MAX_NB1 + b] = f;
+      s_bd[r * BC_MAX_NB1 + b] = (uint16_t)p;
+      mine += (f + TILE - 1) / TILE;
+    }
+    unsigned long long u = block_exclusive_scan64<NT>(mine, s_scan, &tot[r]);
+    for (uint32_t b = b0; b < b1; ++b) {
+      s_cst[r * BC_MAX_NB1 + b] = (uint32_t)u;
+      u += (s_bfill[r * BC_MAX_NB1 + b] + TILE - 1) / TILE;
+    }
+    if (threadIdx.x == 0) {
+      s_cst[r * BC_MAX_NB1 + nb] = (uint32_t)tot[r];
+      s_cst[2 * BC_MAX_NB1 - 1 - r] = nb;  // bucket counts in the two spare top slots
+    }
+  }
+  if (threadIdx.x == 0) {
+    s_cst[2 * BC_MAX_NB1 - 3] = (uint32_t)tot[0];
+    s_cst[2 * BC_MAX_NB1 - 4] = (uint32_t)(tot[0] + tot[1]);
+  }
+}
+
+template <typename K, int MODE, int NT, int ITEMS, bool GD, bool BC = false>
 __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -440,8 +516,11 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
   uint32_t* s_loc = s_cnt + F + 4;                                                 // F
   __shared__ uint32_t s_wt[NT / 32];
   __shared__ uint32_t s_hot, s_hot_next;
-  __shared__ uint32_t s_cst[MODE == 2 ? 2 * 1025 : 1];
-  __shared__ unsigned long long s_pst[MODE == 2 ? 2 * 1025 : 1];
+  __shared__ uint32_t s_cst[MODE == 2 ? 2 * (BC ? BC_MAX_NB1 : 1025) : 1];
+  __shared__ unsigned long long s_pst[MODE == 2 && !BC ? 2 * 1025 : 1];
+  __shared__ uint32_t s_bfill[MODE == 2 && BC ? 2 * BC_MAX_NB1 : 1];  // bucket chains: pass-1 bucket fills
+  __shared__ uint16_t s_bd[MODE == 2 && BC ? 2 * BC_MAX_NB1 : 1];     // and their partitions D
+  __shared__ BcRel s_bc[BC ? 2 : 1];                                  // bucket chains: the plan's BcRel
 
   // digit of a key in this pass: D (pass 1, possibly widened by rank bits) or d2 (pass 2);
   // shifts and masks live in registers (not re-read from the parameter struct per tuple)
@@ -458,10 +537,18 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
 
   if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
   if (threadIdx.x == 0) s_hot = s_hot_next = 0xffffffffu;
-  UnitWalker<K, MODE, TILE> W;
+  UnitWalker<K, MODE, TILE, BC> W;
   if (MODE == 1) {
     W.units0 = P.tiles1[0];
     W.units = W.units0 + P.tiles1[1];
+  } else if (BC) {
+    if (threadIdx.x == 0) {
+      s_bc[0] = P.bc_rel[0];
+      s_bc[1] = P.bc_rel[1];
+    }
+    __syncthreads();
+    bc_pass2_units<NT, TILE>(s_bc, P.counters, 1u << P.b1, s_cst, s_bfill, s_bd);
+    W.units0 = W.units = 0;  // unused: get() reads the counts from s_cst
   } else {
     const uint32_t npc = P.npieces();  // <= 1024
     for (uint32_t i = threadIdx.x; i <= npc; i += NT) {
@@ -478,10 +565,14 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
   // unit descriptors live in a 3-slot shared ring: one thread computes unit i+2 during unit i's
   // phase 2 (slot (i+2) % 3 held unit i-1, whose fields were copied to registers already)
   __shared__ PassUnit<K> s_desc[3];
+  if (BC && MODE == 1 && threadIdx.x == 0) {
+    s_bc[0] = P.bc_rel[0];
+    s_bc[1] = P.bc_rel[1];
+  }
   const unsigned long long G = gridDim.x;
   if (threadIdx.x == NT - 1) {
-    W.get(P, blockIdx.x, s_desc[0], s_cst, s_pst);
-    W.get(P, blockIdx.x + G, s_desc[1], s_cst, s_pst);
+    W.get(P, blockIdx.x, s_desc[0], s_cst, s_pst, s_bfill, s_bd);
+    W.get(P, blockIdx.x + G, s_desc[1], s_cst, s_pst, s_bfill, s_bd);
   }
   __syncthreads();
   T* prev_dst = nullptr;  // unit i-1 awaiting write-out
@@ -575,12 +666,19 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
       if (d < F) {
         s_loc[d] = loc;
         s_cnt[d] = 0;
-        if (c) gd[d] = atomicAdd(s_desc[slot].cur + d, (unsigned long long)c) - loc;
+        if (c) {
+          if (BC) {
+            const int r = (int)s_desc[slot].rel;
+            gd[d] = bc_reserve<MODE>(&s_bc[r], &P.counters[(MODE == 1 ? CNT_BC_NB1 : CNT_BC_NB2) + r],
+                               &P.results[RES_BC_OVERFLOW], s_desc[slot].pbase + d, c) - loc;
+          }
+          else gd[d] = atomicAdd(s_desc[slot].cur + d, (unsigned long long)c) - loc;
+        }
         if (c > TILE / 4) atomicExch(&s_hot_next, d);  // predicts the next unit's hot digit (any one)
       }
     }
     if (threadIdx.x == NT - 1)  // publish unit i+2
-      W.get(P, u + 2 * G, s_desc[nslot == 2 ? 0 : nslot + 1], s_cst, s_pst);
+      W.get(P, u + 2 * G, s_desc[nslot == 2 ? 0 : nslot + 1], s_cst, s_pst, s_bfill, s_bd);
     write_out(s_gd + ((it + 1) & 1) * F);
     __syncthreads();
 

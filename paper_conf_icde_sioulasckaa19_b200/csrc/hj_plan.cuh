@@ -31,8 +31,37 @@ struct RelDev {
   uint32_t* cst;              // [npieces + 1] pass-2 chunk prefix (chunks of C2 tuples per piece)
 };
 
+// NEXT-1: the paper's histogram-free partitioner (§III-A). Each pass writes,
+// per output partition, a chain of fixed-capacity buckets taken from a pool with atomics; no
+// histogram is read and partitions are not contiguous (see hj_bucket.cuh).
+struct BcRel {
+  void* pool1;                // pass-1 buckets: bucket b holds tuples [b * bsz1, b * bsz1 + fill1[b])
+  void* pool2;                // pass-2 buckets
+  unsigned long long* st1;    // [2^b1] pass-1 partition state: j << 32 | fill, current bucket =
+                              //        p (j = 0, the partition's initial bucket) or np + j - 1
+  unsigned long long* st2;    // [2^B]  pass-2 partition state (index q = D << b2 | d2)
+  uint32_t* fill1;            // [nbmax1] tuples in each pass-1 bucket
+  uint32_t* part1;            // [nbmax1] pass-1 partition D of each overflow bucket (b >= np1)
+  uint32_t* fill2;            // [nbmax2]
+  uint32_t* part2;            // [nbmax2] co-partition q of each bucket
+  uint4* sl;                  // join slices {offset lo, offset hi, tuples, 0}, grouped by q
+  uint32_t* nsl;              // [2^B] join slices of each co-partition's closed buckets
+  uint32_t* sst;              // [2^B + 1] first slice of each co-partition
+  uint32_t* scur;             // [2^B] slice scatter cursors
+  uint32_t np1, np2;          // partitions per pass (2^b1, 2^B): buckets [0, np) are the initial ones
+  uint32_t cap1, cap2;        // bucket capacities: a bucket closes once fill >= cap
+  uint32_t nbmax1, nbmax2;    // pool sizes in buckets (proven bounds)
+  unsigned long long bsz1, bsz2;  // bucket stride in tuples = cap + tile (slack for the closing run)
+  uint32_t csl;               // join slice capacity: C_R (R) or C_S (S)
+};
+enum { CNT_BC_NB1 = 2, CNT_BC_NB2 = 4 };  // + relation: overflow buckets taken from the pool
+constexpr uint32_t BC_MAX_NB1 = 1542;  // per relation: <= 1.5 * 2^b1 + 1 pass-1 buckets (cap1 >= 2 x mean) + prefix end + spare
+enum { RES_BC_OVERFLOW = 3 };
+
 struct Plan {
   RelDev rel[2];  // 0 = R (build), 1 = S (probe)
+  int bc;         // 1: bucket-chain partitioner (NEXT-1), rel[r].t2 = bc[r].pool2
+  BcRel bc_rel[2];
   int B, b1, b2;  // local radix field
   int g;          // rank bits in the pass-1 digit (PLAN_SEND), else 0
   int nsrc;       // count rows / piece sources (PLAN_RECV: ranks), else 1
@@ -47,8 +76,8 @@ struct Plan {
   uint32_t C2;           // pass-2 chunk (tile) size in tuples
   uint32_t CR, CS;       // join item capacities: R tuples (smem build) and S tuples per item
   uint32_t* ist;         // [2^B + 1] join item prefix (q-order)
-  uint32_t* counters;    // [8]: 0 next join item, 1 planner blocks done, 2.. reserved
-  unsigned long long* results;  // [4]: 0 matches, 1 checksum, 2 output cursor, 3 unused
+  uint32_t* counters;    // [8]: 0 next join item, 1 planner blocks done, 2..7 bucket-chain counters
+  unsigned long long* results;  // [4]: 0 matches, 1 checksum, 2 output cursor, 3 bucket pool overflow
   void* out_r;           // materialized payloads of R (pay width), capacity out_cap
   void* out_s;
   unsigned long long out_cap;

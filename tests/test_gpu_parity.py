@@ -122,6 +122,100 @@ def test_knob_invariance_block_nested_loops(hj, cap_r, chunk_s):
     ctx.close()
 
 
+JOIN_SHAPES = 15  # number of k_join shapes in hj_api.cu (HJ_OPT_JOIN_VARIANT 1..15)
+
+
+@pytest.mark.parametrize("variant", range(1, JOIN_SHAPES + 1))
+def test_join_shape_invariance(hj, variant):
+    """Every selectable join-kernel shape (block size, tuples per thread, blocks/SM, R buffers,
+    hash-slot count, 16-bit heads) gives the oracle's result, on skewed and duplicate-heavy keys,
+    4- and 8-byte tuples."""
+    rng = np.random.default_rng(40 + variant)
+    for kb in (4, 8):
+        ctx = hj.Context(0, kb, kb)
+        ctx.set_option(hj.OPT_JOIN_VARIANT, variant)
+        dt = np.uint32 if kb == 4 else np.uint64
+        w = W.Workload("v", 30011, 50021, "zipf", keys="sparse" if kb == 4 else "k8", z=1.2, seed=400 + variant)
+        Rk, Rp, Sk, Sp = W.np_generate(w)
+        for bits in (-1, 2, 7):
+            check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True, ctx=ctx)
+        Rk = rng.integers(0, 700, 9000).astype(dt)
+        Sk = rng.integers(0, 700, 7000).astype(dt)
+        check_against_oracle(hj, Rk, np.arange(len(Rk), dtype=dt), Sk, np.arange(len(Sk), dtype=dt), bits=3,
+                             mat=True, ctx=ctx)
+        ctx.close()
+    with pytest.raises(Exception):
+        hj.Context(0, 4, 4).set_option(hj.OPT_JOIN_VARIANT, JOIN_SHAPES + 1)
+
+
+def _bc_ctx(hj, kb=4, **opts):
+    ctx = hj.Context(0, kb, kb)
+    ctx.set_option(hj.OPT_PARTITIONER, 1)
+    for k, v in opts.items():
+        ctx.set_option(getattr(hj, k), v)
+    return ctx
+
+
+@pytest.mark.parametrize("name", CASES)
+@pytest.mark.parametrize("bits", [-1, 0, 1, 5, 13])
+def test_bucket_chains_adversarial(hj, name, bits):
+    """NEXT-1 (HJ_OPT_PARTITIONER = 1, the paper's histogram-free bucket chains)
+    gives the oracle's result on the adversarial inputs."""
+    rng = np.random.default_rng(98)
+    Rk, Sk = adversarial(rng)[name]
+    Rp = rng.integers(0, 1 << 32, len(Rk), dtype=np.uint64).astype(np.uint32)
+    Sp = rng.integers(0, 1 << 32, len(Sk), dtype=np.uint64).astype(np.uint32)
+    ctx = _bc_ctx(hj)
+    check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True, ctx=ctx)
+    ctx.close()
+
+
+@pytest.mark.parametrize("cfg", [
+    dict(nR=1 << 18, nS=1 << 20, dist="fk", keys="sparse", bits=2),   # pass-1 buckets close many times
+    dict(nR=1 << 16, nS=1 << 20, dist="zipf", z=1.5, keys="sparse", bits=8),  # a hot co-partition: long pass-2 chains
+    dict(nR=100_003, nS=300_007, dist="zipf_build", z=1.0, keys="dense", bits=6),
+    dict(nR=1 << 15, nS=1 << 15, dist="replicas", rep=4, keys="dense", bits=4),
+    dict(nR=70_001, nS=90_001, dist="fk", keys="k8", bits=7),
+    dict(nR=1 << 17, nS=1 << 17, dist="1to1", keys="dense", bits=-1),
+])
+def test_bucket_chains_generated(hj, cfg):
+    cfg = dict(cfg)
+    bits = cfg.pop("bits")
+    w = W.Workload("bc", seed=500 + cfg["nR"] % 97, **cfg)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    ctx = _bc_ctx(hj, w.key_bytes)
+    check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True, ctx=ctx)
+    ctx.close()
+
+
+@pytest.mark.parametrize("cap_r,chunk_s", [(7, 0), (100, 33), (4096, 5)])
+def test_bucket_chains_slices(hj, cap_r, chunk_s):
+    """Tiny C_R / C_S cut the final buckets into many join slices (block nested loops)."""
+    rng = np.random.default_rng(6)
+    Rk = rng.integers(0, 3000, 20000).astype(np.uint32)
+    Sk = rng.integers(0, 3000, 15000).astype(np.uint32)
+    ctx = _bc_ctx(hj, OPT_CAP_R=cap_r, OPT_CHUNK_S=chunk_s, OPT_OUT_CAPACITY=1000)
+    for bits in (0, 4, 9):
+        check_against_oracle(hj, Rk, np.arange(len(Rk), dtype=np.uint32), Sk, np.arange(len(Sk), dtype=np.uint32),
+                             bits=bits, mat=True, ctx=ctx)
+    ctx.close()
+
+
+def test_bucket_chains_equal_histogram_path_and_repeat(hj):
+    """Same ctx, alternating partitioners and repeated calls: identical results (no state leaks
+    between calls through the pools or the zeroed metadata)."""
+    w = W.Workload("bc2", 1 << 19, 1 << 21, "zipf", z=1.0, keys="sparse", seed=510)
+    cols = [dev(a) for a in W.np_generate(w)]
+    ctx = hj.Context(0, 4, 4)
+    ref = oracle.hash_join(*W.np_generate(w))
+    for part in (1, 0, 1, 1):
+        ctx.set_option(hj.OPT_PARTITIONER, part)
+        r = ctx.join(*cols)
+        torch.cuda.synchronize()
+        assert (r.matches, r.checksum) == ref, part
+    ctx.close()
+
+
 def test_materialize_overflow_regrows(hj):
     """More matches than the initial capacity: grow and re-run the join phase (reading S11)."""
     ctx = hj.Context(0, 4, 4)
