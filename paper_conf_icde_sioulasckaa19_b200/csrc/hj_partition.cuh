@@ -160,7 +160,10 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P, uint32_t blocks_r) {
 // pieces.
 // ------------------------------------------------------------------------------------------
 __device__ __forceinline__ unsigned long long plan_items(const Plan& P, unsigned long long cr, unsigned long long cs) {
-  return (cr && cs) ? ((cr + P.CR - 1) / P.CR) * ((cs + P.CS - 1) / P.CS) : 0ull;
+  if (!cr || !cs) return 0ull;
+  if (((cr | cs) >> 31) == 0)  // 32-bit division (a 64-bit one is ~10x the instructions)
+    return (unsigned long long)(((uint32_t)cr + P.CR - 1) / P.CR) * (((uint32_t)cs + P.CS - 1) / P.CS);
+  return ((cr + P.CR - 1) / P.CR) * ((cs + P.CS - 1) / P.CS);
 }
 
 __device__ __forceinline__ unsigned long long plan_count(const RelDev& R, int nsrc, uint32_t np, uint32_t q) {
@@ -180,13 +183,22 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   const bool items = P.mode != PLAN_SEND;
   // ---- prefix of everything below this block's range -------------------------------------
   unsigned long long sR = 0, sS = 0, sI = 0;
-  #pragma unroll 8
-  for (uint32_t k = 0; k < b; ++k) {
-    const unsigned long long cr = plan_count(P.rel[0], nsrc, np, k * NT + threadIdx.x);
-    const unsigned long long cs = plan_count(P.rel[1], nsrc, np, k * NT + threadIdx.x);
-    sR += cr;
-    sS += cs;
-    if (items) sI += plan_items(P, cr, cs);
+  // batches of 8 earlier blocks: all 16 count loads are issued before any is used (the loop is
+  // latency-bound: one L2 round trip per batch instead of per block)
+  for (uint32_t k0 = 0; k0 < b; k0 += 8) {
+    unsigned long long cr[8], cs[8];
+    #pragma unroll
+    for (int u = 0; u < 8; ++u) {
+      const bool ok = k0 + u < b;
+      cr[u] = ok ? plan_count(P.rel[0], nsrc, np, (k0 + u) * NT + threadIdx.x) : 0ull;
+      cs[u] = ok ? plan_count(P.rel[1], nsrc, np, (k0 + u) * NT + threadIdx.x) : 0ull;
+    }
+    #pragma unroll
+    for (int u = 0; u < 8; ++u) {
+      sR += cr[u];
+      sS += cs[u];
+      if (items) sI += plan_items(P, cr[u], cs[u]);
+    }
   }
   unsigned long long tot;
   block_exclusive_scan64<NT>(sR, s_tmp, &tot);
