@@ -81,6 +81,16 @@ enum hj_option {
                                device memory (bucket slack); ms_kernel[0..1] are 0 and
                                ms_kernel[2..3] include each pass's bucket bookkeeping. Ignored by
                                hj_join_host / hj_partition / the exchange calls and by graph mode */
+  HJ_OPT_FUSE = 13,         /* hj_join: 1 = pass 2 and the join run as ONE persistent kernel that
+                               joins each pass-1 partition's co-partitions while they are still in
+                               L2 (opt-in: measured slower than separate kernels on c3, DESIGN.md
+                               §5; needs radix_bits >= 2, the histogram partitioner and join
+                               algorithm 0, else ignored); 0 = separate pass-2 and join kernels
+                               (default). ms_kernel[3] is then the fused kernel, ms_kernel[4] 0  */
+  HJ_OPT_FUSE_WINDOW_MB = 14, /* fused: MB of pass-2 output allowed ahead of the join (0 = no
+                               throttle; default 32)                                            */
+  HJ_OPT_FUSE_PASS_SLOTS = 15, /* fused: blocks per SM that start in the pass-2 role (default 1 of
+                               2; the others join; pass-2 blocks join once pass 2 is done)      */
   HJ_OPT_STREAM_CHUNK = 8   /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
                                least 2^22; >= |S| = copy everything, then join)                   */
 };
@@ -102,6 +112,7 @@ typedef struct hj_result {
   float ms_kernel[5];    /* per step, CUDA events on the ctx stream: 0 histogram, 1 planner,
                             2 pass 1, 3 pass 2, 4 join (HJ_OPT_TIMING = 1)                       */
   uint32_t kernels;      /* kernels this call launched                                           */
+  uint32_t fused;        /* 1: pass 2 and the join ran fused (HJ_OPT_FUSE); ms_kernel[3] covers both */
 } hj_result;
 
 /* Create a context on CUDA device `device` for key/payload widths 4/4 or 8/8 bytes.

@@ -41,6 +41,9 @@ OPT_JOIN_ALGO = 9
 OPT_PASS1_BASES = 10
 OPT_GRAPH = 11
 OPT_PARTITIONER = 12  # 0 = histogram (default), 1 = bucket chains (NEXT-1)
+OPT_FUSE = 13  # 1 = pass 2 + join in one L2-resident kernel (opt-in), 0 = separate kernels (default)
+OPT_FUSE_WINDOW_MB = 14
+OPT_FUSE_PASS_SLOTS = 15
 ALGO_HASH, ALGO_NLJ, ALGO_NONPARTITIONED = 0, 1, 2
 
 _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4: "HJ_ERR_CUDA", -5: "HJ_ERR_COMM"}
@@ -60,7 +63,8 @@ class _Result(ctypes.Structure):
     _fields_ = [("matches", ctypes.c_uint64), ("checksum", ctypes.c_uint64), ("r_pay_out", ctypes.c_void_p),
                 ("s_pay_out", ctypes.c_void_p), ("n_items", ctypes.c_uint64), ("radix_bits", ctypes.c_int),
                 ("passes", ctypes.c_int), ("ms_total", ctypes.c_float), ("ms_partition", ctypes.c_float),
-                ("ms_join", ctypes.c_float), ("ms_kernel", ctypes.c_float * 5), ("kernels", ctypes.c_uint32)]
+                ("ms_join", ctypes.c_float), ("ms_kernel", ctypes.c_float * 5), ("kernels", ctypes.c_uint32),
+                ("fused", ctypes.c_uint32)]
 
 
 def _load_lib():
@@ -119,6 +123,7 @@ class JoinResult:
     ms_join: float = 0.0
     ms_kernel: tuple = ()
     kernels: int = 0
+    fused: bool = False  # pass 2 + join ran as one kernel: ms_kernel[3] covers both, ms_kernel[4] = 0
 
 
 class Context:
@@ -268,7 +273,7 @@ def _result(res: _Result) -> JoinResult:
     return JoinResult(matches=int(res.matches), checksum=int(res.checksum), n_items=int(res.n_items),
                       radix_bits=res.radix_bits, passes=res.passes, ms_total=res.ms_total,
                       ms_partition=res.ms_partition, ms_join=res.ms_join,
-                      ms_kernel=tuple(res.ms_kernel), kernels=int(res.kernels))
+                      ms_kernel=tuple(res.ms_kernel), kernels=int(res.kernels), fused=bool(res.fused))
 
 
 def _as_device_col(t, width: int):

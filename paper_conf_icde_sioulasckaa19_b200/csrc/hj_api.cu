@@ -10,6 +10,7 @@
 #include <string>
 
 #include "../../include/hj.h"
+#include "hj_fused.cuh"
 #include "hj_join.cuh"
 #include "hj_partition.cuh"
 #include "hj_variants.cuh"
@@ -56,7 +57,7 @@ struct Ctx {
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
           opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0, opt_graph = 0,
-          opt_partitioner = 0;
+          opt_partitioner = 0, opt_fuse = 0, opt_fuse_window_mb = 32, opt_fuse_pass_slots = 1;
   DevBuf bc_pool1[2], bc_pool2[2], bc_meta;  // HJ_OPT_PARTITIONER = 1 (NEXT-1 bucket chains)
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2], np_heads, np_next;
@@ -123,6 +124,9 @@ struct HostPlan {
   size_t o_cnt[2], o_off[2], o_cur1[2], o_cur2[2], o_pst[2], o_cst[2], o_ist, o_counters, o_results;
   size_t o_cntb = 0, o_relb = 0;  // pass-1 per-block digit counts / bases
   bool bases = false;             // pass 1 = k_pass1b (per-block bases, TMA bulk write-out)
+  bool fused = false;             // pass 2 + join = k_fused (HJ_OPT_FUSE)
+  size_t o_fz = 0;
+  size_t pass2_smem = 0;
   uint32_t g1max = 0;
   size_t zero_bytes = 0;  // [0, zero_bytes) is memset to 0 per call
   size_t meta_bytes = 0;
@@ -157,7 +161,7 @@ int choose_bits(unsigned long long nR) {
 // mode PLAN_FULL: one GPU; PLAN_SEND: exchange sender (g rank bits); PLAN_RECV: exchange
 // receiver (nsrc count rows). nR / nS are the tuples this GPU partitions / joins.
 int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat, int g = 0,
-              int nsrc = 1, int mode = PLAN_FULL) {
+              int nsrc = 1, int mode = PLAN_FULL, bool want_fused = false) {
   const size_t tb = (size_t)c->key_bytes + c->pay_bytes;  // AoS tuple bytes
   hp.B = radix_bits < 0 ? choose_bits(nR) : radix_bits;
   if (hp.B > 20) return fail(c, HJ_ERR_UNSUPPORTED, "radix_bits %d > 20", hp.B);
@@ -174,6 +178,9 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   // 1024-thread block. The pass-2 chunk is that kernel's tile.
   hp.tile = pass_threads(c, hp.pb(), items) * items;
   hp.C2 = (uint32_t)(pass_threads(c, hp.b2, items) * items);
+  // fused pass 2 + join (one GPU, two passes, the smem hash join): 512-thread pass-2 units
+  hp.fused = want_fused && mode == PLAN_FULL && hp.B >= 2 && c->opt_join_algo == 0 && c->opt_partitioner == 0;
+  if (hp.fused) hp.C2 = (uint32_t)(FZ_NT * items);
 
   // join capacities
   const unsigned long long mean = (nR + (1ull << hp.B) - 1) >> hp.B;
@@ -185,14 +192,16 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   uint32_t CS;
   if (c->opt_chunk_s > 0) CS = (uint32_t)std::min<int64_t>(c->opt_chunk_s, 1ll << 30);
   else CS = std::max<uint32_t>(8 * CR, 32768);
-  const int rbuf = JOIN_SHAPES[join_variant(c)].rbuf;
-  const int nbsh = JOIN_SHAPES[join_variant(c)].nbsh;
-  const size_t head_bytes = JOIN_SHAPES[join_variant(c)].h16 ? 2 : 4;
+  const int rbuf = hp.fused ? 1 : JOIN_SHAPES[join_variant(c)].rbuf;
+  const int nbsh = hp.fused ? 1 : JOIN_SHAPES[join_variant(c)].nbsh;
+  const size_t head_bytes = !hp.fused && JOIN_SHAPES[join_variant(c)].h16 ? 2 : 4;
   int lg_nb = std::max(6, ilog2_ceil(CR) - nbsh);
   auto join_smem = [&](uint32_t cr, int lg) {  // R tile buffer(s) (TMA) + heads + next
     return (size_t)rbuf * ((cr + 3) & ~1u) * tb + (head_bytes << lg) + (size_t)cr * 2;
   };
-  while (join_smem(CR, lg_nb) > cap_max_smem - 8 * 1024 && CR > 256) {
+  // fused: two blocks per SM, each with the pass-2 statics (~25 KB) beside the dynamic region
+  const size_t join_cap = hp.fused ? (cap_max_smem / 2 - 28 * 1024) : cap_max_smem - 8 * 1024;
+  while (join_smem(CR, lg_nb) > join_cap && CR > 256) {
     CR /= 2;
     lg_nb = std::max(6, ilog2_ceil(CR) - nbsh);
   }
@@ -200,6 +209,7 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   hp.CS = CS;
   hp.lg_nb = lg_nb;
   hp.join_smem = join_smem(CR, lg_nb);
+  hp.pass2_smem = (size_t)hp.C2 * tb + ((size_t)1 << hp.b2) * 24 + 16;
 
   // metadata layout
   const size_t nq = (size_t)1 << hp.qbits(), F1 = (size_t)1 << hp.pb(), npc = hp.npieces();
@@ -213,6 +223,7 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   hp.o_counters = take(64);
   hp.o_results = take(64);
   for (int r = 0; r < 2; ++r) hp.o_cnt[r] = take(mode == PLAN_RECV ? 0 : nq * 4);
+  if (hp.fused) hp.o_fz = take((size_t)FZ_WORDS * 4);
   hp.zero_bytes = o;
   for (int r = 0; r < 2; ++r) {
     hp.o_off[r] = take((nq + 1) * 8);
@@ -273,6 +284,8 @@ int set_kernel_attrs(Ctx* c) {
   attr((const void*)k_pass<K, 1, 512, pass_items<K>(), false, true>);
   attr((const void*)k_pass<K, 2, 1024, pass_items<K>(), false, true>);
   attr((const void*)k_pass<K, 2, 512, pass_items<K>(), false, true>);
+  attr((const void*)k_fused<K, false>);
+  attr((const void*)k_fused<K, true>);
   attr_join<K, 0>(attr);
   attr_join<K, 1>(attr);
   attr_join<K, 2>(attr);
@@ -341,6 +354,14 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   }
   P.counters = (uint32_t*)(m + hp.o_counters);
   P.results = (unsigned long long*)(m + hp.o_results);
+  if (hp.fused) {
+    P.fz = (uint32_t*)(m + hp.o_fz);
+    P.fz_pass_slots = (uint32_t)std::max<int64_t>(c->opt_fuse_pass_slots, 0);
+    // window: pass-1 partitions of pass-2 output (R + S) allowed ahead of the join
+    const double part_bytes = (double)(nR + nS) * (c->key_bytes + c->pay_bytes) / (double)(1u << hp.b1);
+    P.fz_window = c->opt_fuse_window_mb <= 0 ? 0u
+                  : (uint32_t)std::max(1.0, std::floor((double)c->opt_fuse_window_mb * 1048576.0 / std::max(part_bytes, 1.0)));
+  }
   P.out_r = c->out_r.p;
   P.out_s = c->out_s.p;
   P.out_cap = c->out_r.bytes / c->pay_bytes;
@@ -524,9 +545,9 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   return HJ_OK;
 }
 
-int prepare(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat, int g = 0,
+int prepare(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat, bool want_fused, int g = 0,
             int nsrc = 1, int mode = PLAN_FULL) {
-  int rc = make_plan(c, hp, nR, nS, radix_bits, mat, g, nsrc, mode);
+  int rc = make_plan(c, hp, nR, nS, radix_bits, mat, g, nsrc, mode, want_fused);
   if (rc) return rc;
   const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
   const unsigned long long ns[2] = {nR, nS};
@@ -545,23 +566,53 @@ int prepare(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, 
   return HJ_OK;
 }
 
-// Join phase + result readback shared by hj_join and hj_join_received.
-int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res) {
+// a4-a8 in one persistent kernel (hj_fused.cuh): a full wave of 512-thread blocks (two per SM).
+// Events 4 and 5 (ms_kernel[3] = the fused kernel, ms_kernel[4] = 0).
+template <typename K>
+int launch_fused(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
+  const size_t sm = std::max(hp.join_smem, hp.pass2_smem);
+  const void* f = mat ? (const void*)k_fused<K, true> : (const void*)k_fused<K, false>;
+  int per_sm = 0;
+  CUDA_TRY(c, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, f, FZ_NT, sm));
+  if (per_sm < 1) return fail(c, HJ_ERR_UNSUPPORTED, "fused kernel does not fit an SM (%zu B smem)", sm);
+  const int g = per_sm * c->num_sms;
+  Plan Q = P;
+  // the throttle waits on join-role blocks: none exist when every slot of an SM runs pass 2
+  if (std::max<uint32_t>(Q.fz_pass_slots, 1) >= (uint32_t)per_sm) Q.fz_window = 0;
+  if (mat) k_fused<K, true><<<g, FZ_NT, sm, c->stream>>>(Q);
+  else k_fused<K, false><<<g, FZ_NT, sm, c->stream>>>(Q);
+  CUDA_TRY(c, cudaGetLastError());
+  c->launches += 1;
+  mark(c, 4);
+  mark(c, 5);
+  return HJ_OK;
+}
+
+constexpr int HJ_RERUN = 1;  // finish_join: fused materialization overflowed; output grown, re-run
+
+// Join phase + result readback shared by hj_join and hj_join_received. `joined`: the join
+// already ran inside the fused kernel.
+int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res, bool joined = false) {
   cudaStream_t st = c->stream;
   const bool timing = c->opt_timing != 0;
-  int rc = c->key_bytes == 4 ? launch_join<uint32_t>(c, hp, P, mat) : launch_join<uint64_t>(c, hp, P, mat);
+  int rc = joined ? HJ_OK : c->key_bytes == 4 ? launch_join<uint32_t>(c, hp, P, mat) : launch_join<uint64_t>(c, hp, P, mat);
   if (rc) return rc;
   unsigned long long* h = (unsigned long long*)c->h_res;
   CUDA_TRY(c, cudaMemcpyAsync(h, P.results, 4 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st));
   CUDA_TRY(c, cudaMemcpyAsync(h + 4, P.ist + (1ull << hp.B), sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
+  h[5] = 0;
+  if (joined) CUDA_TRY(c, cudaMemcpyAsync(h + 5, P.fz + FZ_ERR, sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
   if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[6], st));
   CUDA_TRY(c, cudaStreamSynchronize(st));
   if (P.bc && h[RES_BC_OVERFLOW]) return fail(c, HJ_ERR_CUDA, "bucket pool overflow (pool bound violated)");
+  if (joined && (uint32_t)h[5]) return fail(c, HJ_ERR_CUDA, "fused kernel watchdog: wait site %u timed out", (uint32_t)h[5]);
   unsigned long long matches = h[RES_MATCHES];
   if (mat && matches > P.out_cap) {
     // materialization overflow (reading S11): grow to the exact size and re-run only the join
     if ((rc = ensure(c, c->out_r, matches * c->pay_bytes))) return rc;
     if ((rc = ensure(c, c->out_s, matches * c->pay_bytes))) return rc;
+    // the fused kernel discarded T2's lines: the caller re-runs the whole call unfused
+    if (joined) return HJ_RERUN;
     P.out_r = c->out_r.p;
     P.out_s = c->out_s.p;
     P.out_cap = matches;
@@ -856,7 +907,7 @@ int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, cons
     return c->key_bytes == 4 ? run_join_bc<uint32_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, mat, res)
                              : run_join_bc<uint64_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, mat, res);
   HostPlan hp;
-  int rc = prepare(c, hp, nR, nS, radix_bits, mat);
+  int rc = prepare(c, hp, nR, nS, radix_bits, mat, c->opt_fuse && !c->opt_graph);
   if (rc) return rc;
   Plan P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
   if (c->opt_graph) {
@@ -869,6 +920,19 @@ int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, cons
   }
   c->launches = 0;
   if ((rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P))) return rc;
+  if (hp.fused) {
+    if ((rc = c->key_bytes == 4 ? launch_fused<uint32_t>(c, hp, P, mat) : launch_fused<uint64_t>(c, hp, P, mat))) return rc;
+    rc = finish_join(c, hp, P, mat, res, true);
+    if (rc == HJ_RERUN) {  // rare: materialization overflow (exact size now allocated)
+      const int64_t f = c->opt_fuse;
+      c->opt_fuse = 0;
+      rc = run_join(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
+      c->opt_fuse = f;
+    } else if (!rc) {
+      res->fused = 1;
+    }
+    return rc;
+  }
   if ((rc = c->key_bytes == 4 ? launch_pass2<uint32_t>(c, hp, P) : launch_pass2<uint64_t>(c, hp, P))) return rc;
   return finish_join(c, hp, P, mat, res);
 }
@@ -915,7 +979,7 @@ int join_host_stream(Ctx* c, const void* Rk, const void* Rp, uint64_t nR, const 
               ev_free[2] = {c->sev[4], c->sev[5]}, ev_j[2] = {c->sev[6], c->sev[7]}, ev_d = c->sev[8],
               ev_end = c->sev[9];
   HostPlan hp;
-  int rc = prepare(c, hp, nR, chunk, radix_bits, mat);
+  int rc = prepare(c, hp, nR, chunk, radix_bits, mat, false);
   if (rc) return rc;
   const unsigned long long cap = c->opt_out_cap > 0 ? (unsigned long long)c->opt_out_cap : std::max<unsigned long long>(nS, 1 << 20);
   if (mat) {
@@ -1148,6 +1212,9 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_BLOCKS_PER_SM: c->opt_bps = v; break;
     case HJ_OPT_STREAM_CHUNK: c->opt_stream_chunk = v; break;
     case HJ_OPT_PASS1_BASES: c->opt_pass1_bases = v; break;
+    case HJ_OPT_FUSE: c->opt_fuse = v; break;
+    case HJ_OPT_FUSE_WINDOW_MB: c->opt_fuse_window_mb = v; break;
+    case HJ_OPT_FUSE_PASS_SLOTS: c->opt_fuse_pass_slots = v; break;
     case HJ_OPT_PARTITIONER:
       if (v > 1) return fail(c, HJ_ERR_INVALID, "partitioner must be 0 (histogram) or 1 (bucket chains)");
       c->opt_partitioner = v;
@@ -1226,7 +1293,7 @@ int hj_partition(hj_ctx* h, const void* keys, const void* pays, uint64_t n, int 
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
   HostPlan hp;
-  int rc = prepare(c, hp, n, 0, radix_bits, false);
+  int rc = prepare(c, hp, n, 0, radix_bits, false, false);
   if (rc == HJ_OK) {
     Plan P = device_plan(c, hp, keys, pays, n, nullptr, nullptr, 0);
     c->launches = 0;
@@ -1267,7 +1334,7 @@ int hj_exchange_pack(hj_ctx* h, int rel, const void* keys, const void* pays, uin
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
   HostPlan hp;
-  int rc = prepare(c, hp, n, 0, local_bits, false, gpu_bits, 1, PLAN_SEND);
+  int rc = prepare(c, hp, n, 0, local_bits, false, false, gpu_bits, 1, PLAN_SEND);
   const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
   const size_t nq = (size_t)1 << hp.qbits();
   if (rc == HJ_OK) rc = ensure(c, c->xsend[rel], n * tb + 16);
@@ -1315,7 +1382,7 @@ int hj_join_received(hj_ctx* h, const void* R_recv, uint64_t nR, const uint32_t*
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
   HostPlan hp;
-  int rc = prepare(c, hp, nR, nS, local_bits, mat, 0, nsrc, PLAN_RECV);
+  int rc = prepare(c, hp, nR, nS, local_bits, mat, false, 0, nsrc, PLAN_RECV);
   if (rc == HJ_OK) {
     Plan P = device_plan(c, hp, nullptr, nullptr, nR, nullptr, nullptr, nS);
     P.rel[0].t1 = const_cast<void*>(R_recv);

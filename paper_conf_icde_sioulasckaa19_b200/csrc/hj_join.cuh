@@ -27,9 +27,10 @@ struct JoinJob {
   unsigned long long rb, sb, se;
 };
 
+
 // Claim the next work item and decode it (item -> co-partition q by binary search over the
 // planner's item prefix; then the R chunk and S chunk of q it covers). One lane.
-template <typename T>
+template <typename T, bool FUSE = false>
 __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items) {
   JoinJob j;
   j.item = atomicAdd(&P.counters[CNT_NEXT_ITEM], 1u);
@@ -66,6 +67,13 @@ __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items
     j.se = j.sb + min((unsigned long long)P.CS, sn - sc * P.CS);
     const uintptr_t a = reinterpret_cast<uintptr_t>((const T*)P.rel[0].t2 + j.rb);
     j.shift = (uint32_t)((a & 15) / sizeof(T));  // tuples between the 16 B aligned copy start and rb
+    if (FUSE) {
+      // wait until pass 2 has written (and signalled) every unit of q's pass-1 partition
+      const uint32_t d = q >> P.b2;
+      const uint32_t need = (P.rel[0].cst[d + 1] - P.rel[0].cst[d] + P.rel[1].cst[d + 1] - P.rel[1].cst[d]) * FZ_PASS_WARPS;
+      wait_geq(&P.fz[FZ_DONE + d], need, &P.fz[FZ_ERR], 1u);
+      fence_proxy_async_global();  // the R chunk is read by the TMA (async proxy)
+    }
   }
   return j;
 }
@@ -114,8 +122,13 @@ __device__ __forceinline__ uint32_t exch16(unsigned short* a, uint32_t v) {
 }
 
 // H16: 16-bit chain heads (half the head array -> one more block per SM fits in shared memory)
-template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false>
-__global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
+// FUSE (join role of the fused pass-2 + join kernel, hj_fused.cuh): an item waits for its
+// pass-1 partition's pass-2 signals (claim_job); S tuples are read L2-only (ld.global.cg: the
+// co-partitions were just written by other SMs); the pairs are streamed out with evict-first
+// stores; after the item every compute warp bumps the completed-item counter that throttles
+// pass 2.
+template <typename K, int NT, int SPT, bool MAT, int RBUF, bool H16 = false, bool FUSE = false>
+__device__ __forceinline__ void join_body(const Plan& P) {
   using TT = Tup<K>;
   using T = typename TT::T;
   extern __shared__ __align__(16) unsigned char s_raw[];
@@ -144,7 +157,7 @@ __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
     mbar_init(&s_bar[0], 1);
     mbar_init(&s_bar[1], 1);
     fence_mbar_init();
-    JoinJob j = claim_job<T>(P, total_items);
+    JoinJob j = claim_job<T, FUSE>(P, total_items);
     if (j.item < total_items) issue_r_copy<T>(P, j, s_rtb, &s_bar[0]);
     s_jobs[0] = j;
   }
@@ -156,7 +169,7 @@ __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
     if (sched) {
       JoinJob j;
       if (lane == 0) {
-        j = claim_job<T>(P, total_items);
+        j = claim_job<T, FUSE>(P, total_items);
         if (RBUF == 2 && j.item < total_items) issue_r_copy<T>(P, j, s_rtb + ((it + 1) & 1) * cap, &s_bar[(it + 1) & 1]);
         s_jobs[(it + 1) & 1] = j;
       }
@@ -172,7 +185,7 @@ __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
       for (int j = 0; j < SPT; ++j) {
         const unsigned long long s = base + (unsigned long long)j * NT + threadIdx.x;
         if (s < job.se) {
-          const T t = __ldcs(ssrc + s);
+          const T t = FUSE ? __ldcg(ssrc + s) : __ldcs(ssrc + s);
           sk[j] = TT::key(t);
           sp[j] = TT::pay(t);
         }
@@ -263,8 +276,13 @@ __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
           pos0 += wtot;
           if (m[j] == 1) {
             if (pos < P.out_cap) {
-              out_r[pos] = rfirst[j];
-              out_s[pos] = sp[j];
+              if (FUSE) {
+                __stcs(out_r + pos, rfirst[j]);
+                __stcs(out_s + pos, sp[j]);
+              } else {
+                out_r[pos] = rfirst[j];
+                out_s[pos] = sp[j];
+              }
             }
           } else if (m[j] > 1) {
             for (uint32_t i = s_head[slot_of(sk[j], H)]; i != NIL16; i = s_next[i]) {
@@ -282,6 +300,9 @@ __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
         bar_compute(NT);  // s_base / s_wsum are reused by the next round
       }
     }
+    // FUSE: this warp is done with the item (counted per warp, before the end-of-item barrier:
+    // the scheduler may be waiting on pass 2 for the next item, and pass 2 on this count)
+    if (FUSE && lane == 0) red_add_gpu(&P.fz[FZ_JCOMP], 1u);
     bar_item(NT + 32);  // end of item: the tile buffer and s_head are reused, s_jobs[it+1] is ready
   }
 
@@ -307,6 +328,11 @@ __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
       atomicAdd(&P.results[RES_CHECKSUM], h);
     }
   }
+}
+
+template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false>
+__global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
+  join_body<K, NT, SPT, MAT, RBUF, H16, false>(P);
 }
 
 }  // namespace hj

@@ -332,12 +332,13 @@ struct __align__(16) PassUnit {
   uint32_t valid;
   uint32_t rel;    // bucket chains (BC): relation and first partition index of the unit's digits
   uint32_t pbase;
+  uint32_t grp;    // fused pass 2 (FUSE): the pass-1 partition (piece) of the unit
 };
 
 // Unit u (round-robin: u = blockIdx.x + k * gridDim.x) -> its descriptor. MODE 2 maps the chunk
 // to its piece by binary search in the shared-memory chunk prefix (stateless: no registers live
 // across the unit loop).
-template <typename K, int MODE, int TILE, bool BC = false>
+template <typename K, int MODE, int TILE, bool BC = false, bool FUSE = false>
 struct UnitWalker {
   unsigned long long units0, units;
   __device__ __forceinline__ bool get(const Plan& P, unsigned long long u, PassUnit<K>& U, const uint32_t* s_cst,
@@ -348,6 +349,32 @@ struct UnitWalker {
     // no registers live across k_pass's tile loop
     const unsigned long long n0 = (BC && MODE == 2) ? s_cst[2 * BC_MAX_NB1 - 3] : units0;
     const unsigned long long nn = (BC && MODE == 2) ? s_cst[2 * BC_MAX_NB1 - 4] : units;
+    if (FUSE) {  // pass-1 partition major: R chunks of piece i, then S chunks of piece i, then i + 1
+      const uint32_t npc = P.npieces();
+      const uint32_t* cR = s_cst;
+      const uint32_t* cS = s_cst + 1025;
+      U.valid = u < (unsigned long long)(cR[npc] + cS[npc]);
+      if (!U.valid) return false;
+      const uint32_t uc = (uint32_t)u;
+      uint32_t lo = 0, hi = npc;  // largest piece with cR + cS <= uc
+      while (hi - lo > 1) {
+        const uint32_t mid = (lo + hi) >> 1;
+        if (cR[mid] + cS[mid] <= uc) lo = mid; else hi = mid;
+      }
+      const uint32_t k = uc - (cR[lo] + cS[lo]), nr = cR[lo + 1] - cR[lo];
+      const int r = k < nr ? 0 : 1;
+      const RelDev& R = P.rel[r];
+      const unsigned long long s0 = s_pst[r * 1025 + lo] + (unsigned long long)(r ? k - nr : k) * TILE;
+      U.rel = r;
+      U.pbase = 0;
+      U.grp = lo;
+      U.src_k = (const T*)R.t1 + s0;
+      U.src_p = nullptr;
+      U.dst = R.t2;
+      U.cur = R.cur2 + ((unsigned long long)lo << P.b2);
+      U.len = (uint32_t)min((unsigned long long)TILE, s_pst[r * 1025 + lo + 1] - s0);
+      return true;
+    }
     U.valid = u < nn;
     if (!U.valid) return false;
     const int r = (u < n0) ? 0 : 1;
@@ -355,6 +382,7 @@ struct UnitWalker {
     const RelDev& R = P.rel[r];
     U.rel = r;
     U.pbase = 0;
+    U.grp = 0;
     if (BC) {  // bucket chains: pass 1 as below into the pass-1 pool; pass 2 = one bucket unit
       const BcRel& Bc = P.bc_rel[r];
       if (MODE == 1) {
@@ -513,8 +541,15 @@ __device__ __noinline__ void bc_pass2_units(const BcRel* s_bc, const uint32_t* c
   }
 }
 
-template <typename K, int MODE, int NT, int ITEMS, bool GD, bool BC = false>
-__global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits) {
+// FUSE (pass 2 inside the fused pass-2 + join kernel, hj_fused.cuh): units are claimed from a
+// global counter in pass-1-partition order (R then S chunks of each piece); each warp signals
+// the completion of its part of a unit's write-out (fence.acq_rel.gpu + red on the piece's
+// counter, issued one iteration later, when the stores have long been acknowledged); T2 stores
+// are plain write-back stores so the co-partitions stay in L2 for the join; a unit more than
+// fz_window pieces ahead of the join's completed items waits (bounds the L2 footprint).
+template <typename K, int MODE, int NT, int ITEMS, bool GD, bool BC = false, bool FUSE = false>
+__device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
+  static_assert(!FUSE || (MODE == 2 && !BC && !GD), "fused pass 2 only");
   using TT = Tup<K>;
   using T = typename TT::T;
   constexpr int TILE = NT * ITEMS;
@@ -549,7 +584,7 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
 
   if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
   if (threadIdx.x == 0) s_hot = s_hot_next = 0xffffffffu;
-  UnitWalker<K, MODE, TILE, BC> W;
+  UnitWalker<K, MODE, TILE, BC, FUSE> W;
   if (MODE == 1) {
     W.units0 = P.tiles1[0];
     W.units = W.units0 + P.tiles1[1];
@@ -583,12 +618,27 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
   }
   const unsigned long long G = gridDim.x;
   if (threadIdx.x == NT - 1) {
-    W.get(P, blockIdx.x, s_desc[0], s_cst, s_pst, s_bfill, s_bd);
-    W.get(P, blockIdx.x + G, s_desc[1], s_cst, s_pst, s_bfill, s_bd);
+    if (FUSE) {
+      W.get(P, atomicAdd(&P.fz[FZ_UNIT], 1u), s_desc[0], s_cst, s_pst, s_bfill, s_bd);
+      W.get(P, atomicAdd(&P.fz[FZ_UNIT], 1u), s_desc[1], s_cst, s_pst, s_bfill, s_bd);
+    } else {
+      W.get(P, blockIdx.x, s_desc[0], s_cst, s_pst, s_bfill, s_bd);
+      W.get(P, blockIdx.x + G, s_desc[1], s_cst, s_pst, s_bfill, s_bd);
+    }
   }
   __syncthreads();
   T* prev_dst = nullptr;  // unit i-1 awaiting write-out
   uint32_t prev_len = 0;
+  uint32_t prev_grp = 0, sig_grp = 0;  // FUSE: piece of unit i-1; piece of the unit written out last iteration
+  bool sig = false;
+  // FUSE: this warp's part of the write-out issued last iteration is complete -> signal its piece
+  auto signal = [&](uint32_t grp) {
+    __syncwarp();
+    if (lane == 0) {
+      fence_acq_rel_gpu();
+      red_add_gpu(&P.fz[FZ_DONE + grp], 1u);
+    }
+  };
   K kk[ITEMS], pp[ITEMS], kn[ITEMS], pn[ITEMS];
   unsigned long long u = blockIdx.x;
   if (s_desc[0].valid) pass_load<K, MODE, NT, ITEMS>(s_desc[0], kn, pn);
@@ -600,7 +650,8 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
       for (int j = 0; j < ITEMS; ++j) {
         const uint32_t i = j * NT + threadIdx.x;
         const T t = s_buf[i];
-        __stcs(prev_dst + (gd[digit(TT::key(t))] + i), t);
+        if (FUSE) prev_dst[gd[digit(TT::key(t))] + i] = t;
+        else __stcs(prev_dst + (gd[digit(TT::key(t))] + i), t);
       }
     } else {
       #pragma unroll
@@ -608,7 +659,8 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
         const uint32_t i = j * NT + threadIdx.x;
         if (i < prev_len) {
           const T t = s_buf[i];
-          __stcs(prev_dst + (gd[digit(TT::key(t))] + i), t);
+          if (FUSE) prev_dst[gd[digit(TT::key(t))] + i] = t;
+          else __stcs(prev_dst + (gd[digit(TT::key(t))] + i), t);
         }
       }
     }
@@ -621,6 +673,7 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
       kk[j] = kn[j];
       pp[j] = pn[j];
     }
+    if (FUSE && sig) signal(sig_grp);  // before the prefetch: the fence then waits only for old stores
     // prefetch the next unit (in flight across this unit's barriers)
     if (s_desc[nslot].valid) pass_load<K, MODE, NT, ITEMS>(s_desc[nslot], kn, pn);
 
@@ -689,8 +742,25 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
         if (c > TILE / 4) atomicExch(&s_hot_next, d);  // predicts the next unit's hot digit (any one)
       }
     }
-    if (threadIdx.x == NT - 1)  // publish unit i+2
-      W.get(P, u + 2 * G, s_desc[nslot == 2 ? 0 : nslot + 1], s_cst, s_pst, s_bfill, s_bd);
+    if (threadIdx.x == NT - 1) {  // publish unit i+2
+      PassUnit<K>& Dn = s_desc[nslot == 2 ? 0 : nslot + 1];
+      if (FUSE) {
+        W.get(P, atomicAdd(&P.fz[FZ_UNIT], 1u), Dn, s_cst, s_pst, s_bfill, s_bd);
+        if (Dn.valid && P.fz_window) {
+          // throttle: wait until the join completed the items of the pieces more than fz_window
+          // below unit i+2's -- never of a piece this block still has to signal (no deadlock)
+          const uint32_t low = prev_dst ? prev_grp : s_desc[slot].grp;
+          int tg = (int)Dn.grp - (int)P.fz_window;
+          if (tg > (int)low) tg = (int)low;
+          if (tg > 0) {
+            const uint32_t need = P.ist[(uint32_t)tg << P.b2] * FZ_JOIN_WARPS;  // warp counts
+            wait_geq(&P.fz[FZ_JCOMP], need, &P.fz[FZ_ERR], 2u);
+          }
+        }
+      } else {
+        W.get(P, u + 2 * G, Dn, s_cst, s_pst, s_bfill, s_bd);
+      }
+    }
     write_out(s_gd + ((it + 1) & 1) * F);
     __syncthreads();
 
@@ -705,14 +775,26 @@ __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits)
         s_buf[s_loc[digit(kk[j])] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = TT::make(kk[j], pp[j]);
     // (no barrier: the next unit's phase 1 touches only s_cnt; its phase 2 reads s_buf / s_gd
     //  after the next phase-1 barrier)
+    sig = prev_dst != nullptr;  // unit i-1 was written out in this iteration's phase 2
+    sig_grp = prev_grp;
     prev_dst = (T*)s_desc[slot].dst;
     prev_len = ulen;
+    prev_grp = s_desc[slot].grp;
     u += G;
     slot = nslot;
     ++it;
   }
   __syncthreads();
   write_out(s_gd + ((it + 1) & 1) * F);  // the last unit (it was incremented past it)
+  if (FUSE) {
+    if (sig) signal(sig_grp);
+    if (prev_dst) signal(prev_grp);
+  }
+}
+
+template <typename K, int MODE, int NT, int ITEMS, bool GD, bool BC = false>
+__global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits) {
+  pass_body<K, MODE, NT, ITEMS, GD, BC, false>(P, fanout_bits);
 }
 
 // ------------------------------------------------------------------------------------------

@@ -83,6 +83,10 @@ struct Plan {
   unsigned long long out_cap;
   unsigned long long tiles1[2];  // pass-1 tiles per relation (host-known)
   SlotHash H;            // in-partition slot hash (lg = log2 of hash-table slots per join item)
+  // fused pass 2 + join (hj_fused.cuh): zeroed counters, see FZ_* below
+  uint32_t* fz;
+  uint32_t fz_pass_slots;  // blocks per SM that start in the pass-2 role
+  uint32_t fz_window;      // pass 2 may run at most this many pass-1 partitions ahead of the join
   __host__ __device__ int pb() const { return g + b1; }
   __host__ __device__ int qbits() const { return g + B; }
   __host__ __device__ uint32_t npieces() const { return (uint32_t)nsrc << (g + b1); }
@@ -105,6 +109,12 @@ __device__ __forceinline__ uint32_t qbin(K key, const Plan& P) {
 }
 
 enum { CNT_NEXT_ITEM = 0, CNT_PLAN_DONE = 1 };
+// fused-kernel counters (u32 offsets into Plan::fz): next pass-2 unit, join items completed,
+// watchdog error site (0 = none), per-SM role slots, per-pass-1-partition pass-2 completion
+// (warp signals)
+enum { FZ_UNIT = 0, FZ_JCOMP = 1, FZ_ERR = 2, FZ_SLOT = 8, FZ_NSLOT = 1024, FZ_DONE = FZ_SLOT + FZ_NSLOT, FZ_WORDS = FZ_DONE + 1024 };
+constexpr int FZ_PASS_WARPS = 16;  // warps of a pass-2 block in the fused kernel (signals per unit)
+constexpr int FZ_JOIN_WARPS = 15;  // compute warps of a join block in the fused kernel (counts per item)
 enum { RES_MATCHES = 0, RES_CHECKSUM = 1, RES_CURSOR = 2 };
 
 }  // namespace hj

@@ -510,3 +510,62 @@ def test_graph_replay_matches_oracle(hj):
                                bits=3, mat=True, ctx=ctx)
     assert res.matches == 50 * 40 * 30
     ctx.close()
+
+
+FUSE_KNOBS = [(32, 1), (0, 1), (1, 1), (32, 0), (32, 2), (1, 2)]  # (window MB, pass-role blocks/SM; 0 -> 1)
+
+
+@pytest.mark.parametrize("window,slots", FUSE_KNOBS)
+def test_fused_pass2_join_knobs_vs_oracle(hj, window, slots):
+    """HJ_OPT_FUSE (pass 2 + join in one L2-resident kernel): every throttle window and role
+    split gives the oracle's result -- skewed probe side (long S co-partitions split over
+    items), block nested loops (tiny C_R) and 8-byte tuples."""
+    rng = np.random.default_rng(300 + window + slots)
+    for kb, dist, cap_r, chunk_s in [(4, "zipf", 0, 0), (4, "fk", 64, 0), (8, "1to1", 0, 0), (4, "zipf", 300, 2000)]:
+        w = W.Workload("f", 1 << 15, (1 << 15) if dist == "1to1" else (3 << 14), dist,
+                       keys="sparse" if kb == 4 else "k8", z=1.2, seed=int(rng.integers(100, 10_000)))
+        Rk, Rp, Sk, Sp = W.np_generate(w)
+        ctx = hj.Context(0, kb, kb)
+        for opt, v in [(hj.OPT_FUSE, 1), (hj.OPT_FUSE_WINDOW_MB, window), (hj.OPT_FUSE_PASS_SLOTS, slots),
+                       (hj.OPT_CAP_R, cap_r), (hj.OPT_CHUNK_S, chunk_s)]:
+            ctx.set_option(opt, v)
+        for bits in (-1, 2, 9):
+            res = check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True, ctx=ctx)
+            assert res.fused, "the fused kernel ran"
+        ctx.close()
+
+
+@pytest.mark.parametrize("cfg", ["c1"])
+def test_fused_generated_config_repeats(hj, cfg):
+    """The fused kernel on a BASELINE config, called repeatedly: identical to the closed form."""
+    w = W.CONFIGS[cfg]
+    cols = W.torch_generate(w, device="cuda")
+    ctx = hj.Context(0, w.key_bytes, w.key_bytes)
+    ctx.set_option(hj.OPT_FUSE, 0)
+    ref = ctx.join(*cols, radix_bits=w.radix_bits)
+    assert ref.matches == w.nS
+    ctx.set_option(hj.OPT_FUSE, 1)
+    for _ in range(10):
+        r = ctx.join(*cols, radix_bits=w.radix_bits)
+        assert r.fused and (r.matches, r.checksum) == (ref.matches, ref.checksum)
+    ctx.close()
+
+
+def test_fused_equals_unfused_and_repeats(hj):
+    """Fused and unfused paths give identical results call after call on one context (the fused
+    kernel's counters are reset per call)."""
+    w = W.Workload("f", 1 << 17, 1 << 18, "fk", keys="dense", seed=310)
+    cols = [dev(a) for a in W.np_generate(w)]
+    ctx = hj.Context(0, 4, 4)
+    ref = None
+    for fuse in (1, 0, 1, 1, 0):
+        ctx.set_option(hj.OPT_FUSE, fuse)
+        r = ctx.join(*cols)
+        assert r.fused == bool(fuse)
+        ref = ref or (r.matches, r.checksum)
+        assert (r.matches, r.checksum) == ref
+        rm = ctx.join(*cols, out_mode=hj.OUT_MATERIALIZE)
+        assert rm.matches == ref[0]
+        pairs = oracle.pairs_sorted(to_np(rm.r_pay, 4), to_np(rm.s_pay, 4))
+        assert int(np_sig(pairs[:, 0], pairs[:, 1]).sum(dtype=np.uint64)) == ref[1]
+    ctx.close()

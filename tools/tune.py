@@ -16,7 +16,8 @@ import workloads as W  # noqa: E402
 OPTS = {"join_variant": hj.OPT_JOIN_VARIANT, "cap_r": hj.OPT_CAP_R, "chunk_s": hj.OPT_CHUNK_S,
         "blocks_per_sm": hj.OPT_BLOCKS_PER_SM, "pass_threads": hj.OPT_PASS_THREADS, "join_algo": hj.OPT_JOIN_ALGO,
         "stream_chunk": hj.OPT_STREAM_CHUNK, "pass1_bases": hj.OPT_PASS1_BASES,
-        "partitioner": hj.OPT_PARTITIONER}
+        "partitioner": hj.OPT_PARTITIONER, "fuse": hj.OPT_FUSE,
+        "fuse_window_mb": hj.OPT_FUSE_WINDOW_MB, "fuse_pass_slots": hj.OPT_FUSE_PASS_SLOTS}
 
 
 def main():
