@@ -29,11 +29,14 @@ thread_local std::string g_create_error;
 struct JoinShape {
   int nt, spt, minb, rbuf, nbsh;  // nbsh: hash slots = 2^(ceil(log2 C_R) - nbsh)
   bool h16;                       // 16-bit chain heads
+  bool pf;                        // next probe round's S loads issued before the current walk
 };
 constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1, 1}, {256, 8, 2, 2, 1}, {224, 8, 3, 1, 1}, {256, 12, 3, 1, 1},
                                      {192, 8, 3, 1, 1}, {256, 4, 2, 1, 1}, {512, 4, 1, 1, 1}, {256, 8, 2, 1, 1},
                                      {384, 4, 1, 2, 1}, {192, 8, 4, 1, 2}, {256, 8, 3, 1, 2}, {160, 8, 4, 1, 2},
-                                     {224, 8, 4, 1, 1, true}, {192, 8, 4, 1, 1, true}, {256, 8, 3, 1, 1, true}};
+                                     {224, 8, 4, 1, 1, true}, {192, 8, 4, 1, 1, true}, {256, 8, 3, 1, 1, true},
+                                     {256, 4, 3, 1, 1, false, true}, {256, 6, 3, 1, 1, false, true},
+                                     {256, 8, 3, 1, 1, false, true}, {192, 6, 4, 1, 1, false, true}};
 constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
 
@@ -140,10 +143,14 @@ constexpr int pass_items() {
   return sizeof(K) == 4 ? 8 : 4;  // 8192-tuple tiles of 8 B, 4096-tuple tiles of 16 B (64 KB)
 }
 
-// default join shape per key width (measured with tools/tune.py): 4 B -> shape 0, 8 B -> shape 5
-int join_variant(const Ctx* c) {
+// default join shape per key width and output mode (measured with tools/tune.py on B200):
+//   4 B materialize -> shape 0 (c3 0.75 ms; the prefetching shapes 15-17 0.78)
+//   4 B count       -> shape 16 (256 x 6, S prefetch: c2 0.815 vs 0.873 ms, c4 z=1.5 0.83 vs 0.88)
+//   8 B             -> shape 15 (256 x 4, S prefetch: c5_gpu 4.09 vs 4.21 ms for shape 5)
+int join_variant(const Ctx* c, bool mat) {
   if (c->opt_join_variant >= 0) return (int)c->opt_join_variant;
-  return c->key_bytes == 4 ? 0 : 5;
+  if (c->key_bytes == 8) return 15;
+  return mat ? 0 : 16;
 }
 
 int pass_threads(const Ctx* c, int fanout_bits, int items) {
@@ -192,9 +199,9 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   uint32_t CS;
   if (c->opt_chunk_s > 0) CS = (uint32_t)std::min<int64_t>(c->opt_chunk_s, 1ll << 30);
   else CS = std::max<uint32_t>(8 * CR, 32768);
-  const int rbuf = hp.fused ? 1 : JOIN_SHAPES[join_variant(c)].rbuf;
-  const int nbsh = hp.fused ? 1 : JOIN_SHAPES[join_variant(c)].nbsh;
-  const size_t head_bytes = !hp.fused && JOIN_SHAPES[join_variant(c)].h16 ? 2 : 4;
+  const int rbuf = hp.fused ? 1 : JOIN_SHAPES[join_variant(c, mat)].rbuf;
+  const int nbsh = hp.fused ? 1 : JOIN_SHAPES[join_variant(c, mat)].nbsh;
+  const size_t head_bytes = !hp.fused && JOIN_SHAPES[join_variant(c, mat)].h16 ? 2 : 4;
   int lg_nb = std::max(6, ilog2_ceil(CR) - nbsh);
   auto join_smem = [&](uint32_t cr, int lg) {  // R tile buffer(s) (TMA) + heads + next
     return (size_t)rbuf * ((cr + 3) & ~1u) * tb + (head_bytes << lg) + (size_t)cr * 2;
@@ -250,8 +257,8 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
 template <typename K, int V, typename F>
 void attr_join(F&& attr) {
   constexpr JoinShape S = JOIN_SHAPES[V];
-  attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16>);
-  attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16>);
+  attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf>);
+  attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf>);
 }
 
 template <typename K>
@@ -301,6 +308,10 @@ int set_kernel_attrs(Ctx* c) {
   attr_join<K, 12>(attr);
   attr_join<K, 13>(attr);
   attr_join<K, 14>(attr);
+  attr_join<K, 15>(attr);
+  attr_join<K, 16>(attr);
+  attr_join<K, 17>(attr);
+  attr_join<K, 18>(attr);
   return rc;
 }
 
@@ -499,11 +510,11 @@ template <typename K, int V>
 int launch_join_v(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   constexpr JoinShape S = JOIN_SHAPES[V];
   cudaStream_t st = c->stream;
-  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16>
-                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16>;
+  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf>
+                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf>;
   int g = grid_for(c, f, S.nt + 32, hp.join_smem, 1ull << 40);
-  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16><<<g, S.nt + 32, hp.join_smem, st>>>(P);
-  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
   CUDA_TRY(c, cudaGetLastError());
   return HJ_OK;
 }
@@ -522,10 +533,14 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
     c->launches += 1;
     return HJ_OK;
   }
-  switch (join_variant(c)) {
+  switch (join_variant(c, mat)) {
     case 12: rc = launch_join_v<K, 12>(c, hp, P, mat); break;
     case 13: rc = launch_join_v<K, 13>(c, hp, P, mat); break;
     case 14: rc = launch_join_v<K, 14>(c, hp, P, mat); break;
+    case 15: rc = launch_join_v<K, 15>(c, hp, P, mat); break;
+    case 16: rc = launch_join_v<K, 16>(c, hp, P, mat); break;
+    case 17: rc = launch_join_v<K, 17>(c, hp, P, mat); break;
+    case 18: rc = launch_join_v<K, 18>(c, hp, P, mat); break;
     case 9: rc = launch_join_v<K, 9>(c, hp, P, mat); break;
     case 10: rc = launch_join_v<K, 10>(c, hp, P, mat); break;
     case 11: rc = launch_join_v<K, 11>(c, hp, P, mat); break;

@@ -127,7 +127,9 @@ __device__ __forceinline__ uint32_t exch16(unsigned short* a, uint32_t v) {
 // co-partitions were just written by other SMs); the pairs are streamed out with evict-first
 // stores; after the item every compute warp bumps the completed-item counter that throttles
 // pass 2.
-template <typename K, int NT, int SPT, bool MAT, int RBUF, bool H16 = false, bool FUSE = false>
+// PF: the next probe round's S tuples are loaded (into registers) before the current round's
+// chains are walked, so the S load latency overlaps the walk instead of opening each round.
+template <typename K, int NT, int SPT, bool MAT, int RBUF, bool H16 = false, bool FUSE = false, bool PF = false>
 __device__ __forceinline__ void join_body(const Plan& P) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -191,6 +193,14 @@ __device__ __forceinline__ void join_body(const Plan& P) {
         }
       }
     };
+    T nx[PF ? SPT : 1];  // PF: the next round's tuples
+    auto load_next = [&](unsigned long long base) {
+      #pragma unroll
+      for (int j = 0; j < SPT; ++j) {
+        const unsigned long long s = base + (unsigned long long)j * NT + threadIdx.x;
+        if (s < job.se) nx[j] = FUSE ? __ldcg(ssrc + s) : __ldcs(ssrc + s);
+      }
+    };
     load_s(job.sb);
     for (uint32_t i = threadIdx.x; i < nb; i += NT) s_head[i] = NIL16;
     const T* s_rt = s_rtb + (RBUF == 2 ? (it & 1) * cap : 0) + job.shift;
@@ -204,7 +214,18 @@ __device__ __forceinline__ void join_body(const Plan& P) {
 
     // ---- probe (a7) + output (a8), SPT tuples per thread per round --------------------------
     for (unsigned long long base = job.sb; base < job.se; base += (unsigned long long)NT * SPT) {
-      if (base != job.sb) load_s(base);
+      if (PF) {
+        if (base != job.sb) {
+          #pragma unroll
+          for (int j = 0; j < SPT; ++j) {
+            sk[j] = TT::key(nx[j]);
+            sp[j] = TT::pay(nx[j]);
+          }
+        }
+        if (base + (unsigned long long)NT * SPT < job.se) load_next(base + (unsigned long long)NT * SPT);
+      } else if (base != job.sb) {
+        load_s(base);
+      }
       uint32_t idx[SPT], m[SPT];
       K rfirst[SPT];
       #pragma unroll
@@ -330,9 +351,9 @@ __device__ __forceinline__ void join_body(const Plan& P) {
   }
 }
 
-template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false>
+template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false, bool PF = false>
 __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
-  join_body<K, NT, SPT, MAT, RBUF, H16, false>(P);
+  join_body<K, NT, SPT, MAT, RBUF, H16, false, PF>(P);
 }
 
 }  // namespace hj
