@@ -30,13 +30,16 @@ struct JoinShape {
   int nt, spt, minb, rbuf, nbsh;  // nbsh: hash slots = 2^(ceil(log2 C_R) - nbsh)
   bool h16;                       // 16-bit chain heads
   bool pf;                        // next probe round's S loads issued before the current walk
+  bool l2pf;                      // claimed item's R chunk + first S round prefetched into L2
 };
 constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1, 1}, {256, 8, 2, 2, 1}, {224, 8, 3, 1, 1}, {256, 12, 3, 1, 1},
                                      {192, 8, 3, 1, 1}, {256, 4, 2, 1, 1}, {512, 4, 1, 1, 1}, {256, 8, 2, 1, 1},
                                      {384, 4, 1, 2, 1}, {192, 8, 4, 1, 2}, {256, 8, 3, 1, 2}, {160, 8, 4, 1, 2},
                                      {224, 8, 4, 1, 1, true}, {192, 8, 4, 1, 1, true}, {256, 8, 3, 1, 1, true},
                                      {256, 4, 3, 1, 1, false, true}, {256, 6, 3, 1, 1, false, true},
-                                     {256, 8, 3, 1, 1, false, true}, {192, 6, 4, 1, 1, false, true}};
+                                     {256, 8, 3, 1, 1, false, true}, {192, 6, 4, 1, 1, false, true},
+                                     {256, 8, 3, 1, 1, false, false, true}, {256, 6, 3, 1, 1, false, true, true},
+                                     {256, 4, 3, 1, 1, false, true, true}};
 constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
 
@@ -144,13 +147,15 @@ constexpr int pass_items() {
 }
 
 // default join shape per key width and output mode (measured with tools/tune.py on B200):
-//   4 B materialize -> shape 0 (c3 0.75 ms; the prefetching shapes 15-17 0.78)
-//   4 B count       -> shape 16 (256 x 6, S prefetch: c2 0.815 vs 0.873 ms, c4 z=1.5 0.83 vs 0.88)
-//   8 B             -> shape 15 (256 x 4, S prefetch: c5_gpu 4.09 vs 4.21 ms for shape 5)
+//   4 B materialize -> shape 19 (shape 0 + L2 prefetch of the next item: c3 0.749 -> 0.730 ms;
+//                      the register-prefetching shapes 15-17 0.78)
+//   4 B count       -> shape 20 (256 x 6, S prefetch + L2 prefetch: c2 0.873 -> 0.814 ms,
+//                      c4 z=1.5 0.881 -> 0.829)
+//   8 B             -> shape 21 (256 x 4, S prefetch + L2 prefetch: c5_gpu 4.21 -> 4.03 ms)
 int join_variant(const Ctx* c, bool mat) {
   if (c->opt_join_variant >= 0) return (int)c->opt_join_variant;
-  if (c->key_bytes == 8) return 15;
-  return mat ? 0 : 16;
+  if (c->key_bytes == 8) return 21;
+  return mat ? 19 : 20;
 }
 
 int pass_threads(const Ctx* c, int fanout_bits, int items) {
@@ -257,8 +262,8 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
 template <typename K, int V, typename F>
 void attr_join(F&& attr) {
   constexpr JoinShape S = JOIN_SHAPES[V];
-  attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf>);
-  attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf>);
+  attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf>);
+  attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf>);
 }
 
 template <typename K>
@@ -312,6 +317,9 @@ int set_kernel_attrs(Ctx* c) {
   attr_join<K, 16>(attr);
   attr_join<K, 17>(attr);
   attr_join<K, 18>(attr);
+  attr_join<K, 19>(attr);
+  attr_join<K, 20>(attr);
+  attr_join<K, 21>(attr);
   return rc;
 }
 
@@ -510,11 +518,11 @@ template <typename K, int V>
 int launch_join_v(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   constexpr JoinShape S = JOIN_SHAPES[V];
   cudaStream_t st = c->stream;
-  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf>
-                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf>;
+  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf>
+                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf>;
   int g = grid_for(c, f, S.nt + 32, hp.join_smem, 1ull << 40);
-  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
-  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
   CUDA_TRY(c, cudaGetLastError());
   return HJ_OK;
 }
@@ -541,6 +549,9 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
     case 16: rc = launch_join_v<K, 16>(c, hp, P, mat); break;
     case 17: rc = launch_join_v<K, 17>(c, hp, P, mat); break;
     case 18: rc = launch_join_v<K, 18>(c, hp, P, mat); break;
+    case 19: rc = launch_join_v<K, 19>(c, hp, P, mat); break;
+    case 20: rc = launch_join_v<K, 20>(c, hp, P, mat); break;
+    case 21: rc = launch_join_v<K, 21>(c, hp, P, mat); break;
     case 9: rc = launch_join_v<K, 9>(c, hp, P, mat); break;
     case 10: rc = launch_join_v<K, 10>(c, hp, P, mat); break;
     case 11: rc = launch_join_v<K, 11>(c, hp, P, mat); break;

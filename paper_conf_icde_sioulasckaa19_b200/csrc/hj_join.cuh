@@ -89,6 +89,19 @@ __device__ __forceinline__ void issue_r_copy(const Plan& P, const JoinJob& j, T*
   bulk_g2s(buf, reinterpret_cast<const void*>(a0), bytes, bar);
 }
 
+// L2 prefetch of a claimed item's R chunk and first probe round (TMA prefetch, no smem): the
+// R copy issued after the end-of-item barrier and the first S loads then hit L2.
+template <typename T>
+__device__ __forceinline__ void prefetch_item_l2(const Plan& P, const JoinJob& j, uint32_t s_round) {
+  auto pf = [](const T* b, unsigned long long n) {
+    const uintptr_t a = reinterpret_cast<uintptr_t>(b), a0 = a & ~(uintptr_t)15;
+    const uintptr_t a1 = (a + n * sizeof(T) + 15) & ~(uintptr_t)15;
+    if (a1 > a0) bulk_prefetch_l2(reinterpret_cast<const void*>(a0), (uint32_t)(a1 - a0));
+  };
+  pf((const T*)P.rel[0].t2 + j.rb, j.nr);
+  pf((const T*)P.rel[1].t2 + j.sb, min((unsigned long long)s_round, j.se - j.sb));
+}
+
 __device__ __forceinline__ void bar_compute(int nthreads) {  // named barrier 1: compute warps only
   asm volatile("barrier.sync 1, %0;" ::"r"(nthreads) : "memory");
 }
@@ -129,7 +142,8 @@ __device__ __forceinline__ uint32_t exch16(unsigned short* a, uint32_t v) {
 // pass 2.
 // PF: the next probe round's S tuples are loaded (into registers) before the current round's
 // chains are walked, so the S load latency overlaps the walk instead of opening each round.
-template <typename K, int NT, int SPT, bool MAT, int RBUF, bool H16 = false, bool FUSE = false, bool PF = false>
+template <typename K, int NT, int SPT, bool MAT, int RBUF, bool H16 = false, bool FUSE = false, bool PF = false,
+          bool L2PF = false>
 __device__ __forceinline__ void join_body(const Plan& P) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -172,6 +186,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
       JoinJob j;
       if (lane == 0) {
         j = claim_job<T, FUSE>(P, total_items);
+        if (L2PF && RBUF == 1 && j.item < total_items) prefetch_item_l2<T>(P, j, NT * SPT);
         if (RBUF == 2 && j.item < total_items) issue_r_copy<T>(P, j, s_rtb + ((it + 1) & 1) * cap, &s_bar[(it + 1) & 1]);
         s_jobs[(it + 1) & 1] = j;
       }
@@ -351,9 +366,10 @@ __device__ __forceinline__ void join_body(const Plan& P) {
   }
 }
 
-template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false, bool PF = false>
+template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false, bool PF = false,
+          bool L2PF = false>
 __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
-  join_body<K, NT, SPT, MAT, RBUF, H16, false, PF>(P);
+  join_body<K, NT, SPT, MAT, RBUF, H16, false, PF, L2PF>(P);
 }
 
 }  // namespace hj
