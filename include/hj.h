@@ -91,6 +91,9 @@ enum hj_option {
                                throttle; default 32)                                            */
   HJ_OPT_FUSE_PASS_SLOTS = 15, /* fused: blocks per SM that start in the pass-2 role (default 1 of
                                2; the others join; pass-2 blocks join once pass 2 is done)      */
+  HJ_OPT_PASS_L2PF = 17,    /* partition passes: 1 = TMA-prefetch each block's unit-after-next into L2
+                               (cp.async.bulk.prefetch.L2) when its descriptor is published; 0 = off;
+                               2 = auto (default: on for 8-byte keys, where it was measured faster) */
   HJ_OPT_STREAM_CHUNK = 8   /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
                                least 2^22; >= |S| = copy everything, then join)                   */
 };

@@ -44,6 +44,7 @@ OPT_PARTITIONER = 12  # 0 = histogram (default), 1 = bucket chains (NEXT-1)
 OPT_FUSE = 13  # 1 = pass 2 + join in one L2-resident kernel (opt-in), 0 = separate kernels (default)
 OPT_FUSE_WINDOW_MB = 14
 OPT_FUSE_PASS_SLOTS = 15
+OPT_PASS_L2PF = 17
 ALGO_HASH, ALGO_NLJ, ALGO_NONPARTITIONED = 0, 1, 2
 
 _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4: "HJ_ERR_CUDA", -5: "HJ_ERR_COMM"}

@@ -62,7 +62,7 @@ struct Ctx {
   std::string err;
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
-          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0, opt_graph = 0,
+          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0, opt_graph = 0, opt_pass_l2pf = 2,
           opt_partitioner = 0, opt_fuse = 0, opt_fuse_window_mb = 32, opt_fuse_pass_slots = 1;
   DevBuf bc_pool1[2], bc_pool2[2], bc_meta;  // HJ_OPT_PARTITIONER = 1 (NEXT-1 bucket chains)
   // workspace
@@ -364,6 +364,9 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   P.nsrc = hp.nsrc;
   P.mode = hp.mode;
   P.C2 = hp.C2;
+  // measured (tools/tune.py pass_l2pf): 8 B tuples pass 1 4.02 -> 3.59 ms on c5_gpu; 4 B pass 1
+  // slower (c3 0.939 -> 0.983), pass 2 unchanged -> auto (2) = on for 8-byte keys only
+  P.pass_l2pf = c->opt_pass_l2pf == 2 ? (c->key_bytes == 8) : (c->opt_pass_l2pf ? 1 : 0);
   P.CR = hp.CR;
   P.CS = hp.CS;
   P.ist = (uint32_t*)(m + hp.o_ist);
@@ -1239,6 +1242,7 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_STREAM_CHUNK: c->opt_stream_chunk = v; break;
     case HJ_OPT_PASS1_BASES: c->opt_pass1_bases = v; break;
     case HJ_OPT_FUSE: c->opt_fuse = v; break;
+    case HJ_OPT_PASS_L2PF: c->opt_pass_l2pf = v; break;
     case HJ_OPT_FUSE_WINDOW_MB: c->opt_fuse_window_mb = v; break;
     case HJ_OPT_FUSE_PASS_SLOTS: c->opt_fuse_pass_slots = v; break;
     case HJ_OPT_PARTITIONER:

@@ -760,6 +760,14 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
       } else {
         W.get(P, u + 2 * G, Dn, s_cst, s_pst, s_bfill, s_bd);
       }
+      if (P.pass_l2pf && Dn.valid && Dn.len) {  // unit i+2's input -> L2 (its register loads come next iteration)
+        const uint32_t bytes = MODE == 1 ? Dn.len * (uint32_t)sizeof(K) : Dn.len * (uint32_t)sizeof(T);
+        const uintptr_t a = reinterpret_cast<uintptr_t>(Dn.src_k);
+        if (((a | bytes) & 15) == 0) {
+          bulk_prefetch_l2(Dn.src_k, bytes);
+          if (MODE == 1 && (reinterpret_cast<uintptr_t>(Dn.src_p) & 15) == 0) bulk_prefetch_l2(Dn.src_p, bytes);
+        }
+      }
     }
     write_out(s_gd + ((it + 1) & 1) * F);
     __syncthreads();

@@ -67,6 +67,7 @@ struct Plan {
   int nsrc;       // count rows / piece sources (PLAN_RECV: ranks), else 1
   int mode;       // PLAN_FULL, PLAN_SEND, PLAN_RECV
   int skip_r;     // streaming S chunks: R is already partitioned (its pass-2 units are skipped)
+  int pass_l2pf;  // partition passes: TMA-prefetch unit i+2's input into L2 when it is published
   // pass 1 with precomputed per-block bases (k_pass1b): the histogram kernel runs with the same
   // grid and tile -> block assignment as pass 1 and also counts each block's pass-1 digits
   uint32_t g1;                  // pass-1 grid (0 = bases not used)
