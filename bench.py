@@ -43,6 +43,8 @@ def parse():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--cpu-slice-bits", type=int, default=2, help="cpu_baseline sample = 1 of 2^bits key slices")
     ap.add_argument("--e2e-steps", type=int, default=3)
+    ap.add_argument("--clock-period", type=float, default=0.01,
+                    help="NVML clock / throttle sampling period (s) during the timed region; 0 = off (testing only)")
     ap.add_argument("--dist", action="store_true", help="use the multi-GPU exchange path even at N=1")
     return ap.parse_args()
 
@@ -112,6 +114,9 @@ class ClockSampler:
             time.sleep(self.period)
 
     def __enter__(self):
+        if self.nv and self.period <= 0:  # testing only: no sampling
+            self.nv = None
+            self.err = "sampling disabled (--clock-period 0)"
         if self.nv:
             self.t = threading.Thread(target=self._run, daemon=True)
             self.t.start()
@@ -255,7 +260,7 @@ def main():
     launches = 0
     sent = 0
     barrier()
-    with ClockSampler(local) as clk:
+    with ClockSampler(local, args.clock_period) as clk:
         e0 = torch.cuda.Event(enable_timing=True)
         e1 = torch.cuda.Event(enable_timing=True)
         e0.record(stream)

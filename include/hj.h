@@ -94,6 +94,8 @@ enum hj_option {
   HJ_OPT_PASS_L2PF = 17,    /* partition passes: 1 = TMA-prefetch each block's unit-after-next into L2
                                (cp.async.bulk.prefetch.L2) when its descriptor is published; 0 = off;
                                2 = auto (default: on for 8-byte keys, where it was measured faster) */
+  HJ_OPT_PASS1_BITS = 18,   /* radix bits of pass 1 (0 = auto = ceil(B/2)); pass 2 takes the rest.
+                               Each pass's fan-out must stay <= 2^10                              */
   HJ_OPT_STREAM_CHUNK = 8   /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
                                least 2^22; >= |S| = copy everything, then join)                   */
 };

@@ -45,6 +45,7 @@ OPT_FUSE = 13  # 1 = pass 2 + join in one L2-resident kernel (opt-in), 0 = separ
 OPT_FUSE_WINDOW_MB = 14
 OPT_FUSE_PASS_SLOTS = 15
 OPT_PASS_L2PF = 17
+OPT_PASS1_BITS = 18
 ALGO_HASH, ALGO_NLJ, ALGO_NONPARTITIONED = 0, 1, 2
 
 _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4: "HJ_ERR_CUDA", -5: "HJ_ERR_COMM"}
@@ -141,6 +142,7 @@ class Context:
         self.pay_bytes = pay_bytes
 
     def close(self):
+        self._view_key = self._view_val = None  # views of memory hj_destroy frees
         if getattr(self, "_h", None):
             _lib.hj_destroy(self._h)
             self._h = None
@@ -174,9 +176,18 @@ class Context:
         self._check(rc)
         out = _result(res)
         if out_mode == OUT_MATERIALIZE and res.matches:
-            out.r_pay = _wrap_device(res.r_pay_out, res.matches, self.pay_bytes, cols[0].device)
-            out.s_pay = _wrap_device(res.s_pay_out, res.matches, self.pay_bytes, cols[0].device)
+            out.r_pay, out.s_pay = self._views(res, cols[0].device)
         return out
+
+    def _views(self, res, device):
+        # the ctx-owned output buffers are stable across calls (until regrown): the torch views
+        # are built once per (pointers, count) instead of per call (host overhead between calls)
+        key = (res.r_pay_out, res.s_pay_out, res.matches, device)
+        if getattr(self, "_view_key", None) != key:
+            self._view_val = (_wrap_device(res.r_pay_out, res.matches, self.pay_bytes, device),
+                              _wrap_device(res.s_pay_out, res.matches, self.pay_bytes, device))
+            self._view_key = key
+        return self._view_val
 
     def join_host(self, Rk, Rp, Sk, Sp, radix_bits: int = -1, out_mode: int = OUT_COUNT_CHECKSUM,
                   copy: bool = True) -> JoinResult:

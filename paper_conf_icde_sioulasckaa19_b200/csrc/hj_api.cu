@@ -7,7 +7,9 @@
 #include <cstdarg>
 #include <cstdio>
 #include <cstring>
+#include <map>
 #include <string>
+#include <tuple>
 
 #include "../../include/hj.h"
 #include "hj_fused.cuh"
@@ -62,7 +64,7 @@ struct Ctx {
   std::string err;
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
-          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0, opt_graph = 0, opt_pass_l2pf = 2,
+          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0, opt_graph = 0, opt_pass_l2pf = 2, opt_pass1_bits = 0,
           opt_partitioner = 0, opt_fuse = 0, opt_fuse_window_mb = 32, opt_fuse_pass_slots = 1;
   DevBuf bc_pool1[2], bc_pool2[2], bc_meta;  // HJ_OPT_PARTITIONER = 1 (NEXT-1 bucket chains)
   // workspace
@@ -73,6 +75,7 @@ struct Ctx {
   DevBuf part_off_host_dummy;
   cudaEvent_t ev[8] = {};
   uint32_t launches = 0;
+  std::map<std::tuple<const void*, int, size_t>, int> occ;  // occupancy() cache
   // HJ_OPT_GRAPH: the launch sequence of the last hj_join, captured once and replayed while the
   // call signature (columns, sizes, radix bits, mode, workspace) is unchanged
   cudaGraphExec_t graph = nullptr;
@@ -177,8 +180,9 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   const size_t tb = (size_t)c->key_bytes + c->pay_bytes;  // AoS tuple bytes
   hp.B = radix_bits < 0 ? choose_bits(nR) : radix_bits;
   if (hp.B > 20) return fail(c, HJ_ERR_UNSUPPORTED, "radix_bits %d > 20", hp.B);
-  hp.b1 = (hp.B + 1) / 2;
-  hp.b2 = hp.B / 2;
+  hp.b1 = (hp.B + 1) / 2;  // reading S6; HJ_OPT_PASS1_BITS overrides (results never change)
+  if (c->opt_pass1_bits > 0 && hp.B >= 2) hp.b1 = (int)std::min<int64_t>(c->opt_pass1_bits, hp.B - 1);
+  hp.b2 = hp.B - hp.b1;
   hp.g = g;
   hp.nsrc = nsrc;
   hp.mode = mode;
@@ -323,9 +327,23 @@ int set_kernel_attrs(Ctx* c) {
   return rc;
 }
 
-int grid_for(Ctx* c, const void* f, int nt, size_t smem, unsigned long long units) {
+// resident blocks per SM of (kernel, block size, dynamic smem), cached per context: the occupancy
+// query is host work on every launch otherwise (it sits between back-to-back calls)
+int occupancy(Ctx* c, const void* f, int nt, size_t smem) {
+  const auto key = std::make_tuple(f, nt, smem);
+  auto it = c->occ.find(key);
+  if (it != c->occ.end()) return it->second;
   int per_sm = 0;
-  cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, f, nt, smem);
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, f, nt, smem) != cudaSuccess) {
+    cudaGetLastError();
+    per_sm = 0;
+  }
+  c->occ[key] = per_sm;
+  return per_sm;
+}
+
+int grid_for(Ctx* c, const void* f, int nt, size_t smem, unsigned long long units) {
+  int per_sm = occupancy(c, f, nt, smem);
   if (per_sm < 1) per_sm = 1;
   if (c->opt_bps > 0) per_sm = std::min<int>(per_sm, (int)c->opt_bps);
   unsigned long long g = (unsigned long long)per_sm * c->num_sms;
@@ -601,8 +619,7 @@ template <typename K>
 int launch_fused(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   const size_t sm = std::max(hp.join_smem, hp.pass2_smem);
   const void* f = mat ? (const void*)k_fused<K, true> : (const void*)k_fused<K, false>;
-  int per_sm = 0;
-  CUDA_TRY(c, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, f, FZ_NT, sm));
+  const int per_sm = occupancy(c, f, FZ_NT, sm);
   if (per_sm < 1) return fail(c, HJ_ERR_UNSUPPORTED, "fused kernel does not fit an SM (%zu B smem)", sm);
   const int g = per_sm * c->num_sms;
   Plan Q = P;
@@ -1243,6 +1260,7 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_PASS1_BASES: c->opt_pass1_bases = v; break;
     case HJ_OPT_FUSE: c->opt_fuse = v; break;
     case HJ_OPT_PASS_L2PF: c->opt_pass_l2pf = v; break;
+    case HJ_OPT_PASS1_BITS: c->opt_pass1_bits = v; break;
     case HJ_OPT_FUSE_WINDOW_MB: c->opt_fuse_window_mb = v; break;
     case HJ_OPT_FUSE_PASS_SLOTS: c->opt_fuse_pass_slots = v; break;
     case HJ_OPT_PARTITIONER:
