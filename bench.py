@@ -46,6 +46,9 @@ def parse():
     ap.add_argument("--clock-period", type=float, default=0.01,
                     help="NVML clock / throttle sampling period (s) during the timed region; 0 = off (testing only)")
     ap.add_argument("--dist", action="store_true", help="use the multi-GPU exchange path even at N=1")
+    ap.add_argument("--exchange", default="direct", choices=["direct", "nccl"],
+                    help="multi-GPU exchange: direct = pass 1 stores into the owners' windows over peer memory "
+                         "(hj_xd_*); nccl = pack + NCCL all_to_all (hj_exchange_pack)")
     return ap.parse_args()
 
 
@@ -245,7 +248,7 @@ def main():
     def step():
         if not use_dist:
             return ctx.join(Rk, Rp, Sk, Sp, radix_bits=w.radix_bits, out_mode=w.out_mode)
-        return hjdist.join(Rk, Rp, Sk, Sp, out_mode=w.out_mode, ctx=ctx)
+        return hjdist.join(Rk, Rp, Sk, Sp, out_mode=w.out_mode, ctx=ctx, exchange=args.exchange)
 
     for _ in range(args.warmup):
         res = step()
@@ -268,7 +271,8 @@ def main():
             res = step()
             loc = res if not use_dist else res.local
             per_k += np.array(loc.ms_kernel)
-            launches += loc.kernels if not use_dist else loc.kernels + 2 * 3  # + pack (hist, plan, pass 1) x2
+            # + the sender side: direct = hist, plan, count rows, pass 1, barrier; nccl = (hist, plan, pass 1) x 2
+            launches += loc.kernels if not use_dist else loc.kernels + (5 if args.exchange == "direct" else 6)
             sent += 0 if not use_dist else res.sent_bytes
         e1.record(stream)
         barrier()
@@ -311,13 +315,17 @@ def main():
                       "join_items": loc.n_items,
                       "l2": "inputs larger than L2 (2 GiB in + 4 GiB partition buffers vs 126 MB L2); no flush",
                       "parallelism": "1 GPU" if not use_dist else
-                      f"{ws} rank(s): rows sharded, radix exchange over NCCL all_to_all, per-rank 2-pass join"},
+                      f"{ws} rank(s): rows sharded, radix exchange "
+                      + ("fused into pass 1 (direct peer stores, hj_xd_*)" if args.exchange == "direct"
+                         else "over NCCL all_to_all") + ", per-rank 2-pass join"},
            "roofline": roof, "roofline_path": roof_path, "kernels_ms": kms, "clocks": clk.summary(),
            "gpu_launches": launches}
     if use_dist:
         out["nvlink"] = {"bytes_sent_per_gpu_per_step": sent / args.steps,
                          "achieved_GBps": sent / args.steps / (ms * 1e-3) / 1e9, "peak_GBps": 900.0,
-                         "note": "tuple bytes rank 0 sent to other ranks / step time; all_to_all_single over NCCL"}
+                         "note": "tuple bytes rank 0 sent to other ranks / step time; "
+                                 + ("pass-1 peer stores over NVLink (CUDA IPC mappings)" if args.exchange == "direct"
+                                    else "all_to_all_single over NCCL")}
 
     if not args.no_e2e and not use_dist:
         # end to end through the public API from pinned host memory: H2D of the inputs, the join,

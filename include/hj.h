@@ -53,7 +53,7 @@ enum hj_status {
   HJ_ERR_UNSUPPORTED = -2, /* key/payload widths other than 4/4 and 8/8; radix_bits > 20     */
   HJ_ERR_OOM = -3,         /* device or pinned-host allocation failed                         */
   HJ_ERR_CUDA = -4,        /* any CUDA runtime error; message in hj_last_error()              */
-  HJ_ERR_COMM = -5         /* reserved for the multi-GPU exchange                             */
+  HJ_ERR_COMM = -5         /* multi-GPU exchange: a peer missed the hj_xd_barrier deadline    */
 };
 
 enum hj_option {
@@ -199,6 +199,115 @@ int hj_exchange_pack(hj_ctx* ctx, int rel, const void* keys, const void* pays, u
 int hj_join_received(hj_ctx* ctx, const void* R_recv, uint64_t nR, const uint32_t* R_counts,
                      const void* S_recv, uint64_t nS, const uint32_t* S_counts, int nsrc, int local_bits,
                      int out_mode, hj_result* res);
+
+/* ---- Direct-store exchange (multi-GPU over NVLink / NVSwitch peer memory) -----------------
+ * The B200-native form of SURVEY.md §8(e): instead of pack -> NCCL all-to-all -> receive, pass 1
+ * of every sender stores each tuple straight into the receive window of the rank that owns its
+ * co-partition (peer stores over NVLink; the WC-staged runs arrive as full lines), so the
+ * exchange is fused into the partitioning pass and the 2w B/tuple staging round trip and the
+ * separate collective disappear. Co-partitions are independent, so rank j owns the
+ * co-partitions with (key >> local_bits) & (G - 1) == j, exactly as for hj_exchange_pack.
+ *
+ * Protocol per join (G = 2^gpu_bits ranks, one context per rank, all calls on ctx's stream):
+ *   1. hj_xd_count     rows a1-a2 for R and S: histogram over (rank bits, local bits) + plan;
+ *                      returns the tuples this rank sends to every rank.
+ *   2. (caller)        all-gather of those [2][G] totals -> totals[2][G][G] on every rank;
+ *                      grow windows if needed (hj_xd_window) and exchange their IPC handles.
+ *   3. hj_xd_store     row a3: pass 1 writing into the peers' windows, plus this rank's count
+ *                      rows into every peer's window header.
+ *   4. hj_xd_barrier   every rank's stores are visible before any rank reads its window.
+ *   5. hj_join_received(window_R + H, nR_in, window_R, window_S + H, nS_in, window_S, G, ...)
+ *                      rows a4-a8 on what arrived (H = hj_xd_header_bytes(G, local_bits)).
+ *
+ * Receive window of relation r on rank j (ctx-owned device allocation, exported by IPC):
+ *   [0, H)      count rows, [G][2^local_bits] uint32, row s = what source s sent (q-order, as
+ *               hj_exchange_pack's counts_out rows)
+ *   [H, ...)    tuples (AoS as hj_partition), source-major: source s's segment starts at
+ *               sum_{s' < s} totals[r][s'][j] tuples and is grouped by the local pass-1 digit.
+ * Board window (slot 2, HJ_XD_BOARD_BYTES): starts with uint64[HJ_XD_MAX_RANKS] barrier flags,
+ * flag s = last barrier epoch source s reached (the rest serves hj_xd_join).
+ * Requires G <= HJ_XD_MAX_RANKS and gpu_bits + ceil(local_bits / 2) <= 10. */
+#define HJ_XD_MAX_RANKS 64
+/* Board window (slot 2) bytes: barrier / phase flags, the totals board [src][2][dst] and the
+ * results board [src][2] of hj_xd_join, all uint64. */
+#define HJ_XD_BOARD_BYTES 69632
+/* hj_xd_join return value (not an error): some rank's receive window is too small for this
+ * call; nothing was joined; grow every window to the size `totals` implies and call again. */
+#define HJ_XD_REGROW 1
+
+/* hj_xd_window: (re)allocate ctx's window `slot` (0 = R receive, 1 = S receive, 2 = board) to
+ * at least `bytes` (zero-filled when (re)allocated; kept when already large enough).
+ *   *dptr:       device pointer of the window in this process (ctx-owned until hj_destroy or
+ *                the next growth of the same slot).
+ *   ipc_handle:  if non-NULL, 64 bytes receiving cudaIpcGetMemHandle of the window.
+ *   *grew:       if non-NULL, 1 when the window was (re)allocated (peers must re-open it). */
+int hj_xd_window(hj_ctx* ctx, int slot, uint64_t bytes, void** dptr, void* ipc_handle, int* grew);
+
+/* Bytes of a receive window's count-row header: round_up(G * 2^local_bits * 4, 256). */
+uint64_t hj_xd_header_bytes(int G, int local_bits);
+
+/* hj_ipc_open: map a peer's window (64-byte handle from its hj_xd_window) into this process on
+ * ctx's device (cudaIpcMemLazyEnablePeerAccess); hj_ipc_close unmaps it. A handle exported by
+ * this same process cannot be opened here (CUDA IPC rule): use the window pointer directly. */
+int hj_ipc_open(hj_ctx* ctx, const void* ipc_handle, void** dptr);
+int hj_ipc_close(hj_ctx* ctx, void* dptr);
+
+/* hj_xd_count: rows a1-a2 on this rank's SoA rows of R (nR) and S (nS) with the radix field
+ * widened by gpu_bits rank bits above local_bits. Synchronous. The plan is kept in ctx for the
+ * next hj_xd_store. dest_counts: HOST uint64[2][G] (caller-allocated), dest_counts[r*G + j] =
+ * tuples of relation r this rank sends to rank j. Columns must stay unchanged until hj_xd_store. */
+int hj_xd_count(hj_ctx* ctx, const void* R_keys, const void* R_pay, uint64_t nR, const void* S_keys,
+                const void* S_pay, uint64_t nS, int gpu_bits, int local_bits, uint64_t* dest_counts);
+
+/* hj_xd_store: row a3 of the last hj_xd_count, writing into the peers' receive windows.
+ *   rank:       this rank, 0 <= rank < G.
+ *   totals:     HOST uint64[2][G][G], totals[(r*G + s)*G + j] = tuples of relation r rank s
+ *               sends to rank j (the all-gathered dest_counts of every rank).
+ *   win_R/win_S: HOST arrays of G device pointers, valid in this process: every rank's R / S
+ *               receive window (this rank's own window at [rank]); each at least
+ *               H + (sum_s totals[r][s][j]) * (key_bytes + pay_bytes) bytes.
+ * Asynchronous on ctx's stream. */
+int hj_xd_store(hj_ctx* ctx, int rank, const uint64_t* totals, void* const* win_R, void* const* win_S);
+
+/* hj_xd_barrier: on ctx's stream, a one-block kernel publishes this rank's epoch to flag
+ * [rank] of every rank's flag window (system-scope release after a system fence) and waits
+ * until its own flag window holds the epoch of every rank (acquire). The epoch is a per-ctx
+ * counter: all ranks must call it the same number of times. flags: HOST array of G device
+ * pointers (every rank's flag window, this rank's at [rank]). A rank that waits longer than
+ * timeout_ms gives up; the next hj_join_received on ctx then fails with HJ_ERR_COMM.
+ * Asynchronous. */
+int hj_xd_barrier(hj_ctx* ctx, int rank, int G, void* const* flags, uint32_t timeout_ms);
+
+/* hj_xd_join: the whole multi-GPU join of this rank, driven from the device -- no host round
+ * trip and no host collective between the histogram and the result (steps 1-5 above, with the
+ * totals exchange and the result reduction done through the peers' boards):
+ *   a1-a2 histogram + plan over the rank-widened field; phase A: this rank's [2][G] destination
+ *   totals stored into every rank's board, flag A; wait for all flags A; pass-1 cursors from the
+ *   board (window capacities checked on the device, identically on every rank); count rows to
+ *   the peers' window headers; a3 pass 1 storing into the peers' windows; phase B barrier; a4-a8
+ *   on this rank's window; phase C: (matches, checksum) into every board, flag C, wait, sum.
+ *   rank, gpu_bits:   this rank, G = 2^gpu_bits ranks (G <= HJ_XD_MAX_RANKS).
+ *   columns:          this rank's SoA rows of R and S (device, as hj_join).
+ *   win_R, win_S, board: HOST arrays of G device pointers valid in this process (this rank's own
+ *                     windows at [rank]; the board of HJ_XD_BOARD_BYTES, zeroed at creation).
+ *   win_bytes:        HOST uint64[2][G], the byte size of every rank's R / S window.
+ *   res:              this rank's share (as hj_join_received; materialized pairs stay local).
+ *   totals:           HOST out uint64[2][G][G], totals[(r*G + s)*G + j] = tuples of relation r
+ *                     rank s sent to rank j.
+ *   all:              HOST out uint64[2]: matches and checksum summed over all ranks (mod 2^64).
+ * Returns HJ_OK, HJ_XD_REGROW (every rank returns it in the same call), or an error;
+ * HJ_ERR_COMM when a phase wait exceeded timeout_ms. Synchronous. */
+int hj_xd_join(hj_ctx* ctx, int rank, int gpu_bits, const void* R_keys, const void* R_pay, uint64_t nR,
+               const void* S_keys, const void* S_pay, uint64_t nS, int local_bits, int out_mode, void* const* win_R,
+               void* const* win_S, void* const* board, const uint64_t* win_bytes, uint32_t timeout_ms,
+               hj_result* res, uint64_t* totals, uint64_t* all);
+
+/* hj_xd_reserve: every allocation the hj_xd_join call with these sizes (and this rank's window
+ * sizes) would make, without launching anything. hj_xd_join synchronizes only at its end, but a
+ * first-time device allocation inside it can synchronize the device; ranks that share one GPU
+ * (tests) reserve first so no allocation runs while a peer's kernels wait on this rank. */
+int hj_xd_reserve(hj_ctx* ctx, int gpu_bits, uint64_t nR, uint64_t nS, int local_bits, int out_mode,
+                  uint64_t win_R_bytes, uint64_t win_S_bytes);
 
 /* Library build string (compile flags, arch). */
 const char* hj_version(void);

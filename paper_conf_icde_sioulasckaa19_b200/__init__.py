@@ -52,7 +52,12 @@ _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4:
 
 # every symbol include/hj.h declares (checked by tests/test_abi.py)
 EXPORTS = ("hj_create", "hj_destroy", "hj_last_error", "hj_set_stream", "hj_set_option", "hj_join",
-           "hj_join_host", "hj_partition", "hj_exchange_pack", "hj_join_received", "hj_version")
+           "hj_join_host", "hj_partition", "hj_exchange_pack", "hj_join_received", "hj_xd_window",
+           "hj_xd_header_bytes", "hj_ipc_open", "hj_ipc_close", "hj_xd_count", "hj_xd_store", "hj_xd_barrier",
+           "hj_xd_join", "hj_xd_reserve", "hj_version")
+XD_MAX_RANKS = 64
+XD_BOARD_BYTES = 69632  # HJ_XD_BOARD_BYTES
+XD_REGROW = 1           # HJ_XD_REGROW
 
 
 class HJError(RuntimeError):
@@ -95,6 +100,26 @@ def _load_lib():
     lib.hj_exchange_pack.restype = i32
     lib.hj_join_received.argtypes = [vp, vp, u64, vp, vp, u64, vp, i32, i32, i32, ctypes.POINTER(_Result)]
     lib.hj_join_received.restype = i32
+    lib.hj_xd_window.argtypes = [vp, i32, u64, ctypes.POINTER(vp), vp, ctypes.POINTER(i32)]
+    lib.hj_xd_window.restype = i32
+    lib.hj_xd_header_bytes.argtypes = [i32, i32]
+    lib.hj_xd_header_bytes.restype = u64
+    lib.hj_ipc_open.argtypes = [vp, vp, ctypes.POINTER(vp)]
+    lib.hj_ipc_open.restype = i32
+    lib.hj_ipc_close.argtypes = [vp, vp]
+    lib.hj_ipc_close.restype = i32
+    lib.hj_xd_count.argtypes = [vp, vp, vp, u64, vp, vp, u64, i32, i32, ctypes.POINTER(u64)]
+    lib.hj_xd_count.restype = i32
+    lib.hj_xd_store.argtypes = [vp, i32, ctypes.POINTER(u64), ctypes.POINTER(vp), ctypes.POINTER(vp)]
+    lib.hj_xd_store.restype = i32
+    lib.hj_xd_barrier.argtypes = [vp, i32, i32, ctypes.POINTER(vp), ctypes.c_uint32]
+    lib.hj_xd_barrier.restype = i32
+    lib.hj_xd_join.argtypes = [vp, i32, i32, vp, vp, u64, vp, vp, u64, i32, i32, ctypes.POINTER(vp),
+                               ctypes.POINTER(vp), ctypes.POINTER(vp), ctypes.POINTER(u64), ctypes.c_uint32,
+                               ctypes.POINTER(_Result), ctypes.POINTER(u64), ctypes.POINTER(u64)]
+    lib.hj_xd_join.restype = i32
+    lib.hj_xd_reserve.argtypes = [vp, i32, u64, u64, i32, i32, u64, u64]
+    lib.hj_xd_reserve.restype = i32
     lib.hj_version.argtypes = []
     lib.hj_version.restype = ctypes.c_char_p
     return lib
@@ -279,6 +304,104 @@ class Context:
             out.r_pay = _wrap_device(res.r_pay_out, res.matches, self.pay_bytes, dev_)
             out.s_pay = _wrap_device(res.s_pay_out, res.matches, self.pay_bytes, dev_)
         return out
+
+
+    # ---- direct-store exchange (hj_xd_*; orchestrated by dist.DirectExchange) -----------------
+    def xd_window(self, slot: int, nbytes: int, want_handle: bool = True):
+        """(re)allocate window `slot` (0 R, 1 S, 2 flags) to >= nbytes -> (dptr, handle bytes | None, grew)."""
+        d = ctypes.c_void_p()
+        grew = ctypes.c_int()
+        hb = ctypes.create_string_buffer(64) if want_handle else None
+        self._check(_lib.hj_xd_window(self._h, slot, int(nbytes), ctypes.byref(d), hb, ctypes.byref(grew)))
+        return int(d.value), (hb.raw if hb is not None else None), bool(grew.value)
+
+    def ipc_open(self, handle: bytes) -> int:
+        d = ctypes.c_void_p()
+        self._check(_lib.hj_ipc_open(self._h, ctypes.create_string_buffer(handle, 64), ctypes.byref(d)))
+        return int(d.value)
+
+    def ipc_close(self, dptr: int):
+        self._check(_lib.hj_ipc_close(self._h, ctypes.c_void_p(dptr)))
+
+    def xd_count(self, Rk, Rp, Sk, Sp, gpu_bits: int, local_bits: int):
+        """Rows a1-a2 (hj_xd_count) -> numpy uint64 [2, G]: tuples of R / S sent to each rank."""
+        import torch
+
+        cols = [_as_device_col(Rk, self.key_bytes), _as_device_col(Rp, self.pay_bytes),
+                _as_device_col(Sk, self.key_bytes), _as_device_col(Sp, self.pay_bytes)]
+        self.set_stream(torch.cuda.current_stream(cols[0].device).cuda_stream)
+        G = 1 << gpu_bits
+        dest = (ctypes.c_uint64 * (2 * G))()
+        self._check(_lib.hj_xd_count(self._h, _ptr(cols[0]), _ptr(cols[1]), cols[0].numel(), _ptr(cols[2]),
+                                     _ptr(cols[3]), cols[2].numel(), gpu_bits, local_bits, dest))
+        return np.frombuffer(dest, dtype=np.uint64).reshape(2, G).copy()
+
+    def xd_store(self, rank: int, totals, win_R, win_S):
+        """Row a3 into the peers' windows (hj_xd_store). totals: uint64 [2, G, G]; win_*: G device addresses."""
+        t = np.ascontiguousarray(totals, dtype=np.uint64)
+        G = t.shape[1]
+        wr = (ctypes.c_void_p * G)(*[int(x) for x in win_R])
+        ws = (ctypes.c_void_p * G)(*[int(x) for x in win_S])
+        self._check(_lib.hj_xd_store(self._h, rank, t.ctypes.data_as(ctypes.POINTER(ctypes.c_uint64)), wr, ws))
+
+    def xd_header_bytes(self, G: int, local_bits: int) -> int:
+        return xd_header_bytes(G, local_bits)
+
+    def xd_views(self, dptr: int, G: int, local_bits: int, n: int, device):
+        """Torch views of a receive window: (tuples as int64 words, count rows int32 [G, 2^local_bits])."""
+        H = xd_header_bytes(G, local_bits)
+        words = n * (self.key_bytes + self.pay_bytes) // 8
+        recv = _wrap_device(dptr + H, max(words, 1), 8, device)[:words]
+        cnt = _wrap_device(dptr, G << local_bits, 4, device).view(G, 1 << local_bits)
+        return recv, cnt
+
+    def xd_barrier(self, rank: int, flags, timeout_ms: int = 10000):
+        G = len(flags)
+        f = (ctypes.c_void_p * G)(*[int(x) for x in flags])
+        self._check(_lib.hj_xd_barrier(self._h, rank, G, f, timeout_ms))
+
+
+    def xd_join(self, rank: int, gpu_bits: int, Rk, Rp, Sk, Sp, local_bits: int, out_mode: int, win_R, win_S,
+                board, win_bytes, timeout_ms: int = 10000):
+        """The device-driven multi-GPU join of this rank (hj_xd_join).
+        Returns (status, JoinResult of this rank's share, totals uint64 [2, G, G], (matches, checksum)
+        over all ranks); status XD_REGROW = windows too small, nothing joined (grow and call again)."""
+        import torch
+
+        cols = [_as_device_col(Rk, self.key_bytes), _as_device_col(Rp, self.pay_bytes),
+                _as_device_col(Sk, self.key_bytes), _as_device_col(Sp, self.pay_bytes)]
+        dev_ = cols[0].device
+        self.set_stream(torch.cuda.current_stream(dev_).cuda_stream)
+        G = 1 << gpu_bits
+        wr = (ctypes.c_void_p * G)(*[int(x) for x in win_R])
+        ws = (ctypes.c_void_p * G)(*[int(x) for x in win_S])
+        wb = (ctypes.c_void_p * G)(*[int(x) for x in board])
+        cap = np.ascontiguousarray(win_bytes, dtype=np.uint64).reshape(2, G)
+        tot = np.zeros((2, G, G), dtype=np.uint64)
+        allv = np.zeros(2, dtype=np.uint64)
+        res = _Result()
+        rc = _lib.hj_xd_join(self._h, rank, gpu_bits, _ptr(cols[0]), _ptr(cols[1]), cols[0].numel(), _ptr(cols[2]),
+                             _ptr(cols[3]), cols[2].numel(), local_bits, out_mode, wr, ws, wb,
+                             cap.ctypes.data_as(ctypes.POINTER(ctypes.c_uint64)), timeout_ms, ctypes.byref(res),
+                             tot.ctypes.data_as(ctypes.POINTER(ctypes.c_uint64)),
+                             allv.ctypes.data_as(ctypes.POINTER(ctypes.c_uint64)))
+        if rc not in (0, XD_REGROW):
+            self._check(rc)
+        out = _result(res)
+        if rc == 0 and out_mode == OUT_MATERIALIZE and res.matches:
+            out.r_pay = _wrap_device(res.r_pay_out, res.matches, self.pay_bytes, dev_)
+            out.s_pay = _wrap_device(res.s_pay_out, res.matches, self.pay_bytes, dev_)
+        return rc, out, tot, (int(allv[0]), int(allv[1]))
+
+
+    def xd_reserve(self, gpu_bits: int, nR: int, nS: int, local_bits: int, out_mode: int, win_R_bytes: int,
+                   win_S_bytes: int):
+        self._check(_lib.hj_xd_reserve(self._h, gpu_bits, nR, nS, local_bits, out_mode, int(win_R_bytes),
+                                       int(win_S_bytes)))
+
+
+def xd_header_bytes(G: int, local_bits: int) -> int:
+    return int(_lib.hj_xd_header_bytes(G, local_bits))
 
 
 def _result(res: _Result) -> JoinResult:

@@ -10,8 +10,10 @@
 #include <map>
 #include <string>
 #include <tuple>
+#include <vector>
 
 #include "../../include/hj.h"
+#include "hj_exchange.cuh"
 #include "hj_fused.cuh"
 #include "hj_join.cuh"
 #include "hj_partition.cuh"
@@ -50,6 +52,8 @@ struct DevBuf {
   size_t bytes = 0;
 };
 
+struct HostPlan;
+
 struct Ctx {
   int device = 0;
   int key_bytes = 4, pay_bytes = 4;
@@ -78,6 +82,16 @@ struct Ctx {
   std::map<std::tuple<const void*, int, size_t>, int> occ;  // occupancy() cache
   // HJ_OPT_GRAPH: the launch sequence of the last hj_join, captured once and replayed while the
   // call signature (columns, sizes, radix bits, mode, workspace) is unchanged
+  // direct-store exchange (hj_xd_*): windows [R recv, S recv, flags], the plan of the last
+  // hj_xd_count, its pass-1 piece starts, the barrier epoch and the timeout word
+  DevBuf xd_win[3], xd_meta;
+  HostPlan* xd_hp = nullptr;
+  Plan* xd_P = nullptr;
+  std::vector<unsigned long long> xd_pst[2];
+  unsigned long long* h_xd_cur = nullptr;  // pinned: cursor table upload / totals board readback (64 KB)
+  uint32_t* h_xd_err = nullptr;            // pinned, mapped: barrier timeout flag
+  uint32_t* d_xd_err = nullptr;
+  unsigned long long xd_epoch = 0;
   cudaGraphExec_t graph = nullptr;
   unsigned long long graph_key[12] = {};
   uint32_t graph_launches = 0;
@@ -353,10 +367,10 @@ int grid_for(Ctx* c, const void* f, int nt, size_t smem, unsigned long long unit
 
 // Fill the device Plan for one call; rel 1 may be empty (hj_partition, hj_exchange_pack).
 Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, unsigned long long nR, const void* Sk,
-                 const void* Sp, unsigned long long nS) {
+                 const void* Sp, unsigned long long nS, void* meta = nullptr) {
   Plan P;
   memset(&P, 0, sizeof P);
-  char* m = (char*)c->meta.p;
+  char* m = (char*)(meta ? meta : c->meta.p);
   const void* ks[2] = {Rk, Sk};
   const void* ps[2] = {Rp, Sp};
   const unsigned long long ns[2] = {nR, nS};
@@ -430,13 +444,24 @@ size_t pass1b_smem(const HostPlan& hp, int nt) {
   return ((size_t)nt * pass_items<K>() + 2 * F) * tb + 16 * F + 4 * (F + 4) + 8 * F;
 }
 
+// stage: 0 = all of a1-a3; 1 = a1-a2 only (hj_xd_count); 2 = a3 only (hj_xd_store, after stage 1
+// with the same plan)
 template <typename K>
-int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false) {
+int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false, int stage = 0) {
   cudaStream_t st = c->stream;
   const bool gd = hp.g > 0;
+  if (stage == 2) {
+    mark(c, 2);
+    int rc = hp.tile == 512 * pass_items<K>()
+                 ? (gd ? launch_pass<K, 1, 512, true>(c, hp, P, hp.pb()) : launch_pass<K, 1, 512, false>(c, hp, P, hp.pb()))
+                 : (gd ? launch_pass<K, 1, 1024, true>(c, hp, P, hp.pb()) : launch_pass<K, 1, 1024, false>(c, hp, P, hp.pb()));
+    if (rc) return rc;
+    mark(c, 3);
+    return HJ_OK;
+  }
   mark(c, 0);
   if (!chunk) {
-    CUDA_TRY(c, cudaMemsetAsync(c->meta.p, 0, hp.zero_bytes, st));
+    CUDA_TRY(c, cudaMemsetAsync(P.counters, 0, hp.zero_bytes, st));  // the zeroed region starts at o_counters = 0
   } else {  // streaming S chunk: keep R's counts and the accumulated results
     CUDA_TRY(c, cudaMemsetAsync((char*)c->meta.p + hp.o_counters, 0, 64, st));
     CUDA_TRY(c, cudaMemsetAsync((char*)c->meta.p + hp.o_cnt[1], 0, (size_t)4 << hp.qbits(), st));
@@ -481,6 +506,7 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false) 
   CUDA_TRY(c, cudaGetLastError());
   c->launches += 1;
   mark(c, 2);
+  if (stage == 1) return HJ_OK;
   if (hp.mode != PLAN_RECV && Pb.g1) {
     const int nt = hp.tile == 512 * pass_items<K>() ? 512 : 1024;
     const size_t sm = pass1b_smem<K>(hp, nt);
@@ -638,14 +664,21 @@ constexpr int HJ_RERUN = 1;  // finish_join: fused materialization overflowed; o
 
 // Join phase + result readback shared by hj_join and hj_join_received. `joined`: the join
 // already ran inside the fused kernel.
-int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res, bool joined = false) {
+int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res, bool joined = false,
+                const XdJoin* xd = nullptr) {
   cudaStream_t st = c->stream;
   const bool timing = c->opt_timing != 0;
   int rc = joined ? HJ_OK : c->key_bytes == 4 ? launch_join<uint32_t>(c, hp, P, mat) : launch_join<uint64_t>(c, hp, P, mat);
   if (rc) return rc;
   unsigned long long* h = (unsigned long long*)c->h_res;
+  if (xd) {  // hj_xd_join: phase C (results of every rank summed on the device) before the readback
+    k_xd_results<<<1, XD_MAX, 0, st>>>(*xd);
+    CUDA_TRY(c, cudaGetLastError());
+    c->launches += 1;
+  }
   CUDA_TRY(c, cudaMemcpyAsync(h, P.results, 4 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st));
   CUDA_TRY(c, cudaMemcpyAsync(h + 4, P.ist + (1ull << hp.B), sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
+  if (xd) CUDA_TRY(c, cudaMemcpyAsync(h + 6, P.results + 4, 3 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st));
   h[5] = 0;
   if (joined) CUDA_TRY(c, cudaMemcpyAsync(h + 5, P.fz + FZ_ERR, sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
   if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[6], st));
@@ -1145,6 +1178,35 @@ int join_host_serial(Ctx* c, const void* Rk, const void* Rp, uint64_t nR, const 
   return rc;
 }
 
+// hj_xd_join's host side: pinned staging, the send plan (c->xd_hp, own metadata buffer), the
+// receive plan `hr` (sized by this rank's window capacity capt[] in tuples: the received counts
+// are known only on the device), and every device buffer both need. No launches.
+int xd_prepare(Ctx* c, int gpu_bits, unsigned long long nR, unsigned long long nS, int local_bits, bool mat,
+               const unsigned long long capt[2], HostPlan& hr) {
+  const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
+  if (!c->xd_hp) {
+    c->xd_hp = new HostPlan();
+    c->xd_P = new Plan();
+  }
+  if (!c->h_xd_cur) {
+    if (cudaMallocHost(&c->h_xd_cur, (size_t)XD_MAX * 2 * XD_MAX * 8) != cudaSuccess ||
+        cudaHostAlloc(&c->h_xd_err, 64, cudaHostAllocMapped) != cudaSuccess ||
+        cudaHostGetDevicePointer((void**)&c->d_xd_err, c->h_xd_err, 0) != cudaSuccess)
+      return fail(c, HJ_ERR_OOM, "pinned exchange staging");
+    *c->h_xd_err = 0;
+  }
+  HostPlan& hs = *c->xd_hp;
+  int rc = prepare(c, hs, nR, nS, local_bits, false, false, gpu_bits, 1, PLAN_SEND);
+  hs.bases = false;
+  if (rc == HJ_OK) rc = ensure(c, c->xd_meta, hs.meta_bytes);
+  if (rc == HJ_OK) rc = ensure(c, c->t1[0], nR * tb + 16);  // overflow scratch for pass 1
+  if (rc == HJ_OK) rc = ensure(c, c->t1[1], nS * tb + 16);
+  if (rc == HJ_OK) rc = prepare(c, hr, capt[0], capt[1], local_bits, mat, false, 0, 1 << gpu_bits, PLAN_RECV);
+  if (rc == HJ_OK && (hr.npieces() > 1024 || hs.pb() > 10))
+    rc = fail(c, HJ_ERR_UNSUPPORTED, "too many pass-1 pieces (G=%d, local_bits=%d)", 1 << gpu_bits, local_bits);
+  return rc;
+}
+
 }  // namespace
 
 struct hj_ctx {
@@ -1221,6 +1283,13 @@ void hj_destroy(hj_ctx* h) {
   for (DevBuf* b : bufs)
     if (b->p) cudaFree(b->p);
   if (c->graph) cudaGraphExecDestroy(c->graph);
+  for (auto& b : c->xd_win)
+    if (b.p) cudaFree(b.p);
+  if (c->xd_meta.p) cudaFree(c->xd_meta.p);
+  delete c->xd_hp;
+  delete c->xd_P;
+  if (c->h_xd_cur) cudaFreeHost(c->h_xd_cur);
+  if (c->h_xd_err) cudaFreeHost(c->h_xd_err);
   if (c->h_res) cudaFreeHost(c->h_res);
   if (c->h_out) cudaFreeHost(c->h_out);
   for (auto& ev : c->ev)
@@ -1441,6 +1510,422 @@ int hj_join_received(hj_ctx* h, const void* R_recv, uint64_t nR, const uint32_t*
     rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P);
     if (rc == HJ_OK) rc = c->key_bytes == 4 ? launch_pass2<uint32_t>(c, hp, P) : launch_pass2<uint64_t>(c, hp, P);
     if (rc == HJ_OK) rc = finish_join(c, hp, P, mat, res);
+  }
+  if (rc == HJ_OK && c->h_xd_err && *(volatile uint32_t*)c->h_xd_err) {
+    *c->h_xd_err = 0;
+    rc = fail(c, HJ_ERR_COMM, "exchange barrier timed out: a peer never reached hj_xd_barrier");
+  }
+  cudaSetDevice(prev);
+  return rc;
+}
+
+// ---- direct-store exchange -----------------------------------------------------------------
+
+int hj_xd_window(hj_ctx* h, int slot, uint64_t bytes, void** dptr, void* ipc_handle, int* grew) {
+  if (!h || !dptr) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  if (slot < 0 || slot > 2) return fail(c, HJ_ERR_INVALID, "window slot must be 0 (R), 1 (S) or 2 (flags)");
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  int rc = HJ_OK;
+  DevBuf& b = c->xd_win[slot];
+  const size_t want = std::max<size_t>(align_up(bytes, 256), 256);
+  const bool g = !b.p || b.bytes < want;
+  if (g) {
+    // plain cudaMalloc (IPC-exportable); peers that mapped the old window must re-open it
+    if (b.p) {
+      cudaStreamSynchronize(c->stream);
+      cudaFree(b.p);
+      b.p = nullptr;
+      b.bytes = 0;
+    }
+    cudaError_t e = cudaMalloc(&b.p, want);
+    if (e == cudaSuccess) e = cudaMemset(b.p, 0, want);
+    if (e != cudaSuccess) {
+      b.p = nullptr;
+      rc = fail(c, e == cudaErrorMemoryAllocation ? HJ_ERR_OOM : HJ_ERR_CUDA, "window: %s", cudaGetErrorString(e));
+    } else {
+      b.bytes = want;
+    }
+  }
+  if (rc == HJ_OK) {
+    *dptr = b.p;
+    if (grew) *grew = g ? 1 : 0;
+    if (ipc_handle) {
+      cudaIpcMemHandle_t mh;
+      cudaError_t e = cudaIpcGetMemHandle(&mh, b.p);
+      if (e != cudaSuccess) rc = fail(c, HJ_ERR_CUDA, "cudaIpcGetMemHandle: %s", cudaGetErrorString(e));
+      else memcpy(ipc_handle, &mh, sizeof mh);
+    }
+  }
+  cudaSetDevice(prev);
+  return rc;
+}
+
+uint64_t hj_xd_header_bytes(int G, int local_bits) {
+  if (G < 1 || local_bits < 0 || local_bits > 20) return 0;
+  return align_up((size_t)G * ((size_t)4 << local_bits), 256);
+}
+
+int hj_ipc_open(hj_ctx* h, const void* ipc_handle, void** dptr) {
+  if (!h || !ipc_handle || !dptr) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  static_assert(sizeof(cudaIpcMemHandle_t) == 64, "64-byte IPC handle");
+  cudaIpcMemHandle_t mh;
+  memcpy(&mh, ipc_handle, sizeof mh);
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  cudaError_t e = cudaIpcOpenMemHandle(dptr, mh, cudaIpcMemLazyEnablePeerAccess);
+  cudaSetDevice(prev);
+  if (e != cudaSuccess) {
+    cudaGetLastError();
+    return fail(c, HJ_ERR_CUDA, "cudaIpcOpenMemHandle: %s", cudaGetErrorString(e));
+  }
+  return HJ_OK;
+}
+
+int hj_ipc_close(hj_ctx* h, void* dptr) {
+  if (!h || !dptr) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  cudaError_t e = cudaIpcCloseMemHandle(dptr);
+  cudaSetDevice(prev);
+  if (e != cudaSuccess) return fail(c, HJ_ERR_CUDA, "cudaIpcCloseMemHandle: %s", cudaGetErrorString(e));
+  return HJ_OK;
+}
+
+int hj_xd_count(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const void* Sk, const void* Sp, uint64_t nS,
+                int gpu_bits, int local_bits, uint64_t* dest_counts) {
+  if (!h || !dest_counts) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  if (gpu_bits < 0 || (1 << gpu_bits) > XD_MAX || local_bits < 0 || local_bits > 20)
+    return fail(c, HJ_ERR_INVALID, "gpu_bits 0..6, local_bits 0..20");
+  if ((nR && (!Rk || !Rp)) || (nS && (!Sk || !Sp))) return fail(c, HJ_ERR_INVALID, "null column with n > 0");
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  if (!c->xd_hp) {
+    c->xd_hp = new HostPlan();
+    c->xd_P = new Plan();
+  }
+  HostPlan& hp = *c->xd_hp;
+  int rc = prepare(c, hp, nR, nS, local_bits, false, false, gpu_bits, 1, PLAN_SEND);
+  hp.bases = false;  // pass 1 = k_pass with pre-set cursors
+  if (rc == HJ_OK && !c->h_xd_cur) {
+    if (cudaMallocHost(&c->h_xd_cur, (size_t)XD_MAX * 2 * XD_MAX * 8) != cudaSuccess ||
+        cudaHostAlloc(&c->h_xd_err, 64, cudaHostAllocMapped) != cudaSuccess ||
+        cudaHostGetDevicePointer((void**)&c->d_xd_err, c->h_xd_err, 0) != cudaSuccess)
+      rc = fail(c, HJ_ERR_OOM, "pinned exchange staging");
+    else
+      *c->h_xd_err = 0;
+  }
+  if (rc == HJ_OK) {
+    Plan& P = *c->xd_P;
+    P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
+    c->launches = 0;
+    rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P, false, 1) : launch_front<uint64_t>(c, hp, P, false, 1);
+    const uint32_t F1 = 1u << hp.pb();
+    unsigned long long* pst = c->h_xd_cur;  // 2 x (F1 + 1) <= 2 x 1025 (staging reused below)
+    for (int r = 0; r < 2 && rc == HJ_OK; ++r) {
+      cudaError_t e = cudaMemcpyAsync(pst + r * 1025, P.rel[r].pst, (F1 + 1) * 8, cudaMemcpyDeviceToHost, c->stream);
+      if (e != cudaSuccess) rc = fail(c, HJ_ERR_CUDA, "xd_count: %s", cudaGetErrorString(e));
+    }
+    if (rc == HJ_OK) {
+      cudaError_t e = cudaStreamSynchronize(c->stream);
+      if (e != cudaSuccess) rc = fail(c, HJ_ERR_CUDA, "xd_count: %s", cudaGetErrorString(e));
+    }
+    if (rc == HJ_OK) {
+      const int G = 1 << gpu_bits;
+      for (int r = 0; r < 2; ++r) {
+        c->xd_pst[r].assign(pst + r * 1025, pst + r * 1025 + F1 + 1);
+        for (int j = 0; j < G; ++j)
+          dest_counts[r * G + j] = c->xd_pst[r][(size_t)(j + 1) << hp.b1] - c->xd_pst[r][(size_t)j << hp.b1];
+      }
+    }
+  }
+  cudaSetDevice(prev);
+  return rc;
+}
+
+int hj_xd_store(hj_ctx* h, int rank, const uint64_t* totals, void* const* win_R, void* const* win_S) {
+  if (!h || !totals || !win_R || !win_S) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  if (!c->xd_hp || c->xd_pst[0].empty()) return fail(c, HJ_ERR_INVALID, "hj_xd_store without hj_xd_count");
+  HostPlan& hp = *c->xd_hp;
+  Plan P = *c->xd_P;
+  const int G = 1 << hp.g;
+  if (rank < 0 || rank >= G) return fail(c, HJ_ERR_INVALID, "rank %d outside 0..%d", rank, G - 1);
+  void* const* win[2] = {win_R, win_S};
+  for (int r = 0; r < 2; ++r)
+    for (int j = 0; j < G; ++j)
+      if (!win[r][j]) return fail(c, HJ_ERR_INVALID, "null window pointer (relation %d, rank %d)", r, j);
+  const long long tb = c->key_bytes + c->pay_bytes;
+  const size_t H = hj_xd_header_bytes(G, hp.B);
+  const uint32_t F1 = 1u << hp.pb();
+  // cursor of pass-1 digit D = (j, d1): element offset, from this rank's own window tuples, of
+  // where this rank's d1 run for rank j starts in rank j's window (source-major layout, then d1)
+  for (int r = 0; r < 2; ++r) {
+    const char* base = (const char*)win[r][rank] + H;
+    const std::vector<unsigned long long>& pst = c->xd_pst[r];
+    for (int j = 0; j < G; ++j) {
+      const long long diff = (long long)((const char*)win[r][j] + H - base);
+      if (diff % tb) return fail(c, HJ_ERR_INVALID, "window of rank %d not aligned to the tuple size", j);
+      unsigned long long seg = 0;
+      for (int s = 0; s < rank; ++s) seg += totals[((size_t)r * G + s) * G + j];
+      const unsigned long long rel0 = (unsigned long long)(diff / tb) + seg;
+      for (uint32_t d1 = 0; d1 < (1u << hp.b1); ++d1) {
+        const size_t D = ((size_t)j << hp.b1) | d1;
+        c->h_xd_cur[r * 1024 + D] = rel0 + (pst[D] - pst[(size_t)j << hp.b1]);
+      }
+    }
+    P.rel[r].t1 = const_cast<char*>(base);
+  }
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  int rc = HJ_OK;
+  cudaError_t e = cudaSuccess;
+  for (int r = 0; r < 2 && e == cudaSuccess; ++r)
+    e = cudaMemcpyAsync(P.rel[r].cur1, c->h_xd_cur + r * 1024, (size_t)F1 * 8, cudaMemcpyHostToDevice, c->stream);
+  if (e != cudaSuccess) rc = fail(c, HJ_ERR_CUDA, "xd_store: %s", cudaGetErrorString(e));
+  c->launches = 0;
+  if (rc == HJ_OK) {
+    XdRows a;
+    memset(&a, 0, sizeof a);
+    a.rowlen = 1u << hp.B;
+    for (int r = 0; r < 2; ++r) {
+      a.cnt[r] = P.rel[r].cnt;
+      for (int j = 0; j < G; ++j) a.dst[r][j] = (uint32_t*)win[r][j] + (size_t)rank * a.rowlen;
+    }
+    k_xd_rows<<<dim3(G, 2), 256, 0, c->stream>>>(a);
+    e = cudaGetLastError();
+    if (e != cudaSuccess) rc = fail(c, HJ_ERR_CUDA, "k_xd_rows: %s", cudaGetErrorString(e));
+    else c->launches += 1;
+  }
+  if (rc == HJ_OK)
+    rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P, false, 2) : launch_front<uint64_t>(c, hp, P, false, 2);
+  c->xd_pst[0].clear();  // one store per count
+  cudaSetDevice(prev);
+  return rc;
+}
+
+int hj_xd_barrier(hj_ctx* h, int rank, int G, void* const* flags, uint32_t timeout_ms) {
+  if (!h || !flags) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  if (G < 1 || G > XD_MAX || rank < 0 || rank >= G) return fail(c, HJ_ERR_INVALID, "G 1..64, 0 <= rank < G");
+  if (!c->d_xd_err) return fail(c, HJ_ERR_INVALID, "hj_xd_barrier before hj_xd_count");
+  XdBarrier b;
+  memset(&b, 0, sizeof b);
+  for (int j = 0; j < G; ++j) {
+    if (!flags[j]) return fail(c, HJ_ERR_INVALID, "null flag window of rank %d", j);
+    b.flags[j] = (unsigned long long*)flags[j];
+  }
+  b.own = (const unsigned long long*)flags[rank];
+  b.epoch = ++c->xd_epoch;
+  b.timeout_ns = (unsigned long long)timeout_ms * 1000000ull;
+  b.err = c->d_xd_err;
+  b.G = G;
+  b.rank = rank;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  k_xd_barrier<<<1, XD_MAX, 0, c->stream>>>(b);
+  cudaError_t e = cudaGetLastError();
+  cudaSetDevice(prev);
+  if (e != cudaSuccess) return fail(c, HJ_ERR_CUDA, "k_xd_barrier: %s", cudaGetErrorString(e));
+  return HJ_OK;
+}
+
+int hj_xd_reserve(hj_ctx* h, int gpu_bits, uint64_t nR, uint64_t nS, int local_bits, int out_mode, uint64_t win_R_bytes,
+                  uint64_t win_S_bytes) {
+  if (!h) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  if (gpu_bits < 0 || (1 << gpu_bits) > XD_MAX || local_bits < 0 || local_bits > 20)
+    return fail(c, HJ_ERR_INVALID, "gpu_bits 0..6, local_bits 0..20");
+  const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
+  const size_t H = hj_xd_header_bytes(1 << gpu_bits, local_bits);
+  const unsigned long long capt[2] = {win_R_bytes > H + 64 ? (win_R_bytes - H - 64) / tb : 0,
+                                      win_S_bytes > H + 64 ? (win_S_bytes - H - 64) / tb : 0};
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  HostPlan hr;
+  int rc = xd_prepare(c, gpu_bits, nR, nS, local_bits, out_mode == HJ_OUT_MATERIALIZE, capt, hr);
+  cudaSetDevice(prev);
+  return rc;
+}
+
+int hj_xd_join(hj_ctx* h, int rank, int gpu_bits, const void* Rk, const void* Rp, uint64_t nR, const void* Sk,
+               const void* Sp, uint64_t nS, int local_bits, int out_mode, void* const* win_R, void* const* win_S,
+               void* const* board, const uint64_t* win_bytes, uint32_t timeout_ms, hj_result* res, uint64_t* totals,
+               uint64_t* all) {
+  if (!h || !win_R || !win_S || !board || !win_bytes || !res || !totals || !all) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  if (out_mode != HJ_OUT_COUNT_CHECKSUM && out_mode != HJ_OUT_MATERIALIZE)
+    return fail(c, HJ_ERR_INVALID, "bad out_mode %d", out_mode);
+  if (gpu_bits < 0 || (1 << gpu_bits) > XD_MAX || local_bits < 0 || local_bits > 20)
+    return fail(c, HJ_ERR_INVALID, "gpu_bits 0..6, local_bits 0..20");
+  const int G = 1 << gpu_bits;
+  if (rank < 0 || rank >= G) return fail(c, HJ_ERR_INVALID, "rank %d outside 0..%d", rank, G - 1);
+  if ((nR && (!Rk || !Rp)) || (nS && (!Sk || !Sp))) return fail(c, HJ_ERR_INVALID, "null column with n > 0");
+  void* const* win[2] = {win_R, win_S};
+  for (int j = 0; j < G; ++j)
+    if (!win_R[j] || !win_S[j] || !board[j]) return fail(c, HJ_ERR_INVALID, "null window of rank %d", j);
+  const bool mat = out_mode == HJ_OUT_MATERIALIZE;
+  const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
+  const size_t H = hj_xd_header_bytes(G, local_bits);
+  XdJoin a;
+  memset(&a, 0, sizeof a);
+  unsigned long long capt[2];
+  for (int r = 0; r < 2; ++r)
+    for (int j = 0; j < G; ++j) {
+      const uint64_t wb = win_bytes[r * G + j];
+      a.cap[r][j] = wb > H + 64 ? (wb - H - 64) / tb : 0;
+      const long long diff = (long long)((const char*)win[r][j] - (const char*)win[r][rank]);
+      if (diff % (long long)tb) return fail(c, HJ_ERR_INVALID, "window of rank %d not aligned to the tuple size", j);
+      a.delta[r][j] = diff / (long long)tb;
+      if (j == rank) capt[r] = a.cap[r][j];
+    }
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  int rc = HJ_OK;
+  HostPlan hr;
+  if (rc == HJ_OK) rc = xd_prepare(c, gpu_bits, nR, nS, local_bits, mat, capt, hr);
+  if (rc != HJ_OK) {
+    cudaSetDevice(prev);
+    return rc;
+  }
+  HostPlan& hs = *c->xd_hp;
+  Plan Ps = device_plan(c, hs, Rk, Rp, nR, Sk, Sp, nS, c->xd_meta.p);
+  Plan Pr = device_plan(c, hr, nullptr, nullptr, capt[0], nullptr, nullptr, capt[1]);
+  for (int r = 0; r < 2; ++r) {
+    char* own = (char*)win[r][rank];
+    Ps.rel[r].t1 = own + H;
+    Pr.rel[r].t1 = own + H;
+    Pr.rel[r].cnt = (uint32_t*)own;
+    a.pst[r] = Ps.rel[r].pst;
+    a.cur1[r] = Ps.rel[r].cur1;
+    a.rows0[r] = (uint32_t*)own;
+    a.scratch[r] = ((const char*)c->t1[r].p - (own + H)) / (long long)tb;
+    if (((const char*)c->t1[r].p - (own + H)) % (long long)tb)
+      rc = fail(c, HJ_ERR_INVALID, "scratch not aligned to the tuple size");
+  }
+  for (int j = 0; j < G; ++j) a.board[j] = (unsigned long long*)board[j];
+  a.own = (const unsigned long long*)board[rank];
+  a.res = Pr.results;
+  a.sums = Pr.results + 4;
+  a.overflow = (uint32_t*)(Pr.results + 6);
+  a.err = c->d_xd_err;
+  a.epoch = ++c->xd_epoch;
+  a.timeout_ns = (unsigned long long)timeout_ms * 1000000ull;
+  a.rows_words = (uint32_t)G << local_bits;
+  a.G = G;
+  a.rank = rank;
+  a.b1 = hs.b1;
+  cudaStream_t st = c->stream;
+  c->launches = 0;
+  auto run = [&]() -> int {
+    const bool k4 = c->key_bytes == 4;
+    mark(c, 0);
+    CUDA_TRY(c, cudaMemsetAsync(Ps.counters, 0, hs.zero_bytes, st));
+    CUDA_TRY(c, cudaMemsetAsync(Pr.counters, 0, hr.zero_bytes, st));
+    {  // a1 over the rank-widened field
+      const size_t sm = hs.qbits() <= 15 ? ((size_t)4 << hs.qbits()) : hs.qbits() <= 16 ? ((size_t)2 << hs.qbits()) : 0;
+      const void* f = sm ? (k4 ? (const void*)k_hist<uint32_t, true, true> : (const void*)k_hist<uint64_t, true, true>)
+                         : (k4 ? (const void*)k_hist<uint32_t, false, false> : (const void*)k_hist<uint64_t, false, false>);
+      int g = std::max(2, grid_for(c, f, HIST_NT, sm, (nR + nS + 4095) / 4096 + 2));
+      uint32_t gr = (uint32_t)((double)g * (double)nR / (double)std::max<unsigned long long>(nR + nS, 1) + 0.5);
+      gr = std::min<uint32_t>(std::max<uint32_t>(gr, 1), (uint32_t)g - 1);
+      if (nR == 0) gr = 0;
+      if (k4) {
+        if (hs.qbits() <= 15) k_hist<uint32_t, true, true, true><<<g, HIST_NT, sm, st>>>(Ps, gr);
+        else if (sm) k_hist<uint32_t, true, true, false><<<g, HIST_NT, sm, st>>>(Ps, gr);
+        else k_hist<uint32_t, false, true><<<g, HIST_NT, 0, st>>>(Ps, gr);
+      } else {
+        if (hs.qbits() <= 15) k_hist<uint64_t, true, true, true><<<g, HIST_NT, sm, st>>>(Ps, gr);
+        else if (sm) k_hist<uint64_t, true, true, false><<<g, HIST_NT, sm, st>>>(Ps, gr);
+        else k_hist<uint64_t, false, true><<<g, HIST_NT, 0, st>>>(Ps, gr);
+      }
+      CUDA_TRY(c, cudaGetLastError());
+      c->launches += 1;
+    }
+    mark(c, 1);
+    k_plan<<<(unsigned)((((size_t)1 << hs.qbits()) + 1023) / 1024), 1024, 0, st>>>(Ps);
+    k_xd_totals<<<1, 256, 0, st>>>(a);
+    k_xd_cursors<<<1, 1024, 0, st>>>(a);
+    CUDA_TRY(c, cudaGetLastError());
+    c->launches += 3;
+    // the totals board is final once every rank's phase A arrived (read back with the results)
+    CUDA_TRY(c, cudaMemcpyAsync(c->h_xd_cur, (const unsigned long long*)board[rank] + XB_TOT, (size_t)G * 2 * XD_MAX * 8,
+                                cudaMemcpyDeviceToHost, st));
+    mark(c, 2);
+    XdRows xr;
+    memset(&xr, 0, sizeof xr);
+    xr.rowlen = 1u << hs.B;
+    xr.skip = a.overflow;
+    for (int r = 0; r < 2; ++r) {
+      xr.cnt[r] = Ps.rel[r].cnt;
+      for (int j = 0; j < G; ++j) xr.dst[r][j] = (uint32_t*)win[r][j] + (size_t)rank * xr.rowlen;
+    }
+    k_xd_rows<<<dim3(G, 2), 256, 0, st>>>(xr);
+    CUDA_TRY(c, cudaGetLastError());
+    c->launches += 1;
+    const bool gd = hs.g > 0;
+    int e = hs.tile == 512 * (k4 ? pass_items<uint32_t>() : pass_items<uint64_t>())
+                ? (k4 ? (gd ? launch_pass<uint32_t, 1, 512, true>(c, hs, Ps, hs.pb()) : launch_pass<uint32_t, 1, 512, false>(c, hs, Ps, hs.pb()))
+                      : (gd ? launch_pass<uint64_t, 1, 512, true>(c, hs, Ps, hs.pb()) : launch_pass<uint64_t, 1, 512, false>(c, hs, Ps, hs.pb())))
+                : (k4 ? (gd ? launch_pass<uint32_t, 1, 1024, true>(c, hs, Ps, hs.pb()) : launch_pass<uint32_t, 1, 1024, false>(c, hs, Ps, hs.pb()))
+                      : (gd ? launch_pass<uint64_t, 1, 1024, true>(c, hs, Ps, hs.pb()) : launch_pass<uint64_t, 1, 1024, false>(c, hs, Ps, hs.pb())));
+    if (e) return e;
+    XdBarrier b;
+    memset(&b, 0, sizeof b);
+    for (int j = 0; j < G; ++j) b.flags[j] = (unsigned long long*)board[j] + XB_FLAGS_B;
+    b.own = (const unsigned long long*)board[rank] + XB_FLAGS_B;
+    b.epoch = a.epoch;
+    b.timeout_ns = a.timeout_ns;
+    b.err = a.err;
+    b.G = G;
+    b.rank = rank;
+    k_xd_barrier<<<1, XD_MAX, 0, st>>>(b);
+    CUDA_TRY(c, cudaGetLastError());
+    c->launches += 1;
+    mark(c, 3);
+    k_plan<<<(unsigned)((((size_t)1 << hr.qbits()) + 1023) / 1024), 1024, 0, st>>>(Pr);
+    CUDA_TRY(c, cudaGetLastError());
+    c->launches += 1;
+    e = k4 ? launch_pass2<uint32_t>(c, hr, Pr) : launch_pass2<uint64_t>(c, hr, Pr);
+    if (e) return e;
+    return finish_join(c, hr, Pr, mat, res, false, &a);
+  };
+  if (rc == HJ_OK) rc = run();
+  if (rc == HJ_OK) {
+    const unsigned long long* hh = (const unsigned long long*)c->h_res;
+    all[0] = hh[6];
+    all[1] = hh[7];
+    const bool over = (uint32_t)hh[8] != 0;
+    for (int s = 0; s < G; ++s)
+        for (int r = 0; r < 2; ++r)
+          for (int j = 0; j < G; ++j) totals[((size_t)r * G + s) * G + j] = c->h_xd_cur[((size_t)s * 2 + r) * XD_MAX + j];
+    if (*(volatile uint32_t*)c->h_xd_err) {
+      *c->h_xd_err = 0;
+      rc = fail(c, HJ_ERR_COMM, "exchange timed out: a peer never reached hj_xd_join's phase waits");
+    }
+    if (rc == HJ_OK && over) {
+      rc = HJ_XD_REGROW;
+      c->err = "receive windows too small: grow them to the sizes `totals` implies and call again";
+    }
   }
   cudaSetDevice(prev);
   return rc;
