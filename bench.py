@@ -245,10 +245,14 @@ def main():
     stream = torch.cuda.current_stream(dev)
     from paper_conf_icde_sioulasckaa19_b200 import dist as hjdist
 
+    # the local radix bits of the exchange path, fixed once (the whole workload's |R| is known)
+    local_bits = hjdist._local_bits(w.nR, ws)
+
     def step():
         if not use_dist:
             return ctx.join(Rk, Rp, Sk, Sp, radix_bits=w.radix_bits, out_mode=w.out_mode)
-        return hjdist.join(Rk, Rp, Sk, Sp, out_mode=w.out_mode, ctx=ctx, exchange=args.exchange)
+        return hjdist.join(Rk, Rp, Sk, Sp, local_bits=local_bits, out_mode=w.out_mode, ctx=ctx,
+                           exchange=args.exchange)
 
     for _ in range(args.warmup):
         res = step()
