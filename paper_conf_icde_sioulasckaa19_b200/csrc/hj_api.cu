@@ -1705,7 +1705,7 @@ int hj_xd_store(hj_ctx* h, int rank, const uint64_t* totals, void* const* win_R,
       a.cnt[r] = P.rel[r].cnt;
       for (int j = 0; j < G; ++j) a.dst[r][j] = (uint32_t*)win[r][j] + (size_t)rank * a.rowlen;
     }
-    k_xd_rows<<<dim3(G, 2), 256, 0, c->stream>>>(a);
+    k_xd_rows<<<dim3(G, 2, std::max(1u, std::min(32u, (a.rowlen / 4) / 256))), 256, 0, c->stream>>>(a);
     e = cudaGetLastError();
     if (e != cudaSuccess) rc = fail(c, HJ_ERR_CUDA, "k_xd_rows: %s", cudaGetErrorString(e));
     else c->launches += 1;
@@ -1879,7 +1879,7 @@ int hj_xd_join(hj_ctx* h, int rank, int gpu_bits, const void* Rk, const void* Rp
       xr.cnt[r] = Ps.rel[r].cnt;
       for (int j = 0; j < G; ++j) xr.dst[r][j] = (uint32_t*)win[r][j] + (size_t)rank * xr.rowlen;
     }
-    k_xd_rows<<<dim3(G, 2), 256, 0, st>>>(xr);
+    k_xd_rows<<<dim3(G, 2, std::max(1u, std::min(32u, (xr.rowlen / 4) / 256))), 256, 0, st>>>(xr);
     CUDA_TRY(c, cudaGetLastError());
     c->launches += 1;
     const bool gd = hs.g > 0;

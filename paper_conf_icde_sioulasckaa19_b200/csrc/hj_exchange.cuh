@@ -28,19 +28,21 @@ struct XdRows {
   const uint32_t* skip;      // hj_xd_join: non-zero = windows too small this call (write nothing)
 };
 
-// grid (G, 2): block (j, r) copies relation r's row j to rank j (16-byte stores when aligned)
+// grid (G, 2, Z): blocks (j, r, *) copy relation r's row j to rank j, 16-byte stores when
+// aligned, the row split over the Z blocks (a row is up to 2^20 words)
 __global__ void __launch_bounds__(256) k_xd_rows(XdRows a) {
   if (a.skip && *a.skip) return;
   const int j = blockIdx.x, r = blockIdx.y;
   const uint32_t* src = a.cnt[r] + (size_t)j * a.rowlen;
   uint32_t* dst = a.dst[r][j];
+  const uint32_t t0 = blockIdx.z * blockDim.x + threadIdx.x, step = gridDim.z * blockDim.x;
   const bool vec = (a.rowlen & 3) == 0 && ((reinterpret_cast<uintptr_t>(src) | reinterpret_cast<uintptr_t>(dst)) & 15) == 0;
   if (vec) {
     const uint4* s4 = reinterpret_cast<const uint4*>(src);
     uint4* d4 = reinterpret_cast<uint4*>(dst);
-    for (uint32_t i = threadIdx.x; i < a.rowlen / 4; i += blockDim.x) d4[i] = s4[i];
+    for (uint32_t i = t0; i < a.rowlen / 4; i += step) d4[i] = s4[i];
   } else {
-    for (uint32_t i = threadIdx.x; i < a.rowlen; i += blockDim.x) dst[i] = src[i];
+    for (uint32_t i = t0; i < a.rowlen; i += step) dst[i] = src[i];
   }
 }
 

@@ -51,4 +51,20 @@ if which == "all":
     # exchange path with 2 virtual ranks
     send, cnt, dest = ctx4.exchange_pack(0, dev(Rk), dev(Rp), 1, 6)
     torch.cuda.synchronize()
+    # direct-store exchange, one rank (the sanitizers serialize kernels, so the phase waits must
+    # be satisfiable by the rank itself): every hj_xd_join kernel, a regrow, both output modes
+    cx = hj.Context(0, 4, 4)
+    m, c, rr, ss = oracle.hash_join(Rk, Rp, Sk, Sp, materialize=True)
+    H = hj.xd_header_bytes(1, 6)
+    for scale, mode in ((0.5, 0), (1.2, 0), (1.2, 1)):
+        cap = [[H + 64 + int(scale * len(Rk)) * 8], [H + 64 + int(scale * len(Sk)) * 8]]
+        wr, _, _ = cx.xd_window(0, cap[0][0], want_handle=False)
+        ws, _, _ = cx.xd_window(1, cap[1][0], want_handle=False)
+        wb, _, _ = cx.xd_window(2, hj.XD_BOARD_BYTES, want_handle=False)
+        rc, res, tot, allv = cx.xd_join(0, 0, dev(Rk), dev(Rp), dev(Sk), dev(Sp), 6, mode, [wr], [ws], [wb], cap)
+        if scale < 1:
+            assert rc == hj.XD_REGROW and int(tot[1].sum()) == len(Sk)
+        else:
+            assert rc == 0 and allv[0] == m and (mode or allv[1] == c)
+    cx.close()
 print("sanitize cases ok", flush=True)
