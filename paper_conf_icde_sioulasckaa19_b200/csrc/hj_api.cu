@@ -35,6 +35,7 @@ struct JoinShape {
   bool h16;                       // 16-bit chain heads
   bool pf;                        // next probe round's S loads issued before the current walk
   bool l2pf;                      // claimed item's R chunk + first S round prefetched into L2
+  int spf = 0;                    // S stream prefetched into L2 this many probe rounds ahead (0 = off)
 };
 constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1, 1}, {256, 8, 2, 2, 1}, {224, 8, 3, 1, 1}, {256, 12, 3, 1, 1},
                                      {192, 8, 3, 1, 1}, {256, 4, 2, 1, 1}, {512, 4, 1, 1, 1}, {256, 8, 2, 1, 1},
@@ -43,7 +44,10 @@ constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1, 1}, {256, 8, 2, 2, 1}, {224,
                                      {256, 4, 3, 1, 1, false, true}, {256, 6, 3, 1, 1, false, true},
                                      {256, 8, 3, 1, 1, false, true}, {192, 6, 4, 1, 1, false, true},
                                      {256, 8, 3, 1, 1, false, false, true}, {256, 6, 3, 1, 1, false, true, true},
-                                     {256, 4, 3, 1, 1, false, true, true}};
+                                     {256, 4, 3, 1, 1, false, true, true},
+                                     {256, 6, 3, 1, 1, false, true, true, 4}, {256, 8, 3, 1, 1, false, false, true, 4},
+                                     {256, 4, 3, 1, 1, false, true, true, 4}, {256, 6, 3, 1, 1, false, true, true, 8},
+                                     {256, 6, 3, 1, 1, false, true, true, 2}, {256, 8, 3, 1, 1, false, false, true, 2}};
 constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
 
@@ -164,15 +168,17 @@ constexpr int pass_items() {
 }
 
 // default join shape per key width and output mode (measured with tools/tune.py on B200):
-//   4 B materialize -> shape 19 (shape 0 + L2 prefetch of the next item: c3 0.749 -> 0.730 ms;
-//                      the register-prefetching shapes 15-17 0.78)
+//   4 B materialize -> shape 27 (shape 19 + the S stream L2-prefetched 2 rounds ahead: c3 join
+//                      0.730 -> 0.704 ms; 4 rounds ahead also 0.704; shape 19 = shape 0 + L2
+//                      prefetch of the next item: 0.749 -> 0.730; register-prefetching 15-17 0.78)
 //   4 B count       -> shape 20 (256 x 6, S prefetch + L2 prefetch: c2 0.873 -> 0.814 ms,
-//                      c4 z=1.5 0.881 -> 0.829)
+//                      c4 z=1.5 0.881 -> 0.829; streaming S through L2 2-8 rounds ahead, shapes
+//                      22/25/26, is slower here: 0.84 -- this probe is issue-bound on the checksum)
 //   8 B             -> shape 21 (256 x 4, S prefetch + L2 prefetch: c5_gpu 4.21 -> 4.03 ms)
 int join_variant(const Ctx* c, bool mat) {
   if (c->opt_join_variant >= 0) return (int)c->opt_join_variant;
   if (c->key_bytes == 8) return 21;
-  return mat ? 19 : 20;
+  return mat ? 27 : 20;
 }
 
 int pass_threads(const Ctx* c, int fanout_bits, int items) {
@@ -280,8 +286,8 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
 template <typename K, int V, typename F>
 void attr_join(F&& attr) {
   constexpr JoinShape S = JOIN_SHAPES[V];
-  attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf>);
-  attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf>);
+  attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf>);
+  attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf>);
 }
 
 template <typename K>
@@ -338,6 +344,12 @@ int set_kernel_attrs(Ctx* c) {
   attr_join<K, 19>(attr);
   attr_join<K, 20>(attr);
   attr_join<K, 21>(attr);
+  attr_join<K, 22>(attr);
+  attr_join<K, 23>(attr);
+  attr_join<K, 24>(attr);
+  attr_join<K, 25>(attr);
+  attr_join<K, 26>(attr);
+  attr_join<K, 27>(attr);
   return rc;
 }
 
@@ -565,11 +577,11 @@ template <typename K, int V>
 int launch_join_v(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   constexpr JoinShape S = JOIN_SHAPES[V];
   cudaStream_t st = c->stream;
-  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf>
-                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf>;
+  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf>
+                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf>;
   int g = grid_for(c, f, S.nt + 32, hp.join_smem, 1ull << 40);
-  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
-  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
   CUDA_TRY(c, cudaGetLastError());
   return HJ_OK;
 }
@@ -589,6 +601,12 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
     return HJ_OK;
   }
   switch (join_variant(c, mat)) {
+    case 22: rc = launch_join_v<K, 22>(c, hp, P, mat); break;
+    case 23: rc = launch_join_v<K, 23>(c, hp, P, mat); break;
+    case 24: rc = launch_join_v<K, 24>(c, hp, P, mat); break;
+    case 25: rc = launch_join_v<K, 25>(c, hp, P, mat); break;
+    case 26: rc = launch_join_v<K, 26>(c, hp, P, mat); break;
+    case 27: rc = launch_join_v<K, 27>(c, hp, P, mat); break;
     case 12: rc = launch_join_v<K, 12>(c, hp, P, mat); break;
     case 13: rc = launch_join_v<K, 13>(c, hp, P, mat); break;
     case 14: rc = launch_join_v<K, 14>(c, hp, P, mat); break;

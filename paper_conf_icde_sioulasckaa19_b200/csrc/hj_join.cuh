@@ -142,8 +142,12 @@ __device__ __forceinline__ uint32_t exch16(unsigned short* a, uint32_t v) {
 // pass 2.
 // PF: the next probe round's S tuples are loaded (into registers) before the current round's
 // chains are walked, so the S load latency overlaps the walk instead of opening each round.
+// SPF > 0: the S chunk is streamed through L2 ahead of the probe: at the item's first round one
+// compute thread issues a TMA L2 prefetch of rounds 1..SPF, then at round k of rounds k+SPF (one
+// cp.async.bulk.prefetch.L2 of NT*SPT tuples per round), so the bytes in flight per SM no longer
+// depend on the registers of the probing threads.
 template <typename K, int NT, int SPT, bool MAT, int RBUF, bool H16 = false, bool FUSE = false, bool PF = false,
-          bool L2PF = false>
+          bool L2PF = false, int SPF = 0>
 __device__ __forceinline__ void join_body(const Plan& P) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -229,6 +233,16 @@ __device__ __forceinline__ void join_body(const Plan& P) {
 
     // ---- probe (a7) + output (a8), SPT tuples per thread per round --------------------------
     for (unsigned long long base = job.sb; base < job.se; base += (unsigned long long)NT * SPT) {
+      if (SPF > 0 && threadIdx.x == 0) {
+        constexpr unsigned long long RND = (unsigned long long)NT * SPT;
+        const unsigned long long lo = base == job.sb ? base + RND : base + SPF * RND;
+        const unsigned long long hi = min(base + (SPF + 1) * RND, job.se);
+        if (lo < hi) {
+          const uintptr_t a = reinterpret_cast<uintptr_t>(ssrc + lo), a0 = a & ~(uintptr_t)15;
+          const uintptr_t a1 = (reinterpret_cast<uintptr_t>(ssrc + hi) + 15) & ~(uintptr_t)15;
+          bulk_prefetch_l2(reinterpret_cast<const void*>(a0), (uint32_t)(a1 - a0));
+        }
+      }
       if (PF) {
         if (base != job.sb) {
           #pragma unroll
@@ -367,9 +381,9 @@ __device__ __forceinline__ void join_body(const Plan& P) {
 }
 
 template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false, bool PF = false,
-          bool L2PF = false>
+          bool L2PF = false, int SPF = 0>
 __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
-  join_body<K, NT, SPT, MAT, RBUF, H16, false, PF, L2PF>(P);
+  join_body<K, NT, SPT, MAT, RBUF, H16, false, PF, L2PF, SPF>(P);
 }
 
 }  // namespace hj
