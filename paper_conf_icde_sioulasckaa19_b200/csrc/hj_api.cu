@@ -169,7 +169,8 @@ constexpr int pass_items() {
 
 // default join shape per key width and output mode (measured with tools/tune.py on B200):
 //   4 B materialize -> shape 27 (shape 19 + the S stream L2-prefetched 2 rounds ahead: c3 join
-//                      0.730 -> 0.704 ms; 4 rounds ahead also 0.704; shape 19 = shape 0 + L2
+//                      0.730 -> 0.704 ms, 0.679 -> 0.646 after the 32-bit-shared-address
+//                      probe; 4 rounds ahead the same; shape 19 = shape 0 + L2
 //                      prefetch of the next item: 0.749 -> 0.730; register-prefetching 15-17 0.78)
 //   4 B count       -> shape 20 (256 x 6, S prefetch + L2 prefetch: c2 0.873 -> 0.814 ms,
 //                      c4 z=1.5 0.881 -> 0.829; streaming S through L2 2-8 rounds ahead, shapes

@@ -102,6 +102,19 @@ __device__ __forceinline__ void prefetch_item_l2(const Plan& P, const JoinJob& j
   pf((const T*)P.rel[1].t2 + j.sb, min((unsigned long long)s_round, j.se - j.sb));
 }
 
+// a tuple of the R tile from its 32-bit shared-window address (keeps the tile base in a register:
+// through the generic pointer the compiler rematerialized the shared-window base per access)
+__device__ __forceinline__ unsigned long long lds_tuple(uint32_t a, unsigned long long*) {
+  unsigned long long v;
+  asm volatile("ld.shared.u64 %0, [%1];" : "=l"(v) : "r"(a));
+  return v;
+}
+__device__ __forceinline__ ulonglong2 lds_tuple(uint32_t a, ulonglong2*) {
+  ulonglong2 v;
+  asm volatile("ld.shared.v2.u64 {%0, %1}, [%2];" : "=l"(v.x), "=l"(v.y) : "r"(a));
+  return v;
+}
+
 __device__ __forceinline__ void bar_compute(int nthreads) {  // named barrier 1: compute warps only
   asm volatile("barrier.sync 1, %0;" ::"r"(nthreads) : "memory");
 }
@@ -202,11 +215,12 @@ __device__ __forceinline__ void join_body(const Plan& P) {
     // ---- first probe round's S loads (in flight during the build) --------------------------
     K sk[SPT], sp[SPT];
     auto load_s = [&](unsigned long long base) {
+      const uint32_t rem = (uint32_t)min(job.se - base, (unsigned long long)NT * SPT);
+      const T* src = ssrc + base + threadIdx.x;
       #pragma unroll
       for (int j = 0; j < SPT; ++j) {
-        const unsigned long long s = base + (unsigned long long)j * NT + threadIdx.x;
-        if (s < job.se) {
-          const T t = FUSE ? __ldcg(ssrc + s) : __ldcs(ssrc + s);
+        if ((uint32_t)(j * NT) + threadIdx.x < rem) {
+          const T t = FUSE ? __ldcg(src + j * NT) : __ldcs(src + j * NT);
           sk[j] = TT::key(t);
           sp[j] = TT::pay(t);
         }
@@ -214,21 +228,24 @@ __device__ __forceinline__ void join_body(const Plan& P) {
     };
     T nx[PF ? SPT : 1];  // PF: the next round's tuples
     auto load_next = [&](unsigned long long base) {
+      const uint32_t rem = (uint32_t)min(job.se - base, (unsigned long long)NT * SPT);
+      const T* src = ssrc + base + threadIdx.x;
       #pragma unroll
-      for (int j = 0; j < SPT; ++j) {
-        const unsigned long long s = base + (unsigned long long)j * NT + threadIdx.x;
-        if (s < job.se) nx[j] = FUSE ? __ldcg(ssrc + s) : __ldcs(ssrc + s);
-      }
+      for (int j = 0; j < SPT; ++j)
+        if ((uint32_t)(j * NT) + threadIdx.x < rem) nx[j] = FUSE ? __ldcg(src + j * NT) : __ldcs(src + j * NT);
     };
     load_s(job.sb);
     for (uint32_t i = threadIdx.x; i < nb; i += NT) s_head[i] = NIL16;
     const T* s_rt = s_rtb + (RBUF == 2 ? (it & 1) * cap : 0) + job.shift;
+    const uint32_t s_rt_sh = (uint32_t)__cvta_generic_to_shared(s_rt);
     mbar_wait(&s_bar[it & 1], (it >> 1) & 1);  // R chunk landed (TMA)
     bar_compute(NT);
     // ---- build (a6): wait-free push-front insert (Listing 2) ----------------------
-    for (uint32_t i = threadIdx.x; i < job.nr; i += NT)
-      s_next[i] = H16 ? (uint16_t)exch16(reinterpret_cast<unsigned short*>(&s_head[slot_of(TT::key(s_rt[i]), H)]), i)
-                      : (uint16_t)atomicExch(reinterpret_cast<uint32_t*>(&s_head[slot_of(TT::key(s_rt[i]), H)]), i);
+    for (uint32_t i = threadIdx.x; i < job.nr; i += NT) {
+      const K k = TT::key(lds_tuple(s_rt_sh + i * (uint32_t)sizeof(T), (T*)nullptr));
+      s_next[i] = H16 ? (uint16_t)exch16(reinterpret_cast<unsigned short*>(&s_head[slot_of(k, H)]), i)
+                      : (uint16_t)atomicExch(reinterpret_cast<uint32_t*>(&s_head[slot_of(k, H)]), i);
+    }
     bar_compute(NT);
 
     // ---- probe (a7) + output (a8), SPT tuples per thread per round --------------------------
@@ -257,10 +274,11 @@ __device__ __forceinline__ void join_body(const Plan& P) {
       }
       uint32_t idx[SPT], m[SPT];
       K rfirst[SPT];
+      // this round's tuples in the item (32-bit: rounds hold NT * SPT tuples)
+      const uint32_t rem = (uint32_t)min(job.se - base, (unsigned long long)NT * SPT);
       #pragma unroll
       for (int j = 0; j < SPT; ++j) {
-        const unsigned long long s = base + (unsigned long long)j * NT + threadIdx.x;
-        idx[j] = (s < job.se) ? s_head[slot_of(sk[j], H)] : NIL16;
+        idx[j] = ((uint32_t)(j * NT) + threadIdx.x < rem) ? s_head[slot_of(sk[j], H)] : NIL16;
         m[j] = 0;
       }
       // chains of all SPT tuples advance together (independent shared-memory loads in flight)
@@ -270,7 +288,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
         #pragma unroll
         for (int j = 0; j < SPT; ++j) {
           if (idx[j] != NIL16) {
-            const T r = s_rt[idx[j]];
+            const T r = lds_tuple(s_rt_sh + idx[j] * (uint32_t)sizeof(T), (T*)nullptr);
             if (TT::key(r) == sk[j]) {
               if (MAT) {
                 if (m[j] == 0) rfirst[j] = TT::pay(r);
