@@ -96,6 +96,11 @@ enum hj_option {
                                2 = auto (default: on for 8-byte keys, where it was measured faster) */
   HJ_OPT_PASS1_BITS = 18,   /* radix bits of pass 1 (0 = auto = ceil(B/2)); pass 2 takes the rest.
                                Each pass's fan-out must stay <= 2^10                              */
+  HJ_OPT_PASS_VARIANT = 19, /* partition passes with 1024-thread tiles: either 1024 threads with the
+                               next tile prefetched into registers, or the same tile as 512 threads
+                               x twice the tuples, no register prefetch, two blocks per SM. Value =
+                               1 + mask of the passes using the second form (bit 0 pass 1, bit 1
+                               pass 2); 0 = auto (pass 1 of 8-byte tuples, where it measured faster) */
   HJ_OPT_STREAM_CHUNK = 8   /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
                                least 2^22; >= |S| = copy everything, then join)                   */
 };

@@ -46,6 +46,7 @@ OPT_FUSE_WINDOW_MB = 14
 OPT_FUSE_PASS_SLOTS = 15
 OPT_PASS_L2PF = 17
 OPT_PASS1_BITS = 18
+OPT_PASS_VARIANT = 19
 ALGO_HASH, ALGO_NLJ, ALGO_NONPARTITIONED = 0, 1, 2
 
 _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4: "HJ_ERR_CUDA", -5: "HJ_ERR_COMM"}

@@ -73,7 +73,7 @@ struct Ctx {
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
           opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0, opt_graph = 0, opt_pass_l2pf = 2, opt_pass1_bits = 0,
-          opt_partitioner = 0, opt_fuse = 0, opt_fuse_window_mb = 32, opt_fuse_pass_slots = 1;
+          opt_partitioner = 0, opt_pass_variant = 0, opt_fuse = 0, opt_fuse_window_mb = 32, opt_fuse_pass_slots = 1;
   DevBuf bc_pool1[2], bc_pool2[2], bc_meta;  // HJ_OPT_PARTITIONER = 1 (NEXT-1 bucket chains)
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2], np_heads, np_next;
@@ -321,6 +321,11 @@ int set_kernel_attrs(Ctx* c) {
   attr((const void*)k_pass<K, 1, 512, pass_items<K>(), false, true>);
   attr((const void*)k_pass<K, 2, 1024, pass_items<K>(), false, true>);
   attr((const void*)k_pass<K, 2, 512, pass_items<K>(), false, true>);
+  attr((const void*)k_pass<K, 1, 512, 2 * pass_items<K>(), false, false, false>);
+  attr((const void*)k_pass<K, 1, 512, 2 * pass_items<K>(), true, false, false>);
+  attr((const void*)k_pass<K, 2, 512, 2 * pass_items<K>(), false, false, false>);
+  attr((const void*)k_pass<K, 1, 512, 2 * pass_items<K>(), false, true, false>);
+  attr((const void*)k_pass<K, 2, 512, 2 * pass_items<K>(), false, true, false>);
   attr((const void*)k_fused<K, false>);
   attr((const void*)k_fused<K, true>);
   attr_join<K, 0>(attr);
@@ -544,6 +549,31 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false, 
 template <typename K, int MODE, int NT, bool GD, bool BC>
 int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
   constexpr int IT = pass_items<K>();
+  // HJ_OPT_PASS_VARIANT 1: the 1024 x IT tile as 512 threads x 2 IT without register prefetch,
+  // two blocks per SM (the unit after next still goes to L2 by TMA prefetch)
+  // per pass (bit MODE - 1 of the mask); auto = pass 1 of 8-byte tuples (measured: c5_gpu pass 1
+  // 3.60 -> 3.29 ms, but pass 2 3.24 -> 3.49 and c3 pass 1 0.94 -> 1.00)
+  const int mask = c->opt_pass_variant > 0 ? (int)c->opt_pass_variant - 1 : (c->key_bytes == 8 ? 1 : 0);
+  if (NT == 1024 && ((mask >> (MODE - 1)) & 1) && (1 << fanout_bits) <= 512) {
+    const void* f2 = (const void*)k_pass<K, MODE, 512, 2 * IT, GD, BC, false>;
+    const size_t sm2 = (size_t)NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << fanout_bits) * 24 + 16;
+    const unsigned long long tile2 = (unsigned long long)NT * IT;
+    Plan Q = P;
+    Q.C2 = (uint32_t)tile2;
+    if (c->opt_pass_l2pf == 2) Q.pass_l2pf = 1;
+    unsigned long long units = MODE == 1 ? (P.rel[0].n + tile2 - 1) / tile2 + (P.rel[1].n + tile2 - 1) / tile2
+                                         : (P.rel[0].n + P.rel[1].n) / tile2 + 2ull * hp.npieces() + 2;
+    if (BC && MODE == 2) units = (P.rel[0].n + P.rel[1].n) / tile2 + P.bc_rel[0].nbmax1 + P.bc_rel[1].nbmax1 + 2;
+    if (MODE == 1) {
+      Q.tiles1[0] = (P.rel[0].n + tile2 - 1) / tile2;
+      Q.tiles1[1] = (P.rel[1].n + tile2 - 1) / tile2;
+    }
+    int g = grid_for(c, f2, 512, sm2, units);
+    k_pass<K, MODE, 512, 2 * IT, GD, BC, false><<<g, 512, sm2, c->stream>>>(Q, fanout_bits);
+    CUDA_TRY(c, cudaGetLastError());
+    c->launches += 1;
+    return HJ_OK;
+  }
   const void* f = (const void*)k_pass<K, MODE, NT, IT, GD, BC>;
   const size_t sm = (size_t)NT * IT * sizeof(typename Tup<K>::T) + ((size_t)1 << fanout_bits) * 24 + 16;
   const unsigned long long tile = (unsigned long long)NT * IT;
@@ -1365,6 +1395,10 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_JOIN_ALGO:
       if (v > 2) return fail(c, HJ_ERR_INVALID, "join algorithm must be 0, 1 or 2");
       c->opt_join_algo = v;
+      break;
+    case HJ_OPT_PASS_VARIANT:
+      if (v < 0 || v > 4) return fail(c, HJ_ERR_INVALID, "pass variant must be 0..4");
+      c->opt_pass_variant = v;
       break;
     case HJ_OPT_PASS_THREADS:
       if (v != 0 && v != 512 && v != 1024) return fail(c, HJ_ERR_INVALID, "pass threads must be 0, 512 or 1024");

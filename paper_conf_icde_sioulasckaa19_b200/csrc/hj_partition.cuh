@@ -547,7 +547,10 @@ __device__ __noinline__ void bc_pass2_units(const BcRel* s_bc, const uint32_t* c
 // counter, issued one iteration later, when the stores have long been acknowledged); T2 stores
 // are plain write-back stores so the co-partitions stay in L2 for the join; a unit more than
 // fz_window pieces ahead of the join's completed items waits (bounds the L2 footprint).
-template <typename K, int MODE, int NT, int ITEMS, bool GD, bool BC = false, bool FUSE = false>
+// RPF: the next unit's tuples are prefetched into registers during the current unit (default);
+// RPF = false loads each unit at the top of its iteration (half the data registers: twice the
+// tuples per thread at the same register budget, for two blocks per SM whose barriers overlap).
+template <typename K, int MODE, int NT, int ITEMS, bool GD, bool BC = false, bool FUSE = false, bool RPF = true>
 __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
   static_assert(!FUSE || (MODE == 2 && !BC && !GD), "fused pass 2 only");
   using TT = Tup<K>;
@@ -639,9 +642,11 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
       red_add_gpu(&P.fz[FZ_DONE + grp], 1u);
     }
   };
-  K kk[ITEMS], pp[ITEMS], kn[ITEMS], pn[ITEMS];
+  K kk[ITEMS], pp[ITEMS], kn[RPF ? ITEMS : 1], pn[RPF ? ITEMS : 1];
   unsigned long long u = blockIdx.x;
-  if (s_desc[0].valid) pass_load<K, MODE, NT, ITEMS>(s_desc[0], kn, pn);
+  if constexpr (RPF) {
+    if (s_desc[0].valid) pass_load<K, MODE, NT, ITEMS>(s_desc[0], kn, pn);
+  }
   uint32_t it = 0, slot = 0;
 
   auto write_out = [&](const unsigned long long* gd) {
@@ -668,14 +673,20 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
 
   while (s_desc[slot].valid) {
     const uint32_t nslot = slot == 2 ? 0 : slot + 1;
-    #pragma unroll
-    for (int j = 0; j < ITEMS; ++j) {
-      kk[j] = kn[j];
-      pp[j] = pn[j];
+    if constexpr (RPF) {
+      #pragma unroll
+      for (int j = 0; j < ITEMS; ++j) {
+        kk[j] = kn[j];
+        pp[j] = pn[j];
+      }
+    } else {
+      pass_load<K, MODE, NT, ITEMS>(s_desc[slot], kk, pp);
     }
     if (FUSE && sig) signal(sig_grp);  // before the prefetch: the fence then waits only for old stores
     // prefetch the next unit (in flight across this unit's barriers)
-    if (s_desc[nslot].valid) pass_load<K, MODE, NT, ITEMS>(s_desc[nslot], kn, pn);
+    if constexpr (RPF) {
+      if (s_desc[nslot].valid) pass_load<K, MODE, NT, ITEMS>(s_desc[nslot], kn, pn);
+    }
 
     // ---- phase 1: rank ------------------------------------------------------------------------
     // elements past the unit's end count into the spare counter s_cnt[F] (no branches)
@@ -800,9 +811,9 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
   }
 }
 
-template <typename K, int MODE, int NT, int ITEMS, bool GD, bool BC = false>
+template <typename K, int MODE, int NT, int ITEMS, bool GD, bool BC = false, bool RPF = true>
 __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits) {
-  pass_body<K, MODE, NT, ITEMS, GD, BC, false>(P, fanout_bits);
+  pass_body<K, MODE, NT, ITEMS, GD, BC, false, RPF>(P, fanout_bits);
 }
 
 // ------------------------------------------------------------------------------------------

@@ -569,3 +569,23 @@ def test_fused_equals_unfused_and_repeats(hj):
         pairs = oracle.pairs_sorted(to_np(rm.r_pay, 4), to_np(rm.s_pay, 4))
         assert int(np_sig(pairs[:, 0], pairs[:, 1]).sum(dtype=np.uint64)) == ref[1]
     ctx.close()
+
+
+@pytest.mark.parametrize("variant", [1, 2, 3, 4])
+def test_pass_variant_invariance(hj, variant):
+    """HJ_OPT_PASS_VARIANT (1024-thread register-prefetch tiles vs 512 threads x twice the tuples,
+    per pass) never changes results: skewed, duplicate-heavy and ragged inputs, 4/4 and 8/8."""
+    rng = np.random.default_rng(70 + variant)
+    for kb in (4, 8):
+        ctx = hj.Context(0, kb, kb)
+        ctx.set_option(hj.OPT_PASS_VARIANT, variant)
+        dt = np.uint32 if kb == 4 else np.uint64
+        w = W.Workload("pv", 70001, 90011, "zipf", keys="sparse" if kb == 4 else "k8", z=1.3, seed=420 + variant)
+        Rk, Rp, Sk, Sp = W.np_generate(w)
+        for bits in (-1, 9, 16):
+            check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=bits == 9, ctx=ctx)
+        Rk = rng.integers(0, 900, 20000).astype(dt)
+        Sk = rng.integers(0, 900, 15000).astype(dt)
+        check_against_oracle(hj, Rk, np.arange(len(Rk), dtype=dt), Sk, np.arange(len(Sk), dtype=dt), bits=18,
+                             mat=True, ctx=ctx)
+        ctx.close()

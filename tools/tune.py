@@ -18,7 +18,8 @@ OPTS = {"join_variant": hj.OPT_JOIN_VARIANT, "cap_r": hj.OPT_CAP_R, "chunk_s": h
         "stream_chunk": hj.OPT_STREAM_CHUNK, "pass1_bases": hj.OPT_PASS1_BASES,
         "partitioner": hj.OPT_PARTITIONER, "fuse": hj.OPT_FUSE,
         "fuse_window_mb": hj.OPT_FUSE_WINDOW_MB, "fuse_pass_slots": hj.OPT_FUSE_PASS_SLOTS,
-        "pass_l2pf": hj.OPT_PASS_L2PF, "pass1_bits": hj.OPT_PASS1_BITS}
+        "pass_l2pf": hj.OPT_PASS_L2PF, "pass1_bits": hj.OPT_PASS1_BITS,
+        "pass_variant": hj.OPT_PASS_VARIANT}
 
 
 def main():
