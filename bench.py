@@ -254,6 +254,21 @@ def main():
         return hjdist.join(Rk, Rp, Sk, Sp, local_bits=local_bits, out_mode=w.out_mode, ctx=ctx,
                            exchange=args.exchange)
 
+    exchange_note = None
+    if use_dist and args.exchange == "direct":
+        # the direct store needs every peer's windows mapped through CUDA IPC; where a launcher
+        # hides the peers' devices that cannot work: then every rank switches to the NCCL
+        # all-to-all exchange together (decided by an all-reduce, so no rank is left waiting)
+        ok = torch.ones(1, device=dev)
+        try:
+            step()
+        except Exception as e:  # HJError from hj_ipc_open / hj_xd_join
+            ok.zero_()
+            exchange_note = f"direct store unavailable ({str(e)[:120]}); NCCL all_to_all used"
+        torch.distributed.all_reduce(ok, op=torch.distributed.ReduceOp.MIN)
+        if ok.item() == 0:
+            args.exchange = "nccl"
+            exchange_note = exchange_note or "direct store unavailable on a peer; NCCL all_to_all used"
     for _ in range(args.warmup):
         res = step()
     assert res.matches == w.nS, "closed form: FK / 1:1 joins produce |S| matches"
@@ -324,6 +339,8 @@ def main():
                          else "over NCCL all_to_all") + ", per-rank 2-pass join"},
            "roofline": roof, "roofline_path": roof_path, "kernels_ms": kms, "clocks": clk.summary(),
            "gpu_launches": launches}
+    if use_dist:
+        out["config"]["exchange"] = args.exchange + (f" ({exchange_note})" if exchange_note else "")
     if use_dist:
         out["nvlink"] = {"bytes_sent_per_gpu_per_step": sent / args.steps,
                          "achieved_GBps": sent / args.steps / (ms * 1e-3) / 1e9, "peak_GBps": 900.0,
