@@ -72,8 +72,10 @@ enum hj_option {
                                TMA bulk-store write-out instead of atomic run reservation (opt-in;
                                measured slower on B200, kept for comparison)                      */
   HJ_OPT_GRAPH = 11,        /* 1 = hj_join captures its launch sequence in a CUDA graph and replays
-                               it while the call signature is unchanged (launch-bound small joins;
-                               per-kernel ms_kernel are not reported in this mode)               */
+                               it while the call signature is unchanged (launch gaps and host
+                               preparation leave the critical path: c3 2.73 -> 2.68 ms/call; only
+                               ms_total is reported in this mode). Any hj_set_option call drops
+                               the captured graph                                                */
   HJ_OPT_PARTITIONER = 12,  /* hj_join only: 0 = histogram + prefix sum + exact placement (north
                                star, default); 1 = the paper's histogram-free bucket chains
                                (NEXT-1): no histogram pass, partitions are chains of

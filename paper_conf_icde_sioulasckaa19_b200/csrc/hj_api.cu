@@ -98,6 +98,7 @@ struct Ctx {
   unsigned long long xd_epoch = 0;
   cudaGraphExec_t graph = nullptr;
   unsigned long long graph_key[12] = {};
+  bool capturing = false;  // a graph capture is in progress on c->stream
   uint32_t graph_launches = 0;
 };
 
@@ -448,7 +449,9 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
 }
 
 void mark(Ctx* c, int i) {
-  if (c->opt_timing) cudaEventRecord(c->ev[i], c->stream);
+  // inside a graph capture the record must be an external event-record node to be timed
+  if (c->opt_timing)
+    cudaEventRecordWithFlags(c->ev[i], c->stream, c->capturing ? cudaEventRecordExternal : cudaEventRecordDefault);
 }
 
 // a1 (histogram), a2/a5 (planner), a3 (pass 1). PLAN_RECV skips a1 and a3 (counts and the
@@ -769,6 +772,7 @@ int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res, b
     cudaEventElapsedTime(&res->ms_partition, c->ev[0], c->ev[4]);
     cudaEventElapsedTime(&res->ms_join, c->ev[4], c->ev[6]);
     for (int k = 0; k < 5; ++k) cudaEventElapsedTime(&res->ms_kernel[k], c->ev[k], c->ev[k + 1]);
+    cudaGetLastError();  // a phase that recorded no event (e.g. skipped) must not fail the next call
   }
   return HJ_OK;
 }
@@ -864,10 +868,13 @@ int run_join_graph_on(Ctx* c, HostPlan& hp, Plan& P, bool mat, const unsigned lo
   if (!c->graph || memcmp(key, c->graph_key, sizeof c->graph_key) != 0) {
     if (c->graph) cudaGraphExecDestroy(c->graph);
     c->graph = nullptr;
+    // no event records inside the capture: as external event-record nodes they cost the replay
+    // its gain (c3: 2.69 -> 2.74-2.89 ms/call, measured), so a replay reports ms_total only
     const int64_t timing = c->opt_timing;
-    c->opt_timing = 0;  // no event records inside the capture
+    c->opt_timing = 0;
     c->launches = 0;
     CUDA_TRY(c, cudaStreamBeginCapture(st, cudaStreamCaptureModeThreadLocal));
+    c->capturing = true;
     int rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P);
     if (!rc) rc = c->key_bytes == 4 ? launch_pass2<uint32_t>(c, hp, P) : launch_pass2<uint64_t>(c, hp, P);
     if (!rc) rc = c->key_bytes == 4 ? launch_join<uint32_t>(c, hp, P, mat) : launch_join<uint64_t>(c, hp, P, mat);
@@ -877,6 +884,7 @@ int run_join_graph_on(Ctx* c, HostPlan& hp, Plan& P, bool mat, const unsigned lo
       rc = fail(c, HJ_ERR_CUDA, "capture: items copy");
     cudaGraph_t g = nullptr;
     cudaError_t e = cudaStreamEndCapture(st, &g);
+    c->capturing = false;
     c->opt_timing = timing;
     if (rc) {
       if (g) cudaGraphDestroy(g);
@@ -1368,6 +1376,10 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
   if (!h) return HJ_ERR_INVALID;
   Ctx* c = &h->c;
   if (v < 0) return fail(c, HJ_ERR_INVALID, "negative option value");
+  if (c->graph) {  // any option may change the captured launch sequence: capture again
+    cudaGraphExecDestroy(c->graph);
+    c->graph = nullptr;
+  }
   switch (opt) {
     case HJ_OPT_CAP_R: c->opt_cap_r = v; break;
     case HJ_OPT_CHUNK_S: c->opt_chunk_s = v; break;

@@ -499,6 +499,7 @@ def test_graph_replay_matches_oracle(hj):
         for _ in range(3):
             res = ctx.join(*cols)
             assert (res.matches, res.checksum) == (m, c)
+            assert res.ms_total > 0
         for _ in range(2):
             res = ctx.join(*cols, out_mode=hj.OUT_MATERIALIZE)
             assert res.matches == m
