@@ -702,23 +702,30 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
         if (j & 1) rk[j / 2] |= r << 16; else rk[j / 2] = r & 0xffffu;
       }
     } else {
-      // skew: lanes on the hot digit are ranked with one ballot + one atomic per warp instead
-      // of serialising on the same shared counter (Zipf probe sides)
+      // skew: lanes on the hot digit do not touch its shared counter item by item (same-address
+      // atomics serialise); they are ranked inside the warp by ballot + popc, the warp reserves
+      // its hot total with ONE atomic after all ITEMS and adds that base to its hot items' ranks
+      // (Zipf probe sides). Branch-free per item: the other lanes' atomic is
+      // the only per-item shared-memory access.
+      uint32_t hacc = 0, hbits = 0;  // this warp's hot items so far; this thread's hot items (bit j)
+      const uint32_t lt = lanemask_lt();
       #pragma unroll
       for (int j = 0; j < ITEMS; ++j) {
         const uint32_t d = (full || pass_elem<K, MODE, NT>(j) < ulen) ? digit(kk[j]) : F;
-        const uint32_t hm = __ballot_sync(0xffffffffu, d == hot);
-        uint32_t r;
-        if (hm) {
-          const int leader = __ffs(hm) - 1;
-          uint32_t base = 0;
-          if (lane == leader) base = atomicAdd(&s_cnt[hot], (uint32_t)__popc(hm));
-          base = __shfl_sync(0xffffffffu, base, leader);
-          r = (d == hot) ? base + __popc(hm & lanemask_lt()) : atomicAdd(&s_cnt[d], 1u);
-        } else {
-          r = atomicAdd(&s_cnt[d], 1u);
-        }
+        const bool ih = d == hot;
+        const uint32_t hm = __ballot_sync(0xffffffffu, ih);
+        const uint32_t r = ih ? hacc + __popc(hm & lt) : atomicAdd(&s_cnt[d], 1u);
+        hacc += __popc(hm);
+        hbits |= (uint32_t)ih << j;
         if (j & 1) rk[j / 2] |= r << 16; else rk[j / 2] = r & 0xffffu;
+      }
+      if (hacc) {  // warp-uniform
+        uint32_t base = 0;
+        if (lane == 0) base = atomicAdd(&s_cnt[hot], hacc);
+        base = __shfl_sync(0xffffffffu, base, 0);
+        #pragma unroll
+        for (int j = 0; j < ITEMS; ++j)
+          if ((hbits >> j) & 1) rk[j / 2] += base << (16 * (j & 1));
       }
     }
     __syncthreads();
