@@ -47,7 +47,15 @@ constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1, 1}, {256, 8, 2, 2, 1}, {224,
                                      {256, 4, 3, 1, 1, false, true, true},
                                      {256, 6, 3, 1, 1, false, true, true, 4}, {256, 8, 3, 1, 1, false, false, true, 4},
                                      {256, 4, 3, 1, 1, false, true, true, 4}, {256, 6, 3, 1, 1, false, true, true, 8},
-                                     {256, 6, 3, 1, 1, false, true, true, 2}, {256, 8, 3, 1, 1, false, false, true, 2}};
+                                     {256, 6, 3, 1, 1, false, true, true, 2}, {256, 8, 3, 1, 1, false, false, true, 2},
+                                     {512, 4, 2, 1, 1, false, true, true}, {512, 2, 2, 1, 1, false, true, true},
+                                     {384, 4, 2, 1, 1, false, true, true}, {384, 2, 2, 1, 1, false, true, true},
+                                     {512, 4, 2, 1, 1, true, true, true}, {512, 2, 2, 1, 1, false, false, true},
+                                     {512, 2, 2, 1, 1, false, true, true, 2}, {640, 2, 2, 1, 1, false, true, true},
+                                     {640, 1, 2, 1, 1, false, true, true}, {512, 1, 2, 1, 1, false, true, true},
+                                     {768, 1, 2, 1, 1, false, true, true}, {512, 1, 2, 1, 1, false, false, true},
+                                     {512, 2, 3, 1, 1, false, true, true}, {512, 1, 3, 1, 1, false, true, true},
+                                     {384, 1, 4, 1, 1, false, true, true}};
 constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
 
@@ -176,10 +184,16 @@ constexpr int pass_items() {
 //   4 B count       -> shape 20 (256 x 6, S prefetch + L2 prefetch: c2 0.873 -> 0.814 ms,
 //                      c4 z=1.5 0.881 -> 0.829; streaming S through L2 2-8 rounds ahead, shapes
 //                      22/25/26, is slower here: 0.84 -- this probe is issue-bound on the checksum)
-//   8 B             -> shape 21 (256 x 4, S prefetch + L2 prefetch: c5_gpu 4.21 -> 4.03 ms)
+//   8 B             -> shape 37 (512 x 1, S and L2 prefetch, two blocks per SM: the 16-byte R
+//                      tile limits blocks to two per SM, so more threads per block -- not more
+//                      tuples per thread -- hide the chain-walk latency: c5_gpu join 3.54 ->
+//                      2.69 ms; 512 x 2: 2.90, 640 x 1: 2.85, 768 x 1: 3.34, 384 x 2: 2.98;
+//                      shape 21 = 256 x 4: 4.21 -> 4.03 before the 32-bit-shared-address probe,
+//                      3.54 after). For 4-byte tuples three 256-thread blocks per SM fit and the
+//                      512-thread shapes are slower (c2 0.74 -> 0.95, c3 0.645 -> 0.86)
 int join_variant(const Ctx* c, bool mat) {
   if (c->opt_join_variant >= 0) return (int)c->opt_join_variant;
-  if (c->key_bytes == 8) return 21;
+  if (c->key_bytes == 8) return 37;
   return mat ? 27 : 20;
 }
 
@@ -357,6 +371,21 @@ int set_kernel_attrs(Ctx* c) {
   attr_join<K, 25>(attr);
   attr_join<K, 26>(attr);
   attr_join<K, 27>(attr);
+  attr_join<K, 28>(attr);
+  attr_join<K, 29>(attr);
+  attr_join<K, 30>(attr);
+  attr_join<K, 31>(attr);
+  attr_join<K, 32>(attr);
+  attr_join<K, 33>(attr);
+  attr_join<K, 34>(attr);
+  attr_join<K, 35>(attr);
+  attr_join<K, 36>(attr);
+  attr_join<K, 37>(attr);
+  attr_join<K, 38>(attr);
+  attr_join<K, 39>(attr);
+  attr_join<K, 40>(attr);
+  attr_join<K, 41>(attr);
+  attr_join<K, 42>(attr);
   return rc;
 }
 
@@ -635,6 +664,21 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
     return HJ_OK;
   }
   switch (join_variant(c, mat)) {
+    case 38: rc = launch_join_v<K, 38>(c, hp, P, mat); break;
+    case 39: rc = launch_join_v<K, 39>(c, hp, P, mat); break;
+    case 40: rc = launch_join_v<K, 40>(c, hp, P, mat); break;
+    case 41: rc = launch_join_v<K, 41>(c, hp, P, mat); break;
+    case 42: rc = launch_join_v<K, 42>(c, hp, P, mat); break;
+    case 33: rc = launch_join_v<K, 33>(c, hp, P, mat); break;
+    case 34: rc = launch_join_v<K, 34>(c, hp, P, mat); break;
+    case 35: rc = launch_join_v<K, 35>(c, hp, P, mat); break;
+    case 36: rc = launch_join_v<K, 36>(c, hp, P, mat); break;
+    case 37: rc = launch_join_v<K, 37>(c, hp, P, mat); break;
+    case 28: rc = launch_join_v<K, 28>(c, hp, P, mat); break;
+    case 29: rc = launch_join_v<K, 29>(c, hp, P, mat); break;
+    case 30: rc = launch_join_v<K, 30>(c, hp, P, mat); break;
+    case 31: rc = launch_join_v<K, 31>(c, hp, P, mat); break;
+    case 32: rc = launch_join_v<K, 32>(c, hp, P, mat); break;
     case 22: rc = launch_join_v<K, 22>(c, hp, P, mat); break;
     case 23: rc = launch_join_v<K, 23>(c, hp, P, mat); break;
     case 24: rc = launch_join_v<K, 24>(c, hp, P, mat); break;
