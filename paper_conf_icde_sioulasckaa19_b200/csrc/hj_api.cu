@@ -55,7 +55,8 @@ constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1, 1}, {256, 8, 2, 2, 1}, {224,
                                      {640, 1, 2, 1, 1, false, true, true}, {512, 1, 2, 1, 1, false, true, true},
                                      {768, 1, 2, 1, 1, false, true, true}, {512, 1, 2, 1, 1, false, false, true},
                                      {512, 2, 3, 1, 1, false, true, true}, {512, 1, 3, 1, 1, false, true, true},
-                                     {384, 1, 4, 1, 1, false, true, true}};
+                                     {384, 1, 4, 1, 1, false, true, true}, {256, 6, 4, 1, 1, true, true, true},
+                                     {224, 6, 4, 1, 1, true, true, true}, {256, 4, 4, 1, 1, true, true, true}};
 constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
 
@@ -386,6 +387,9 @@ int set_kernel_attrs(Ctx* c) {
   attr_join<K, 40>(attr);
   attr_join<K, 41>(attr);
   attr_join<K, 42>(attr);
+  attr_join<K, 43>(attr);
+  attr_join<K, 44>(attr);
+  attr_join<K, 45>(attr);
   return rc;
 }
 
@@ -664,6 +668,9 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
     return HJ_OK;
   }
   switch (join_variant(c, mat)) {
+    case 43: rc = launch_join_v<K, 43>(c, hp, P, mat); break;
+    case 44: rc = launch_join_v<K, 44>(c, hp, P, mat); break;
+    case 45: rc = launch_join_v<K, 45>(c, hp, P, mat); break;
     case 38: rc = launch_join_v<K, 38>(c, hp, P, mat); break;
     case 39: rc = launch_join_v<K, 39>(c, hp, P, mat); break;
     case 40: rc = launch_join_v<K, 40>(c, hp, P, mat); break;

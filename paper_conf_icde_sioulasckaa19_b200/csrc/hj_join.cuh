@@ -281,9 +281,31 @@ __device__ __forceinline__ void join_body(const Plan& P) {
         idx[j] = ((uint32_t)(j * NT) + threadIdx.x < rem) ? s_head[slot_of(sk[j], H)] : NIL16;
         m[j] = 0;
       }
+      // first chain step of every tuple without branches (unique build keys: chains of length
+      // <= 1, so this is usually the whole probe): the head's tuple is read even for an empty
+      // slot (index 0 instead, discarded), the signature is computed for every tuple and added
+      // only on a hit; the general walk below runs only while some lane still has a chain
+      // (4-byte tuples; for 8-byte tuples the branchy walk below measured faster: c5_gpu join
+      // 2.69 vs 2.84-2.90 ms)
+      bool live = sizeof(K) != 4;
+      #pragma unroll
+      for (int j = 0; j < SPT && sizeof(K) == 4; ++j) {
+        const bool v = idx[j] != NIL16;
+        const uint32_t i0 = v ? idx[j] : 0u;
+        const T r = lds_tuple(s_rt_sh + i0 * (uint32_t)sizeof(T), (T*)nullptr);
+        const bool hit = v && TT::key(r) == sk[j];
+        if (MAT) {
+          rfirst[j] = TT::pay(r);
+        } else {
+          const uint64_t sg = pair_sig((uint64_t)TT::pay(r), (uint64_t)sp[j]);
+          my_chk += hit ? sg : 0ull;
+        }
+        m[j] = hit ? 1u : 0u;
+        idx[j] = v ? (uint32_t)s_next[i0] : NIL16;
+        live |= idx[j] != NIL16;
+      }
       // chains of all SPT tuples advance together (independent shared-memory loads in flight)
-      bool live = true;
-      while (live) {
+      while (sizeof(K) == 4 ? __any_sync(0xffffffffu, live) : live) {
         live = false;
         #pragma unroll
         for (int j = 0; j < SPT; ++j) {
