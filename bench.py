@@ -46,6 +46,9 @@ def parse():
     ap.add_argument("--clock-period", type=float, default=0.01,
                     help="NVML clock / throttle sampling period (s) during the timed region; 0 = off (testing only)")
     ap.add_argument("--dist", action="store_true", help="use the multi-GPU exchange path even at N=1")
+    ap.add_argument("--debug-one-device", action="store_true",
+                    help="testing only: every rank on cuda:0 with a gloo process group (validates the multi-rank "
+                         "flow on a one-GPU box; not a scaling measurement)")
     ap.add_argument("--exchange", default="direct", choices=["direct", "nccl"],
                     help="multi-GPU exchange: direct = pass 1 stores into the owners' windows over peer memory "
                          "(hj_xd_*); nccl = pack + NCCL all_to_all (hj_exchange_pack)")
@@ -137,10 +140,10 @@ class ClockSampler:
         return {"sm_mhz": med, "sm_max_mhz": self.max_mhz, "reasons": sorted(self.reasons), "samples": len(self.samples)}
 
 
-def dist_env():
+def dist_env(one_device: bool = False):
     ws = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
-    local = int(os.environ.get("LOCAL_RANK", "0"))
+    local = 0 if one_device else int(os.environ.get("LOCAL_RANK", "0"))
     return ws, rank, local
 
 
@@ -218,7 +221,7 @@ def main():
 
     import torch
 
-    ws, rank, local = dist_env()
+    ws, rank, local = dist_env(args.debug_one_device)
     use_dist = ws > 1 or args.dist
     if use_dist:
         import torch.distributed as dist
@@ -229,7 +232,7 @@ def main():
             os.environ.setdefault("MASTER_PORT", "29531")
             os.environ.setdefault("RANK", "0")
             os.environ.setdefault("WORLD_SIZE", "1")
-        dist.init_process_group("nccl")
+        dist.init_process_group("gloo" if args.debug_one_device else "nccl")
     dev = torch.device("cuda", local)
     torch.cuda.set_device(dev)
     import paper_conf_icde_sioulasckaa19_b200 as hj
@@ -259,7 +262,7 @@ def main():
         # the direct store needs every peer's windows mapped through CUDA IPC; where a launcher
         # hides the peers' devices that cannot work: then every rank switches to the NCCL
         # all-to-all exchange together (decided by an all-reduce, so no rank is left waiting)
-        ok = torch.ones(1, device=dev)
+        ok = torch.ones(1, device="cpu" if args.debug_one_device else dev)
         try:
             step()
         except Exception as e:  # HJError from hj_ipc_open / hj_xd_join
@@ -297,7 +300,7 @@ def main():
         barrier()
     ms = e0.elapsed_time(e1) / args.steps
     if use_dist:
-        t = torch.tensor([ms], device=dev)
+        t = torch.tensor([ms], device="cpu" if args.debug_one_device else dev)
         torch.distributed.all_reduce(t, op=torch.distributed.ReduceOp.MAX)
         ms = float(t.item())
     per_k /= args.steps

@@ -81,6 +81,18 @@ def _allgather_u64(arr: np.ndarray, group, dev) -> np.ndarray:
     return out.cpu().numpy().view(np.uint64).reshape(G, *arr.shape)
 
 
+def _a2a(out, inp, out_split, in_split, group):
+    """all_to_all_single; under gloo (CPU collectives, tests) CUDA tensors travel through host copies."""
+    import torch.distributed as dist
+
+    if out.is_cuda and dist.get_backend(group) != "nccl":
+        o = out.cpu()
+        dist.all_to_all_single(o, inp.cpu(), out_split, in_split, group=group)
+        out.copy_(o)
+        return
+    dist.all_to_all_single(out, inp, out_split, in_split, group=group)
+
+
 class DirectExchange:
     """Direct-store exchange state of one rank (include/hj.h hj_xd_*): its context, its three
     windows (R receive, S receive, barrier flags), the peers' windows mapped into this process,
@@ -210,12 +222,12 @@ def join(Rk, Rp, Sk, Sp, group=None, local_bits: int = -1, out_mode: int = 0, ct
     for rel, (k, p) in enumerate(((Rk, Rp), (Sk, Sp))):
         send, cnt, dest = ctx.exchange_pack(rel, k, p, g, local_bits)
         cnt_recv = torch.empty_like(cnt)
-        dist.all_to_all_single(cnt_recv, cnt, group=group)
+        _a2a(cnt_recv, cnt, None, None, group)
         in_split = [int(x) * words_per_tuple for x in dest]
         out_tuples = [int(x) for x in cnt_recv.view(G, -1).to(torch.int64).sum(1).tolist()]
         out_split = [x * words_per_tuple for x in out_tuples]
         buf = torch.empty(sum(out_split), dtype=torch.int64, device=dev)
-        dist.all_to_all_single(buf, send[: sum(in_split)], out_split, in_split, group=group)
+        _a2a(buf, send[: sum(in_split)], out_split, in_split, group)
         sent += (sum(int(x) for x in dest) - int(dest[rank])) * tb
         recv.append((buf, sum(out_tuples), cnt_recv.contiguous()))
     (rb, nr, rc), (sb, ns, sc) = recv

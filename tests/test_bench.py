@@ -6,6 +6,7 @@ import subprocess
 import sys
 
 import numpy as np
+import pytest
 
 import oracle
 import workloads as W
@@ -45,3 +46,37 @@ def test_reference_arm_runs_on_cpu():
     assert d["impl"] == "reference" and d["value"] > 0 and d["unit"] == "tuples/s"
     assert d["cpu_baseline"]["kind"] == "oracle" and d["cpu_baseline"]["cores"] == 1
     assert d["e2e"]["h2d_bytes_per_step"] == 0
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("exchange", ["direct", "nccl"])
+def test_bench_multi_rank_flow_on_one_gpu(exchange):
+    """bench.py --gpus 2 under torchrun, both ranks on cuda:0 (--debug-one-device, gloo): the
+    multi-rank flow the driver's scaling run uses -- row sharding, the exchange (direct: windows
+    over CUDA IPC between the two processes), max-over-ranks timing, one JSON line from rank 0
+    with the NVLink byte count -- with the closed-form check (matches = |S|) inside bench.py."""
+    import json
+    import socket
+    import subprocess
+    import sys
+
+    import torch
+
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    port = s.getsockname()[1]
+    s.close()
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", "--nproc-per-node", "2", "--master-addr",
+           "127.0.0.1", "--master-port", str(port), os.path.join(root, "bench.py"), "--gpus", "2",
+           "--debug-one-device", "--config", "c1", "--exchange", exchange, "--steps", "3", "--warmup", "3",
+           "--no-e2e", "--no-cpu-baseline", "--clock-period", "0"]
+    out = subprocess.run(cmd, capture_output=True, text=True, timeout=600, cwd=root)
+    assert out.returncode == 0, out.stderr[-4000:]
+    lines = [ln for ln in out.stdout.splitlines() if ln.startswith("{")]
+    assert len(lines) == 1, out.stdout[-2000:]
+    d = json.loads(lines[0])
+    assert d["n_gpus"] == 2 and d["value"] > 0 and d["config"]["exchange"].startswith(exchange)
+    assert d["nvlink"]["bytes_sent_per_gpu_per_step"] > 0
