@@ -194,7 +194,9 @@ int hj_partition(hj_ctx* ctx, const void* keys, const void* pays, uint64_t n, in
  *   *counts_out: device, [G][2^local_bits] uint32 per-co-partition counts (q-order, see the
  *                implementation notes in DESIGN.md §7); row j goes to rank j. ctx-owned.
  *   dest_counts: HOST array of G uint64 (caller-allocated): tuples destined to each rank.
- * Requires gpu_bits + ceil(local_bits / 2) <= 10. */
+ * The pass-1 digit gets b1 = min(ceil(local_bits / 2), 10 - gpu_bits) local bits (pass 2 the
+ * rest, which must stay <= 10), so the fan-out stays <= 2^10 and hj_join_received with
+ * nsrc = 2^gpu_bits derives the same split. */
 int hj_exchange_pack(hj_ctx* ctx, int rel, const void* keys, const void* pays, uint64_t n, int gpu_bits,
                      int local_bits, const void** send_out, const uint32_t** counts_out, uint64_t* dest_counts);
 
@@ -233,7 +235,8 @@ int hj_join_received(hj_ctx* ctx, const void* R_recv, uint64_t nR, const uint32_
  *               sum_{s' < s} totals[r][s'][j] tuples and is grouped by the local pass-1 digit.
  * Board window (slot 2, HJ_XD_BOARD_BYTES): starts with uint64[HJ_XD_MAX_RANKS] barrier flags,
  * flag s = last barrier epoch source s reached (the rest serves hj_xd_join).
- * Requires G <= HJ_XD_MAX_RANKS and gpu_bits + ceil(local_bits / 2) <= 10. */
+ * Requires G <= HJ_XD_MAX_RANKS; the pass split is hj_exchange_pack's (b1 = min(ceil(local_bits
+ * / 2), 10 - gpu_bits)). */
 #define HJ_XD_MAX_RANKS 64
 /* Board window (slot 2) bytes: barrier / phase flags, the totals board [src][2][dst] and the
  * results board [src][2] of hj_xd_join, all uint64. */

@@ -219,6 +219,11 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   if (hp.B > 20) return fail(c, HJ_ERR_UNSUPPORTED, "radix_bits %d > 20", hp.B);
   hp.b1 = (hp.B + 1) / 2;  // reading S6; HJ_OPT_PASS1_BITS overrides (results never change)
   if (c->opt_pass1_bits > 0 && hp.B >= 2) hp.b1 = (int)std::min<int64_t>(c->opt_pass1_bits, hp.B - 1);
+  // multi-GPU: pass 1's fan-out (rank bits + b1) and the receiver's pass-2 pieces
+  // (sources x 2^b1) stay <= 2^10, so b1 = min(ceil(B/2), 10 - log2 G); sender (g rank bits)
+  // and receiver (nsrc = G sources) derive the same b1 (c5 at G = 8: B = 16 -> 7 + 9)
+  const int gl = std::max(g, ilog2_ceil((unsigned long long)std::max(nsrc, 1)));
+  if (gl > 0 && hp.b1 > 10 - gl) hp.b1 = std::max(0, 10 - gl);
   hp.b2 = hp.B - hp.b1;
   hp.g = g;
   hp.nsrc = nsrc;

@@ -624,3 +624,19 @@ def test_gpu_xd_join_regrow_and_8byte():
     m, c = oracle.hash_join(*cols)
     for outs in calls:
         assert all(o[0] == 0 and o[3] == (m, c) for o in outs)
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("G,lb", [(8, 16), (4, 17), (2, 18)])
+def test_gpu_exchange_c5_local_bits(G, lb):
+    """The local radix bits c5 needs at G = 2/4/8 (2^31 rows: 18/17/16 bits): the pass-1 fan-out
+    (rank bits + b1) and the receiver's pieces stay <= 2^10 by b1 = min(ceil(B/2), 10 - log2 G),
+    on both exchange paths, 8-byte tuples."""
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_icde_sioulasckaa19_b200 as hj
+
+    w = W.Workload("c5s", 1 << 15, 1 << 15, "1to1", keys="k8", seed=198)
+    cols, calls = _xd_join_threads(hj, w, G, lb, 0, width=8, calls=1, cap_scale=2.0)
+    m, c = oracle.hash_join(*cols)
+    assert all(o[0] == 0 and o[3] == (m, c) for o in calls[0])
