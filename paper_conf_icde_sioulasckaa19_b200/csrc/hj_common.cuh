@@ -210,4 +210,44 @@ __device__ __forceinline__ unsigned long long block_exclusive_scan64(unsigned lo
   return res;
 }
 
+// M independent 64-bit exclusive scans in one pass (one pair of barriers instead of M): v[m] ->
+// exclusive prefix of v[m] over the block, total[m] = block sum. tmp: >= M * (NT / 32 + 1).
+template <int NT, int M>
+__device__ __forceinline__ void block_exclusive_scan64xM(unsigned long long (&v)[M], unsigned long long* tmp,
+                                                         unsigned long long (&total)[M]) {
+  constexpr int NW = NT / 32;
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  unsigned long long x[M];
+  #pragma unroll
+  for (int m = 0; m < M; ++m) {
+    x[m] = v[m];
+    #pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      unsigned long long y = __shfl_up_sync(0xffffffffu, x[m], o);
+      if (lane >= o) x[m] += y;
+    }
+    if (lane == 31) tmp[m * (NW + 1) + warp] = x[m];
+  }
+  __syncthreads();
+  if (warp < M) {  // warp m scans the warp totals of value m
+    unsigned long long* t = tmp + warp * (NW + 1);
+    unsigned long long w = (lane < NW) ? t[lane] : 0ull;
+    unsigned long long s = w;
+    #pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      unsigned long long y = __shfl_up_sync(0xffffffffu, s, o);
+      if (lane >= o) s += y;
+    }
+    if (lane < NW) t[lane] = s - w;
+    if (lane == NW - 1) t[NW] = s;
+  }
+  __syncthreads();
+  #pragma unroll
+  for (int m = 0; m < M; ++m) {
+    v[m] = tmp[m * (NW + 1) + warp] + x[m] - v[m];
+    total[m] = tmp[m * (NW + 1) + NW];
+  }
+  __syncthreads();
+}
+
 }  // namespace hj

@@ -175,7 +175,7 @@ __device__ __forceinline__ unsigned long long plan_count(const RelDev& R, int ns
 
 __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   constexpr int NT = 1024;
-  __shared__ unsigned long long s_tmp[NT / 32 + 1];
+  __shared__ unsigned long long s_tmp6[6 * (NT / 32 + 1)];
   __shared__ bool s_last;
   const uint32_t np = 1u << P.qbits();
   const uint32_t b = blockIdx.x;
@@ -200,13 +200,6 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
       if (items) sI += plan_items(P, cr[u], cs[u]);
     }
   }
-  unsigned long long tot;
-  block_exclusive_scan64<NT>(sR, s_tmp, &tot);
-  const unsigned long long bR = tot;
-  block_exclusive_scan64<NT>(sS, s_tmp, &tot);
-  const unsigned long long bS = tot;
-  block_exclusive_scan64<NT>(sI, s_tmp, &tot);
-  const unsigned long long bI = tot;
   // ---- own range ---------------------------------------------------------------------------
   const uint32_t q = b * NT + threadIdx.x;
   unsigned long long cr = 0, cs = 0;
@@ -214,10 +207,13 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
     cr = plan_count(P.rel[0], nsrc, np, q);
     cs = plan_count(P.rel[1], nsrc, np, q);
   }
-  unsigned long long tR, tS, tI;
-  const unsigned long long oR = bR + block_exclusive_scan64<NT>(cr, s_tmp, &tR);
-  const unsigned long long oS = bS + block_exclusive_scan64<NT>(cs, s_tmp, &tS);
-  const unsigned long long oI = bI + block_exclusive_scan64<NT>(items ? plan_items(P, cr, cs) : 0ull, s_tmp, &tI);
+  // the block totals of the prefix (reductions: exclusive scans whose totals are used) and this
+  // range's three scans, all in ONE multi-value scan (one pair of barriers)
+  unsigned long long v[6] = {sR, sS, sI, cr, cs, items ? plan_items(P, cr, cs) : 0ull}, tt[6];
+  block_exclusive_scan64xM<NT, 6>(v, s_tmp6, tt);
+  const unsigned long long bR = tt[0], bS = tt[1], bI = tt[2];
+  const unsigned long long tR = tt[3], tS = tt[4], tI = tt[5];
+  const unsigned long long oR = bR + v[3], oS = bS + v[4], oI = bI + v[5];
   if (q < np) {
     P.rel[0].off[q] = oR;
     P.rel[0].cur2[q] = oR;
@@ -276,9 +272,11 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   __syncthreads();
   if (!s_last) return;
   __threadfence();
+  const uint32_t i = threadIdx.x;
+  unsigned long long pv[4], ptt[4];  // (piece size, its pass-2 chunks) of R, then of S
+  #pragma unroll
   for (int rel = 0; rel < 2; ++rel) {
     const RelDev& R = P.rel[rel];
-    const uint32_t i = threadIdx.x;
     unsigned long long sz = 0;
     if (i < npieces) {
       if (nsrc == 1)
@@ -286,19 +284,21 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
       else
         sz = __ldcg(&R.pst[i + 1]);
     }
-    unsigned long long ptot;
-    const unsigned long long ps = block_exclusive_scan64<NT>(sz, s_tmp, &ptot);
-    const unsigned long long nch = (sz + P.C2 - 1) / P.C2;
-    unsigned long long ctot;
-    const unsigned long long cb = block_exclusive_scan64<NT>(nch, s_tmp, &ctot);
+    pv[2 * rel] = sz;
+    pv[2 * rel + 1] = (sz + P.C2 - 1) / P.C2;
+  }
+  block_exclusive_scan64xM<NT, 4>(pv, s_tmp6, ptt);
+  #pragma unroll
+  for (int rel = 0; rel < 2; ++rel) {
+    const RelDev& R = P.rel[rel];
     if (i < npieces) {
-      R.pst[i] = ps;
-      R.cst[i] = (uint32_t)cb;
-      if (nsrc == 1) R.cur1[i] = ps;
+      R.pst[i] = pv[2 * rel];
+      R.cst[i] = (uint32_t)pv[2 * rel + 1];
+      if (nsrc == 1) R.cur1[i] = pv[2 * rel];
     }
     if (i == 0) {
-      R.pst[npieces] = ptot;
-      R.cst[npieces] = (uint32_t)ctot;
+      R.pst[npieces] = ptt[2 * rel];
+      R.cst[npieces] = (uint32_t)ptt[2 * rel + 1];
     }
   }
 }
