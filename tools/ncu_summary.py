@@ -26,6 +26,18 @@ def main(path, as_json=False):
             if w in hdr:
                 i = hdr.index(w)
                 d[w] = f"{r[i]} {units[i]}".strip()
+        def val(name, scale):
+            if name not in hdr:
+                return None
+            i = hdr.index(name)
+            u = units[i].lower()
+            f = {"byte": 1, "kbyte": 1e3, "mbyte": 1e6, "gbyte": 1e9, "nsecond": 1e-9, "usecond": 1e-6,
+                 "msecond": 1e-3, "second": 1, "ns": 1e-9, "us": 1e-6, "ms": 1e-3, "s": 1}.get(u, scale)
+            return float(r[i].replace(",", "") or 0) * f
+        rd, wr = val("dram__bytes_read.sum", 1), val("dram__bytes_write.sum", 1)
+        t = val("gpu__time_duration.sum", 1e-9)
+        if rd is not None and wr is not None and t:
+            d["achieved_dram_GBps"] = f"{(rd + wr) / t / 1e9:.0f} GB/s (read + write / duration; cold-cache replay)"
         st = sorted(((float(r[i] or 0), hdr[i].replace("smsp__average_warps_issue_stalled_", "")
                       .replace("_per_issue_active.ratio", "")) for i in stall), reverse=True)[:6]
         d["top_stalls"] = ", ".join(f"{n}={v:.2f}" for v, n in st)
