@@ -322,6 +322,21 @@ int set_kernel_attrs(Ctx* c) {
                              (int)(c->smem_optin - fa.sharedSizeBytes)) != cudaSuccess)
       rc = -1;
   };
+  // kernels without a shared-memory attribute are still touched here: under lazy module
+  // loading (the CUDA 12 default) a kernel's first launch loads it, which can synchronize the
+  // context -- inside hj_xd_join that would wait on kernels that wait on this rank
+  auto load = [&](const void* f) {
+    cudaFuncAttributes fa;
+    if (cudaFuncGetAttributes(&fa, f) != cudaSuccess) rc = -1;
+  };
+  load((const void*)k_hist<K, false, false>);
+  load((const void*)k_hist<K, false, true>);
+  load((const void*)k_plan);
+  load((const void*)k_xd_rows);
+  load((const void*)k_xd_totals);
+  load((const void*)k_xd_cursors);
+  load((const void*)k_xd_barrier);
+  load((const void*)k_xd_results);
   attr((const void*)k_join_nlj<K, 256, false>);
   attr((const void*)k_join_nlj<K, 256, true>);
   attr((const void*)k_hist<K, true, false, true>);
@@ -1633,8 +1648,9 @@ int hj_join_received(hj_ctx* h, const void* R_recv, uint64_t nR, const uint32_t*
     if (rc == HJ_OK) rc = finish_join(c, hp, P, mat, res);
   }
   if (rc == HJ_OK && c->h_xd_err && *(volatile uint32_t*)c->h_xd_err) {
+    const uint32_t xe = *(volatile uint32_t*)c->h_xd_err;
     *c->h_xd_err = 0;
-    rc = fail(c, HJ_ERR_COMM, "exchange barrier timed out: a peer never reached hj_xd_barrier");
+    rc = fail(c, HJ_ERR_COMM, "exchange barrier timed out: rank %u never reached hj_xd_barrier", xe >> 4);
   }
   cudaSetDevice(prev);
   return rc;
@@ -2039,9 +2055,11 @@ int hj_xd_join(hj_ctx* h, int rank, int gpu_bits, const void* Rk, const void* Rp
     for (int s = 0; s < G; ++s)
         for (int r = 0; r < 2; ++r)
           for (int j = 0; j < G; ++j) totals[((size_t)r * G + s) * G + j] = c->h_xd_cur[((size_t)s * 2 + r) * XD_MAX + j];
-    if (*(volatile uint32_t*)c->h_xd_err) {
+    const uint32_t xe = *(volatile uint32_t*)c->h_xd_err;
+    if (xe) {
       *c->h_xd_err = 0;
-      rc = fail(c, HJ_ERR_COMM, "exchange timed out: a peer never reached hj_xd_join's phase waits");
+      static const char* phase[] = {"?", "totals (phase A)", "barrier (phase B)", "results (phase C)"};
+      rc = fail(c, HJ_ERR_COMM, "exchange timed out at the %s wait: rank %u never arrived", phase[xe & 3], xe >> 4);
     }
     if (rc == HJ_OK && over) {
       rc = HJ_XD_REGROW;

@@ -77,8 +77,8 @@ __global__ void __launch_bounds__(XD_MAX) k_xd_barrier(XdBarrier b) {
   if (t < b.G) {
     const unsigned long long t0 = global_ns();
     while (ld_acquire_sys(b.own + t) < b.epoch) {
-      if (global_ns() - t0 > b.timeout_ns) {
-        asm volatile("st.relaxed.sys.global.u32 [%0], %1;" ::"l"(b.err), "r"(1u) : "memory");
+      if (global_ns() - t0 > b.timeout_ns) {  // site 2: the barrier (phase B); bit 4+: the missing rank
+        asm volatile("st.relaxed.sys.global.u32 [%0], %1;" ::"l"(b.err), "r"(2u | ((uint32_t)t << 4)) : "memory");
         break;
       }
       __nanosleep(256);
@@ -90,13 +90,13 @@ __global__ void __launch_bounds__(XD_MAX) k_xd_barrier(XdBarrier b) {
 
 // wait (acquire, system scope) until flags[t] >= epoch for every t < G; thread t waits on flag t
 __device__ __forceinline__ void xd_wait_all(const unsigned long long* flags, int G, unsigned long long epoch,
-                                            unsigned long long timeout_ns, uint32_t* err) {
+                                            unsigned long long timeout_ns, uint32_t* err, uint32_t site) {
   const int t = threadIdx.x;
   if (t < G) {
     const unsigned long long t0 = global_ns();
     while (ld_acquire_sys(flags + t) < epoch) {
-      if (global_ns() - t0 > timeout_ns) {
-        asm volatile("st.relaxed.sys.global.u32 [%0], %1;" ::"l"(err), "r"(1u) : "memory");
+      if (global_ns() - t0 > timeout_ns) {  // site: 1 totals (phase A), 3 results (phase C); bit 4+: rank
+        asm volatile("st.relaxed.sys.global.u32 [%0], %1;" ::"l"(err), "r"(site | ((uint32_t)t << 4)) : "memory");
         break;
       }
       __nanosleep(128);
@@ -145,7 +145,7 @@ __global__ void __launch_bounds__(256) k_xd_totals(XdJoin a) {
 // and join then do nothing) and the host grows the windows and calls again.
 __global__ void __launch_bounds__(1024) k_xd_cursors(XdJoin a) {
   const int G = a.G;
-  xd_wait_all(a.own + XB_FLAGS_A, G, a.epoch, a.timeout_ns, a.err);
+  xd_wait_all(a.own + XB_FLAGS_A, G, a.epoch, a.timeout_ns, a.err, 1u);
   __shared__ unsigned long long s_seg[2][XD_MAX];
   __shared__ uint32_t s_over;
   if (threadIdx.x == 0) s_over = 0;
@@ -189,7 +189,7 @@ __global__ void __launch_bounds__(XD_MAX) k_xd_results(XdJoin a) {
   asm volatile("fence.sc.sys;" ::: "memory");
   __syncthreads();
   if (t < G) st_release_sys(a.board[t] + XB_FLAGS_C + a.rank, a.epoch);
-  xd_wait_all(a.own + XB_FLAGS_C, G, a.epoch, a.timeout_ns, a.err);
+  xd_wait_all(a.own + XB_FLAGS_C, G, a.epoch, a.timeout_ns, a.err, 3u);
   if (t == 0) {
     unsigned long long m = 0, c = 0;
     for (int s = 0; s < G; ++s) {

@@ -640,3 +640,19 @@ def test_gpu_exchange_c5_local_bits(G, lb):
     cols, calls = _xd_join_threads(hj, w, G, lb, 0, width=8, calls=1, cap_scale=2.0)
     m, c = oracle.hash_join(*cols)
     assert all(o[0] == 0 and o[3] == (m, c) for o in calls[0])
+
+
+@pytest.mark.gpu
+@pytest.mark.parametrize("nR,nS", [(3, 5000), (5000, 2), (1, 1)])
+def test_gpu_xd_join_ranks_without_rows(nR, nS):
+    """A rank with no local rows of R or S still takes part in every phase of hj_xd_join (its
+    peers wait on its flags): tiny relations over 4 virtual ranks."""
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_icde_sioulasckaa19_b200 as hj
+
+    w = W.Workload("tiny", nR, nS, "fk", keys="sparse", seed=199)
+    cols, calls = _xd_join_threads(hj, w, 4, 2, 0, calls=2, cap_scale=8.0)
+    m, c = oracle.hash_join(*cols)
+    for outs in calls:
+        assert all(o[0] == 0 and o[3] == (m, c) for o in outs)
