@@ -331,7 +331,11 @@ int set_kernel_attrs(Ctx* c) {
   };
   load((const void*)k_hist<K, false, false>);
   load((const void*)k_hist<K, false, true>);
-  load((const void*)k_plan);
+  load((const void*)k_plan<false, false, true>);
+  load((const void*)k_plan<false, true, true>);
+  load((const void*)k_plan<false, false, false>);
+  load((const void*)k_plan<false, true, false>);
+  load((const void*)k_plan<true, false, true>);
   load((const void*)k_xd_rows);
   load((const void*)k_xd_totals);
   load((const void*)k_xd_cursors);
@@ -518,6 +522,21 @@ size_t pass1b_smem(const HostPlan& hp, int nt) {
   return ((size_t)nt * pass_items<K>() + 2 * F) * tb + 16 * F + 4 * (F + 4) + 8 * F;
 }
 
+// a2: the planner instance for this plan (several sources / per-block bases / join items)
+int launch_plan(Ctx* c, const HostPlan& hp, const Plan& P) {
+  const unsigned g = (unsigned)((((size_t)1 << hp.qbits()) + 1023) / 1024);
+  const bool ms = P.nsrc > 1, bs = P.g1 != 0, it = P.mode != PLAN_SEND;
+  cudaStream_t st = c->stream;
+  if (ms) k_plan<true, false, true><<<g, 1024, 0, st>>>(P);
+  else if (bs && it) k_plan<false, true, true><<<g, 1024, 0, st>>>(P);
+  else if (bs) k_plan<false, true, false><<<g, 1024, 0, st>>>(P);
+  else if (it) k_plan<false, false, true><<<g, 1024, 0, st>>>(P);
+  else k_plan<false, false, false><<<g, 1024, 0, st>>>(P);
+  CUDA_TRY(c, cudaGetLastError());
+  c->launches += 1;
+  return HJ_OK;
+}
+
 // stage: 0 = all of a1-a3; 1 = a1-a2 only (hj_xd_count); 2 = a3 only (hj_xd_store, after stage 1
 // with the same plan)
 template <typename K>
@@ -576,9 +595,7 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false, 
     c->launches += 1;
   }
   mark(c, 1);
-  k_plan<<<(unsigned)((((size_t)1 << hp.qbits()) + 1023) / 1024), 1024, 0, st>>>(Pb);
-  CUDA_TRY(c, cudaGetLastError());
-  c->launches += 1;
+  if (int rc = launch_plan(c, hp, Pb)) return rc;
   mark(c, 2);
   if (stage == 1) return HJ_OK;
   if (hp.mode != PLAN_RECV && Pb.g1) {
@@ -1999,11 +2016,11 @@ int hj_xd_join(hj_ctx* h, int rank, int gpu_bits, const void* Rk, const void* Rp
       c->launches += 1;
     }
     mark(c, 1);
-    k_plan<<<(unsigned)((((size_t)1 << hs.qbits()) + 1023) / 1024), 1024, 0, st>>>(Ps);
+    if (int e0 = launch_plan(c, hs, Ps)) return e0;
     k_xd_totals<<<1, 256, 0, st>>>(a);
     k_xd_cursors<<<1, 1024, 0, st>>>(a);
     CUDA_TRY(c, cudaGetLastError());
-    c->launches += 3;
+    c->launches += 2;
     // the totals board is final once every rank's phase A arrived (read back with the results)
     CUDA_TRY(c, cudaMemcpyAsync(c->h_xd_cur, (const unsigned long long*)board[rank] + XB_TOT, (size_t)G * 2 * XD_MAX * 8,
                                 cudaMemcpyDeviceToHost, st));
@@ -2039,9 +2056,7 @@ int hj_xd_join(hj_ctx* h, int rank, int gpu_bits, const void* Rk, const void* Rp
     CUDA_TRY(c, cudaGetLastError());
     c->launches += 1;
     mark(c, 3);
-    k_plan<<<(unsigned)((((size_t)1 << hr.qbits()) + 1023) / 1024), 1024, 0, st>>>(Pr);
-    CUDA_TRY(c, cudaGetLastError());
-    c->launches += 1;
+    if (int e1 = launch_plan(c, hr, Pr)) return e1;
     e = k4 ? launch_pass2<uint32_t>(c, hr, Pr) : launch_pass2<uint64_t>(c, hr, Pr);
     if (e) return e;
     return finish_join(c, hr, Pr, mat, res, false, &a);

@@ -173,14 +173,17 @@ __device__ __forceinline__ unsigned long long plan_count(const RelDev& R, int ns
   return c;
 }
 
+// MS: several sources (exchange receiver); BS: per-block bases (HJ_OPT_PASS1_BASES); IT: join items
+// (not on the exchange sender). Specialised so each launch runs (and fetches) only its own code.
+template <bool MS, bool BS, bool IT>
 __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   constexpr int NT = 1024;
   __shared__ unsigned long long s_tmp6[6 * (NT / 32 + 1)];
   __shared__ bool s_last;
   const uint32_t np = 1u << P.qbits();
   const uint32_t b = blockIdx.x;
-  const int nsrc = P.nsrc;
-  const bool items = P.mode != PLAN_SEND;
+  const int nsrc = MS ? P.nsrc : 1;
+  constexpr bool items = IT;
   // ---- prefix of everything below this block's range -------------------------------------
   unsigned long long sR = 0, sS = 0, sI = 0;
   // batches of 8 earlier blocks: all 16 count loads are issued before any is used (the loop is
@@ -229,7 +232,7 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   // ---- several sources: piece sizes, a warp per piece (stored in pst[i + 1]) --------------
   const uint32_t npieces = P.npieces();
   const int pb = P.pb(), b2 = P.b2;
-  if (nsrc > 1) {
+  if (MS && nsrc > 1) {
     const uint32_t lane = threadIdx.x & 31, gw = b * (NT / 32) + (threadIdx.x >> 5), nw = gridDim.x * (NT / 32);
     for (int rel = 0; rel < 2; ++rel) {
       const RelDev& R = P.rel[rel];
@@ -245,7 +248,7 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
     }
   }
   // ---- pass-1 bases: exclusive prefix over pass-1 blocks of each (relation, digit) column ----
-  if (P.g1) {
+  if (BS && P.g1) {
     const uint32_t F1 = 1u << pb, g1 = P.g1;
     const uint32_t lane = threadIdx.x & 31, gw = b * (NT / 32) + (threadIdx.x >> 5), nw = gridDim.x * (NT / 32);
     for (uint32_t col = gw; col < 2 * F1; col += nw) {
