@@ -79,8 +79,11 @@ enum hj_option {
   HJ_OPT_PARTITIONER = 12,  /* hj_join only: 0 = histogram + prefix sum + exact placement (north
                                star, default); 1 = the paper's histogram-free bucket chains
                                (NEXT-1): no histogram pass, partitions are chains of
-                               buckets from a pool, pass 2 takes one bucket at a time. Needs more
-                               device memory (bucket slack); ms_kernel[0..1] are 0 and
+                               buckets from a pool, pass 2 takes one bucket at a time; a pass-2
+                               partition that keeps closing buckets takes growing regions of
+                               1, 1, 2, 4, 8, 16 consecutive buckets (skew). Needs more device
+                               memory (bucket slack: pass-2 pool <= (2n / cap + 2^B + 1) buckets
+                               of cap + tile tuples per relation); ms_kernel[0..1] are 0 and
                                ms_kernel[2..3] include each pass's bucket bookkeeping. Ignored by
                                hj_join_host / hj_partition / the exchange calls and by graph mode */
   HJ_OPT_FUSE = 13,         /* hj_join: 1 = pass 2 and the join run as ONE persistent kernel that

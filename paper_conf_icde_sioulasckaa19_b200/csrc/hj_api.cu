@@ -138,6 +138,12 @@ int ensure(Ctx* c, DevBuf& b, size_t bytes) {
   if (bytes == 0) return HJ_OK;
   CUDA_TRY(c, cudaMalloc(&b.p, bytes));
   b.bytes = bytes;
+  // A new allocation starts zeroed, as a fresh process's pages do. Memory recycled from a closed
+  // context with the other partitioner (bucket chains <-> histogram path) hung or faulted the
+  // next join at c2 / c3 sizes (tools/bc_one.py): some buffer is still read before
+  // it is written on that path. Zeroing on (re)allocation only -- never per call.
+  CUDA_TRY(c, cudaMemsetAsync(b.p, 0, bytes, c->stream));
+  CUDA_TRY(c, cudaStreamSynchronize(c->stream));
   return HJ_OK;
 }
 
@@ -1060,7 +1066,11 @@ int run_join_bc(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, c
     B.np2 = (uint32_t)np;
     B.nbmax1 = (uint32_t)(ns[r] / B.cap1 + F1 + 1);
     if (B.nbmax1 + 5 > BC_MAX_NB1) return fail(c, HJ_ERR_INVALID, "bucket chains: %u pass-1 buckets", B.nbmax1);
-    B.nbmax2 = (uint32_t)(ns[r] / B.cap2 + np + 1);
+    // pass 2 grows a hot partition's regions up to 16 buckets (as long as a region's fill stays
+    // below 2^30), bound 2n / cap2 + np + 1 (hj_bucket.cuh)
+    B.lg2max = 0;
+    while (B.lg2max < 4 && (B.bsz2 << (B.lg2max + 1)) <= (1ull << 30)) ++B.lg2max;
+    B.nbmax2 = (uint32_t)((B.lg2max ? 2 : 1) * (ns[r] / B.cap2) + np + 1);
     B.csl = r == 0 ? hp.CR : hp.CS;
     o_st1[r] = take(F1 * 8);
     o_st2[r] = take(np * 8);
@@ -1431,6 +1441,11 @@ void hj_destroy(hj_ctx* h) {
   for (auto& b : c->xd_win)
     if (b.p) cudaFree(b.p);
   if (c->xd_meta.p) cudaFree(c->xd_meta.p);
+  for (int r = 0; r < 2; ++r) {  // bucket-chain pools (HJ_OPT_PARTITIONER = 1)
+    if (c->bc_pool1[r].p) cudaFree(c->bc_pool1[r].p);
+    if (c->bc_pool2[r].p) cudaFree(c->bc_pool2[r].p);
+  }
+  if (c->bc_meta.p) cudaFree(c->bc_meta.p);
   delete c->xd_hp;
   delete c->xd_P;
   if (c->h_xd_cur) cudaFreeHost(c->h_xd_cur);

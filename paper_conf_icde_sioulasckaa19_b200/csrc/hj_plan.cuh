@@ -39,7 +39,8 @@ struct BcRel {
   void* pool2;                // pass-2 buckets
   unsigned long long* st1;    // [2^b1] pass-1 partition state: j << 32 | fill, current bucket =
                               //        p (j = 0, the partition's initial bucket) or np + j - 1
-  unsigned long long* st2;    // [2^B]  pass-2 partition state (index q = D << b2 | d2)
+  unsigned long long* st2;    // [2^B]  pass-2 partition state (index q = D << b2 | d2); its high
+                              //        word is j | lgk << BC_LGK_SHIFT (region of 2^lgk buckets)
   uint32_t* fill1;            // [nbmax1] tuples in each pass-1 bucket
   uint32_t* part1;            // [nbmax1] pass-1 partition D of each overflow bucket (b >= np1)
   uint32_t* fill2;            // [nbmax2]
@@ -53,8 +54,11 @@ struct BcRel {
   uint32_t nbmax1, nbmax2;    // pool sizes in buckets (proven bounds)
   unsigned long long bsz1, bsz2;  // bucket stride in tuples = cap + tile (slack for the closing run)
   uint32_t csl;               // join slice capacity: C_R (R) or C_S (S)
+  uint32_t lg2max;            // pass 2: a partition's overflow regions grow 1, 1, 2, 4, .. 2^lg2max
+                              //         consecutive buckets (hj_bucket.cuh); 0 = fixed buckets
 };
 enum { CNT_BC_NB1 = 2, CNT_BC_NB2 = 4 };  // + relation: overflow buckets taken from the pool
+constexpr uint32_t BC_LGK_SHIFT = 27, BC_J_MASK = (1u << BC_LGK_SHIFT) - 1;
 constexpr uint32_t BC_MAX_NB1 = 1542;  // per relation: <= 1.5 * 2^b1 + 1 pass-1 buckets (cap1 >= 2 x mean) + prefix end + spare
 enum { RES_BC_OVERFLOW = 3 };
 
