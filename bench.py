@@ -163,20 +163,67 @@ def key_slices(w: W.Workload, Rk, Rp, Sk, Sp, slices: int):
             for t in range(slices)]
 
 
+def cpu_model() -> str:
+    try:
+        for line in open("/proc/cpuinfo"):
+            if line.startswith("model name"):
+                return line.split(":", 1)[1].strip()
+    except OSError:
+        pass
+    return "unknown"
+
+
+class PinnedCore:
+    """Run the (single-threaded) oracle pinned to one host core, like `taskset -c <core>`."""
+
+    def __init__(self, core: int = 0):
+        self.core = core
+
+    def __enter__(self):
+        try:
+            self.prev = os.sched_getaffinity(0)
+            cores = sorted(self.prev)
+            self.core = self.core if self.core in self.prev else cores[0]
+            os.sched_setaffinity(0, {self.core})
+            self.pinned = True
+        except (AttributeError, OSError):
+            self.pinned = False
+        return self
+
+    def __exit__(self, *a):
+        if self.pinned:
+            os.sched_setaffinity(0, self.prev)
+
+
 def cpu_oracle_sample(w: W.Workload, Rk, Rp, Sk, Sp, slices: int):
-    """Time the oracle (as it stands, single thread) on key slice 0 of `slices` of the workload
-    (pre-filtered, untimed); throughput = (|R|+|S|) / (slices * t_slice)."""
+    """Time the oracle (as it stands, single thread, pinned to one core) on key slice 0 of
+    `slices` of the workload (pre-filtered, untimed); throughput = (|R|+|S|) / (slices * t_slice)."""
     import oracle
 
     sl = key_slices(w, Rk, Rp, Sk, Sp, slices)[0]
-    t0 = time.perf_counter()
-    res = oracle.hash_join(*sl, materialize=bool(w.out_mode))
-    dt = time.perf_counter() - t0
+    with PinnedCore(0) as pin:
+        t0 = time.perf_counter()
+        res = oracle.hash_join(*sl, materialize=bool(w.out_mode))
+        dt = time.perf_counter() - t0
     v = w.n / (slices * dt)
     sample = (f"key slice 0 of {slices} (top bits of fmix64(key), pre-filtered) of the full {w.name} input: "
               f"|R|={len(sl[0])} |S|={len(sl[2])}, {'materialized' if w.out_mode else 'count'}, {res[0]} matches in "
               f"{dt:.2f} s; value = (|R|+|S|)/({slices}*t_slice)")
-    return {"value": v, "unit": UNIT, "cores": 1, "kind": "oracle", "sample": sample, "host_cpus": os.cpu_count()}
+    return {"value": v, "unit": UNIT, "cores": 1, "kind": "oracle", "sample": sample, "host_cpus": os.cpu_count(),
+            "cpu_model": cpu_model(), "pinned_core": pin.core if pin.pinned else None}
+
+
+def closed_form(w: W.Workload):
+    """(matches, checksum) the generator fixes for FK / 1:1 / Zipf-FK inputs:
+    every S row j matches exactly R row rho(j), so matches = |S| and checksum = sum_j sig(rho(j), j)
+    (sig = fmix64(r_pay ^ s_pay * golden), payloads are row ids). Computed on the host, untimed;
+    every timed step's result is compared with it."""
+    j = np.arange(w.nS, dtype=np.uint64)
+    cdf = W.zipf_cdf(w.nR, w.z) if w.dist == "zipf" else None
+    rho = W.np_rho_for(w, j, cdf)
+    with np.errstate(over="ignore"):
+        chk = int(W.np_fmix64(rho ^ (j * np.uint64(0x9E3779B97F4A7C15))).sum(dtype=np.uint64))
+    return w.nS, chk
 
 
 def run_reference(args, w: W.Workload):
@@ -196,14 +243,16 @@ def run_reference(args, w: W.Workload):
     parts = key_slices(w, Rk, Rp, Sk, Sp, slices)
     del Rk, Rp, Sk, Sp
     times = []
-    for i in range(steps):
-        t0 = time.perf_counter()
-        oracle.hash_join(*parts[i % slices], materialize=bool(w.out_mode))
-        if i >= args.warmup:
-            times.append(time.perf_counter() - t0)
+    with PinnedCore(0) as pin:
+        for i in range(steps):
+            t0 = time.perf_counter()
+            oracle.hash_join(*parts[i % slices], materialize=bool(w.out_mode))
+            if i >= args.warmup:
+                times.append(time.perf_counter() - t0)
     t = float(np.mean(times))
     v = w.n / (slices * t)
     cpu = {"value": v, "unit": UNIT, "cores": 1, "kind": "oracle", "host_cpus": os.cpu_count(),
+           "cpu_model": cpu_model(), "pinned_core": pin.core if pin.pinned else None,
            "sample": f"each step one key slice (1 of {slices}, top bits of fmix64(key), pre-filtered) of the full "
                      f"{w.name} input; value = (|R|+|S|)/({slices}*mean t_slice)"}
     print(json.dumps({"impl": "reference", "metric": METRIC, "value": v, "unit": UNIT, "n_gpus": ws,
@@ -273,9 +322,10 @@ def main():
         if ok.item() == 0:
             args.exchange = "nccl"
             exchange_note = exchange_note or "direct store unavailable on a peer; NCCL all_to_all used"
+    expect = closed_form(w)  # untimed; every step below is checked against it
     for _ in range(args.warmup):
         res = step()
-    assert res.matches == w.nS, "closed form: FK / 1:1 joins produce |S| matches"
+        assert (res.matches, res.checksum) == expect, ("closed form", res.matches, res.checksum, expect)
 
     def barrier():
         if use_dist:
@@ -290,8 +340,10 @@ def main():
         e0 = torch.cuda.Event(enable_timing=True)
         e1 = torch.cuda.Event(enable_timing=True)
         e0.record(stream)
+        results = []
         for _ in range(args.steps):
             res = step()
+            results.append((res.matches, res.checksum))
             loc = res if not use_dist else res.local
             per_k += np.array(loc.ms_kernel)
             # + the sender side: direct = hist, plan, count rows, pass 1, barrier; nccl = (hist, plan, pass 1) x 2
@@ -299,6 +351,8 @@ def main():
             sent += 0 if not use_dist else res.sent_bytes
         e1.record(stream)
         barrier()
+    bad = [k for k, r in enumerate(results) if r != expect]
+    assert not bad, f"timed steps {bad[:5]} differ from the closed form {expect}"
     ms = e0.elapsed_time(e1) / args.steps
     if use_dist:
         t = torch.tensor([ms], device="cpu" if args.debug_one_device else dev)
@@ -343,7 +397,8 @@ def main():
                       + ("fused into pass 1 (direct peer stores, hj_xd_*)" if args.exchange == "direct"
                          else "over NCCL all_to_all") + ", per-rank 2-pass join"},
            "roofline": roof, "roofline_path": roof_path, "kernels_ms": kms, "clocks": clk.summary(),
-           "gpu_launches": launches}
+           "gpu_launches": launches,
+           "validated": f"every warm-up and timed step: (matches, checksum) == closed form {list(expect)}"}
     if use_dist:
         out["config"]["exchange"] = args.exchange + (f" ({exchange_note})" if exchange_note else "")
     if use_dist:

@@ -53,7 +53,11 @@ enum hj_status {
   HJ_ERR_UNSUPPORTED = -2, /* key/payload widths other than 4/4 and 8/8; radix_bits > 20     */
   HJ_ERR_OOM = -3,         /* device or pinned-host allocation failed                         */
   HJ_ERR_CUDA = -4,        /* any CUDA runtime error; message in hj_last_error()              */
-  HJ_ERR_COMM = -5         /* multi-GPU exchange: a peer missed the hj_xd_barrier deadline    */
+  HJ_ERR_COMM = -5,        /* multi-GPU exchange: a peer missed the hj_xd_barrier deadline    */
+  HJ_ERR_WORKSPACE = -6    /* hj_join with a caller workspace (hj_set_workspace): the workspace
+                              is smaller than hj_workspace_bytes() for this call, or the
+                              materialized pairs outgrew HJ_OPT_OUT_CAPACITY -- then res->matches
+                              holds the exact count; raise the capacity, resize, call again      */
 };
 
 enum hj_option {
@@ -63,14 +67,12 @@ enum hj_option {
   HJ_OPT_OUT_CAPACITY = 3, /* initial materialization capacity in pairs; 0 = max(nS, 1M)      */
   HJ_OPT_TIMING = 4,       /* 1 = record per-phase CUDA events into hj_result (default 1)     */
   HJ_OPT_BLOCKS_PER_SM = 5, /* persistent-grid residency override for the passes (0 = auto)   */
-  HJ_OPT_JOIN_VARIANT = 6,  /* join kernel shape (tuning; 0 = auto, k = shape k-1 of hj_api.cu)  */
+  HJ_OPT_JOIN_VARIANT = 6,  /* join kernel shape (tuning; 0 = auto, k = shape k-1 of hj_api.cu's
+                               JOIN_SHAPES, 1..6)                                                */
   HJ_OPT_PASS_THREADS = 7,  /* partition-pass block size 512 / 1024 (0 = auto)                   */
   HJ_OPT_JOIN_ALGO = 9,     /* 0 = radix-partitioned + smem hash table (default); 1 = radix-
                                partitioned + ballot nested loops (Listing 1); 2 = non-
                                partitioned hash join on a device-memory table (Fig. 8) */
-  HJ_OPT_PASS1_BASES = 10,  /* 1 = pass 1 uses per-block bases computed by the histogram kernel and
-                               TMA bulk-store write-out instead of atomic run reservation (opt-in;
-                               measured slower on B200, kept for comparison)                      */
   HJ_OPT_GRAPH = 11,        /* 1 = hj_join captures its launch sequence in a CUDA graph and replays
                                it while the call signature is unchanged (launch gaps and host
                                preparation leave the critical path: c3 2.73 -> 2.68 ms/call; only
@@ -86,16 +88,6 @@ enum hj_option {
                                of cap + tile tuples per relation); ms_kernel[0..1] are 0 and
                                ms_kernel[2..3] include each pass's bucket bookkeeping. Ignored by
                                hj_join_host / hj_partition / the exchange calls and by graph mode */
-  HJ_OPT_FUSE = 13,         /* hj_join: 1 = pass 2 and the join run as ONE persistent kernel that
-                               joins each pass-1 partition's co-partitions while they are still in
-                               L2 (opt-in: measured slower than separate kernels on c3, DESIGN.md
-                               §5; needs radix_bits >= 2, the histogram partitioner and join
-                               algorithm 0, else ignored); 0 = separate pass-2 and join kernels
-                               (default). ms_kernel[3] is then the fused kernel, ms_kernel[4] 0  */
-  HJ_OPT_FUSE_WINDOW_MB = 14, /* fused: MB of pass-2 output allowed ahead of the join (0 = no
-                               throttle; default 32)                                            */
-  HJ_OPT_FUSE_PASS_SLOTS = 15, /* fused: blocks per SM that start in the pass-2 role (default 1 of
-                               2; the others join; pass-2 blocks join once pass 2 is done)      */
   HJ_OPT_PASS_L2PF = 17,    /* partition passes: 1 = TMA-prefetch each block's unit-after-next into L2
                                (cp.async.bulk.prefetch.L2) when its descriptor is published; 0 = off;
                                2 = auto (default: on for 8-byte keys, where it was measured faster) */
@@ -106,14 +98,17 @@ enum hj_option {
                                x twice the tuples, no register prefetch, two blocks per SM. Value =
                                1 + mask of the passes using the second form (bit 0 pass 1, bit 1
                                pass 2); 0 = auto (pass 1 of 8-byte tuples, where it measured faster) */
-  HJ_OPT_STREAM_CHUNK = 8   /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
+  HJ_OPT_STREAM_CHUNK = 8,  /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
                                least 2^22; >= |S| = copy everything, then join)                   */
+  HJ_OPT_MAT_CHECKSUM = 20  /* 1 (default) = MATERIALIZE also fills res->checksum (the pairs'
+                               signatures are summed by the probe, so every materialized result is
+                               self-checking); 0 = checksum left 0 in MATERIALIZE (measurement)   */
 };
 
 typedef struct hj_result {
   uint64_t matches;      /* |R ⋈ S| (always filled)                                              */
-  uint64_t checksum;     /* sum of sig(r_pay, s_pay) mod 2^64 in COUNT_CHECKSUM mode; 0 in
-                            MATERIALIZE mode, whose result is the pairs themselves               */
+  uint64_t checksum;     /* sum of sig(r_pay, s_pay) mod 2^64 over the matched pairs, in both
+                            modes (MATERIALIZE: unless HJ_OPT_MAT_CHECKSUM = 0)                  */
   const void* r_pay_out; /* MATERIALIZE: `matches` payloads of R, pay_bytes each (device memory
                             for hj_join, pinned host memory for hj_join_host); owned by the ctx,
                             valid until the next join on this ctx or hj_destroy                   */
@@ -127,11 +122,12 @@ typedef struct hj_result {
   float ms_kernel[5];    /* per step, CUDA events on the ctx stream: 0 histogram, 1 planner,
                             2 pass 1, 3 pass 2, 4 join (HJ_OPT_TIMING = 1)                       */
   uint32_t kernels;      /* kernels this call launched                                           */
-  uint32_t fused;        /* 1: pass 2 and the join ran fused (HJ_OPT_FUSE); ms_kernel[3] covers both */
+  uint32_t reserved;
 } hj_result;
 
 /* Create a context on CUDA device `device` for key/payload widths 4/4 or 8/8 bytes.
- * cuda_stream: a cudaStream_t to issue all work on (NULL = a ctx-owned non-blocking stream).
+ * cuda_stream: a cudaStream_t to issue all work on (NULL = a ctx-owned non-blocking stream; the
+ * caller then orders it after its own producers, or re-targets it with hj_set_stream).
  * Returns HJ_OK and *out, or HJ_ERR_INVALID / HJ_ERR_UNSUPPORTED / HJ_ERR_CUDA. */
 int hj_create(hj_ctx** out, int device, int key_bytes, int pay_bytes, void* cuda_stream);
 
@@ -141,7 +137,10 @@ void hj_destroy(hj_ctx* ctx);
 /* Message of the last failure on ctx ("" if none). NULL ctx -> message of the last hj_create. */
 const char* hj_last_error(const hj_ctx* ctx);
 
-/* Re-target the context to another stream (NULL = the ctx-owned stream). */
+/* Re-target the context to another stream. NULL = the legacy default stream ("stream 0", e.g.
+ * torch's default stream): the join is then ordered after every kernel the caller issued there.
+ * Every call is stream-ordered after prior work on the ctx's stream; inputs produced on another
+ * stream must be synchronized by the caller. */
 int hj_set_stream(hj_ctx* ctx, void* cuda_stream);
 
 /* Set a tuning / test knob (enum hj_option). Results never depend on knobs. */
@@ -159,6 +158,20 @@ int hj_join(hj_ctx* ctx,
             const void* R_keys, const void* R_pay, uint64_t nR,
             const void* S_keys, const void* S_pay, uint64_t nS,
             int radix_bits, int out_mode, hj_result* res);
+
+/* Caller-provided device workspace (device buffers reserved up front).
+ * hj_workspace_bytes: the device bytes hj_join(ctx, nR, nS, radix_bits, out_mode) needs with the
+ *   ctx's current options (partitioner, join algorithm, HJ_OPT_OUT_CAPACITY); 0 if nR or nS is 0
+ *   or an argument is invalid. Host-only, no device work.
+ * hj_set_workspace: from now on hj_join carves every device buffer from [dptr, dptr + bytes)
+ *   (256-byte aligned; e.g. a torch tensor) instead of allocating: no cudaMalloc and no
+ *   synchronization inside hj_join before its final result readback. The buffer is caller-owned
+ *   and must stay valid (and unused by the caller) while the ctx may use it; materialized pairs
+ *   are returned inside it. dptr = NULL returns to ctx-owned allocations. Synchronizes the ctx's
+ *   streams and frees hj_join's ctx-owned buffers. hj_join_host / hj_partition / the exchange
+ *   calls keep ctx-owned allocations. A too-small workspace -> HJ_ERR_WORKSPACE. */
+uint64_t hj_workspace_bytes(const hj_ctx* ctx, uint64_t nR, uint64_t nS, int radix_bits, int out_mode);
+int hj_set_workspace(hj_ctx* ctx, void* dptr, uint64_t bytes);
 
 /* Same join from HOST columns (pinned for full overlap; pageable works): the streaming probe
  * of the paper's out-of-GPU strategy (NEXT-3). R is copied and

@@ -38,22 +38,21 @@ OPT_JOIN_VARIANT = 6
 OPT_PASS_THREADS = 7
 OPT_STREAM_CHUNK = 8
 OPT_JOIN_ALGO = 9
-OPT_PASS1_BASES = 10
 OPT_GRAPH = 11
 OPT_PARTITIONER = 12  # 0 = histogram (default), 1 = bucket chains (NEXT-1)
-OPT_FUSE = 13  # 1 = pass 2 + join in one L2-resident kernel (opt-in), 0 = separate kernels (default)
-OPT_FUSE_WINDOW_MB = 14
-OPT_FUSE_PASS_SLOTS = 15
 OPT_PASS_L2PF = 17
 OPT_PASS1_BITS = 18
 OPT_PASS_VARIANT = 19
+OPT_MAT_CHECKSUM = 20  # 1 (default): MATERIALIZE also returns the checksum
 ALGO_HASH, ALGO_NLJ, ALGO_NONPARTITIONED = 0, 1, 2
 
-_ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4: "HJ_ERR_CUDA", -5: "HJ_ERR_COMM"}
+ERR_WORKSPACE = -6
+_ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4: "HJ_ERR_CUDA", -5: "HJ_ERR_COMM",
+           -6: "HJ_ERR_WORKSPACE"}
 
 # every symbol include/hj.h declares (checked by tests/test_abi.py)
 EXPORTS = ("hj_create", "hj_destroy", "hj_last_error", "hj_set_stream", "hj_set_option", "hj_join",
-           "hj_join_host", "hj_partition", "hj_exchange_pack", "hj_join_received", "hj_xd_window",
+           "hj_workspace_bytes", "hj_set_workspace", "hj_join_host", "hj_partition", "hj_exchange_pack", "hj_join_received", "hj_xd_window",
            "hj_xd_header_bytes", "hj_ipc_open", "hj_ipc_close", "hj_xd_count", "hj_xd_store", "hj_xd_barrier",
            "hj_xd_join", "hj_xd_reserve", "hj_version")
 XD_MAX_RANKS = 64
@@ -72,7 +71,7 @@ class _Result(ctypes.Structure):
                 ("s_pay_out", ctypes.c_void_p), ("n_items", ctypes.c_uint64), ("radix_bits", ctypes.c_int),
                 ("passes", ctypes.c_int), ("ms_total", ctypes.c_float), ("ms_partition", ctypes.c_float),
                 ("ms_join", ctypes.c_float), ("ms_kernel", ctypes.c_float * 5), ("kernels", ctypes.c_uint32),
-                ("fused", ctypes.c_uint32)]
+                ("reserved", ctypes.c_uint32)]
 
 
 def _load_lib():
@@ -94,6 +93,10 @@ def _load_lib():
     for f in (lib.hj_join, lib.hj_join_host):
         f.argtypes = [vp, vp, vp, u64, vp, vp, u64, i32, i32, ctypes.POINTER(_Result)]
         f.restype = i32
+    lib.hj_workspace_bytes.argtypes = [vp, u64, u64, i32, i32]
+    lib.hj_workspace_bytes.restype = u64
+    lib.hj_set_workspace.argtypes = [vp, vp, u64]
+    lib.hj_set_workspace.restype = i32
     lib.hj_partition.argtypes = [vp, vp, vp, u64, i32, ctypes.POINTER(vp), ctypes.POINTER(u64), ctypes.POINTER(u64)]
     lib.hj_partition.restype = i32
     lib.hj_exchange_pack.argtypes = [vp, i32, vp, vp, u64, i32, i32, ctypes.POINTER(vp), ctypes.POINTER(vp),
@@ -151,13 +154,17 @@ class JoinResult:
     ms_join: float = 0.0
     ms_kernel: tuple = ()
     kernels: int = 0
-    fused: bool = False  # pass 2 + join ran as one kernel: ms_kernel[3] covers both, ms_kernel[4] = 0
 
 
 class Context:
-    """One hj_ctx (device, widths). Not thread-safe; the module keeps one per thread."""
+    """One hj_ctx (device, widths). Not thread-safe; the module keeps one per thread.
 
-    def __init__(self, device: int = 0, key_bytes: int = 4, pay_bytes: int = 4, stream: int | None = None):
+    With workspace=True (default) hj_join's device memory is a torch tensor this object owns
+    (hj_workspace_bytes / hj_set_workspace): PyTorch's caching allocator supplies it, and the
+    library neither allocates nor synchronizes inside hj_join before the result readback."""
+
+    def __init__(self, device: int = 0, key_bytes: int = 4, pay_bytes: int = 4, stream: int | None = None,
+                 workspace: bool = True):
         h = ctypes.c_void_p()
         rc = _lib.hj_create(ctypes.byref(h), device, key_bytes, pay_bytes, stream)
         if rc != 0:
@@ -166,12 +173,15 @@ class Context:
         self.device = device
         self.key_bytes = key_bytes
         self.pay_bytes = pay_bytes
+        self.use_workspace = workspace
+        self._ws = None  # torch uint8 tensor backing hj_join's buffers
 
     def close(self):
         self._view_key = self._view_val = None  # views of memory hj_destroy frees
         if getattr(self, "_h", None):
             _lib.hj_destroy(self._h)
             self._h = None
+        self._ws = None  # after hj_destroy: the ctx no longer touches it
 
     def __del__(self):
         try:
@@ -189,20 +199,45 @@ class Context:
     def set_stream(self, stream_handle: int | None):
         self._check(_lib.hj_set_stream(self._h, stream_handle))
 
+    def workspace_bytes(self, nR: int, nS: int, radix_bits: int = -1, out_mode: int = OUT_COUNT_CHECKSUM) -> int:
+        return int(_lib.hj_workspace_bytes(self._h, nR, nS, radix_bits, out_mode))
+
+    def _ensure_workspace(self, nbytes: int, device):
+        import torch
+
+        if self._ws is not None and self._ws.numel() >= nbytes:
+            return
+        self._view_key = self._view_val = None
+        self._check(_lib.hj_set_workspace(self._h, None, 0))  # drop the old one before torch frees it
+        self._ws = None
+        # +256: torch's allocations are 512-byte aligned already; the slack keeps the size a multiple
+        self._ws = torch.empty(nbytes + 256, dtype=torch.uint8, device=device)
+        self._check(_lib.hj_set_workspace(self._h, ctypes.c_void_p(self._ws.data_ptr()), self._ws.numel()))
+
     def join(self, Rk, Rp, Sk, Sp, radix_bits: int = -1, out_mode: int = OUT_COUNT_CHECKSUM) -> JoinResult:
         import torch
 
         cols = [_as_device_col(t, self.key_bytes if i % 2 == 0 else self.pay_bytes) for i, t in enumerate((Rk, Rp, Sk, Sp))]
         if cols[0].numel() != cols[1].numel() or cols[2].numel() != cols[3].numel():
             raise ValueError("key and payload columns differ in length")
-        self.set_stream(torch.cuda.current_stream(cols[0].device).cuda_stream)
+        dev_ = cols[0].device
+        self.set_stream(torch.cuda.current_stream(dev_).cuda_stream)
+        nR, nS = cols[0].numel(), cols[2].numel()
         res = _Result()
-        rc = _lib.hj_join(self._h, _ptr(cols[0]), _ptr(cols[1]), cols[0].numel(), _ptr(cols[2]), _ptr(cols[3]),
-                          cols[2].numel(), radix_bits, out_mode, ctypes.byref(res))
+        for _ in range(3):
+            if self.use_workspace and nR and nS:
+                self._ensure_workspace(self.workspace_bytes(nR, nS, radix_bits, out_mode), dev_)
+            rc = _lib.hj_join(self._h, _ptr(cols[0]), _ptr(cols[1]), nR, _ptr(cols[2]), _ptr(cols[3]), nS,
+                              radix_bits, out_mode, ctypes.byref(res))
+            if rc != ERR_WORKSPACE or not self.use_workspace:
+                break
+            # materialized pairs outgrew the capacity (reading S11: never overwrite): the exact
+            # count came back in res.matches -> grow the output part of the workspace, re-run
+            self.set_option(OPT_OUT_CAPACITY, max(int(res.matches), 1))
         self._check(rc)
         out = _result(res)
         if out_mode == OUT_MATERIALIZE and res.matches:
-            out.r_pay, out.s_pay = self._views(res, cols[0].device)
+            out.r_pay, out.s_pay = self._views(res, dev_)
         return out
 
     def _views(self, res, device):
@@ -414,7 +449,7 @@ def _result(res: _Result) -> JoinResult:
     return JoinResult(matches=int(res.matches), checksum=int(res.checksum), n_items=int(res.n_items),
                       radix_bits=res.radix_bits, passes=res.passes, ms_total=res.ms_total,
                       ms_partition=res.ms_partition, ms_join=res.ms_join,
-                      ms_kernel=tuple(res.ms_kernel), kernels=int(res.kernels), fused=bool(res.fused))
+                      ms_kernel=tuple(res.ms_kernel), kernels=int(res.kernels))
 
 
 def _as_device_col(t, width: int):

@@ -14,7 +14,6 @@
 
 #include "../../include/hj.h"
 #include "hj_exchange.cuh"
-#include "hj_fused.cuh"
 #include "hj_join.cuh"
 #include "hj_partition.cuh"
 #include "hj_variants.cuh"
@@ -37,32 +36,23 @@ struct JoinShape {
   bool l2pf;                      // claimed item's R chunk + first S round prefetched into L2
   int spf = 0;                    // S stream prefetched into L2 this many probe rounds ahead (0 = off)
 };
-constexpr JoinShape JOIN_SHAPES[] = {{256, 8, 3, 1, 1}, {256, 8, 2, 2, 1}, {224, 8, 3, 1, 1}, {256, 12, 3, 1, 1},
-                                     {192, 8, 3, 1, 1}, {256, 4, 2, 1, 1}, {512, 4, 1, 1, 1}, {256, 8, 2, 1, 1},
-                                     {384, 4, 1, 2, 1}, {192, 8, 4, 1, 2}, {256, 8, 3, 1, 2}, {160, 8, 4, 1, 2},
-                                     {224, 8, 4, 1, 1, true}, {192, 8, 4, 1, 1, true}, {256, 8, 3, 1, 1, true},
-                                     {256, 4, 3, 1, 1, false, true}, {256, 6, 3, 1, 1, false, true},
-                                     {256, 8, 3, 1, 1, false, true}, {192, 6, 4, 1, 1, false, true},
-                                     {256, 8, 3, 1, 1, false, false, true}, {256, 6, 3, 1, 1, false, true, true},
-                                     {256, 4, 3, 1, 1, false, true, true},
-                                     {256, 6, 3, 1, 1, false, true, true, 4}, {256, 8, 3, 1, 1, false, false, true, 4},
-                                     {256, 4, 3, 1, 1, false, true, true, 4}, {256, 6, 3, 1, 1, false, true, true, 8},
-                                     {256, 6, 3, 1, 1, false, true, true, 2}, {256, 8, 3, 1, 1, false, false, true, 2},
-                                     {512, 4, 2, 1, 1, false, true, true}, {512, 2, 2, 1, 1, false, true, true},
-                                     {384, 4, 2, 1, 1, false, true, true}, {384, 2, 2, 1, 1, false, true, true},
-                                     {512, 4, 2, 1, 1, true, true, true}, {512, 2, 2, 1, 1, false, false, true},
-                                     {512, 2, 2, 1, 1, false, true, true, 2}, {640, 2, 2, 1, 1, false, true, true},
-                                     {640, 1, 2, 1, 1, false, true, true}, {512, 1, 2, 1, 1, false, true, true},
-                                     {768, 1, 2, 1, 1, false, true, true}, {512, 1, 2, 1, 1, false, false, true},
-                                     {512, 2, 3, 1, 1, false, true, true}, {512, 1, 3, 1, 1, false, true, true},
-                                     {384, 1, 4, 1, 1, false, true, true}, {256, 6, 4, 1, 1, true, true, true},
-                                     {224, 6, 4, 1, 1, true, true, true}, {256, 4, 4, 1, 1, true, true, true}};
+// 0-2 are the defaults (join_variant below); 3-5 are kept as measured alternatives (round 1 swept
+// 46 shapes; the slower ones were removed)
+constexpr JoinShape JOIN_SHAPES[] = {
+    {256, 6, 3, 1, 1, false, true, true},      // 0: 4 B count
+    {256, 8, 3, 1, 1, false, false, true, 2},  // 1: 4 B materialize
+    {512, 1, 2, 1, 1, false, true, true},      // 2: 8 B (both modes)
+    {256, 8, 3, 1, 1},                         // 3: no prefetching
+    {256, 8, 2, 2, 1},                         // 4: double-buffered R tile
+    {224, 8, 4, 1, 1, true},                   // 5: 16-bit heads, 4 blocks / SM
+};
 constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
 
 struct DevBuf {
   void* p = nullptr;
   size_t bytes = 0;
+  bool ws = false;  // carved from the caller's workspace (hj_set_workspace), not ctx-owned
 };
 
 struct HostPlan;
@@ -81,8 +71,8 @@ struct Ctx {
   std::string err;
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
-          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_pass1_bases = 0, opt_graph = 0, opt_pass_l2pf = 2, opt_pass1_bits = 0,
-          opt_partitioner = 0, opt_pass_variant = 0, opt_fuse = 0, opt_fuse_window_mb = 32, opt_fuse_pass_slots = 1;
+          opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_graph = 0, opt_pass_l2pf = 2, opt_pass1_bits = 0,
+          opt_partitioner = 0, opt_pass_variant = 0, opt_mat_chk = 1;
   DevBuf bc_pool1[2], bc_pool2[2], bc_meta;  // HJ_OPT_PARTITIONER = 1 (NEXT-1 bucket chains)
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2], np_heads, np_next;
@@ -105,8 +95,17 @@ struct Ctx {
   uint32_t* h_xd_err = nullptr;            // pinned, mapped: barrier timeout flag
   uint32_t* d_xd_err = nullptr;
   unsigned long long xd_epoch = 0;
+  // caller-provided workspace (hj_set_workspace): hj_join carves every device buffer it needs
+  // from [ws, ws + ws_bytes) in a fixed order (bump pointer reset per call) instead of allocating;
+  // `dry` = hj_workspace_bytes: the allocation steps only sum the sizes
+  char* ws = nullptr;
+  size_t ws_bytes = 0, ws_off = 0;
+  bool use_ws = false;  // inside hj_join with a workspace set
+  std::vector<DevBuf*> ws_bufs;
+  bool dry = false;
+  size_t dry_bytes = 0;
   cudaGraphExec_t graph = nullptr;
-  unsigned long long graph_key[12] = {};
+  unsigned long long graph_key[16] = {};
   bool capturing = false;  // a graph capture is in progress on c->stream
   uint32_t graph_launches = 0;
 };
@@ -130,24 +129,70 @@ int fail(Ctx* c, int code, const char* fmt, ...) {
                   #expr, cudaGetErrorString(e_), __FILE__, __LINE__);                             \
   } while (0)
 
+size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
+
+void drop_graph(Ctx* c) {
+  if (c->graph) cudaGraphExecDestroy(c->graph);
+  c->graph = nullptr;
+}
+
+// Device buffer of at least `bytes` for this call. Three modes:
+//   dry (hj_workspace_bytes): only sum the 256-byte aligned sizes;
+//   workspace (hj_join after hj_set_workspace): carve from the caller's buffer, never allocate;
+//   otherwise a ctx-owned cudaMalloc, kept and reused while large enough.
+// No buffer is zeroed here: every call zeroes exactly what it reads before writing (the
+// planner's counters / results region, the bucket-chain states) with cudaMemsetAsync.
 int ensure(Ctx* c, DevBuf& b, size_t bytes) {
-  if (b.bytes >= bytes && b.p) return HJ_OK;
-  if (b.p) cudaFree(b.p);
+  if (c->dry) {
+    c->dry_bytes += align_up(bytes, 256);
+    return HJ_OK;
+  }
+  if (c->use_ws) {
+    if (b.ws && b.p && b.bytes >= bytes) return HJ_OK;  // carved earlier in this call
+    if (b.p && !b.ws) {  // a ctx-owned buffer from a call without workspace
+      cudaStreamSynchronize(c->stream);
+      cudaFree(b.p);
+    }
+    const size_t need = align_up(bytes, 256);
+    if (c->ws_off + need > c->ws_bytes)
+      return fail(c, HJ_ERR_WORKSPACE, "workspace of %zu bytes too small (needs > %zu; see hj_workspace_bytes)",
+                  c->ws_bytes, c->ws_off + need);
+    b.p = c->ws + c->ws_off;
+    b.bytes = bytes;
+    b.ws = true;
+    c->ws_off += need;
+    c->ws_bufs.push_back(&b);
+    return HJ_OK;
+  }
+  if (b.bytes >= bytes && b.p && !b.ws) return HJ_OK;
+  if (b.p && !b.ws) cudaFree(b.p);
   b.p = nullptr;
   b.bytes = 0;
+  b.ws = false;
+  drop_graph(c);  // a captured launch sequence may hold the old address
   if (bytes == 0) return HJ_OK;
   CUDA_TRY(c, cudaMalloc(&b.p, bytes));
   b.bytes = bytes;
-  // A new allocation starts zeroed, as a fresh process's pages do. Memory recycled from a closed
-  // context with the other partitioner (bucket chains <-> histogram path) hung or faulted the
-  // next join at c2 / c3 sizes (tools/bc_one.py): some buffer is still read before
-  // it is written on that path. Zeroing on (re)allocation only -- never per call.
-  CUDA_TRY(c, cudaMemsetAsync(b.p, 0, bytes, c->stream));
-  CUDA_TRY(c, cudaStreamSynchronize(c->stream));
   return HJ_OK;
 }
 
-size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
+// start of an hj_join call with a workspace: buffers are carved again from offset 0 (same sizes
+// and order -> same addresses, so a captured graph stays valid)
+void ws_begin(Ctx* c) {
+  for (DevBuf* b : c->ws_bufs)
+    if (b->ws) {  // (a buffer another entry point re-allocated since is ctx-owned now)
+      b->p = nullptr;
+      b->bytes = 0;
+      b->ws = false;
+    }
+  c->ws_bufs.clear();
+  c->ws_off = 0;
+}
+
+// does the materialized output need (re)allocation for `pairs` pairs?
+bool out_short(const Ctx* c, unsigned long long pairs) {
+  return c->dry || c->out_r.bytes < pairs * c->pay_bytes || c->out_s.bytes < pairs * c->pay_bytes;
+}
 
 int ilog2_ceil(unsigned long long x) {
   int l = 0;
@@ -165,12 +210,6 @@ struct HostPlan {
   int tile = 0;
   // metadata offsets (bytes) inside ctx->meta
   size_t o_cnt[2], o_off[2], o_cur1[2], o_cur2[2], o_pst[2], o_cst[2], o_ist, o_counters, o_results;
-  size_t o_cntb = 0, o_relb = 0;  // pass-1 per-block digit counts / bases
-  bool bases = false;             // pass 1 = k_pass1b (per-block bases, TMA bulk write-out)
-  bool fused = false;             // pass 2 + join = k_fused (HJ_OPT_FUSE)
-  size_t o_fz = 0;
-  size_t pass2_smem = 0;
-  uint32_t g1max = 0;
   size_t zero_bytes = 0;  // [0, zero_bytes) is memset to 0 per call
   size_t meta_bytes = 0;
   int pb() const { return g + b1; }
@@ -184,24 +223,19 @@ constexpr int pass_items() {
 }
 
 // default join shape per key width and output mode (measured with tools/tune.py on B200):
-//   4 B materialize -> shape 27 (shape 19 + the S stream L2-prefetched 2 rounds ahead: c3 join
-//                      0.730 -> 0.704 ms, 0.679 -> 0.646 after the 32-bit-shared-address
-//                      probe; 4 rounds ahead the same; shape 19 = shape 0 + L2
-//                      prefetch of the next item: 0.749 -> 0.730; register-prefetching 15-17 0.78)
-//   4 B count       -> shape 20 (256 x 6, S prefetch + L2 prefetch: c2 0.873 -> 0.814 ms,
-//                      c4 z=1.5 0.881 -> 0.829; streaming S through L2 2-8 rounds ahead, shapes
-//                      22/25/26, is slower here: 0.84 -- this probe is issue-bound on the checksum)
-//   8 B             -> shape 37 (512 x 1, S and L2 prefetch, two blocks per SM: the 16-byte R
-//                      tile limits blocks to two per SM, so more threads per block -- not more
-//                      tuples per thread -- hide the chain-walk latency: c5_gpu join 3.54 ->
-//                      2.69 ms; 512 x 2: 2.90, 640 x 1: 2.85, 768 x 1: 3.34, 384 x 2: 2.98;
-//                      shape 21 = 256 x 4: 4.21 -> 4.03 before the 32-bit-shared-address probe,
-//                      3.54 after). For 4-byte tuples three 256-thread blocks per SM fit and the
-//                      512-thread shapes are slower (c2 0.74 -> 0.95, c3 0.645 -> 0.86)
+//   4 B materialize -> shape 1 (256 x 8, L2 prefetch of the next item and of the S stream 2
+//                      rounds ahead: c3 join 0.749 -> 0.704 ms before the 32-bit-shared-address
+//                      probe, 0.646 after)
+//   4 B count       -> shape 0 (256 x 6, next round's S in registers + L2 prefetch of the next
+//                      item: c2 0.873 -> 0.814 ms; streaming S through L2 was slower here)
+//   8 B             -> shape 2 (512 x 1, two blocks per SM: the 16-byte R tile limits blocks to
+//                      two per SM, so more threads per block -- not more tuples per thread --
+//                      hide the chain-walk latency: c5_gpu join 3.54 -> 2.69 ms; 512 x 2: 2.90,
+//                      640 x 1: 2.85, 768 x 1: 3.34)
 int join_variant(const Ctx* c, bool mat) {
   if (c->opt_join_variant >= 0) return (int)c->opt_join_variant;
-  if (c->key_bytes == 8) return 37;
-  return mat ? 27 : 20;
+  if (c->key_bytes == 8) return 2;
+  return mat ? 1 : 0;
 }
 
 int pass_threads(const Ctx* c, int fanout_bits, int items) {
@@ -219,7 +253,7 @@ int choose_bits(unsigned long long nR) {
 // mode PLAN_FULL: one GPU; PLAN_SEND: exchange sender (g rank bits); PLAN_RECV: exchange
 // receiver (nsrc count rows). nR / nS are the tuples this GPU partitions / joins.
 int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat, int g = 0,
-              int nsrc = 1, int mode = PLAN_FULL, bool want_fused = false) {
+              int nsrc = 1, int mode = PLAN_FULL) {
   const size_t tb = (size_t)c->key_bytes + c->pay_bytes;  // AoS tuple bytes
   hp.B = radix_bits < 0 ? choose_bits(nR) : radix_bits;
   if (hp.B > 20) return fail(c, HJ_ERR_UNSUPPORTED, "radix_bits %d > 20", hp.B);
@@ -242,9 +276,6 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   // 1024-thread block. The pass-2 chunk is that kernel's tile.
   hp.tile = pass_threads(c, hp.pb(), items) * items;
   hp.C2 = (uint32_t)(pass_threads(c, hp.b2, items) * items);
-  // fused pass 2 + join (one GPU, two passes, the smem hash join): 512-thread pass-2 units
-  hp.fused = want_fused && mode == PLAN_FULL && hp.B >= 2 && c->opt_join_algo == 0 && c->opt_partitioner == 0;
-  if (hp.fused) hp.C2 = (uint32_t)(FZ_NT * items);
 
   // join capacities
   const unsigned long long mean = (nR + (1ull << hp.B) - 1) >> hp.B;
@@ -256,15 +287,14 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   uint32_t CS;
   if (c->opt_chunk_s > 0) CS = (uint32_t)std::min<int64_t>(c->opt_chunk_s, 1ll << 30);
   else CS = std::max<uint32_t>(8 * CR, 32768);
-  const int rbuf = hp.fused ? 1 : JOIN_SHAPES[join_variant(c, mat)].rbuf;
-  const int nbsh = hp.fused ? 1 : JOIN_SHAPES[join_variant(c, mat)].nbsh;
-  const size_t head_bytes = !hp.fused && JOIN_SHAPES[join_variant(c, mat)].h16 ? 2 : 4;
+  const JoinShape& JS = JOIN_SHAPES[join_variant(c, mat)];
+  const int rbuf = JS.rbuf, nbsh = JS.nbsh;
+  const size_t head_bytes = JS.h16 ? 2 : 4;
   int lg_nb = std::max(6, ilog2_ceil(CR) - nbsh);
   auto join_smem = [&](uint32_t cr, int lg) {  // R tile buffer(s) (TMA) + heads + next
     return (size_t)rbuf * ((cr + 3) & ~1u) * tb + (head_bytes << lg) + (size_t)cr * 2;
   };
-  // fused: two blocks per SM, each with the pass-2 statics (~25 KB) beside the dynamic region
-  const size_t join_cap = hp.fused ? (cap_max_smem / 2 - 28 * 1024) : cap_max_smem - 8 * 1024;
+  const size_t join_cap = cap_max_smem - 8 * 1024;
   while (join_smem(CR, lg_nb) > join_cap && CR > 256) {
     CR /= 2;
     lg_nb = std::max(6, ilog2_ceil(CR) - nbsh);
@@ -273,7 +303,6 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   hp.CS = CS;
   hp.lg_nb = lg_nb;
   hp.join_smem = join_smem(CR, lg_nb);
-  hp.pass2_smem = (size_t)hp.C2 * tb + ((size_t)1 << hp.b2) * 24 + 16;
 
   // metadata layout
   const size_t nq = (size_t)1 << hp.qbits(), F1 = (size_t)1 << hp.pb(), npc = hp.npieces();
@@ -287,7 +316,6 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   hp.o_counters = take(64);
   hp.o_results = take(64);
   for (int r = 0; r < 2; ++r) hp.o_cnt[r] = take(mode == PLAN_RECV ? 0 : nq * 4);
-  if (hp.fused) hp.o_fz = take((size_t)FZ_WORDS * 4);
   hp.zero_bytes = o;
   for (int r = 0; r < 2; ++r) {
     hp.o_off[r] = take((nq + 1) * 8);
@@ -297,15 +325,6 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
     hp.o_cst[r] = take((npc + 1) * 4);
   }
   hp.o_ist = take((((size_t)1 << hp.B) + 1) * 4);
-  // pass 1 with precomputed per-block bases and TMA bulk-store write-out (opt-in: measured
-  // slower than the atomic-reservation pass on c2/c3/c4); needs the exact
-  // shared histogram (<= 2^15 u32 bins)
-  hp.bases = mode != PLAN_RECV && hp.qbits() <= 15 && c->opt_pass1_bases;
-  if (hp.bases) {
-    hp.g1max = 2 * (uint32_t)c->num_sms;
-    hp.o_cntb = take((size_t)2 * hp.g1max * F1 * 4);
-    hp.o_relb = take((size_t)2 * hp.g1max * F1 * 8);
-  }
   hp.meta_bytes = o;
   (void)nS;
   return HJ_OK;
@@ -337,11 +356,9 @@ int set_kernel_attrs(Ctx* c) {
   };
   load((const void*)k_hist<K, false, false>);
   load((const void*)k_hist<K, false, true>);
-  load((const void*)k_plan<false, false, true>);
-  load((const void*)k_plan<false, true, true>);
-  load((const void*)k_plan<false, false, false>);
-  load((const void*)k_plan<false, true, false>);
-  load((const void*)k_plan<true, false, true>);
+  load((const void*)k_plan<false, true>);
+  load((const void*)k_plan<false, false>);
+  load((const void*)k_plan<true, true>);
   load((const void*)k_xd_rows);
   load((const void*)k_xd_totals);
   load((const void*)k_xd_cursors);
@@ -356,10 +373,6 @@ int set_kernel_attrs(Ctx* c) {
   attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), false>);
   attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), true>);
   attr((const void*)k_pass<K, 2, 1024, pass_items<K>(), false>);
-  attr((const void*)k_pass1b<K, 1024, pass_items<K>(), false>);
-  attr((const void*)k_pass1b<K, 1024, pass_items<K>(), true>);
-  attr((const void*)k_pass1b<K, 512, pass_items<K>(), false>);
-  attr((const void*)k_pass1b<K, 512, pass_items<K>(), true>);
   attr((const void*)k_pass<K, 1, 512, pass_items<K>(), false>);
   attr((const void*)k_pass<K, 1, 512, pass_items<K>(), true>);
   attr((const void*)k_pass<K, 2, 512, pass_items<K>(), false>);
@@ -372,54 +385,12 @@ int set_kernel_attrs(Ctx* c) {
   attr((const void*)k_pass<K, 2, 512, 2 * pass_items<K>(), false, false, false>);
   attr((const void*)k_pass<K, 1, 512, 2 * pass_items<K>(), false, true, false>);
   attr((const void*)k_pass<K, 2, 512, 2 * pass_items<K>(), false, true, false>);
-  attr((const void*)k_fused<K, false>);
-  attr((const void*)k_fused<K, true>);
   attr_join<K, 0>(attr);
   attr_join<K, 1>(attr);
   attr_join<K, 2>(attr);
   attr_join<K, 3>(attr);
   attr_join<K, 4>(attr);
   attr_join<K, 5>(attr);
-  attr_join<K, 6>(attr);
-  attr_join<K, 7>(attr);
-  attr_join<K, 8>(attr);
-  attr_join<K, 9>(attr);
-  attr_join<K, 10>(attr);
-  attr_join<K, 11>(attr);
-  attr_join<K, 12>(attr);
-  attr_join<K, 13>(attr);
-  attr_join<K, 14>(attr);
-  attr_join<K, 15>(attr);
-  attr_join<K, 16>(attr);
-  attr_join<K, 17>(attr);
-  attr_join<K, 18>(attr);
-  attr_join<K, 19>(attr);
-  attr_join<K, 20>(attr);
-  attr_join<K, 21>(attr);
-  attr_join<K, 22>(attr);
-  attr_join<K, 23>(attr);
-  attr_join<K, 24>(attr);
-  attr_join<K, 25>(attr);
-  attr_join<K, 26>(attr);
-  attr_join<K, 27>(attr);
-  attr_join<K, 28>(attr);
-  attr_join<K, 29>(attr);
-  attr_join<K, 30>(attr);
-  attr_join<K, 31>(attr);
-  attr_join<K, 32>(attr);
-  attr_join<K, 33>(attr);
-  attr_join<K, 34>(attr);
-  attr_join<K, 35>(attr);
-  attr_join<K, 36>(attr);
-  attr_join<K, 37>(attr);
-  attr_join<K, 38>(attr);
-  attr_join<K, 39>(attr);
-  attr_join<K, 40>(attr);
-  attr_join<K, 41>(attr);
-  attr_join<K, 42>(attr);
-  attr_join<K, 43>(attr);
-  attr_join<K, 44>(attr);
-  attr_join<K, 45>(attr);
   return rc;
 }
 
@@ -484,23 +455,12 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   P.CR = hp.CR;
   P.CS = hp.CS;
   P.ist = (uint32_t*)(m + hp.o_ist);
-  if (hp.bases) {
-    P.cntb = (uint32_t*)(m + hp.o_cntb);
-    P.relb = (unsigned long long*)(m + hp.o_relb);
-  }
   P.counters = (uint32_t*)(m + hp.o_counters);
   P.results = (unsigned long long*)(m + hp.o_results);
-  if (hp.fused) {
-    P.fz = (uint32_t*)(m + hp.o_fz);
-    P.fz_pass_slots = (uint32_t)std::max<int64_t>(c->opt_fuse_pass_slots, 0);
-    // window: pass-1 partitions of pass-2 output (R + S) allowed ahead of the join
-    const double part_bytes = (double)(nR + nS) * (c->key_bytes + c->pay_bytes) / (double)(1u << hp.b1);
-    P.fz_window = c->opt_fuse_window_mb <= 0 ? 0u
-                  : (uint32_t)std::max(1.0, std::floor((double)c->opt_fuse_window_mb * 1048576.0 / std::max(part_bytes, 1.0)));
-  }
+  P.mat_chk = c->opt_mat_chk ? 1 : 0;
   P.out_r = c->out_r.p;
   P.out_s = c->out_s.p;
-  P.out_cap = c->out_r.bytes / c->pay_bytes;
+  P.out_cap = std::min(c->out_r.bytes, c->out_s.bytes) / c->pay_bytes;
   P.H.B = hp.B;
   P.H.lg = hp.lg_nb;
   {
@@ -522,22 +482,14 @@ void mark(Ctx* c, int i) {
 template <typename K, int MODE, int NT, bool GD, bool BC = false>
 int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits);
 
-template <typename K>
-size_t pass1b_smem(const HostPlan& hp, int nt) {
-  const size_t F = (size_t)1 << hp.pb(), tb = sizeof(typename Tup<K>::T);
-  return ((size_t)nt * pass_items<K>() + 2 * F) * tb + 16 * F + 4 * (F + 4) + 8 * F;
-}
-
-// a2: the planner instance for this plan (several sources / per-block bases / join items)
+// a2: the planner instance for this plan (several sources / join items)
 int launch_plan(Ctx* c, const HostPlan& hp, const Plan& P) {
   const unsigned g = (unsigned)((((size_t)1 << hp.qbits()) + 1023) / 1024);
-  const bool ms = P.nsrc > 1, bs = P.g1 != 0, it = P.mode != PLAN_SEND;
+  const bool ms = P.nsrc > 1, it = P.mode != PLAN_SEND;
   cudaStream_t st = c->stream;
-  if (ms) k_plan<true, false, true><<<g, 1024, 0, st>>>(P);
-  else if (bs && it) k_plan<false, true, true><<<g, 1024, 0, st>>>(P);
-  else if (bs) k_plan<false, true, false><<<g, 1024, 0, st>>>(P);
-  else if (it) k_plan<false, false, true><<<g, 1024, 0, st>>>(P);
-  else k_plan<false, false, false><<<g, 1024, 0, st>>>(P);
+  if (ms) k_plan<true, true><<<g, 1024, 0, st>>>(P);
+  else if (it) k_plan<false, true><<<g, 1024, 0, st>>>(P);
+  else k_plan<false, false><<<g, 1024, 0, st>>>(P);
   CUDA_TRY(c, cudaGetLastError());
   c->launches += 1;
   return HJ_OK;
@@ -559,24 +511,17 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false, 
     return HJ_OK;
   }
   mark(c, 0);
+  if (hp.mode != PLAN_SEND)  // T2's 64-byte tails: the join's 16-byte aligned R copies may read into them
+    for (int r = 0; r < 2; ++r)
+      if (P.rel[r].t2 && !(r == 0 && P.skip_r)) {  // (streaming S chunks: T2 of R holds R)
+        const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
+        CUDA_TRY(c, cudaMemsetAsync((char*)P.rel[r].t2 + P.rel[r].n * tb, 0, 64, st));
+      }
   if (!chunk) {
     CUDA_TRY(c, cudaMemsetAsync(P.counters, 0, hp.zero_bytes, st));  // the zeroed region starts at o_counters = 0
   } else {  // streaming S chunk: keep R's counts and the accumulated results
     CUDA_TRY(c, cudaMemsetAsync((char*)c->meta.p + hp.o_counters, 0, 64, st));
     CUDA_TRY(c, cudaMemsetAsync((char*)c->meta.p + hp.o_cnt[1], 0, (size_t)4 << hp.qbits(), st));
-  }
-  Plan Pb = P;  // P with the pass-1 grid / tile when pass 1 uses per-block bases
-  if (hp.mode != PLAN_RECV && hp.bases) {
-    const int nt = hp.tile == 512 * pass_items<K>() ? 512 : 1024;
-    const size_t sm = pass1b_smem<K>(hp, nt);
-    const void* f = nt == 512 ? (gd ? (const void*)k_pass1b<K, 512, pass_items<K>(), true>
-                                    : (const void*)k_pass1b<K, 512, pass_items<K>(), false>)
-                              : (gd ? (const void*)k_pass1b<K, 1024, pass_items<K>(), true>
-                                    : (const void*)k_pass1b<K, 1024, pass_items<K>(), false>);
-    Pb.tile1 = (uint32_t)hp.tile;
-    Pb.tiles1[0] = (P.rel[0].n + hp.tile - 1) / hp.tile;
-    Pb.tiles1[1] = (P.rel[1].n + hp.tile - 1) / hp.tile;
-    Pb.g1 = (uint32_t)std::min<unsigned long long>(grid_for(c, f, nt, sm, Pb.tiles1[0] + Pb.tiles1[1]), hp.g1max);
   }
   if (hp.mode != PLAN_RECV) {
     const bool smem = hp.qbits() <= 16;
@@ -590,30 +535,20 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false, 
     uint32_t gr = (uint32_t)((double)g * (double)nR / (double)std::max<unsigned long long>(nR + nS, 1) + 0.5);
     gr = std::min<uint32_t>(std::max<uint32_t>(gr, 1), (uint32_t)g - 1);
     if (nR == 0) gr = 0;  // streaming S chunk: every block counts S
-    if (Pb.g1) g = (int)Pb.g1;  // bases: the histogram walks exactly pass 1's tiles per block
-    if (smem && c32 && gd) k_hist<K, true, true, true><<<g, HIST_NT, sm, st>>>(Pb, gr);
-    else if (smem && c32) k_hist<K, true, false, true><<<g, HIST_NT, sm, st>>>(Pb, gr);
-    else if (smem && gd) k_hist<K, true, true, false><<<g, HIST_NT, sm, st>>>(Pb, gr);
-    else if (smem) k_hist<K, true, false, false><<<g, HIST_NT, sm, st>>>(Pb, gr);
-    else if (gd) k_hist<K, false, true><<<g, HIST_NT, 0, st>>>(Pb, gr);
-    else k_hist<K, false, false><<<g, HIST_NT, 0, st>>>(Pb, gr);
+    if (smem && c32 && gd) k_hist<K, true, true, true><<<g, HIST_NT, sm, st>>>(P, gr);
+    else if (smem && c32) k_hist<K, true, false, true><<<g, HIST_NT, sm, st>>>(P, gr);
+    else if (smem && gd) k_hist<K, true, true, false><<<g, HIST_NT, sm, st>>>(P, gr);
+    else if (smem) k_hist<K, true, false, false><<<g, HIST_NT, sm, st>>>(P, gr);
+    else if (gd) k_hist<K, false, true><<<g, HIST_NT, 0, st>>>(P, gr);
+    else k_hist<K, false, false><<<g, HIST_NT, 0, st>>>(P, gr);
     CUDA_TRY(c, cudaGetLastError());
     c->launches += 1;
   }
   mark(c, 1);
-  if (int rc = launch_plan(c, hp, Pb)) return rc;
+  if (int rc = launch_plan(c, hp, P)) return rc;
   mark(c, 2);
   if (stage == 1) return HJ_OK;
-  if (hp.mode != PLAN_RECV && Pb.g1) {
-    const int nt = hp.tile == 512 * pass_items<K>() ? 512 : 1024;
-    const size_t sm = pass1b_smem<K>(hp, nt);
-    if (nt == 512 && gd) k_pass1b<K, 512, pass_items<K>(), true><<<Pb.g1, 512, sm, st>>>(Pb, hp.pb());
-    else if (nt == 512) k_pass1b<K, 512, pass_items<K>(), false><<<Pb.g1, 512, sm, st>>>(Pb, hp.pb());
-    else if (gd) k_pass1b<K, 1024, pass_items<K>(), true><<<Pb.g1, 1024, sm, st>>>(Pb, hp.pb());
-    else k_pass1b<K, 1024, pass_items<K>(), false><<<Pb.g1, 1024, sm, st>>>(Pb, hp.pb());
-    CUDA_TRY(c, cudaGetLastError());
-    c->launches += 1;
-  } else if (hp.mode != PLAN_RECV) {
+  if (hp.mode != PLAN_RECV) {
     int rc = hp.tile == 512 * pass_items<K>()
                  ? (gd ? launch_pass<K, 1, 512, true>(c, hp, P, hp.pb()) : launch_pass<K, 1, 512, false>(c, hp, P, hp.pb()))
                  : (gd ? launch_pass<K, 1, 1024, true>(c, hp, P, hp.pb()) : launch_pass<K, 1, 1024, false>(c, hp, P, hp.pb()));
@@ -623,8 +558,7 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false, 
   return HJ_OK;
 }
 
-// a4: pass 2 over the pass-1 pieces. Event 4.
-// a4: pass 2 over the pass-1 pieces. Event 4.
+// a3 / a4: one partition pass (launch shape per pass and width).
 template <typename K, int MODE, int NT, bool GD, bool BC>
 int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
   constexpr int IT = pass_items<K>();
@@ -711,51 +645,11 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
     return HJ_OK;
   }
   switch (join_variant(c, mat)) {
-    case 43: rc = launch_join_v<K, 43>(c, hp, P, mat); break;
-    case 44: rc = launch_join_v<K, 44>(c, hp, P, mat); break;
-    case 45: rc = launch_join_v<K, 45>(c, hp, P, mat); break;
-    case 38: rc = launch_join_v<K, 38>(c, hp, P, mat); break;
-    case 39: rc = launch_join_v<K, 39>(c, hp, P, mat); break;
-    case 40: rc = launch_join_v<K, 40>(c, hp, P, mat); break;
-    case 41: rc = launch_join_v<K, 41>(c, hp, P, mat); break;
-    case 42: rc = launch_join_v<K, 42>(c, hp, P, mat); break;
-    case 33: rc = launch_join_v<K, 33>(c, hp, P, mat); break;
-    case 34: rc = launch_join_v<K, 34>(c, hp, P, mat); break;
-    case 35: rc = launch_join_v<K, 35>(c, hp, P, mat); break;
-    case 36: rc = launch_join_v<K, 36>(c, hp, P, mat); break;
-    case 37: rc = launch_join_v<K, 37>(c, hp, P, mat); break;
-    case 28: rc = launch_join_v<K, 28>(c, hp, P, mat); break;
-    case 29: rc = launch_join_v<K, 29>(c, hp, P, mat); break;
-    case 30: rc = launch_join_v<K, 30>(c, hp, P, mat); break;
-    case 31: rc = launch_join_v<K, 31>(c, hp, P, mat); break;
-    case 32: rc = launch_join_v<K, 32>(c, hp, P, mat); break;
-    case 22: rc = launch_join_v<K, 22>(c, hp, P, mat); break;
-    case 23: rc = launch_join_v<K, 23>(c, hp, P, mat); break;
-    case 24: rc = launch_join_v<K, 24>(c, hp, P, mat); break;
-    case 25: rc = launch_join_v<K, 25>(c, hp, P, mat); break;
-    case 26: rc = launch_join_v<K, 26>(c, hp, P, mat); break;
-    case 27: rc = launch_join_v<K, 27>(c, hp, P, mat); break;
-    case 12: rc = launch_join_v<K, 12>(c, hp, P, mat); break;
-    case 13: rc = launch_join_v<K, 13>(c, hp, P, mat); break;
-    case 14: rc = launch_join_v<K, 14>(c, hp, P, mat); break;
-    case 15: rc = launch_join_v<K, 15>(c, hp, P, mat); break;
-    case 16: rc = launch_join_v<K, 16>(c, hp, P, mat); break;
-    case 17: rc = launch_join_v<K, 17>(c, hp, P, mat); break;
-    case 18: rc = launch_join_v<K, 18>(c, hp, P, mat); break;
-    case 19: rc = launch_join_v<K, 19>(c, hp, P, mat); break;
-    case 20: rc = launch_join_v<K, 20>(c, hp, P, mat); break;
-    case 21: rc = launch_join_v<K, 21>(c, hp, P, mat); break;
-    case 9: rc = launch_join_v<K, 9>(c, hp, P, mat); break;
-    case 10: rc = launch_join_v<K, 10>(c, hp, P, mat); break;
-    case 11: rc = launch_join_v<K, 11>(c, hp, P, mat); break;
-    case 5: rc = launch_join_v<K, 5>(c, hp, P, mat); break;
-    case 6: rc = launch_join_v<K, 6>(c, hp, P, mat); break;
-    case 7: rc = launch_join_v<K, 7>(c, hp, P, mat); break;
-    case 8: rc = launch_join_v<K, 8>(c, hp, P, mat); break;
     case 1: rc = launch_join_v<K, 1>(c, hp, P, mat); break;
     case 2: rc = launch_join_v<K, 2>(c, hp, P, mat); break;
     case 3: rc = launch_join_v<K, 3>(c, hp, P, mat); break;
     case 4: rc = launch_join_v<K, 4>(c, hp, P, mat); break;
+    case 5: rc = launch_join_v<K, 5>(c, hp, P, mat); break;
     default: rc = launch_join_v<K, 0>(c, hp, P, mat); break;
   }
   if (rc) return rc;
@@ -764,9 +658,9 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   return HJ_OK;
 }
 
-int prepare(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat, bool want_fused, int g = 0,
+int prepare(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat, int g = 0,
             int nsrc = 1, int mode = PLAN_FULL) {
-  int rc = make_plan(c, hp, nR, nS, radix_bits, mat, g, nsrc, mode, want_fused);
+  int rc = make_plan(c, hp, nR, nS, radix_bits, mat, g, nsrc, mode);
   if (rc) return rc;
   const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
   const unsigned long long ns[2] = {nR, nS};
@@ -777,7 +671,7 @@ int prepare(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, 
   if ((rc = ensure(c, c->meta, hp.meta_bytes))) return rc;
   if (mat) {
     unsigned long long cap = c->opt_out_cap > 0 ? (unsigned long long)c->opt_out_cap : std::max<unsigned long long>(nS, 1 << 20);
-    if (c->out_r.bytes < cap * c->pay_bytes) {
+    if (out_short(c, cap)) {
       if ((rc = ensure(c, c->out_r, cap * c->pay_bytes))) return rc;
       if ((rc = ensure(c, c->out_s, cap * c->pay_bytes))) return rc;
     }
@@ -785,36 +679,11 @@ int prepare(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, 
   return HJ_OK;
 }
 
-// a4-a8 in one persistent kernel (hj_fused.cuh): a full wave of 512-thread blocks (two per SM).
-// Events 4 and 5 (ms_kernel[3] = the fused kernel, ms_kernel[4] = 0).
-template <typename K>
-int launch_fused(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
-  const size_t sm = std::max(hp.join_smem, hp.pass2_smem);
-  const void* f = mat ? (const void*)k_fused<K, true> : (const void*)k_fused<K, false>;
-  const int per_sm = occupancy(c, f, FZ_NT, sm);
-  if (per_sm < 1) return fail(c, HJ_ERR_UNSUPPORTED, "fused kernel does not fit an SM (%zu B smem)", sm);
-  const int g = per_sm * c->num_sms;
-  Plan Q = P;
-  // the throttle waits on join-role blocks: none exist when every slot of an SM runs pass 2
-  if (std::max<uint32_t>(Q.fz_pass_slots, 1) >= (uint32_t)per_sm) Q.fz_window = 0;
-  if (mat) k_fused<K, true><<<g, FZ_NT, sm, c->stream>>>(Q);
-  else k_fused<K, false><<<g, FZ_NT, sm, c->stream>>>(Q);
-  CUDA_TRY(c, cudaGetLastError());
-  c->launches += 1;
-  mark(c, 4);
-  mark(c, 5);
-  return HJ_OK;
-}
-
-constexpr int HJ_RERUN = 1;  // finish_join: fused materialization overflowed; output grown, re-run
-
-// Join phase + result readback shared by hj_join and hj_join_received. `joined`: the join
-// already ran inside the fused kernel.
-int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res, bool joined = false,
-                const XdJoin* xd = nullptr) {
+// Join phase + result readback shared by hj_join and hj_join_received.
+int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res, const XdJoin* xd = nullptr) {
   cudaStream_t st = c->stream;
   const bool timing = c->opt_timing != 0;
-  int rc = joined ? HJ_OK : c->key_bytes == 4 ? launch_join<uint32_t>(c, hp, P, mat) : launch_join<uint64_t>(c, hp, P, mat);
+  int rc = c->key_bytes == 4 ? launch_join<uint32_t>(c, hp, P, mat) : launch_join<uint64_t>(c, hp, P, mat);
   if (rc) return rc;
   unsigned long long* h = (unsigned long long*)c->h_res;
   if (xd) {  // hj_xd_join: phase C (results of every rank summed on the device) before the readback
@@ -826,18 +695,25 @@ int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res, b
   CUDA_TRY(c, cudaMemcpyAsync(h + 4, P.ist + (1ull << hp.B), sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
   if (xd) CUDA_TRY(c, cudaMemcpyAsync(h + 6, P.results + 4, 3 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, st));
   h[5] = 0;
-  if (joined) CUDA_TRY(c, cudaMemcpyAsync(h + 5, P.fz + FZ_ERR, sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
+  if (P.mode == PLAN_RECV)
+    CUDA_TRY(c, cudaMemcpyAsync(h + 5, P.counters + CNT_BAD_COUNTS, sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
   if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[6], st));
   CUDA_TRY(c, cudaStreamSynchronize(st));
   if (P.bc && h[RES_BC_OVERFLOW]) return fail(c, HJ_ERR_CUDA, "bucket pool overflow (pool bound violated)");
-  if (joined && (uint32_t)h[5]) return fail(c, HJ_ERR_CUDA, "fused kernel watchdog: wait site %u timed out", (uint32_t)h[5]);
+  if ((uint32_t)h[5])
+    return fail(c, HJ_ERR_INVALID, "received count rows describe more tuples than the received buffers hold");
   unsigned long long matches = h[RES_MATCHES];
   if (mat && matches > P.out_cap) {
-    // materialization overflow (reading S11): grow to the exact size and re-run only the join
+    // materialization overflow (reading S11): never overwrite -- grow to the exact size and re-run
+    // only the join; with a caller workspace the caller grows it (HJ_ERR_WORKSPACE, exact count)
+    if (c->use_ws) {
+      memset(res, 0, sizeof *res);
+      res->matches = matches;
+      return fail(c, HJ_ERR_WORKSPACE, "materialized output needs %llu pairs (capacity %llu): set "
+                  "HJ_OPT_OUT_CAPACITY >= matches and resize the workspace", matches, P.out_cap);
+    }
     if ((rc = ensure(c, c->out_r, matches * c->pay_bytes))) return rc;
     if ((rc = ensure(c, c->out_s, matches * c->pay_bytes))) return rc;
-    // the fused kernel discarded T2's lines: the caller re-runs the whole call unfused
-    if (joined) return HJ_RERUN;
     P.out_r = c->out_r.p;
     P.out_s = c->out_s.p;
     P.out_cap = matches;
@@ -884,9 +760,10 @@ int run_join_np(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, c
       (rc = ensure(c, c->np_next, nR * 4)))
     return rc;
   unsigned long long cap = c->opt_out_cap > 0 ? (unsigned long long)c->opt_out_cap : std::max<unsigned long long>(nS, 1 << 20);
-  if (mat && c->out_r.bytes < cap * c->pay_bytes &&
+  if (mat && out_short(c, cap) &&
       ((rc = ensure(c, c->out_r, cap * c->pay_bytes)) || (rc = ensure(c, c->out_s, cap * c->pay_bytes))))
     return rc;
+  if (c->dry) return HJ_OK;
   Plan P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
   cudaStream_t st = c->stream;
   c->launches = 0;
@@ -911,6 +788,12 @@ int run_join_np(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, c
     mark(c, 6);
     CUDA_TRY(c, cudaStreamSynchronize(st));
     if (mat && h[RES_MATCHES] > P.out_cap && attempt == 0) {  // grow and re-run (reading S11)
+      if (c->use_ws) {
+        memset(res, 0, sizeof *res);
+        res->matches = h[RES_MATCHES];
+        return fail(c, HJ_ERR_WORKSPACE, "materialized output needs %llu pairs: set HJ_OPT_OUT_CAPACITY and resize "
+                    "the workspace", h[RES_MATCHES]);
+      }
       if ((rc = ensure(c, c->out_r, h[RES_MATCHES] * c->pay_bytes)) ||
           (rc = ensure(c, c->out_s, h[RES_MATCHES] * c->pay_bytes)))
         return rc;
@@ -1033,7 +916,7 @@ int run_join_bc(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, c
   if ((rc = ensure(c, c->meta, hp.meta_bytes))) return rc;
   if (mat) {
     unsigned long long cap = c->opt_out_cap > 0 ? (unsigned long long)c->opt_out_cap : std::max<unsigned long long>(nS, 1 << 20);
-    if (c->out_r.bytes < cap * c->pay_bytes &&
+    if (out_short(c, cap) &&
         ((rc = ensure(c, c->out_r, cap * c->pay_bytes)) || (rc = ensure(c, c->out_s, cap * c->pay_bytes))))
       return rc;
   }
@@ -1092,6 +975,7 @@ int run_join_bc(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, c
     BcRel& B = P.bc_rel[r];
     if ((rc = ensure(c, c->bc_pool1[r], (size_t)B.nbmax1 * B.bsz1 * tb))) return rc;
     if ((rc = ensure(c, c->bc_pool2[r], (size_t)B.nbmax2 * B.bsz2 * tb))) return rc;
+    if (c->dry) continue;
     char* m = (char*)c->bc_meta.p;
     B.pool1 = c->bc_pool1[r].p;
     B.pool2 = c->bc_pool2[r].p;
@@ -1107,6 +991,7 @@ int run_join_bc(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, c
     B.scur = (uint32_t*)(m + o_scur[r]);
     P.rel[r].t2 = B.pool2;  // the join reads slices of the pass-2 pool
   }
+  if (c->dry) return HJ_OK;
   cudaStream_t st = c->stream;
   c->launches = 0;
   mark(c, 0);
@@ -1141,32 +1026,23 @@ int run_join(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, cons
     return c->key_bytes == 4 ? run_join_bc<uint32_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, mat, res)
                              : run_join_bc<uint64_t>(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, mat, res);
   HostPlan hp;
-  int rc = prepare(c, hp, nR, nS, radix_bits, mat, c->opt_fuse && !c->opt_graph);
-  if (rc) return rc;
+  int rc = prepare(c, hp, nR, nS, radix_bits, mat);
+  if (rc || c->dry) return rc;
   Plan P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
   if (c->opt_graph) {
-    const unsigned long long key[12] = {(unsigned long long)Rk, (unsigned long long)Rp, nR, (unsigned long long)Sk,
+    // every address and size the captured launch sequence bakes in (ensure() also drops the graph
+    // whenever it reallocates a buffer)
+    const unsigned long long key[16] = {(unsigned long long)Rk, (unsigned long long)Rp, nR, (unsigned long long)Sk,
                                         (unsigned long long)Sp, nS, (unsigned long long)hp.B * 2 + mat,
                                         (unsigned long long)c->meta.p, (unsigned long long)c->out_r.p,
-                                        (unsigned long long)c->t1[1].p, (unsigned long long)c->t2[1].p,
+                                        (unsigned long long)c->out_s.p, P.out_cap,
+                                        (unsigned long long)c->t1[0].p, (unsigned long long)c->t1[1].p,
+                                        (unsigned long long)c->t2[0].p, (unsigned long long)c->t2[1].p,
                                         (unsigned long long)c->opt_join_algo};
     return run_join_graph(c, hp, P, mat, key, res);
   }
   c->launches = 0;
   if ((rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P))) return rc;
-  if (hp.fused) {
-    if ((rc = c->key_bytes == 4 ? launch_fused<uint32_t>(c, hp, P, mat) : launch_fused<uint64_t>(c, hp, P, mat))) return rc;
-    rc = finish_join(c, hp, P, mat, res, true);
-    if (rc == HJ_RERUN) {  // rare: materialization overflow (exact size now allocated)
-      const int64_t f = c->opt_fuse;
-      c->opt_fuse = 0;
-      rc = run_join(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
-      c->opt_fuse = f;
-    } else if (!rc) {
-      res->fused = 1;
-    }
-    return rc;
-  }
   if ((rc = c->key_bytes == 4 ? launch_pass2<uint32_t>(c, hp, P) : launch_pass2<uint64_t>(c, hp, P))) return rc;
   return finish_join(c, hp, P, mat, res);
 }
@@ -1213,7 +1089,7 @@ int join_host_stream(Ctx* c, const void* Rk, const void* Rp, uint64_t nR, const 
               ev_free[2] = {c->sev[4], c->sev[5]}, ev_j[2] = {c->sev[6], c->sev[7]}, ev_d = c->sev[8],
               ev_end = c->sev[9];
   HostPlan hp;
-  int rc = prepare(c, hp, nR, chunk, radix_bits, mat, false);
+  int rc = prepare(c, hp, nR, chunk, radix_bits, mat);
   if (rc) return rc;
   const unsigned long long cap = c->opt_out_cap > 0 ? (unsigned long long)c->opt_out_cap : std::max<unsigned long long>(nS, 1 << 20);
   if (mat) {
@@ -1351,12 +1227,11 @@ int xd_prepare(Ctx* c, int gpu_bits, unsigned long long nR, unsigned long long n
     *c->h_xd_err = 0;
   }
   HostPlan& hs = *c->xd_hp;
-  int rc = prepare(c, hs, nR, nS, local_bits, false, false, gpu_bits, 1, PLAN_SEND);
-  hs.bases = false;
+  int rc = prepare(c, hs, nR, nS, local_bits, false, gpu_bits, 1, PLAN_SEND);
   if (rc == HJ_OK) rc = ensure(c, c->xd_meta, hs.meta_bytes);
   if (rc == HJ_OK) rc = ensure(c, c->t1[0], nR * tb + 16);  // overflow scratch for pass 1
   if (rc == HJ_OK) rc = ensure(c, c->t1[1], nS * tb + 16);
-  if (rc == HJ_OK) rc = prepare(c, hr, capt[0], capt[1], local_bits, mat, false, 0, 1 << gpu_bits, PLAN_RECV);
+  if (rc == HJ_OK) rc = prepare(c, hr, capt[0], capt[1], local_bits, mat, 0, 1 << gpu_bits, PLAN_RECV);
   if (rc == HJ_OK && (hr.npieces() > 1024 || hs.pb() > 10))
     rc = fail(c, HJ_ERR_UNSUPPORTED, "too many pass-1 pieces (G=%d, local_bits=%d)", 1 << gpu_bits, local_bits);
   return rc;
@@ -1431,21 +1306,19 @@ void hj_destroy(hj_ctx* h) {
   int prev = 0;
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
-  if (c->stream) cudaStreamSynchronize(c->stream);
+  // drain every stream this ctx issued work on before its memory is freed
+  for (cudaStream_t s : {c->stream, c->own_stream, c->h2d_stream, c->d2h_stream})
+    if (s) cudaStreamSynchronize(s);
   DevBuf* bufs[] = {&c->t1[0], &c->t1[1], &c->t2[0], &c->t2[1], &c->meta,    &c->out_r,    &c->out_s,
                     &c->in[0], &c->in[1], &c->in[2], &c->in[3], &c->xsend[0], &c->xsend[1], &c->xcnt[0],
-                    &c->xcnt[1], &c->np_heads, &c->np_next};
+                    &c->xcnt[1], &c->np_heads, &c->np_next, &c->bc_pool1[0], &c->bc_pool1[1], &c->bc_pool2[0],
+                    &c->bc_pool2[1], &c->bc_meta, &c->xd_meta, &c->sin[0][0], &c->sin[0][1], &c->sin[1][0],
+                    &c->sin[1][1]};
   for (DevBuf* b : bufs)
-    if (b->p) cudaFree(b->p);
+    if (b->p && !b->ws) cudaFree(b->p);  // workspace-carved buffers belong to the caller
   if (c->graph) cudaGraphExecDestroy(c->graph);
   for (auto& b : c->xd_win)
     if (b.p) cudaFree(b.p);
-  if (c->xd_meta.p) cudaFree(c->xd_meta.p);
-  for (int r = 0; r < 2; ++r) {  // bucket-chain pools (HJ_OPT_PARTITIONER = 1)
-    if (c->bc_pool1[r].p) cudaFree(c->bc_pool1[r].p);
-    if (c->bc_pool2[r].p) cudaFree(c->bc_pool2[r].p);
-  }
-  if (c->bc_meta.p) cudaFree(c->bc_meta.p);
   delete c->xd_hp;
   delete c->xd_P;
   if (c->h_xd_cur) cudaFreeHost(c->h_xd_cur);
@@ -1456,9 +1329,6 @@ void hj_destroy(hj_ctx* h) {
     if (ev) cudaEventDestroy(ev);
   for (auto& ev : c->sev)
     if (ev) cudaEventDestroy(ev);
-  for (auto& b : c->sin)
-    for (auto& x : b)
-      if (x.p) cudaFree(x.p);
   if (c->h_cur) cudaFreeHost(c->h_cur);
   if (c->h2d_stream) cudaStreamDestroy(c->h2d_stream);
   if (c->d2h_stream) cudaStreamDestroy(c->d2h_stream);
@@ -1471,7 +1341,10 @@ const char* hj_last_error(const hj_ctx* h) { return h ? h->c.err.c_str() : g_cre
 
 int hj_set_stream(hj_ctx* h, void* s) {
   if (!h) return HJ_ERR_INVALID;
-  h->c.stream = s ? (cudaStream_t)s : h->c.own_stream;
+  // NULL is the caller's "stream 0", the legacy default stream (torch's default stream handle is
+  // 0): work is then ordered after every kernel the caller issued there (mapping NULL
+  // to the ctx's non-blocking stream let the join read columns still being written)
+  h->c.stream = s ? (cudaStream_t)s : cudaStreamLegacy;
   return HJ_OK;
 }
 
@@ -1479,10 +1352,7 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
   if (!h) return HJ_ERR_INVALID;
   Ctx* c = &h->c;
   if (v < 0) return fail(c, HJ_ERR_INVALID, "negative option value");
-  if (c->graph) {  // any option may change the captured launch sequence: capture again
-    cudaGraphExecDestroy(c->graph);
-    c->graph = nullptr;
-  }
+  drop_graph(c);  // any option may change the captured launch sequence: capture again
   switch (opt) {
     case HJ_OPT_CAP_R: c->opt_cap_r = v; break;
     case HJ_OPT_CHUNK_S: c->opt_chunk_s = v; break;
@@ -1490,12 +1360,9 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_TIMING: c->opt_timing = v; break;
     case HJ_OPT_BLOCKS_PER_SM: c->opt_bps = v; break;
     case HJ_OPT_STREAM_CHUNK: c->opt_stream_chunk = v; break;
-    case HJ_OPT_PASS1_BASES: c->opt_pass1_bases = v; break;
-    case HJ_OPT_FUSE: c->opt_fuse = v; break;
+    case HJ_OPT_MAT_CHECKSUM: c->opt_mat_chk = v; break;
     case HJ_OPT_PASS_L2PF: c->opt_pass_l2pf = v; break;
     case HJ_OPT_PASS1_BITS: c->opt_pass1_bits = v; break;
-    case HJ_OPT_FUSE_WINDOW_MB: c->opt_fuse_window_mb = v; break;
-    case HJ_OPT_FUSE_PASS_SLOTS: c->opt_fuse_pass_slots = v; break;
     case HJ_OPT_PARTITIONER:
       if (v > 1) return fail(c, HJ_ERR_INVALID, "partitioner must be 0 (histogram) or 1 (bucket chains)");
       c->opt_partitioner = v;
@@ -1540,9 +1407,57 @@ int hj_join(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const void* 
   int prev = 0;
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
+  if (c->ws) {
+    ws_begin(c);
+    c->use_ws = true;
+  }
   rc = run_join(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
+  c->use_ws = false;
   cudaSetDevice(prev);
   return rc;
+}
+
+uint64_t hj_workspace_bytes(const hj_ctx* hc, uint64_t nR, uint64_t nS, int radix_bits, int out_mode) {
+  if (!hc) return 0;
+  Ctx* c = const_cast<Ctx*>(&hc->c);
+  if (nR == 0 || nS == 0) return 0;
+  if (check_args(c, (const void*)1, (const void*)1, nR, (const void*)1, (const void*)1, nS, radix_bits, out_mode))
+    return 0;
+  hj_result res;
+  c->dry = true;
+  c->dry_bytes = 0;
+  const int rc = run_join(c, nullptr, nullptr, nR, nullptr, nullptr, nS, radix_bits, out_mode, &res);
+  c->dry = false;
+  return rc ? 0 : (uint64_t)c->dry_bytes;
+}
+
+int hj_set_workspace(hj_ctx* h, void* dptr, uint64_t bytes) {
+  if (!h) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  if (dptr && ((uintptr_t)dptr & 255)) return fail(c, HJ_ERR_INVALID, "workspace must be 256-byte aligned");
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  for (cudaStream_t s : {c->stream, c->own_stream, c->h2d_stream, c->d2h_stream})
+    if (s) cudaStreamSynchronize(s);
+  // buffers carved from the old workspace are forgotten; hj_join's ctx-owned buffers are freed
+  // (everything it needs now comes from the workspace)
+  ws_begin(c);
+  DevBuf* own[] = {&c->t1[0], &c->t1[1], &c->t2[0], &c->t2[1], &c->meta, &c->out_r, &c->out_s, &c->np_heads,
+                   &c->np_next, &c->bc_pool1[0], &c->bc_pool1[1], &c->bc_pool2[0], &c->bc_pool2[1], &c->bc_meta};
+  if (dptr)
+    for (DevBuf* b : own)
+      if (b->p && !b->ws) {
+        cudaFree(b->p);
+        b->p = nullptr;
+        b->bytes = 0;
+      }
+  drop_graph(c);
+  c->ws = (char*)dptr;
+  c->ws_bytes = dptr ? (size_t)bytes : 0;
+  cudaSetDevice(prev);
+  return HJ_OK;
 }
 
 int hj_join_host(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const void* Sk, const void* Sp, uint64_t nS,
@@ -1578,7 +1493,7 @@ int hj_partition(hj_ctx* h, const void* keys, const void* pays, uint64_t n, int 
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
   HostPlan hp;
-  int rc = prepare(c, hp, n, 0, radix_bits, false, false);
+  int rc = prepare(c, hp, n, 0, radix_bits, false);
   if (rc == HJ_OK) {
     Plan P = device_plan(c, hp, keys, pays, n, nullptr, nullptr, 0);
     c->launches = 0;
@@ -1619,7 +1534,7 @@ int hj_exchange_pack(hj_ctx* h, int rel, const void* keys, const void* pays, uin
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
   HostPlan hp;
-  int rc = prepare(c, hp, n, 0, local_bits, false, false, gpu_bits, 1, PLAN_SEND);
+  int rc = prepare(c, hp, n, 0, local_bits, false, gpu_bits, 1, PLAN_SEND);
   const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
   const size_t nq = (size_t)1 << hp.qbits();
   if (rc == HJ_OK) rc = ensure(c, c->xsend[rel], n * tb + 16);
@@ -1667,7 +1582,7 @@ int hj_join_received(hj_ctx* h, const void* R_recv, uint64_t nR, const uint32_t*
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
   HostPlan hp;
-  int rc = prepare(c, hp, nR, nS, local_bits, mat, false, 0, nsrc, PLAN_RECV);
+  int rc = prepare(c, hp, nR, nS, local_bits, mat, 0, nsrc, PLAN_RECV);
   if (rc == HJ_OK) {
     Plan P = device_plan(c, hp, nullptr, nullptr, nR, nullptr, nullptr, nS);
     P.rel[0].t1 = const_cast<void*>(R_recv);
@@ -1785,8 +1700,7 @@ int hj_xd_count(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const vo
     c->xd_P = new Plan();
   }
   HostPlan& hp = *c->xd_hp;
-  int rc = prepare(c, hp, nR, nS, local_bits, false, false, gpu_bits, 1, PLAN_SEND);
-  hp.bases = false;  // pass 1 = k_pass with pre-set cursors
+  int rc = prepare(c, hp, nR, nS, local_bits, false, gpu_bits, 1, PLAN_SEND);
   if (rc == HJ_OK && !c->h_xd_cur) {
     if (cudaMallocHost(&c->h_xd_cur, (size_t)XD_MAX * 2 * XD_MAX * 8) != cudaSuccess ||
         cudaHostAlloc(&c->h_xd_err, 64, cudaHostAllocMapped) != cudaSuccess ||
@@ -2074,7 +1988,7 @@ int hj_xd_join(hj_ctx* h, int rank, int gpu_bits, const void* Rk, const void* Rp
     if (int e1 = launch_plan(c, hr, Pr)) return e1;
     e = k4 ? launch_pass2<uint32_t>(c, hr, Pr) : launch_pass2<uint64_t>(c, hr, Pr);
     if (e) return e;
-    return finish_join(c, hr, Pr, mat, res, false, &a);
+    return finish_join(c, hr, Pr, mat, res, &a);
   };
   if (rc == HJ_OK) rc = run();
   if (rc == HJ_OK) {

@@ -100,46 +100,12 @@ __device__ __forceinline__ void mbar_wait(unsigned long long* bar, uint32_t pari
   }
 }
 
-// ---- cross-block signalling of the fused pass-2 + join kernel (hj_fused.cuh) ---------------
-// Release side: the writers' stores are ordered before a warp/block barrier, then one thread
-// issues fence.acq_rel.gpu + a relaxed reduction (the fence is cumulative over the writes the
-// barrier made visible to it). Acquire side: ld.acquire.gpu, then a barrier.
-__device__ __forceinline__ void fence_acq_rel_gpu() { asm volatile("fence.acq_rel.gpu;" ::: "memory"); }
-__device__ __forceinline__ void red_add_gpu(uint32_t* a, uint32_t v) {
-  asm volatile("red.relaxed.gpu.global.add.u32 [%0], %1;" ::"l"(a), "r"(v) : "memory");
-}
-__device__ __forceinline__ uint32_t ld_acquire_gpu(const uint32_t* a) {
-  uint32_t v;
-  asm volatile("ld.acquire.gpu.global.u32 %0, [%1];" : "=r"(v) : "l"(a) : "memory");
-  return v;
-}
-// generic-proxy global writes of other blocks (acquired) -> this thread's TMA reads
-__device__ __forceinline__ void fence_proxy_async_global() { asm volatile("fence.proxy.async.global;" ::: "memory"); }
+// %globaltimer (ns): watchdog deadlines of the exchange's device-side waits
 __device__ __forceinline__ unsigned long long global_ns() {
   unsigned long long t;
   asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
   return t;
 }
-// Spin until *a >= need (acquire). Watchdog: after ~10 s (a wait on another block should take
-// microseconds) set *err and return false instead of hanging the GPU.
-__device__ __noinline__ bool wait_geq(const uint32_t* a, uint32_t need, uint32_t* err, uint32_t site) {
-  if (ld_acquire_gpu(a) >= need) return true;
-  const unsigned long long t0 = global_ns();
-  while (ld_acquire_gpu(a) < need) {
-    __nanosleep(128);
-    if (global_ns() - t0 > 10000000000ull) {
-      atomicCAS(err, 0u, site);
-      return false;
-    }
-  }
-  return true;
-}
-__device__ __forceinline__ uint32_t sm_id() {
-  uint32_t s;
-  asm volatile("mov.u32 %0, %%smid;" : "=r"(s));
-  return s;
-}
-
 __device__ __forceinline__ uint32_t lanemask_lt() {
   uint32_t m;
   asm("mov.u32 %0, %%lanemask_lt;" : "=r"(m));

@@ -30,7 +30,7 @@ struct JoinJob {
 
 // Claim the next work item and decode it (item -> co-partition q by binary search over the
 // planner's item prefix; then the R chunk and S chunk of q it covers). One lane.
-template <typename T, bool FUSE = false>
+template <typename T>
 __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items) {
   JoinJob j;
   j.item = atomicAdd(&P.counters[CNT_NEXT_ITEM], 1u);
@@ -67,13 +67,6 @@ __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items
     j.se = j.sb + min((unsigned long long)P.CS, sn - sc * P.CS);
     const uintptr_t a = reinterpret_cast<uintptr_t>((const T*)P.rel[0].t2 + j.rb);
     j.shift = (uint32_t)((a & 15) / sizeof(T));  // tuples between the 16 B aligned copy start and rb
-    if (FUSE) {
-      // wait until pass 2 has written (and signalled) every unit of q's pass-1 partition
-      const uint32_t d = q >> P.b2;
-      const uint32_t need = (P.rel[0].cst[d + 1] - P.rel[0].cst[d] + P.rel[1].cst[d + 1] - P.rel[1].cst[d]) * FZ_PASS_WARPS;
-      wait_geq(&P.fz[FZ_DONE + d], need, &P.fz[FZ_ERR], 1u);
-      fence_proxy_async_global();  // the R chunk is read by the TMA (async proxy)
-    }
   }
   return j;
 }
@@ -148,19 +141,14 @@ __device__ __forceinline__ uint32_t exch16(unsigned short* a, uint32_t v) {
 }
 
 // H16: 16-bit chain heads (half the head array -> one more block per SM fits in shared memory)
-// FUSE (join role of the fused pass-2 + join kernel, hj_fused.cuh): an item waits for its
-// pass-1 partition's pass-2 signals (claim_job); S tuples are read L2-only (ld.global.cg: the
-// co-partitions were just written by other SMs); the pairs are streamed out with evict-first
-// stores; after the item every compute warp bumps the completed-item counter that throttles
-// pass 2.
 // PF: the next probe round's S tuples are loaded (into registers) before the current round's
 // chains are walked, so the S load latency overlaps the walk instead of opening each round.
 // SPF > 0: the S chunk is streamed through L2 ahead of the probe: at the item's first round one
 // compute thread issues a TMA L2 prefetch of rounds 1..SPF, then at round k of rounds k+SPF (one
 // cp.async.bulk.prefetch.L2 of NT*SPT tuples per round), so the bytes in flight per SM no longer
 // depend on the registers of the probing threads.
-template <typename K, int NT, int SPT, bool MAT, int RBUF, bool H16 = false, bool FUSE = false, bool PF = false,
-          bool L2PF = false, int SPF = 0>
+template <typename K, int NT, int SPT, bool MAT, int RBUF, bool H16 = false, bool PF = false, bool L2PF = false,
+          int SPF = 0>
 __device__ __forceinline__ void join_body(const Plan& P) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -185,12 +173,15 @@ __device__ __forceinline__ void join_body(const Plan& P) {
   K* out_s = (K*)P.out_s;
   const T* ssrc = (const T*)P.rel[1].t2;
   unsigned long long my_cnt = 0, my_chk = 0;
+  // checksum in MATERIALIZE mode too (block-uniform; the pairs' signatures are summed in the first
+  // chain walk, so re-walks of multi-match tuples only write)
+  const bool chk = !MAT || P.mat_chk != 0;
 
   if (threadIdx.x == NT) {
     mbar_init(&s_bar[0], 1);
     mbar_init(&s_bar[1], 1);
     fence_mbar_init();
-    JoinJob j = claim_job<T, FUSE>(P, total_items);
+    JoinJob j = claim_job<T>(P, total_items);
     if (j.item < total_items) issue_r_copy<T>(P, j, s_rtb, &s_bar[0]);
     s_jobs[0] = j;
   }
@@ -202,7 +193,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
     if (sched) {
       JoinJob j;
       if (lane == 0) {
-        j = claim_job<T, FUSE>(P, total_items);
+        j = claim_job<T>(P, total_items);
         if (L2PF && RBUF == 1 && j.item < total_items) prefetch_item_l2<T>(P, j, NT * SPT);
         if (RBUF == 2 && j.item < total_items) issue_r_copy<T>(P, j, s_rtb + ((it + 1) & 1) * cap, &s_bar[(it + 1) & 1]);
         s_jobs[(it + 1) & 1] = j;
@@ -220,7 +211,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
       #pragma unroll
       for (int j = 0; j < SPT; ++j) {
         if ((uint32_t)(j * NT) + threadIdx.x < rem) {
-          const T t = FUSE ? __ldcg(src + j * NT) : __ldcs(src + j * NT);
+          const T t = __ldcs(src + j * NT);
           sk[j] = TT::key(t);
           sp[j] = TT::pay(t);
         }
@@ -232,7 +223,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
       const T* src = ssrc + base + threadIdx.x;
       #pragma unroll
       for (int j = 0; j < SPT; ++j)
-        if ((uint32_t)(j * NT) + threadIdx.x < rem) nx[j] = FUSE ? __ldcg(src + j * NT) : __ldcs(src + j * NT);
+        if ((uint32_t)(j * NT) + threadIdx.x < rem) nx[j] = __ldcs(src + j * NT);
     };
     load_s(job.sb);
     for (uint32_t i = threadIdx.x; i < nb; i += NT) s_head[i] = NIL16;
@@ -294,9 +285,8 @@ __device__ __forceinline__ void join_body(const Plan& P) {
         const uint32_t i0 = v ? idx[j] : 0u;
         const T r = lds_tuple(s_rt_sh + i0 * (uint32_t)sizeof(T), (T*)nullptr);
         const bool hit = v && TT::key(r) == sk[j];
-        if (MAT) {
-          rfirst[j] = TT::pay(r);
-        } else {
+        if (MAT) rfirst[j] = TT::pay(r);
+        if (!MAT || chk) {
           const uint64_t sg = pair_sig((uint64_t)TT::pay(r), (uint64_t)sp[j]);
           my_chk += hit ? sg : 0ull;
         }
@@ -312,11 +302,8 @@ __device__ __forceinline__ void join_body(const Plan& P) {
           if (idx[j] != NIL16) {
             const T r = lds_tuple(s_rt_sh + idx[j] * (uint32_t)sizeof(T), (T*)nullptr);
             if (TT::key(r) == sk[j]) {
-              if (MAT) {
-                if (m[j] == 0) rfirst[j] = TT::pay(r);
-              } else {
-                my_chk += pair_sig((uint64_t)TT::pay(r), (uint64_t)sp[j]);
-              }
+              if (MAT && m[j] == 0) rfirst[j] = TT::pay(r);
+              if (!MAT || chk) my_chk += pair_sig((uint64_t)TT::pay(r), (uint64_t)sp[j]);
               ++m[j];
             }
             idx[j] = s_next[idx[j]];
@@ -366,13 +353,8 @@ __device__ __forceinline__ void join_body(const Plan& P) {
           pos0 += wtot;
           if (m[j] == 1) {
             if (pos < P.out_cap) {
-              if (FUSE) {
-                __stcs(out_r + pos, rfirst[j]);
-                __stcs(out_s + pos, sp[j]);
-              } else {
-                out_r[pos] = rfirst[j];
-                out_s[pos] = sp[j];
-              }
+              out_r[pos] = rfirst[j];
+              out_s[pos] = sp[j];
             }
           } else if (m[j] > 1) {
             for (uint32_t i = s_head[slot_of(sk[j], H)]; i != NIL16; i = s_next[i]) {
@@ -390,9 +372,6 @@ __device__ __forceinline__ void join_body(const Plan& P) {
         bar_compute(NT);  // s_base / s_wsum are reused by the next round
       }
     }
-    // FUSE: this warp is done with the item (counted per warp, before the end-of-item barrier:
-    // the scheduler may be waiting on pass 2 for the next item, and pass 2 on this count)
-    if (FUSE && lane == 0) red_add_gpu(&P.fz[FZ_JCOMP], 1u);
     bar_item(NT + 32);  // end of item: the tile buffer and s_head are reused, s_jobs[it+1] is ready
   }
 
@@ -423,7 +402,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
 template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false, bool PF = false,
           bool L2PF = false, int SPF = 0>
 __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
-  join_body<K, NT, SPT, MAT, RBUF, H16, false, PF, L2PF, SPF>(P);
+  join_body<K, NT, SPT, MAT, RBUF, H16, PF, L2PF, SPF>(P);
 }
 
 }  // namespace hj

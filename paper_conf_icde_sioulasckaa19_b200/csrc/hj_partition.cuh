@@ -27,9 +27,12 @@ namespace hj {
 // ------------------------------------------------------------------------------------------
 // Shared-memory counters, one 32-bit atomicAdd per key:
 //   C32 = true : 2^qbits u32 counters (qbits <= 15, <= 128 KB)
-//   C32 = false: 2^qbits u16 counters packed in pairs (qbits == 16, 128 KB). A wrap of a 16-bit
-//                half (old value 0xFFFF) is detected from the atomic's return value: the carry
-//                into the upper half is undone and 65536 is added to the global counter.
+//   C32 = false: 2^qbits u16 counters packed in pairs (qbits == 16, 128 KB). The increment that
+//                takes a half from 0x7FFF to 0x8000 (seen in the atomic's return value) moves
+//                0x8000 to the global counter and subtracts it from the half. The subtract is
+//                issued as soon as that return arrives, long before another 0x8000 increments of
+//                the same address can execute, so a half never passes 0xFFFF: no carry ever
+//                reaches the neighbouring bin, and the flush adds each remainder.
 template <bool C32>
 __device__ __forceinline__ void hist_add(uint32_t* h, uint32_t bin, uint32_t* gcnt) {
   if (C32) {
@@ -37,9 +40,9 @@ __device__ __forceinline__ void hist_add(uint32_t* h, uint32_t bin, uint32_t* gc
   } else {
     const uint32_t sh = (bin & 1) << 4;
     const uint32_t old = atomicAdd(&h[bin >> 1], 1u << sh);
-    if (((old >> sh) & 0xffffu) == 0xffffu) {
-      if (sh == 0) atomicSub(&h[bin >> 1], 1u << 16);
-      atomicAdd(&gcnt[bin], 65536u);
+    if (((old >> sh) & 0xffffu) == 0x7fffu) {
+      atomicSub(&h[bin >> 1], 0x8000u << sh);
+      atomicAdd(&gcnt[bin], 0x8000u);
     }
   }
 }
@@ -47,16 +50,11 @@ __device__ __forceinline__ void hist_add(uint32_t* h, uint32_t bin, uint32_t* gc
 template <typename K, bool SMEM, bool GD, bool C32 = true>
 __global__ void __launch_bounds__(1024) k_hist(Plan P, uint32_t blocks_r) {
   extern __shared__ uint32_t s_hist[];
-  __shared__ uint32_t s_blk[2][1024];  // BLK mode: this block's pass-1 digit counts per relation
   const uint32_t np = 1u << P.qbits();
   const uint32_t nwords = C32 ? np : np / 2;
-  const bool blk = P.g1 != 0;
   if (SMEM) {
     for (uint32_t i = threadIdx.x; i < nwords; i += blockDim.x) s_hist[i] = 0;
   }
-  const uint32_t F1 = 1u << P.pb();
-  if (blk)
-    for (uint32_t i = threadIdx.x; i < 2 * 1024; i += blockDim.x) (&s_blk[0][0])[i] = 0;
   __syncthreads();
   constexpr int VEC = 16 / sizeof(K);
   int rel = 0;
@@ -65,23 +63,13 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P, uint32_t blocks_r) {
     if (SMEM) hist_add<C32>(s_hist, b, P.rel[rel].cnt);
     else atomicAdd(&P.rel[rel].cnt[b], 1u);
   };
-  // merge the shared q-histogram of relation r into the global one and clear it
+  // merge the shared q-histogram of relation r into the global one
   auto flush_q = [&](int r) {
     __syncthreads();
-    if (blk)  // this block's pass-1 digit counts: D = q >> b2 sums 2^b2 consecutive bins
-      for (uint32_t d = threadIdx.x; d < F1; d += blockDim.x) {
-        uint32_t t = 0;
-        for (uint32_t j = d << P.b2; j < (d + 1) << P.b2; ++j)
-          t += C32 ? s_hist[j] : ((s_hist[j >> 1] >> ((j & 1) << 4)) & 0xffffu);
-        s_blk[r][d] = t;
-      }
     for (uint32_t i = threadIdx.x; i < np; i += blockDim.x) {
       const uint32_t c = C32 ? s_hist[i] : ((s_hist[i >> 1] >> ((i & 1) << 4)) & 0xffffu);
       if (c) atomicAdd(&P.rel[r].cnt[i], c);
     }
-    __syncthreads();
-    for (uint32_t i = threadIdx.x; i < nwords; i += blockDim.x) s_hist[i] = 0;
-    __syncthreads();
   };
   auto count_range = [&](const K* keys, unsigned long long lo, unsigned long long hi) {
     if (lo >= hi) return;
@@ -113,35 +101,16 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P, uint32_t blocks_r) {
     }
     for (unsigned long long j = i + threadIdx.x; j < hi; j += blockDim.x) add(keys[j]);
   };
-  if (!blk) {
-    // blocks [0, blocks_r) count R, the rest count S (split proportionally to |R| : |S|)
-    rel = blockIdx.x < blocks_r ? 0 : 1;
-    const unsigned long long n = P.rel[rel].n;
-    const uint32_t nblk = rel ? gridDim.x - blocks_r : blocks_r;
-    const uint32_t bid = rel ? blockIdx.x - blocks_r : blockIdx.x;
-    unsigned long long per = (n + nblk - 1) / nblk;
-    per = (per + VEC - 1) / VEC * VEC;
-    const unsigned long long lo = (unsigned long long)bid * per;
-    count_range((const K*)P.rel[rel].keys, lo, lo + per < n ? lo + per : n);
-  } else {
-    // exactly the tiles pass 1 block blockIdx.x will process: u = blockIdx.x + k * g1
-    const unsigned long long units0 = P.tiles1[0], units = units0 + P.tiles1[1];
-    for (unsigned long long u = blockIdx.x; u < units; u += gridDim.x) {
-      const int r = u < units0 ? 0 : 1;
-      if (SMEM && r != rel) flush_q(rel);  // R's tiles come first; flush R before counting S
-      rel = r;
-      const unsigned long long s0 = (rel ? u - units0 : u) * P.tile1;
-      const unsigned long long n = P.rel[rel].n;
-      count_range((const K*)P.rel[rel].keys, s0, s0 + P.tile1 < n ? s0 + P.tile1 : n);
-    }
-  }
+  // blocks [0, blocks_r) count R, the rest count S (split proportionally to |R| : |S|)
+  rel = blockIdx.x < blocks_r ? 0 : 1;
+  const unsigned long long n = P.rel[rel].n;
+  const uint32_t nblk = rel ? gridDim.x - blocks_r : blocks_r;
+  const uint32_t bid = rel ? blockIdx.x - blocks_r : blockIdx.x;
+  unsigned long long per = (n + nblk - 1) / nblk;
+  per = (per + VEC - 1) / VEC * VEC;
+  const unsigned long long lo = (unsigned long long)bid * per;
+  count_range((const K*)P.rel[rel].keys, lo, lo + per < n ? lo + per : n);
   if (SMEM) flush_q(rel);
-  if (blk) {
-    __syncthreads();
-    for (int r = 0; r < 2; ++r)
-      for (uint32_t d = threadIdx.x; d < F1; d += blockDim.x)
-        P.cntb[((size_t)r * gridDim.x + blockIdx.x) * F1 + d] = s_blk[r][d];
-  }
 }
 
 // ------------------------------------------------------------------------------------------
@@ -173,9 +142,8 @@ __device__ __forceinline__ unsigned long long plan_count(const RelDev& R, int ns
   return c;
 }
 
-// MS: several sources (exchange receiver); BS: per-block bases (HJ_OPT_PASS1_BASES); IT: join items
-// (not on the exchange sender). Specialised so each launch runs (and fetches) only its own code.
-template <bool MS, bool BS, bool IT>
+// MS: several sources (exchange receiver); IT: join items (not on the exchange sender). Specialised so each launch runs (and fetches) only its own code.
+template <bool MS, bool IT>
 __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   constexpr int NT = 1024;
   __shared__ unsigned long long s_tmp6[6 * (NT / 32 + 1)];
@@ -227,7 +195,12 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   if (b == gridDim.x - 1 && threadIdx.x == 0) {
     P.rel[0].off[np] = bR + tR;
     P.rel[1].off[np] = bS + tS;
-    if (items) P.ist[np] = (uint32_t)(bI + tI);
+    bool bad = false;
+    if (P.mode == PLAN_RECV) {  // received count rows must not describe more tuples than the buffers hold
+      bad = bR + tR > P.rel[0].n || bS + tS > P.rel[1].n;
+      if (bad) P.counters[CNT_BAD_COUNTS] = 1u;  // pass 2 and the join then do nothing
+    }
+    if (items) P.ist[np] = bad ? 0u : (uint32_t)(bI + tI);
   }
   // ---- several sources: piece sizes, a warp per piece (stored in pst[i + 1]) --------------
   const uint32_t npieces = P.npieces();
@@ -244,27 +217,6 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
         #pragma unroll
         for (int o = 16; o; o >>= 1) c += __shfl_xor_sync(0xffffffffu, c, o);
         if (lane == 0) R.pst[i + 1] = c;
-      }
-    }
-  }
-  // ---- pass-1 bases: exclusive prefix over pass-1 blocks of each (relation, digit) column ----
-  if (BS && P.g1) {
-    const uint32_t F1 = 1u << pb, g1 = P.g1;
-    const uint32_t lane = threadIdx.x & 31, gw = b * (NT / 32) + (threadIdx.x >> 5), nw = gridDim.x * (NT / 32);
-    for (uint32_t col = gw; col < 2 * F1; col += nw) {
-      const size_t r0 = (size_t)(col / F1) * g1, D = col % F1;
-      unsigned long long run = 0;
-      for (uint32_t b0 = 0; b0 < g1; b0 += 32) {
-        const bool ok = b0 + lane < g1;
-        const unsigned long long v = ok ? P.cntb[(r0 + b0 + lane) * F1 + D] : 0ull;
-        unsigned long long x = v;
-        #pragma unroll
-        for (int o = 1; o < 32; o <<= 1) {
-          const unsigned long long y = __shfl_up_sync(0xffffffffu, x, o);
-          if (lane >= o) x += y;
-        }
-        if (ok) P.relb[(r0 + b0 + lane) * F1 + D] = run + x - v;
-        run += __shfl_sync(0xffffffffu, x, 31);
       }
     }
   }
@@ -335,13 +287,12 @@ struct __align__(16) PassUnit {
   uint32_t valid;
   uint32_t rel;    // bucket chains (BC): relation and first partition index of the unit's digits
   uint32_t pbase;
-  uint32_t grp;    // fused pass 2 (FUSE): the pass-1 partition (piece) of the unit
 };
 
 // Unit u (round-robin: u = blockIdx.x + k * gridDim.x) -> its descriptor. MODE 2 maps the chunk
 // to its piece by binary search in the shared-memory chunk prefix (stateless: no registers live
 // across the unit loop).
-template <typename K, int MODE, int TILE, bool BC = false, bool FUSE = false>
+template <typename K, int MODE, int TILE, bool BC = false>
 struct UnitWalker {
   unsigned long long units0, units;
   __device__ __forceinline__ bool get(const Plan& P, unsigned long long u, PassUnit<K>& U, const uint32_t* s_cst,
@@ -352,32 +303,6 @@ struct UnitWalker {
     // no registers live across k_pass's tile loop
     const unsigned long long n0 = (BC && MODE == 2) ? s_cst[2 * BC_MAX_NB1 - 3] : units0;
     const unsigned long long nn = (BC && MODE == 2) ? s_cst[2 * BC_MAX_NB1 - 4] : units;
-    if (FUSE) {  // pass-1 partition major: R chunks of piece i, then S chunks of piece i, then i + 1
-      const uint32_t npc = P.npieces();
-      const uint32_t* cR = s_cst;
-      const uint32_t* cS = s_cst + 1025;
-      U.valid = u < (unsigned long long)(cR[npc] + cS[npc]);
-      if (!U.valid) return false;
-      const uint32_t uc = (uint32_t)u;
-      uint32_t lo = 0, hi = npc;  // largest piece with cR + cS <= uc
-      while (hi - lo > 1) {
-        const uint32_t mid = (lo + hi) >> 1;
-        if (cR[mid] + cS[mid] <= uc) lo = mid; else hi = mid;
-      }
-      const uint32_t k = uc - (cR[lo] + cS[lo]), nr = cR[lo + 1] - cR[lo];
-      const int r = k < nr ? 0 : 1;
-      const RelDev& R = P.rel[r];
-      const unsigned long long s0 = s_pst[r * 1025 + lo] + (unsigned long long)(r ? k - nr : k) * TILE;
-      U.rel = r;
-      U.pbase = 0;
-      U.grp = lo;
-      U.src_k = (const T*)R.t1 + s0;
-      U.src_p = nullptr;
-      U.dst = R.t2;
-      U.cur = R.cur2 + ((unsigned long long)lo << P.b2);
-      U.len = (uint32_t)min((unsigned long long)TILE, s_pst[r * 1025 + lo + 1] - s0);
-      return true;
-    }
     U.valid = u < nn;
     if (!U.valid) return false;
     const int r = (u < n0) ? 0 : 1;
@@ -385,7 +310,6 @@ struct UnitWalker {
     const RelDev& R = P.rel[r];
     U.rel = r;
     U.pbase = 0;
-    U.grp = 0;
     if (BC) {  // bucket chains: pass 1 as below into the pass-1 pool; pass 2 = one bucket unit
       const BcRel& Bc = P.bc_rel[r];
       if (MODE == 1) {
@@ -544,18 +468,11 @@ __device__ __noinline__ void bc_pass2_units(const BcRel* s_bc, const uint32_t* c
   }
 }
 
-// FUSE (pass 2 inside the fused pass-2 + join kernel, hj_fused.cuh): units are claimed from a
-// global counter in pass-1-partition order (R then S chunks of each piece); each warp signals
-// the completion of its part of a unit's write-out (fence.acq_rel.gpu + red on the piece's
-// counter, issued one iteration later, when the stores have long been acknowledged); T2 stores
-// are plain write-back stores so the co-partitions stay in L2 for the join; a unit more than
-// fz_window pieces ahead of the join's completed items waits (bounds the L2 footprint).
 // RPF: the next unit's tuples are prefetched into registers during the current unit (default);
 // RPF = false loads each unit at the top of its iteration (half the data registers: twice the
 // tuples per thread at the same register budget, for two blocks per SM whose barriers overlap).
-template <typename K, int MODE, int NT, int ITEMS, bool GD, bool BC = false, bool FUSE = false, bool RPF = true>
+template <typename K, int MODE, int NT, int ITEMS, bool GD, bool BC = false, bool RPF = true>
 __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
-  static_assert(!FUSE || (MODE == 2 && !BC && !GD), "fused pass 2 only");
   using TT = Tup<K>;
   using T = typename TT::T;
   constexpr int TILE = NT * ITEMS;
@@ -587,10 +504,12 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
   };
   const uint32_t nscan = F < 32 ? 32u : F;  // threads in the digit scan (whole warps)
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  // the exchange receiver's planner rejected the received count rows: nothing to do (block-uniform)
+  if (MODE == 2 && !BC && P.mode == PLAN_RECV && *(volatile const uint32_t*)&P.counters[CNT_BAD_COUNTS]) return;
 
   if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
   if (threadIdx.x == 0) s_hot = s_hot_next = 0xffffffffu;
-  UnitWalker<K, MODE, TILE, BC, FUSE> W;
+  UnitWalker<K, MODE, TILE, BC> W;
   if (MODE == 1) {
     W.units0 = P.tiles1[0];
     W.units = W.units0 + P.tiles1[1];
@@ -624,27 +543,12 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
   }
   const unsigned long long G = gridDim.x;
   if (threadIdx.x == NT - 1) {
-    if (FUSE) {
-      W.get(P, atomicAdd(&P.fz[FZ_UNIT], 1u), s_desc[0], s_cst, s_pst, s_bfill, s_bd);
-      W.get(P, atomicAdd(&P.fz[FZ_UNIT], 1u), s_desc[1], s_cst, s_pst, s_bfill, s_bd);
-    } else {
-      W.get(P, blockIdx.x, s_desc[0], s_cst, s_pst, s_bfill, s_bd);
-      W.get(P, blockIdx.x + G, s_desc[1], s_cst, s_pst, s_bfill, s_bd);
-    }
+    W.get(P, blockIdx.x, s_desc[0], s_cst, s_pst, s_bfill, s_bd);
+    W.get(P, blockIdx.x + G, s_desc[1], s_cst, s_pst, s_bfill, s_bd);
   }
   __syncthreads();
   T* prev_dst = nullptr;  // unit i-1 awaiting write-out
   uint32_t prev_len = 0;
-  uint32_t prev_grp = 0, sig_grp = 0;  // FUSE: piece of unit i-1; piece of the unit written out last iteration
-  bool sig = false;
-  // FUSE: this warp's part of the write-out issued last iteration is complete -> signal its piece
-  auto signal = [&](uint32_t grp) {
-    __syncwarp();
-    if (lane == 0) {
-      fence_acq_rel_gpu();
-      red_add_gpu(&P.fz[FZ_DONE + grp], 1u);
-    }
-  };
   K kk[ITEMS], pp[ITEMS], kn[RPF ? ITEMS : 1], pn[RPF ? ITEMS : 1];
   unsigned long long u = blockIdx.x;
   if constexpr (RPF) {
@@ -658,8 +562,7 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
       for (int j = 0; j < ITEMS; ++j) {
         const uint32_t i = j * NT + threadIdx.x;
         const T t = s_buf[i];
-        if (FUSE) prev_dst[gd[digit(TT::key(t))] + i] = t;
-        else __stcs(prev_dst + (gd[digit(TT::key(t))] + i), t);
+        __stcs(prev_dst + (gd[digit(TT::key(t))] + i), t);
       }
     } else {
       #pragma unroll
@@ -667,8 +570,7 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
         const uint32_t i = j * NT + threadIdx.x;
         if (i < prev_len) {
           const T t = s_buf[i];
-          if (FUSE) prev_dst[gd[digit(TT::key(t))] + i] = t;
-          else __stcs(prev_dst + (gd[digit(TT::key(t))] + i), t);
+          __stcs(prev_dst + (gd[digit(TT::key(t))] + i), t);
         }
       }
     }
@@ -685,7 +587,6 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
     } else {
       pass_load<K, MODE, NT, ITEMS>(s_desc[slot], kk, pp);
     }
-    if (FUSE && sig) signal(sig_grp);  // before the prefetch: the fence then waits only for old stores
     // prefetch the next unit (in flight across this unit's barriers)
     if constexpr (RPF) {
       if (s_desc[nslot].valid) pass_load<K, MODE, NT, ITEMS>(s_desc[nslot], kn, pn);
@@ -765,22 +666,7 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
     }
     if (threadIdx.x == NT - 1) {  // publish unit i+2
       PassUnit<K>& Dn = s_desc[nslot == 2 ? 0 : nslot + 1];
-      if (FUSE) {
-        W.get(P, atomicAdd(&P.fz[FZ_UNIT], 1u), Dn, s_cst, s_pst, s_bfill, s_bd);
-        if (Dn.valid && P.fz_window) {
-          // throttle: wait until the join completed the items of the pieces more than fz_window
-          // below unit i+2's -- never of a piece this block still has to signal (no deadlock)
-          const uint32_t low = prev_dst ? prev_grp : s_desc[slot].grp;
-          int tg = (int)Dn.grp - (int)P.fz_window;
-          if (tg > (int)low) tg = (int)low;
-          if (tg > 0) {
-            const uint32_t need = P.ist[(uint32_t)tg << P.b2] * FZ_JOIN_WARPS;  // warp counts
-            wait_geq(&P.fz[FZ_JCOMP], need, &P.fz[FZ_ERR], 2u);
-          }
-        }
-      } else {
-        W.get(P, u + 2 * G, Dn, s_cst, s_pst, s_bfill, s_bd);
-      }
+      W.get(P, u + 2 * G, Dn, s_cst, s_pst, s_bfill, s_bd);
       if (P.pass_l2pf && Dn.valid && Dn.len) {  // unit i+2's input -> L2 (its register loads come next iteration)
         const uint32_t bytes = MODE == 1 ? Dn.len * (uint32_t)sizeof(K) : Dn.len * (uint32_t)sizeof(T);
         const uintptr_t a = reinterpret_cast<uintptr_t>(Dn.src_k);
@@ -804,244 +690,19 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
         s_buf[s_loc[digit(kk[j])] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = TT::make(kk[j], pp[j]);
     // (no barrier: the next unit's phase 1 touches only s_cnt; its phase 2 reads s_buf / s_gd
     //  after the next phase-1 barrier)
-    sig = prev_dst != nullptr;  // unit i-1 was written out in this iteration's phase 2
-    sig_grp = prev_grp;
     prev_dst = (T*)s_desc[slot].dst;
     prev_len = ulen;
-    prev_grp = s_desc[slot].grp;
     u += G;
     slot = nslot;
     ++it;
   }
   __syncthreads();
   write_out(s_gd + ((it + 1) & 1) * F);  // the last unit (it was incremented past it)
-  if (FUSE) {
-    if (sig) signal(sig_grp);
-    if (prev_dst) signal(prev_grp);
-  }
 }
 
 template <typename K, int MODE, int NT, int ITEMS, bool GD, bool BC = false, bool RPF = true>
 __global__ void __launch_bounds__(NT, 1024 / NT) k_pass(Plan P, int fanout_bits) {
-  pass_body<K, MODE, NT, ITEMS, GD, BC, false, RPF>(P, fanout_bits);
-}
-
-// ------------------------------------------------------------------------------------------
-// a3 with precomputed per-block bases (default pass 1 when 2^qbits <= 2^15): block b's run of
-// digit d in its k-th tile starts at pst[d] + relb[b][d] + (its earlier tiles' counts of d) --
-// no atomics, and every run's global start is known BEFORE the shuffle. Each run is placed in
-// shared memory at the same 16-byte phase as its destination (one spare slot per digit), so the
-// write-out is one TMA bulk store (cp.async.bulk shared -> global) per run plus at most one
-// scalar tuple at each end, issued by one thread per digit and completed asynchronously.
-// Per tile: rank | scan + wait for the previous tile's bulk reads | shuffle + proxy fence |
-// issue bulk stores (overlapping the next tile's rank).
-// ------------------------------------------------------------------------------------------
-__device__ __forceinline__ void bulk_s2g(void* dst, const void* src, uint32_t bytes) {
-  asm volatile("cp.async.bulk.global.shared::cta.bulk_group [%0], [%1], %2;" ::"l"(dst), "r"(smem_u32(src)), "r"(bytes)
-               : "memory");
-}
-__device__ __forceinline__ void bulk_commit() { asm volatile("cp.async.bulk.commit_group;" ::: "memory"); }
-__device__ __forceinline__ void bulk_wait_read() { asm volatile("cp.async.bulk.wait_group.read 0;" ::: "memory"); }
-__device__ __forceinline__ void bulk_wait_all() { asm volatile("cp.async.bulk.wait_group 0;" ::: "memory"); }
-
-template <typename K, int NT, int ITEMS, bool GD>
-__global__ void __launch_bounds__(NT, 1024 / NT) k_pass1b(Plan P, int fanout_bits) {
-  using TT = Tup<K>;
-  using T = typename TT::T;
-  constexpr int TILE = NT * ITEMS;
-  constexpr int TPS = 16 / sizeof(T);  // tuples per 16-byte segment (2 for 8 B tuples, 1 for 16 B)
-  static_assert(NT == 512 || NT == 1024, "block size");
-  static_assert(TILE <= 65536 && ITEMS % 2 == 0, "16-bit packed ranks");
-  extern __shared__ __align__(16) unsigned char s_raw[];
-  const uint32_t F = 1u << fanout_bits;
-  T* s_buf = reinterpret_cast<T*>(s_raw);                                                  // TILE + 2F tuples
-  unsigned long long* s_cur = reinterpret_cast<unsigned long long*>(s_buf + TILE + 2 * F);  // F: next global slot
-  unsigned long long* s_gst = s_cur + F;                                                   // F: run start (global)
-  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gst + F);                                // F + 1 (spare)
-  uint32_t* s_loc = s_cnt + F + 4;                                                         // F: run start (smem)
-  uint32_t* s_len = s_loc + F;                                                             // F: run length
-  __shared__ uint32_t s_wt[NT / 32];
-  __shared__ uint32_t s_hot, s_hot_next;
-
-  const uint32_t dmask = (1u << P.b1) - 1;
-  const uint32_t gsh = (uint32_t)P.B, gmask = (1u << P.g) - 1, gup = (uint32_t)P.b1;
-  auto digit = [=](K key) -> uint32_t {
-    uint32_t d = (uint32_t)key & dmask;
-    if (GD) d |= ((uint32_t)(key >> gsh) & gmask) << gup;
-    return d;
-  };
-  const uint32_t nscan = F < 32 ? 32u : F;
-  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-  const unsigned long long G = gridDim.x;
-  const unsigned long long units0 = P.tiles1[0], units = units0 + P.tiles1[1];
-
-  if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
-  if (threadIdx.x == 0) s_hot = s_hot_next = 0xffffffffu;
-  int cur_rel = -1;
-  auto load_bases = [&](int r) {  // cursors of this block for relation r
-    if (threadIdx.x < F)
-      s_cur[threadIdx.x] = P.rel[r].pst[threadIdx.x] + P.relb[((size_t)r * G + blockIdx.x) * F + threadIdx.x];
-  };
-  auto unit = [&](unsigned long long u, const K*& kp, const K*& pp_, uint32_t& len, int& r) {
-    r = u < units0 ? 0 : 1;
-    const unsigned long long s0 = (r ? u - units0 : u) * TILE;
-    kp = (const K*)P.rel[r].keys + s0;
-    pp_ = (const K*)P.rel[r].pays + s0;
-    len = (uint32_t)min((unsigned long long)TILE, P.rel[r].n - s0);
-  };
-  K kk[ITEMS], pp[ITEMS], kn[ITEMS], pn[ITEMS];
-  auto load = [&](const K* keys, const K* pays, uint32_t len) {
-    constexpr int VEC = 16 / sizeof(K);
-    const bool vec_ok = (len == TILE) && ((reinterpret_cast<uintptr_t>(keys) & 15) == 0) &&
-                        ((reinterpret_cast<uintptr_t>(pays) & 15) == 0);
-    if (vec_ok) {
-      #pragma unroll
-      for (int j = 0; j < ITEMS / VEC; ++j) {
-        const uint4 kv = __ldcs(reinterpret_cast<const uint4*>(keys) + j * NT + threadIdx.x);
-        const uint4 pv = __ldcs(reinterpret_cast<const uint4*>(pays) + j * NT + threadIdx.x);
-        const K* ke = reinterpret_cast<const K*>(&kv);
-        const K* pe = reinterpret_cast<const K*>(&pv);
-        #pragma unroll
-        for (int t = 0; t < VEC; ++t) {
-          kn[j * VEC + t] = ke[t];
-          pn[j * VEC + t] = pe[t];
-        }
-      }
-    } else {
-      #pragma unroll
-      for (int j = 0; j < ITEMS; ++j) {
-        const uint32_t e = pass_elem<K, 1, NT>(j);
-        if (e < len) {
-          kn[j] = keys[e];
-          pn[j] = pays[e];
-        }
-      }
-    }
-  };
-
-  unsigned long long u = blockIdx.x;
-  const K *ck, *cp;
-  uint32_t clen = 0;
-  int crel = 0;
-  if (u < units) {
-    unit(u, ck, cp, clen, crel);
-    load(ck, cp, clen);
-  }
-  __syncthreads();
-  bool pending = false;  // this thread issued bulk stores not yet known to be read
-  T* dst = nullptr;
-  while (u < units) {
-    const uint32_t ulen = clen;
-    const int urel = crel;
-    #pragma unroll
-    for (int j = 0; j < ITEMS; ++j) {
-      kk[j] = kn[j];
-      pp[j] = pn[j];
-    }
-    const unsigned long long un = u + G;
-    if (un < units) {
-      unit(un, ck, cp, clen, crel);
-      load(ck, cp, clen);
-    }
-    if (urel != cur_rel) {  // block-uniform; the previous relation's stores were waited for below
-      load_bases(urel);
-      cur_rel = urel;
-      dst = (T*)P.rel[urel].t1;
-    }
-    // ---- phase 1: rank (hot-digit aggregation as in k_pass) ---------------------------------
-    uint32_t rk[ITEMS / 2];
-    const bool full = ulen == TILE;
-    const uint32_t hot = s_hot;
-    #pragma unroll
-    for (int j = 0; j < ITEMS; ++j) {
-      const uint32_t d = (full || pass_elem<K, 1, NT>(j) < ulen) ? digit(kk[j]) : F;
-      uint32_t r;
-      if (hot > F) {
-        r = atomicAdd(&s_cnt[d], 1u);
-      } else {
-        const uint32_t hm = __ballot_sync(0xffffffffu, d == hot);
-        if (hm) {
-          const int leader = __ffs(hm) - 1;
-          uint32_t base = 0;
-          if (lane == leader) base = atomicAdd(&s_cnt[hot], (uint32_t)__popc(hm));
-          base = __shfl_sync(0xffffffffu, base, leader);
-          r = (d == hot) ? base + __popc(hm & lanemask_lt()) : atomicAdd(&s_cnt[d], 1u);
-        } else {
-          r = atomicAdd(&s_cnt[d], 1u);
-        }
-      }
-      if (j & 1) rk[j / 2] |= r << 16; else rk[j / 2] = r & 0xffffu;
-    }
-    __syncthreads();
-    // ---- phase 2: scan -> smem run starts aligned to the destination's 16 B phase ------------
-    if (threadIdx.x < nscan) {
-      const uint32_t d = threadIdx.x;
-      const uint32_t c = d < F ? s_cnt[d] : 0u;
-      uint32_t x = c;
-      #pragma unroll
-      for (int o = 1; o < 32; o <<= 1) {
-        const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
-        if (lane >= o) x += y;
-      }
-      if (lane == 31) s_wt[warp] = x;
-      asm volatile("barrier.sync 1, %0;" ::"r"(nscan) : "memory");
-      uint32_t base = 0;
-      for (int w = 0; w < warp; ++w) base += s_wt[w];
-      if (pending) {  // the previous tile's bulk stores must have read s_buf before the shuffle
-        bulk_wait_read();
-        pending = false;
-      }
-      if (d < F) {
-        const uint32_t loc = base + x - c;
-        const unsigned long long g0 = s_cur[d];
-        // digit d owns smem slots [loc + TPS*d, loc + TPS*d + c + TPS - 1]: shift by 0..TPS-1 to
-        // match the destination's phase within a 16-byte segment
-        const uint32_t s0 = loc + (uint32_t)TPS * d;
-        const uint32_t sh = (uint32_t)((g0 + TPS - (s0 % TPS)) % TPS);
-        s_loc[d] = s0 + sh;
-        s_gst[d] = g0;
-        s_len[d] = c;
-        s_cur[d] = g0 + c;
-        s_cnt[d] = 0;
-        if (c > TILE / 4) atomicExch(&s_hot_next, d);
-      }
-    }
-    __syncthreads();
-    // ---- phase 3: shuffle into the aligned run slots; make the writes visible to the TMA -----
-    if (threadIdx.x == 0) {
-      s_hot = s_hot_next;
-      s_hot_next = 0xffffffffu;
-    }
-    #pragma unroll
-    for (int j = 0; j < ITEMS; ++j)
-      if (full || pass_elem<K, 1, NT>(j) < ulen)
-        s_buf[s_loc[digit(kk[j])] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = TT::make(kk[j], pp[j]);
-    fence_proxy_async();
-    __syncthreads();
-    // ---- phase 4: one bulk store per run (+ ragged ends), completed asynchronously -------------
-    if (threadIdx.x < F) {
-      const uint32_t d = threadIdx.x, c = s_len[d];
-      if (c) {
-        const uint32_t sl = s_loc[d];
-        const unsigned long long g0 = s_gst[d];
-        const uint32_t head = (uint32_t)min((unsigned long long)c, (TPS - g0 % TPS) % TPS);
-        for (uint32_t t = 0; t < head; ++t) dst[g0 + t] = s_buf[sl + t];
-        const uint32_t body = (c - head) / TPS * TPS;
-        if (body) {
-          bulk_s2g(dst + g0 + head, s_buf + sl + head, body * (uint32_t)sizeof(T));
-          bulk_commit();
-          pending = true;
-        }
-        for (uint32_t t = head + body; t < c; ++t) dst[g0 + t] = s_buf[sl + t];
-      }
-    }
-    u = un;
-    if (u < units && (u < units0 ? 0 : 1) != cur_rel && pending) {  // before the cursors switch
-      bulk_wait_read();
-      pending = false;
-    }
-  }
-  bulk_wait_all();  // the bulk stores' global writes complete before the kernel (and pass 2) ends
+  pass_body<K, MODE, NT, ITEMS, GD, BC, RPF>(P, fanout_bits);
 }
 
 }  // namespace hj

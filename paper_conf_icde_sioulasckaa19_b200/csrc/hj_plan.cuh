@@ -72,26 +72,18 @@ struct Plan {
   int mode;       // PLAN_FULL, PLAN_SEND, PLAN_RECV
   int skip_r;     // streaming S chunks: R is already partitioned (its pass-2 units are skipped)
   int pass_l2pf;  // partition passes: TMA-prefetch unit i+2's input into L2 when it is published
-  // pass 1 with precomputed per-block bases (k_pass1b): the histogram kernel runs with the same
-  // grid and tile -> block assignment as pass 1 and also counts each block's pass-1 digits
-  uint32_t g1;                  // pass-1 grid (0 = bases not used)
-  uint32_t tile1;               // pass-1 tile (tuples)
-  uint32_t* cntb;               // [2][g1][2^pb] per-block pass-1 digit counts (k_hist)
-  unsigned long long* relb;     // [2][g1][2^pb] exclusive prefix over blocks (k_plan)
   uint32_t C2;           // pass-2 chunk (tile) size in tuples
   uint32_t CR, CS;       // join item capacities: R tuples (smem build) and S tuples per item
   uint32_t* ist;         // [2^B + 1] join item prefix (q-order)
-  uint32_t* counters;    // [8]: 0 next join item, 1 planner blocks done, 2..7 bucket-chain counters
+  uint32_t* counters;    // [8]: 0 next join item, 1 planner blocks done, 2..5 bucket-chain counters,
+                         //      6 bad received counts
   unsigned long long* results;  // [4]: 0 matches, 1 checksum, 2 output cursor, 3 bucket pool overflow
   void* out_r;           // materialized payloads of R (pay width), capacity out_cap
   void* out_s;
   unsigned long long out_cap;
   unsigned long long tiles1[2];  // pass-1 tiles per relation (host-known)
   SlotHash H;            // in-partition slot hash (lg = log2 of hash-table slots per join item)
-  // fused pass 2 + join (hj_fused.cuh): zeroed counters, see FZ_* below
-  uint32_t* fz;
-  uint32_t fz_pass_slots;  // blocks per SM that start in the pass-2 role
-  uint32_t fz_window;      // pass 2 may run at most this many pass-1 partitions ahead of the join
+  int mat_chk;           // MATERIALIZE also accumulates the checksum (HJ_OPT_MAT_CHECKSUM, default 1)
   __host__ __device__ int pb() const { return g + b1; }
   __host__ __device__ int qbits() const { return g + B; }
   __host__ __device__ uint32_t npieces() const { return (uint32_t)nsrc << (g + b1); }
@@ -113,13 +105,9 @@ __device__ __forceinline__ uint32_t qbin(K key, const Plan& P) {
   return (dig1<GD>(key, P) << P.b2) | dig2(key, P);
 }
 
-enum { CNT_NEXT_ITEM = 0, CNT_PLAN_DONE = 1 };
-// fused-kernel counters (u32 offsets into Plan::fz): next pass-2 unit, join items completed,
-// watchdog error site (0 = none), per-SM role slots, per-pass-1-partition pass-2 completion
-// (warp signals)
-enum { FZ_UNIT = 0, FZ_JCOMP = 1, FZ_ERR = 2, FZ_SLOT = 8, FZ_NSLOT = 1024, FZ_DONE = FZ_SLOT + FZ_NSLOT, FZ_WORDS = FZ_DONE + 1024 };
-constexpr int FZ_PASS_WARPS = 16;  // warps of a pass-2 block in the fused kernel (signals per unit)
-constexpr int FZ_JOIN_WARPS = 15;  // compute warps of a join block in the fused kernel (counts per item)
+// counters[CNT_BAD_COUNTS]: the exchange receiver's planner found count rows that do not sum
+// to the tuples received (pass 2 and the join then do nothing; hj_join_received fails)
+enum { CNT_NEXT_ITEM = 0, CNT_PLAN_DONE = 1, CNT_BAD_COUNTS = 6 };
 enum { RES_MATCHES = 0, RES_CHECKSUM = 1, RES_CURSOR = 2 };
 
 }  // namespace hj

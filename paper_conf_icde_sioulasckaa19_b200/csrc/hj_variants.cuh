@@ -120,7 +120,7 @@ __global__ void __launch_bounds__(NT) k_join_nlj(Plan P) {
             if (MAT) warp_emit<K>(P, hit, rpj, sp);
             if (hit) {
               ++my_cnt;
-              if (!MAT) my_chk += pair_sig((uint64_t)rpj, (uint64_t)sp);
+              if (!MAT || P.mat_chk) my_chk += pair_sig((uint64_t)rpj, (uint64_t)sp);
             }
           }
         }
@@ -168,7 +168,7 @@ __global__ void __launch_bounds__(512) k_np_probe(Plan P, const K* __restrict__ 
       if (MAT) warp_emit<K>(P, hit, r, pay);
       if (hit) {
         ++my_cnt;
-        if (!MAT) my_chk += pair_sig((uint64_t)r, (uint64_t)pay);
+        if (!MAT || P.mat_chk) my_chk += pair_sig((uint64_t)r, (uint64_t)pay);
       }
       if (i != 0xffffffffu) i = next[i];
     }

@@ -330,6 +330,31 @@ def _virtual_exchange(hj, w, G, lb, out_mode):
 
 
 @pytest.mark.gpu
+def test_gpu_join_received_rejects_inconsistent_counts():
+    """hj_join_received sizes its buffers from nR / nS: count rows that describe more tuples than
+    that must fail (HJ_ERR_INVALID) without writing out of bounds, and the same
+    context must give the right result on the next, consistent call."""
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_icde_sioulasckaa19_b200 as hj
+
+    w = W.Workload("bad", 20000, 30000, "fk", keys="sparse", seed=133)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    ctx = hj.Context(0, 4, 4)
+    packed = []
+    for rel, (k, p) in enumerate(((Rk, Rp), (Sk, Sp))):
+        send, cnt, dest = ctx.exchange_pack(rel, torch.from_numpy(k.view(np.int32)).cuda(),
+                                            torch.from_numpy(p.view(np.int32)).cuda(), 0, 7)
+        packed.append((send.clone(), cnt.clone()))
+    (rs, rc), (ss, sc) = packed
+    with pytest.raises(hj.HJError, match="INVALID"):
+        ctx.join_received(rs, w.nR - 1000, rc, ss, w.nS, sc, 1, 7)
+    res = ctx.join_received(rs, w.nR, rc, ss, w.nS, sc, 1, 7)
+    assert (res.matches, res.checksum) == oracle.hash_join(Rk, Rp, Sk, Sp)
+    ctx.close()
+
+
+@pytest.mark.gpu
 @pytest.mark.parametrize("G", [1, 2, 4, 8])
 @pytest.mark.parametrize("dist_", ["fk", "zipf"])
 def test_gpu_virtual_ranks_exchange(G, dist_):
@@ -640,6 +665,26 @@ def test_gpu_exchange_c5_local_bits(G, lb):
     cols, calls = _xd_join_threads(hj, w, G, lb, 0, width=8, calls=1, cap_scale=2.0)
     m, c = oracle.hash_join(*cols)
     assert all(o[0] == 0 and o[3] == (m, c) for o in calls[0])
+
+
+@pytest.mark.gpu
+@pytest.mark.slow
+def test_gpu_xd_join_c5_bits_at_scale():
+    """c5's multi-GPU shape at scale: G = 8 virtual ranks, local_bits = 16, 8-byte 1:1 keys,
+    2^23 rows of R and of S per rank (2^26 each): every rank's all-rank result equals the closed
+    form (|S| matches, checksum = sum_j sig(rho(j), j))."""
+    if not torch.cuda.is_available():
+        pytest.skip("no CUDA device")
+    import paper_conf_icde_sioulasckaa19_b200 as hj
+
+    w = W.Workload("c5x", 1 << 26, 1 << 26, "1to1", keys="k8", seed=108)
+    cols, calls = _xd_join_threads(hj, w, 8, 16, 0, width=8, calls=2, cap_scale=1.25)
+    j = np.arange(w.nS, dtype=np.uint64)
+    rho = W.np_rho_for(w, j)
+    with np.errstate(over="ignore"):
+        exp = int(W.np_fmix64(rho ^ (j * np.uint64(0x9E3779B97F4A7C15))).sum(dtype=np.uint64))
+    for outs in calls:
+        assert all(o[0] == 0 and o[3] == (w.nS, exp) for o in outs), [o[:1] + o[3:4] for o in outs]
 
 
 @pytest.mark.gpu

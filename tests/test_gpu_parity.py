@@ -5,6 +5,7 @@ after a lexicographic sort (reading S9), partitions equal as multisets. Inputs a
 generator's (workloads/) or small adversarial arrays; expected values come only from oracle/
 or from the generator's closed forms, never from the CUDA path.
 """
+import ctypes
 import os
 
 import numpy as np
@@ -58,7 +59,7 @@ def check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=-1, mat=True, ctx=None):
     if mat:
         res = gpu_join(hj, Rk, Rp, Sk, Sp, bits, mat=True, ctx=ctx)
         assert res.matches == m, f"materialize mode bits={bits}"
-        assert res.checksum == 0  # MATERIALIZE returns the pairs, not the aggregate
+        assert res.checksum == c, f"materialize-mode checksum bits={bits}"  # HJ_OPT_MAT_CHECKSUM = 1
         if m:
             w = Rp.dtype.itemsize
             got = oracle.pairs_sorted(to_np(res.r_pay, w), to_np(res.s_pay, w))
@@ -122,7 +123,7 @@ def test_knob_invariance_block_nested_loops(hj, cap_r, chunk_s):
     ctx.close()
 
 
-JOIN_SHAPES = 46  # number of k_join shapes in hj_api.cu (HJ_OPT_JOIN_VARIANT 1..46)
+JOIN_SHAPES = 6  # number of k_join shapes in hj_api.cu (HJ_OPT_JOIN_VARIANT 1..6)
 
 
 @pytest.mark.parametrize("variant", range(1, JOIN_SHAPES + 1))
@@ -302,6 +303,8 @@ def test_partition_vs_oracle(hj, bits, width):
         e = np.sort(op[o0:o0 + c])
         assert np.array_equal(g, e), f"partition {p}"
         assert np.all((gk[a:a + c] & dt((1 << bits) - 1)) == p)
+    # key <-> payload pairing survives both passes (payloads are row ids)
+    assert np.array_equal(gk, keys[gp.astype(np.int64)])
     assert int(start.max() + count[np.argmax(start)]) <= n
 
 
@@ -331,7 +334,7 @@ def test_device_generator_matches_host(hj):
 
 
 @pytest.mark.slow
-@pytest.mark.parametrize("cfg", ["c2", "c3", "c4_z0.5", "c4_z1.0", "c4_z1.5"])
+@pytest.mark.parametrize("cfg", ["c2", "c3", "c4_z0.5", "c4_z1.0", "c4_z1.5", "c5_gpu"])
 def test_full_size_closed_form(hj, cfg):
     """Full BASELINE sizes in the bench's launch configuration: matches == |S| and the checksum
     equals sum_j sig(rho(j), j) computed on the host from the generator (closed form); for c3's
@@ -343,26 +346,47 @@ def test_full_size_closed_form(hj, cfg):
     rows = np.random.default_rng(0).integers(0, w.nS, 1 << 16).astype(np.uint64)
     rho_s = W.np_rho_for(w, rows, cdf)
     Rk_h = W.np_generate(w, s_rows=slice(0, 0))[0]  # R keys only
-    assert np.array_equal(to_np(Sk[torch.from_numpy(rows.astype(np.int64)).cuda()], 4), Rk_h[rho_s.astype(np.int64)]), \
+    kb = w.key_bytes
+    assert np.array_equal(to_np(Sk[torch.from_numpy(rows.astype(np.int64)).cuda()], kb), Rk_h[rho_s.astype(np.int64)]), \
         "device generator differs from the host generator"
-    ctx = hj.context(0, 4, 4)
+    del Rk_h
+    ctx = hj.context(0, kb, kb)
     res = ctx.join(Rk, Rp, Sk, Sp, radix_bits=w.radix_bits, out_mode=w.out_mode)
     torch.cuda.synchronize()
     del Rk, Rp, Sk, Sp
     j = np.arange(w.nS, dtype=np.uint64)
     rho = W.np_rho_for(w, j, cdf)
     assert res.matches == w.nS, f"matches {res.matches} != |S| {w.nS} (items {res.n_items})"
-    if w.out_mode == 0:
-        exp = int(np_sig(rho, j).sum(dtype=np.uint64))
-        assert res.checksum == exp, f"checksum {res.checksum:#x} != closed form {exp:#x} (items {res.n_items})"
+    exp = int(np_sig(rho, j).sum(dtype=np.uint64))  # both modes (materialize: HJ_OPT_MAT_CHECKSUM)
+    assert res.checksum == exp, f"checksum {res.checksum:#x} != closed form {exp:#x} (items {res.n_items})"
     if w.out_mode == 1:
         s_pay = res.s_pay
         order = torch.argsort(s_pay)
-        r_sorted = to_np(res.r_pay[order], 4).astype(np.uint64)
-        s_sorted = to_np(s_pay[order], 4).astype(np.uint64)
+        r_sorted = to_np(res.r_pay[order], kb).astype(np.uint64)
+        s_sorted = to_np(s_pay[order], kb).astype(np.uint64)
         assert np.array_equal(s_sorted, j), "materialized s_pay is not a permutation of S's rows"
         bad = np.nonzero(r_sorted != rho)[0]
         assert len(bad) == 0, f"{len(bad)} materialized pairs differ, first at s_pay {bad[:5]}"
+
+
+@pytest.mark.slow
+@pytest.mark.parametrize("slice_id", [0, 11])
+def test_c5_shape_sliced_oracle(hj, slice_id):
+    """c5's shape (1:1, 8-byte fmix64 keys, row-id payloads, B = 16 local bits) at 2^26 x 2^26
+    rows: the oracle's sliced mode (slice = top 4 bits of fmix64(key); the join decomposes over any
+    key partition) on one slice equals the GPU join of that slice's rows, and the GPU
+    join of all rows equals the closed form."""
+    w = W.Workload("c5s", 1 << 26, 1 << 26, "1to1", keys="k8", seed=107, out_mode=0, radix_bits=16)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    bits = 4
+    m, c = oracle.hash_join(Rk, Rp, Sk, Sp, slice_bits=bits, slice_id=slice_id)
+    inR = (W.np_fmix64(Rk) >> np.uint64(64 - bits)) == np.uint64(slice_id)
+    inS = (W.np_fmix64(Sk) >> np.uint64(64 - bits)) == np.uint64(slice_id)
+    assert m == int(inS.sum()) and m > (1 << 21)
+    res = gpu_join(hj, Rk[inR], Rp[inR], Sk[inS], Sp[inS], bits=12)
+    assert (res.matches, res.checksum) == (m, c)
+    full = gpu_join(hj, Rk, Rp, Sk, Sp, bits=w.radix_bits)
+    assert (full.matches, full.checksum) == (w.nS, _closed_form_checksum(w))
 
 
 @pytest.mark.parametrize("width", [4, 8])
@@ -375,6 +399,26 @@ def test_partition_16bit_counters_wrap(hj, width):
     keys = rng.integers(0, 1 << (8 * width - 1), n, dtype=np.uint64).astype(dt)
     keys[: 3 * n // 4] = dt(0x12345)  # 300K copies of one key
     rng.shuffle(keys)
+    pays = np.arange(n, dtype=dt)
+    _, _, offs = oracle.radix_partition(keys, pays, 0, 16)
+    t, start, count = hj.context(0, width, width).partition(dev(keys), dev(pays), 16)
+    torch.cuda.synchronize()
+    assert np.array_equal(count, np.diff(offs.astype(np.int64)).astype(np.uint64))
+
+
+@pytest.mark.parametrize("width", [4, 8])
+def test_partition_16bit_counters_two_hot_bins_one_word(hj, width):
+    """2^16 bins are packed two per 32-bit word: two hot keys whose bins share a word (bins 2k and
+    2k + 1), each far past 65535 occurrences in one histogram block, interleaved so both halves
+    wrap repeatedly while the other is being incremented (a carry between the halves
+    must never be visible to the partner bin)."""
+    rng = np.random.default_rng(18)
+    dt = np.uint32 if width == 4 else np.uint64
+    n = 1_200_000
+    keys = rng.integers(0, 1 << (8 * width - 1), n, dtype=np.uint64).astype(dt)
+    hot = rng.random(n)
+    keys[hot < 0.45] = dt(0x52344)   # bin 0x2344 (even)
+    keys[(hot >= 0.45) & (hot < 0.9)] = dt(0x72345)  # bin 0x2345 (odd): same packed word
     pays = np.arange(n, dtype=dt)
     _, _, offs = oracle.radix_partition(keys, pays, 0, 16)
     t, start, count = hj.context(0, width, width).partition(dev(keys), dev(pays), 16)
@@ -476,7 +520,7 @@ def test_next2_skew_and_replicas_vs_oracle(hj, dist, z, rep):
 
 
 @pytest.mark.slow
-@pytest.mark.parametrize("tool", ["memcheck", "racecheck", "synccheck"])
+@pytest.mark.parametrize("tool", ["memcheck", "racecheck", "synccheck", "initcheck"])
 def test_compute_sanitizer_clean(hj, tool):
     import subprocess
     import sys
@@ -488,23 +532,6 @@ def test_compute_sanitizer_clean(hj, tool):
     txt = out.stdout + out.stderr
     assert "sanitize cases ok" in txt, txt[-2000:]
     assert ("ERROR SUMMARY: 0 errors" in txt) or ("RACECHECK SUMMARY: 0 hazards" in txt), txt[-2000:]
-
-
-@pytest.mark.parametrize("name", ["dups_both", "random_ragged", "sparse_uniform"])
-@pytest.mark.parametrize("width", [4, 8])
-def test_pass1_bases_variant_vs_oracle(hj, name, width):
-    """HJ_OPT_PASS1_BASES: per-block bases from the histogram + TMA bulk-store write-out."""
-    rng = np.random.default_rng(77)
-    Rk, Sk = adversarial(rng)[name]
-    dt = np.uint32 if width == 4 else np.uint64
-    Rk, Sk = Rk.astype(dt) * dt(0x10001), Sk.astype(dt) * dt(0x10001)
-    Rp = np.arange(len(Rk), dtype=dt)
-    Sp = np.arange(len(Sk), dtype=dt)
-    ctx = hj.Context(0, width, width)
-    ctx.set_option(hj.OPT_PASS1_BASES, 1)
-    for bits in (-1, 3, 12):
-        check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True, ctx=ctx)
-    ctx.close()
 
 
 def test_graph_replay_matches_oracle(hj):
@@ -534,65 +561,6 @@ def test_graph_replay_matches_oracle(hj):
     ctx.close()
 
 
-FUSE_KNOBS = [(32, 1), (0, 1), (1, 1), (32, 0), (32, 2), (1, 2)]  # (window MB, pass-role blocks/SM; 0 -> 1)
-
-
-@pytest.mark.parametrize("window,slots", FUSE_KNOBS)
-def test_fused_pass2_join_knobs_vs_oracle(hj, window, slots):
-    """HJ_OPT_FUSE (pass 2 + join in one L2-resident kernel): every throttle window and role
-    split gives the oracle's result -- skewed probe side (long S co-partitions split over
-    items), block nested loops (tiny C_R) and 8-byte tuples."""
-    rng = np.random.default_rng(300 + window + slots)
-    for kb, dist, cap_r, chunk_s in [(4, "zipf", 0, 0), (4, "fk", 64, 0), (8, "1to1", 0, 0), (4, "zipf", 300, 2000)]:
-        w = W.Workload("f", 1 << 15, (1 << 15) if dist == "1to1" else (3 << 14), dist,
-                       keys="sparse" if kb == 4 else "k8", z=1.2, seed=int(rng.integers(100, 10_000)))
-        Rk, Rp, Sk, Sp = W.np_generate(w)
-        ctx = hj.Context(0, kb, kb)
-        for opt, v in [(hj.OPT_FUSE, 1), (hj.OPT_FUSE_WINDOW_MB, window), (hj.OPT_FUSE_PASS_SLOTS, slots),
-                       (hj.OPT_CAP_R, cap_r), (hj.OPT_CHUNK_S, chunk_s)]:
-            ctx.set_option(opt, v)
-        for bits in (-1, 2, 9):
-            res = check_against_oracle(hj, Rk, Rp, Sk, Sp, bits=bits, mat=True, ctx=ctx)
-            assert res.fused, "the fused kernel ran"
-        ctx.close()
-
-
-@pytest.mark.parametrize("cfg", ["c1"])
-def test_fused_generated_config_repeats(hj, cfg):
-    """The fused kernel on a BASELINE config, called repeatedly: identical to the closed form."""
-    w = W.CONFIGS[cfg]
-    cols = W.torch_generate(w, device="cuda")
-    ctx = hj.Context(0, w.key_bytes, w.key_bytes)
-    ctx.set_option(hj.OPT_FUSE, 0)
-    ref = ctx.join(*cols, radix_bits=w.radix_bits)
-    assert ref.matches == w.nS
-    ctx.set_option(hj.OPT_FUSE, 1)
-    for _ in range(10):
-        r = ctx.join(*cols, radix_bits=w.radix_bits)
-        assert r.fused and (r.matches, r.checksum) == (ref.matches, ref.checksum)
-    ctx.close()
-
-
-def test_fused_equals_unfused_and_repeats(hj):
-    """Fused and unfused paths give identical results call after call on one context (the fused
-    kernel's counters are reset per call)."""
-    w = W.Workload("f", 1 << 17, 1 << 18, "fk", keys="dense", seed=310)
-    cols = [dev(a) for a in W.np_generate(w)]
-    ctx = hj.Context(0, 4, 4)
-    ref = None
-    for fuse in (1, 0, 1, 1, 0):
-        ctx.set_option(hj.OPT_FUSE, fuse)
-        r = ctx.join(*cols)
-        assert r.fused == bool(fuse)
-        ref = ref or (r.matches, r.checksum)
-        assert (r.matches, r.checksum) == ref
-        rm = ctx.join(*cols, out_mode=hj.OUT_MATERIALIZE)
-        assert rm.matches == ref[0]
-        pairs = oracle.pairs_sorted(to_np(rm.r_pay, 4), to_np(rm.s_pay, 4))
-        assert int(np_sig(pairs[:, 0], pairs[:, 1]).sum(dtype=np.uint64)) == ref[1]
-    ctx.close()
-
-
 @pytest.mark.parametrize("variant", [1, 2, 3, 4])
 def test_pass_variant_invariance(hj, variant):
     """HJ_OPT_PASS_VARIANT (1024-thread register-prefetch tiles vs 512 threads x twice the tuples,
@@ -613,24 +581,110 @@ def test_pass_variant_invariance(hj, variant):
         ctx.close()
 
 
-@pytest.mark.skip(reason="known issue (DESIGN.md §8): at c3 size, a context created after other "
-                         "contexts in the same process can hang or miscount; repro: "
-                         "python tools/bc_one.py c3 0 c3 1 c3 0")
-@pytest.mark.timeout(300)
+@pytest.mark.slow
+@pytest.mark.timeout(600)
 def test_contexts_in_sequence_recycle_memory(hj):
     """Contexts created and closed one after another in one process, alternating the partitioner
-    (histogram path <-> bucket chains), at c3's size: each new context's buffers are recycled
-    from the closed one's. Before ensure() zeroed new allocations this hung (hist -> chains) or
-    faulted (chains -> hist); every join must give the closed form (1:1 permutation: |S| matches)."""
+    (histogram path <-> bucket chains), at c3's size, joining right after the torch generator
+    with no synchronization: each new context's memory is recycled from the closed one's by
+    torch's caching allocator (workspace) or cudaMalloc (ctx-owned). Round 1 saw a miscount and a
+    hang here: hj_set_stream(NULL) mapped torch's default stream to the ctx's non-blocking
+    stream, so the join could read columns the generator was still writing. Every
+    join must give the closed form (1:1 permutation: |S| matches, checksum = sum sig(rho(j), j))."""
     w = W.CONFIGS["c3"]
-    cols = W.torch_generate(w, device="cuda")
+    exp = _closed_form_checksum(w)
     for part in (0, 1, 0, 1):
+        cols = W.torch_generate(w, device="cuda")  # no synchronize: the join must be stream-ordered
         ctx = hj.Context(0, w.key_bytes, w.key_bytes)
         ctx.set_option(hj.OPT_PARTITIONER, part)
         for out_mode in (0, w.out_mode):
             r = ctx.join(*cols, radix_bits=w.radix_bits, out_mode=out_mode)
-            torch.cuda.synchronize()
-            assert r.matches == w.nS, (part, out_mode)
+            assert (r.matches, r.checksum) == (w.nS, exp), (part, out_mode, r.n_items)
         ctx.close()
-    del cols
+        del cols
     torch.cuda.empty_cache()
+
+
+def _closed_form_checksum(w):
+    j = np.arange(w.nS, dtype=np.uint64)
+    cdf = W.zipf_cdf(w.nR, w.z) if w.dist == "zipf" else None
+    return int(np_sig(W.np_rho_for(w, j, cdf), j).sum(dtype=np.uint64))
+
+
+@pytest.mark.slow
+@pytest.mark.timeout(900)
+def test_context_stress_alternating(hj):
+    """>= 20 contexts in one process, alternating partitioner (histogram / bucket chains), output
+    mode, workspace (torch-owned / ctx-owned) and config (c2 / c3), each joined right after its
+    inputs were generated on torch's stream: every result equals the closed form."""
+    cfgs = {k: (W.CONFIGS[k], _closed_form_checksum(W.CONFIGS[k])) for k in ("c2", "c3")}
+    for i in range(20):
+        name = ("c2", "c3")[i % 2]
+        w, exp = cfgs[name]
+        cols = W.torch_generate(w, device="cuda")
+        ctx = hj.Context(0, 4, 4, workspace=(i // 2) % 2 == 0)
+        ctx.set_option(hj.OPT_PARTITIONER, (i // 4) % 2)
+        mode = (i // 8) % 2
+        r = ctx.join(*cols, radix_bits=w.radix_bits, out_mode=mode)
+        assert (r.matches, r.checksum) == (w.nS, exp), (i, name, mode, r.n_items)
+        ctx.close()
+        del cols
+    torch.cuda.empty_cache()
+
+
+def test_join_right_after_generation_no_sync(hj):
+    """The join is ordered after the producer of its columns on torch's current stream (default
+    and a side stream), with no torch.cuda.synchronize() in between."""
+    w = W.Workload("ns", 1 << 20, 1 << 22, "fk", keys="sparse", seed=131)
+    ref = oracle.hash_join(*W.np_generate(w))
+    for use_side in (False, True):
+        s = torch.cuda.Stream() if use_side else torch.cuda.current_stream()
+        with torch.cuda.stream(s):
+            for _ in range(3):
+                cols = W.torch_generate(w, device="cuda")
+                r = hj.join(*cols)
+                assert (r.matches, r.checksum) == ref, use_side
+
+
+def test_workspace_api(hj):
+    """hj_workspace_bytes / hj_set_workspace: hj_join runs inside a caller (torch) buffer that
+    starts with garbage (nothing is read before it is written), refuses a too-small one, and the
+    binding regrows it when materialized pairs outgrow the capacity (reading S11)."""
+    lib = hj.lib()
+    w = W.Workload("ws", 1 << 17, 1 << 19, "zipf", keys="sparse", z=1.1, seed=132)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    m, c, r, s = oracle.hash_join(Rk, Rp, Sk, Sp, materialize=True)
+    cols = [dev(a) for a in (Rk, Rp, Sk, Sp)]
+    for part in (0, 1):
+        ctx = hj.Context(0, 4, 4, workspace=False)
+        ctx.set_option(hj.OPT_PARTITIONER, part)
+        need = ctx.workspace_bytes(w.nR, w.nS, -1, hj.OUT_MATERIALIZE)
+        assert need > 0 and ctx.workspace_bytes(0, w.nS, -1, 0) == 0
+        buf = torch.full((need,), 0xA5, dtype=torch.uint8, device="cuda")  # garbage
+        assert lib.hj_set_workspace(ctx._h, ctypes.c_void_p(buf.data_ptr() + 8), need) == -1  # unaligned
+        small = torch.empty(need // 2, dtype=torch.uint8, device="cuda")
+        assert lib.hj_set_workspace(ctx._h, ctypes.c_void_p(small.data_ptr()), small.numel()) == 0
+        with pytest.raises(hj.HJError, match="WORKSPACE"):
+            ctx.join(*cols, out_mode=hj.OUT_MATERIALIZE)
+        assert lib.hj_set_workspace(ctx._h, ctypes.c_void_p(buf.data_ptr()), need) == 0
+        for mode in (0, 1, 1):
+            res = ctx.join(*cols, out_mode=mode)
+            assert (res.matches, res.checksum) == (m, c), (part, mode)
+            if mode:
+                assert np.array_equal(oracle.pairs_sorted(to_np(res.r_pay, 4), to_np(res.s_pay, 4)),
+                                      oracle.pairs_sorted(r, s))
+                p0 = res.r_pay.data_ptr()
+                assert buf.data_ptr() <= p0 < buf.data_ptr() + need  # the pairs live in the workspace
+        assert lib.hj_set_workspace(ctx._h, None, 0) == 0  # back to ctx-owned memory
+        res = ctx.join(*cols)
+        assert (res.matches, res.checksum) == (m, c)
+        ctx.close()
+    # the binding's torch workspace regrows on a materialization overflow
+    ctx = hj.Context(0, 4, 4)
+    ctx.set_option(hj.OPT_OUT_CAPACITY, 1000)
+    Rk = np.repeat(np.arange(50, dtype=np.uint32), 40)
+    Sk = np.repeat(np.arange(60, dtype=np.uint32), 30)
+    res = check_against_oracle(hj, Rk, np.arange(len(Rk), dtype=np.uint32), Sk, np.arange(len(Sk), dtype=np.uint32),
+                               bits=3, mat=True, ctx=ctx)
+    assert res.matches == 50 * 40 * 30
+    ctx.close()

@@ -15,11 +15,9 @@ import workloads as W  # noqa: E402
 
 OPTS = {"join_variant": hj.OPT_JOIN_VARIANT, "cap_r": hj.OPT_CAP_R, "chunk_s": hj.OPT_CHUNK_S,
         "blocks_per_sm": hj.OPT_BLOCKS_PER_SM, "pass_threads": hj.OPT_PASS_THREADS, "join_algo": hj.OPT_JOIN_ALGO,
-        "stream_chunk": hj.OPT_STREAM_CHUNK, "pass1_bases": hj.OPT_PASS1_BASES,
-        "partitioner": hj.OPT_PARTITIONER, "fuse": hj.OPT_FUSE,
-        "fuse_window_mb": hj.OPT_FUSE_WINDOW_MB, "fuse_pass_slots": hj.OPT_FUSE_PASS_SLOTS,
+        "stream_chunk": hj.OPT_STREAM_CHUNK, "partitioner": hj.OPT_PARTITIONER,
         "pass_l2pf": hj.OPT_PASS_L2PF, "pass1_bits": hj.OPT_PASS1_BITS,
-        "pass_variant": hj.OPT_PASS_VARIANT}
+        "pass_variant": hj.OPT_PASS_VARIANT, "mat_checksum": hj.OPT_MAT_CHECKSUM}
 
 
 def main():
