@@ -449,6 +449,7 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   P.nsrc = hp.nsrc;
   P.mode = hp.mode;
   P.C2 = hp.C2;
+  P.tuple_bytes = c->key_bytes + c->pay_bytes;
   // measured (tools/tune.py pass_l2pf): 8 B tuples pass 1 4.02 -> 3.59 ms on c5_gpu; 4 B pass 1
   // slower (c3 0.939 -> 0.983), pass 2 unchanged -> auto (2) = on for 8-byte keys only
   P.pass_l2pf = c->opt_pass_l2pf == 2 ? (c->key_bytes == 8) : (c->opt_pass_l2pf ? 1 : 0);
@@ -511,12 +512,6 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false, 
     return HJ_OK;
   }
   mark(c, 0);
-  if (hp.mode != PLAN_SEND)  // T2's 64-byte tails: the join's 16-byte aligned R copies may read into them
-    for (int r = 0; r < 2; ++r)
-      if (P.rel[r].t2 && !(r == 0 && P.skip_r)) {  // (streaming S chunks: T2 of R holds R)
-        const size_t tb = (size_t)c->key_bytes + c->pay_bytes;
-        CUDA_TRY(c, cudaMemsetAsync((char*)P.rel[r].t2 + P.rel[r].n * tb, 0, 64, st));
-      }
   if (!chunk) {
     CUDA_TRY(c, cudaMemsetAsync(P.counters, 0, hp.zero_bytes, st));  // the zeroed region starts at o_counters = 0
   } else {  // streaming S chunk: keep R's counts and the accumulated results

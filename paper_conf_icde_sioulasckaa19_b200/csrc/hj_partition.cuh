@@ -171,6 +171,13 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
       if (items) sI += plan_items(P, cr[u], cs[u]);
     }
   }
+  // T2's 64-byte tails (the join's 16-byte aligned R copies may read into them; streaming S
+  // chunks: T2 of R holds R, its tail is past R's end and stays)
+  if (b == 0 && threadIdx.x < 32 && P.mode != PLAN_SEND) {
+    const int r = threadIdx.x >> 4;
+    if (P.rel[r].t2 && !(r == 0 && P.skip_r))
+      reinterpret_cast<uint32_t*>(reinterpret_cast<char*>(P.rel[r].t2) + P.rel[r].n * (unsigned long long)P.tuple_bytes)[threadIdx.x & 15] = 0u;
+  }
   // ---- own range ---------------------------------------------------------------------------
   const uint32_t q = b * NT + threadIdx.x;
   unsigned long long cr = 0, cs = 0;

@@ -72,6 +72,7 @@ struct Plan {
   int mode;       // PLAN_FULL, PLAN_SEND, PLAN_RECV
   int skip_r;     // streaming S chunks: R is already partitioned (its pass-2 units are skipped)
   int pass_l2pf;  // partition passes: TMA-prefetch unit i+2's input into L2 when it is published
+  int tuple_bytes;  // AoS tuple size (8 or 16): the planner zeroes each T2's 64-byte tail
   uint32_t C2;           // pass-2 chunk (tile) size in tuples
   uint32_t CR, CS;       // join item capacities: R tuples (smem build) and S tuples per item
   uint32_t* ist;         // [2^B + 1] join item prefix (q-order)

@@ -5,6 +5,9 @@
 //   runs  : read SoA, write each 8192-tuple tile as F runs of 8192/F tuples, run d of tile t to
 //           region d at offset t * run (F write streams, one run per warp store group) -- the
 //           pattern a pass with fan-out F produces on uniform keys
+//   scat  : the same F streams, but element i of a tile goes to stream i % F: every lane of a
+//           warp stores to a different stream (no shared-memory shuffle; write combining is
+//           left to L2) -- the ceiling of a pass that scatters tuples straight from registers
 // n = 2^28 tuples (c3's pass 1: R + S). Prints GB/s of (read + write) bytes per variant.
 //   nvcc -gencode arch=compute_100a,code=sm_100a -O3 -o mb_scatter mb_scatter.cu
 #include <cstdint>
@@ -23,7 +26,7 @@ __global__ void __launch_bounds__(NT) k_read(const uint4* __restrict__ k, const 
   if (acc == 0x12345678u) sink[0] = acc;
 }
 
-// MODE 0: sequential AoS write; MODE 1: F runs per tile
+// MODE 0: sequential AoS write; MODE 1: F runs per tile; MODE 2: scattered (element i -> stream i % F)
 template <int MODE>
 __global__ void __launch_bounds__(NT) k_pass(const uint32_t* __restrict__ keys, const uint32_t* __restrict__ pays,
                                              size_t n, unsigned long long* __restrict__ out, int F) {
@@ -43,7 +46,8 @@ __global__ void __launch_bounds__(NT) k_pass(const uint32_t* __restrict__ keys, 
         const unsigned long long v = (unsigned long long)ka[e] | ((unsigned long long)pa[e] << 32);
         size_t dst;
         if (MODE == 0) dst = t * TILE + i;
-        else dst = (size_t)(i / run) * (n / F) + t * run + (i % run);
+        else if (MODE == 1) dst = (size_t)(i / run) * (n / F) + t * run + (i % run);
+        else dst = (size_t)(i % F) * (n / F) + t * run + (i / F);
         __stcs(out + dst, v);
       }
     }
@@ -87,6 +91,10 @@ int main() {
     for (int F : {64, 128, 256, 512, 1024}) {
       snprintf(nm, sizeof nm, "runs F=%d run=%d (grid %d)", F, TILE / F, g);
       time([&] { k_pass<1><<<g, NT>>>(k, p, n, out, F); }, 16.0 * n, nm);
+    }
+    for (int F : {32, 128, 1024, 8192}) {
+      snprintf(nm, sizeof nm, "scat F=%d (grid %d)", F, g);
+      time([&] { k_pass<2><<<g, NT>>>(k, p, n, out, F); }, 16.0 * n, nm);
     }
   }
   cudaError_t e = cudaDeviceSynchronize();
