@@ -100,6 +100,10 @@ enum hj_option {
                                pass 2); 0 = auto (pass 1 of 8-byte tuples, where it measured faster) */
   HJ_OPT_STREAM_CHUNK = 8,  /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
                                least 2^22; >= |S| = copy everything, then join)                   */
+  HJ_OPT_PASS_WS = 21,      /* partition passes (histogram partitioner, fan-out <= 2^9): 1 (default) =
+                               warp-specialized pipeline (TMA-fed input stages, compute warps that
+                               rank and shuffle, writer warps that stream the previous tile out);
+                               0 = every warp of the block in lock step (round-1 kernel)           */
   HJ_OPT_MAT_CHECKSUM = 20  /* 1 (default) = MATERIALIZE also fills res->checksum (the pairs'
                                signatures are summed by the probe, so every materialized result is
                                self-checking); 0 = checksum left 0 in MATERIALIZE (measurement)   */

@@ -44,6 +44,7 @@ OPT_PASS_L2PF = 17
 OPT_PASS1_BITS = 18
 OPT_PASS_VARIANT = 19
 OPT_MAT_CHECKSUM = 20  # 1 (default): MATERIALIZE also returns the checksum
+OPT_PASS_WS = 21  # 1 (default): warp-specialized partition passes
 ALGO_HASH, ALGO_NLJ, ALGO_NONPARTITIONED = 0, 1, 2
 
 ERR_WORKSPACE = -6

@@ -16,6 +16,7 @@
 #include "hj_exchange.cuh"
 #include "hj_join.cuh"
 #include "hj_partition.cuh"
+#include "hj_pass_ws.cuh"
 #include "hj_variants.cuh"
 
 using namespace hj;
@@ -72,7 +73,7 @@ struct Ctx {
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
           opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_graph = 0, opt_pass_l2pf = 2, opt_pass1_bits = 0,
-          opt_partitioner = 0, opt_pass_variant = 0, opt_mat_chk = 1;
+          opt_partitioner = 0, opt_pass_variant = 0, opt_mat_chk = 1, opt_pass_ws = 1;
   DevBuf bc_pool1[2], bc_pool2[2], bc_meta;  // HJ_OPT_PARTITIONER = 1 (NEXT-1 bucket chains)
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2], np_heads, np_next;
@@ -243,6 +244,17 @@ int pass_threads(const Ctx* c, int fanout_bits, int items) {
   return (512 * items) >> fanout_bits >= 32 ? 512 : 1024;
 }
 
+// the warp-specialized pass (hj_pass_ws.cuh) for a fan-out of 2^bits: histogram partitioner,
+// fan-out <= WS_MAXF (shared-memory budget); its unit is a 64 KB tile
+bool use_ws(const Ctx* c, int bits) { return c->opt_pass_ws && c->opt_partitioner == 0 && (1 << bits) <= WS_MAXF; }
+// role split: HJ_OPT_PASS_WS = 1 / 2 / 3 -> 16 / 20 / 24 compute warps
+int ws_cw(const Ctx* c) { return c->opt_pass_ws == 3 ? 24 : c->opt_pass_ws == 2 ? 20 : 16; }
+uint32_t ws_tile(const Ctx* c) {
+  const int cw = ws_cw(c);
+  if (c->key_bytes == 4) return cw == 24 ? WsShape<uint32_t, 24>::TILE : cw == 20 ? WsShape<uint32_t, 20>::TILE : WsShape<uint32_t, 16>::TILE;
+  return cw == 24 ? WsShape<uint64_t, 24>::TILE : cw == 20 ? WsShape<uint64_t, 20>::TILE : WsShape<uint64_t, 16>::TILE;
+}
+
 int choose_bits(unsigned long long nR) {
   // mean R co-partition ~4096 tuples: the paper's shared-memory reservation
   if (nR <= 4096) return 0;
@@ -274,8 +286,8 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   // pass tiles: two 512-thread blocks per SM when a 512-thread tile still averages >= 32 tuples
   // per digit run (measured: shorter runs cost more than the extra block's overlap), else one
   // 1024-thread block. The pass-2 chunk is that kernel's tile.
-  hp.tile = pass_threads(c, hp.pb(), items) * items;
-  hp.C2 = (uint32_t)(pass_threads(c, hp.b2, items) * items);
+  hp.tile = use_ws(c, hp.pb()) ? ws_tile(c) : pass_threads(c, hp.pb(), items) * items;
+  hp.C2 = use_ws(c, hp.b2) ? ws_tile(c) : (uint32_t)(pass_threads(c, hp.b2, items) * items);
 
   // join capacities
   const unsigned long long mean = (nR + (1ull << hp.B) - 1) >> hp.B;
@@ -337,6 +349,19 @@ void attr_join(F&& attr) {
   attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf>);
 }
 
+template <typename K, typename F>
+void for_ws_variants(F&& attr) {
+  attr((const void*)k_pass_ws<K, 1, false, 16>);
+  attr((const void*)k_pass_ws<K, 1, true, 16>);
+  attr((const void*)k_pass_ws<K, 2, false, 16>);
+  attr((const void*)k_pass_ws<K, 1, false, 20>);
+  attr((const void*)k_pass_ws<K, 1, true, 20>);
+  attr((const void*)k_pass_ws<K, 2, false, 20>);
+  attr((const void*)k_pass_ws<K, 1, false, 24>);
+  attr((const void*)k_pass_ws<K, 1, true, 24>);
+  attr((const void*)k_pass_ws<K, 2, false, 24>);
+}
+
 template <typename K>
 int set_kernel_attrs(Ctx* c) {
   int rc = 0;
@@ -370,6 +395,7 @@ int set_kernel_attrs(Ctx* c) {
   attr((const void*)k_hist<K, true, true, true>);
   attr((const void*)k_hist<K, true, false, false>);
   attr((const void*)k_hist<K, true, true, false>);
+  for_ws_variants<K>(attr);
   attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), false>);
   attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), true>);
   attr((const void*)k_pass<K, 2, 1024, pass_items<K>(), false>);
@@ -554,13 +580,38 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false, 
 }
 
 // a3 / a4: one partition pass (launch shape per pass and width).
+template <typename K, int MODE, bool GD, int CW>
+int launch_pass_ws(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
+  using S = WsShape<K, CW>;
+  const void* f = (const void*)k_pass_ws<K, MODE, GD, CW>;
+  const size_t sm = S::smem(fanout_bits);
+  const unsigned long long tile = S::TILE;
+  Plan Q = P;
+  Q.C2 = (uint32_t)tile;
+  const unsigned long long units = MODE == 1 ? (P.rel[0].n + tile - 1) / tile + (P.rel[1].n + tile - 1) / tile
+                                             : (P.rel[0].n + P.rel[1].n) / tile + 2ull * hp.npieces() + 2;
+  if (MODE == 1) {
+    Q.tiles1[0] = (P.rel[0].n + tile - 1) / tile;
+    Q.tiles1[1] = (P.rel[1].n + tile - 1) / tile;
+  }
+  const int g = grid_for(c, f, WS_NT, sm, units);
+  k_pass_ws<K, MODE, GD, CW><<<g, WS_NT, sm, c->stream>>>(Q, fanout_bits);
+  CUDA_TRY(c, cudaGetLastError());
+  c->launches += 1;
+  return HJ_OK;
+}
+
 template <typename K, int MODE, int NT, bool GD, bool BC>
 int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
   constexpr int IT = pass_items<K>();
-  // HJ_OPT_PASS_VARIANT 1: the 1024 x IT tile as 512 threads x 2 IT without register prefetch,
-  // two blocks per SM (the unit after next still goes to L2 by TMA prefetch)
-  // per pass (bit MODE - 1 of the mask); auto = pass 1 of 8-byte tuples (measured: c5_gpu pass 1
-  // 3.60 -> 3.29 ms, but pass 2 3.24 -> 3.49 and c3 pass 1 0.94 -> 1.00)
+  if (!BC && use_ws(c, fanout_bits) && (MODE == 1 ? hp.tile : hp.C2) == ws_tile(c)) {
+    // warp-specialized pipeline: one 1024-thread block per SM
+    switch (ws_cw(c)) {
+      case 24: return launch_pass_ws<K, MODE, GD, 24>(c, hp, P, fanout_bits);
+      case 20: return launch_pass_ws<K, MODE, GD, 20>(c, hp, P, fanout_bits);
+      default: return launch_pass_ws<K, MODE, GD, 16>(c, hp, P, fanout_bits);
+    }
+  }
   const int mask = c->opt_pass_variant > 0 ? (int)c->opt_pass_variant - 1 : (c->key_bytes == 8 ? 1 : 0);
   if (NT == 1024 && ((mask >> (MODE - 1)) & 1) && (1 << fanout_bits) <= 512) {
     const void* f2 = (const void*)k_pass<K, MODE, 512, 2 * IT, GD, BC, false>;
@@ -1356,6 +1407,10 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_BLOCKS_PER_SM: c->opt_bps = v; break;
     case HJ_OPT_STREAM_CHUNK: c->opt_stream_chunk = v; break;
     case HJ_OPT_MAT_CHECKSUM: c->opt_mat_chk = v; break;
+    case HJ_OPT_PASS_WS:
+      if (v > 3) return fail(c, HJ_ERR_INVALID, "pass_ws must be 0..3");
+      c->opt_pass_ws = v;
+      break;
     case HJ_OPT_PASS_L2PF: c->opt_pass_l2pf = v; break;
     case HJ_OPT_PASS1_BITS: c->opt_pass1_bits = v; break;
     case HJ_OPT_PARTITIONER:

@@ -1,0 +1,369 @@
+// hj_pass_ws.cuh -- a3 / a4 (one radix-partition pass) as a warp-specialized pipeline.
+//
+// Same result as k_pass (hj_partition.cuh): every tuple of a unit is ranked within its digit with
+// a shared-memory atomic, each digit's run is reserved in the output with one global atomic per
+// (unit, digit), the unit is shuffled into digit order in shared memory and streamed out so
+// consecutive threads write consecutive addresses of a run (P:142-148 coalescing; P:265-275
+// metadata + shuffle space in shared memory). What changes is how an SM overlaps the steps: k_pass
+// runs rank | write-out of the previous unit | shuffle with every warp of the block in lock step,
+// so each SM's HBM traffic comes in bursts between block barriers (c3 pass 1: 0.95 ms, against
+// 0.68 ms for the same access pattern with no shared-memory work, tools/microbench/mb_scatter.cu).
+// Here one 1024-thread block per SM is three roles joined by mbarriers:
+//   producer (warp 31)   : unit descriptors, and each unit's input copied into one of two
+//                          shared-memory stages by TMA bulk copies (cp.async.bulk, no registers:
+//                          two units of input in flight per SM)
+//   compute  (warps 0-15): rank the stage's keys (shared atomics), scan + reserve (one global
+//                          atomic per digit run), shuffle the stage into the output tile
+//   writer   (warps 16-30): output tile -> HBM, a run per consecutive group of threads
+// so the writer streams unit i-1 while the compute warps rank unit i and TMA fetches unit i+1.
+// Shared memory: 2 input stages + 1 output tile (64 KB each) + run tables: fan-out <= 512.
+// A unit stays in its stage until it is shuffled (only the ranks live in registers). Units whose
+// input is ragged or not 16-byte aligned (the last unit of a relation, a piece whose aligned
+// superset would leave the pass-1 data) are copied into the stage by the compute warps.
+#pragma once
+#include "hj_common.cuh"
+#include "hj_plan.cuh"
+
+namespace hj {
+
+constexpr int WS_NT = 1024;       // compute warps + writer warps + producer warp 31
+constexpr int WS_MAXF = 512;      // fan-out bound (shared-memory budget)
+
+// Role split (HJ_OPT_PASS_WS = 1 + variant): CW compute warps, 31 - CW writer warps; each compute
+// thread ranks CIT tuples of a unit, so a unit (tile) has CW * 32 * CIT tuples.
+template <typename K, int CW>
+struct WsShape {
+  static constexpr int CT = CW * 32, WT = (31 - CW) * 32;
+  static constexpr int CIT = sizeof(K) == 4 ? (CW == 16 ? 16 : CW == 20 ? 12 : 8) : (CW == 16 ? 8 : CW == 20 ? 6 : 4);
+  static constexpr int TILE = CT * CIT;
+  static constexpr uint32_t STAGE = (uint32_t)TILE * 2 * sizeof(K) + 16;  // +16: aligned superset of AoS units
+  static constexpr size_t smem(int fanout_bits) {  // 2 stages + output tile + s_gd (3F) + s_cnt + s_loc
+    return 2 * (size_t)STAGE + (size_t)TILE * 2 * sizeof(K) + ((size_t)1 << fanout_bits) * 32 + 16;
+  }
+};
+
+__device__ __forceinline__ void mbar_arrive(unsigned long long* bar) {
+  asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
+}
+
+struct WsUnit {
+  const void* src_k;  // MODE 1: key column at the unit start; MODE 2: first AoS tuple
+  const void* src_p;  // MODE 1: payload column at the unit start
+  void* dst;          // output buffer (T1 or T2)
+  unsigned long long* cur;  // reservation cursors (MODE 2: &cur2[D << b2])
+  uint32_t len;
+  uint32_t valid;
+  uint32_t tma;    // input is in the stage (else: load from global)
+  uint32_t shift;  // MODE 2: tuples between the stage start and the unit's first tuple
+};
+
+template <typename K, int MODE, bool GD, int CW>
+__global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
+  using TT = Tup<K>;
+  using T = typename TT::T;
+  using S = WsShape<K, CW>;
+  constexpr int WS_CT = S::CT, WS_WT = S::WT, CIT = S::CIT, TILE = S::TILE;
+  constexpr uint32_t WS_STAGE = S::STAGE;
+  constexpr int VEC = 16 / sizeof(K);
+  static_assert(CIT % VEC == 0 && CIT % 2 == 0 && TILE < 65536, "tile shape");
+  extern __shared__ __align__(128) unsigned char s_raw[];
+  unsigned char* s_in = s_raw;                                    // 2 x WS_STAGE
+  T* s_out = reinterpret_cast<T*>(s_raw + 2 * WS_STAGE);          // TILE tuples
+  const uint32_t F = 1u << fanout_bits;
+  unsigned long long* s_gd = reinterpret_cast<unsigned long long*>(s_out + TILE);  // 3 x F: run base - loc
+  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gd + 3 * F);    // F + 1 (spare for ragged lanes)
+  uint32_t* s_loc = s_cnt + F + 4;                                // F
+  __shared__ __align__(8) unsigned long long s_full[2], s_empty[2], s_ofull, s_oempty;
+  __shared__ WsUnit s_desc[4];
+  __shared__ uint32_t s_wt[WS_CT / 32];
+  __shared__ uint32_t s_hot, s_hot_next;
+  __shared__ uint32_t s_cst[MODE == 2 ? 2 * 1025 : 1];
+
+  const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+  if (MODE == 2 && P.mode == PLAN_RECV && *(volatile const uint32_t*)&P.counters[CNT_BAD_COUNTS]) return;
+  const uint32_t dsh = MODE == 1 ? 0u : (uint32_t)P.b1;
+  const uint32_t dmask = MODE == 1 ? ((1u << P.b1) - 1) : ((1u << P.b2) - 1);
+  const uint32_t gsh = (uint32_t)P.B, gmask = (1u << P.g) - 1, gup = (uint32_t)P.b1;
+  auto digit = [=](K key) -> uint32_t {
+    uint32_t d = (uint32_t)(key >> dsh) & dmask;
+    if (MODE == 1 && GD) d |= ((uint32_t)(key >> gsh) & gmask) << gup;
+    return d;
+  };
+
+  unsigned long long units0, units;
+  if (MODE == 1) {
+    units0 = P.tiles1[0];
+    units = units0 + P.tiles1[1];
+  } else {
+    const uint32_t npc = P.npieces();  // <= 1024
+    for (uint32_t i = threadIdx.x; i <= npc; i += WS_NT) {
+      s_cst[i] = P.rel[0].cst[i];
+      s_cst[1025 + i] = P.rel[1].cst[i];
+    }
+    units0 = P.skip_r ? 0ull : P.rel[0].cst[npc];
+    units = units0 + P.rel[1].cst[npc];
+  }
+  if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
+  if (threadIdx.x == 0) {
+    s_hot = s_hot_next = 0xffffffffu;
+    mbar_init(&s_full[0], 1);
+    mbar_init(&s_full[1], 1);
+    mbar_init(&s_empty[0], WS_CT / 32);
+    mbar_init(&s_empty[1], WS_CT / 32);
+    mbar_init(&s_ofull, WS_CT / 32);
+    mbar_init(&s_oempty, WS_WT / 32);
+    fence_mbar_init();
+  }
+  __syncthreads();
+  const unsigned long long G = gridDim.x;
+
+  if (warp == 31) {
+    // ---------------------------------------------------------------- producer ----------------
+    if (lane != 0) return;
+    for (uint32_t i = 0;; ++i) {
+      const uint32_t stage = i & 1;
+      if (i >= 2) mbar_wait(&s_empty[stage], ((i >> 1) - 1) & 1);  // compute consumed unit i-2
+      const unsigned long long u = blockIdx.x + (unsigned long long)i * G;
+      WsUnit D;
+      D.valid = u < units;
+      D.tma = 0;
+      D.shift = 0;
+      if (D.valid) {
+        const int r = u < units0 ? 0 : 1;
+        const RelDev& R = P.rel[r];
+        const unsigned long long ul = r ? u - units0 : u;
+        if (MODE == 1) {
+          const unsigned long long s0 = ul * TILE;
+          D.src_k = (const K*)R.keys + s0;
+          D.src_p = (const K*)R.pays + s0;
+          D.dst = R.t1;
+          D.cur = R.cur1;
+          D.len = (uint32_t)min((unsigned long long)TILE, R.n - s0);
+          D.tma = D.len == TILE && ((reinterpret_cast<uintptr_t>(D.src_k) | reinterpret_cast<uintptr_t>(D.src_p)) & 15) == 0;
+        } else {
+          const uint32_t* cst = s_cst + r * 1025;
+          const uint32_t uc = (uint32_t)ul;
+          uint32_t lo = 0, hi = P.npieces();  // largest piece with cst[piece] <= uc
+          while (hi - lo > 1) {
+            const uint32_t mid = (lo + hi) >> 1;
+            if (cst[mid] <= uc) lo = mid; else hi = mid;
+          }
+          const unsigned long long pa = R.pst[lo], pb = R.pst[lo + 1];
+          const unsigned long long s0 = pa + (unsigned long long)(uc - cst[lo]) * TILE;
+          const uint32_t Dg = lo & ((1u << P.pb()) - 1);  // pass-1 digit of the piece
+          D.src_k = (const T*)R.t1 + s0;
+          D.src_p = nullptr;
+          D.dst = R.t2;
+          D.cur = R.cur2 + ((unsigned long long)Dg << P.b2);
+          D.len = (uint32_t)min((unsigned long long)TILE, pb - s0);
+          // the 16-byte aligned superset must stay inside the relation's pass-1 data
+          const uintptr_t a = reinterpret_cast<uintptr_t>(D.src_k), a0 = a & ~(uintptr_t)15;
+          const uintptr_t a1 = (a + (uintptr_t)D.len * sizeof(T) + 15) & ~(uintptr_t)15;
+          const uintptr_t end = reinterpret_cast<uintptr_t>((const T*)R.t1 + R.pst[P.npieces()]);
+          D.tma = a1 <= end;
+          D.shift = (uint32_t)((a - a0) / sizeof(T));
+        }
+      }
+      s_desc[i & 3] = D;
+      unsigned char* st = s_in + stage * WS_STAGE;
+      if (D.valid && D.tma) {
+        fence_proxy_async();  // the compute warps' reads of this stage (unit i-2) precede the copy
+        if (MODE == 1) {
+          const uint32_t b = TILE * (uint32_t)sizeof(K);
+          mbar_arrive_expect_tx(&s_full[stage], 2 * b);
+          bulk_g2s(st, D.src_k, b, &s_full[stage]);
+          bulk_g2s(st + b, D.src_p, b, &s_full[stage]);
+        } else {
+          const uintptr_t a = reinterpret_cast<uintptr_t>(D.src_k), a0 = a & ~(uintptr_t)15;
+          const uint32_t b = (uint32_t)(((a + (uintptr_t)D.len * sizeof(T) - a0) + 15) & ~(uintptr_t)15);
+          mbar_arrive_expect_tx(&s_full[stage], b);
+          bulk_g2s(st, reinterpret_cast<const void*>(a0), b, &s_full[stage]);
+        }
+      } else {
+        mbar_arrive(&s_full[stage]);  // descriptor only (the end marker, or a unit loaded from global)
+      }
+      if (!D.valid) return;
+    }
+  }
+
+  if (warp >= WS_CT / 32) {
+    // ---------------------------------------------------------------- writer ------------------
+    const uint32_t wt = threadIdx.x - WS_CT;
+    for (uint32_t i = 0;; ++i) {
+      mbar_wait(&s_ofull, i & 1);  // the compute warps shuffled unit i (or reached the end)
+      const WsUnit& D = s_desc[i & 3];
+      if (!D.valid) return;
+      T* dst = (T*)D.dst;
+      const uint32_t len = D.len;
+      const unsigned long long* gd = s_gd + (i % 3) * F;
+      #pragma unroll 4
+      for (uint32_t e = wt; e < len; e += WS_WT) {
+        const T t = s_out[e];
+        __stcs(dst + (gd[digit(TT::key(t))] + e), t);
+      }
+      __syncwarp();
+      if (lane == 0) mbar_arrive(&s_oempty);
+    }
+  }
+
+  // ------------------------------------------------------------------ compute -----------------
+  // The unit stays in its input stage until the shuffle (keys are read there for the ranks, and
+  // key + payload again for the shuffle): only the ranks live in registers across the barriers.
+  const uint32_t nscan = F < 32 ? 32u : F;  // threads in the digit scan (whole warps)
+  // element e of the unit in the stage held by thread (j, v): MODE 1 (j * CT + tid) * VEC + v
+  // (128-bit loads of VEC keys / payloads), MODE 2 j * CT + tid
+  auto elem = [&](int j) -> uint32_t {
+    return MODE == 1 ? (uint32_t)((j / VEC) * WS_CT + threadIdx.x) * VEC + (j % VEC) : (uint32_t)(j * WS_CT + threadIdx.x);
+  };
+  for (uint32_t i = 0;; ++i) {
+    const uint32_t stage = i & 1;
+    mbar_wait(&s_full[stage], (i >> 1) & 1);
+    const WsUnit D = s_desc[i & 3];
+    if (!D.valid) {
+      if (i >= 1) mbar_wait(&s_oempty, (i - 1) & 1);  // the writer finished the last unit
+      __syncwarp();
+      if (lane == 0) mbar_arrive(&s_ofull);  // end marker for the writer
+      break;
+    }
+    const uint32_t ulen = D.len;
+    const bool full = ulen == TILE;
+    unsigned char* st = s_in + stage * WS_STAGE;
+    const K* s_k = reinterpret_cast<const K*>(st);                   // MODE 1: keys
+    const K* s_p = reinterpret_cast<const K*>(st + TILE * sizeof(K));  //         payloads
+    const T* s_t = reinterpret_cast<const T*>(st) + D.shift;         // MODE 2: tuples
+    if (!D.tma) {  // ragged / unaligned unit: the compute warps copy it into the stage
+      for (uint32_t e = threadIdx.x; e < ulen; e += WS_CT) {
+        if (MODE == 1) {
+          const_cast<K*>(s_k)[e] = ((const K*)D.src_k)[e];
+          const_cast<K*>(s_p)[e] = ((const K*)D.src_p)[e];
+        } else {
+          const_cast<T*>(s_t)[e] = __ldcs((const T*)D.src_k + e);
+        }
+      }
+      asm volatile("barrier.sync 1, %0;" ::"r"(WS_CT) : "memory");
+    }
+    // this thread's CIT keys (MODE 1: 128-bit loads of VEC consecutive keys, conflict-free)
+    K kk[CIT];
+    #pragma unroll
+    for (int j0 = 0; j0 < CIT; j0 += (MODE == 1 ? VEC : 1)) {
+      if (MODE == 1) {
+        const uint4 kv = *reinterpret_cast<const uint4*>(s_k + elem(j0));
+        const K* ke = reinterpret_cast<const K*>(&kv);
+        #pragma unroll
+        for (int v = 0; v < VEC; ++v) kk[j0 + v] = ke[v];
+      } else {
+        kk[j0] = TT::key(s_t[elem(j0)]);
+      }
+    }
+
+    // ---- rank (as k_pass: lanes on the predicted hot digit are ranked by ballot) -------------
+    uint32_t rk[CIT / 2];
+    const uint32_t hot = s_hot;
+    if (hot > F) {
+      #pragma unroll
+      for (int j = 0; j < CIT; ++j) {
+        const uint32_t d = (full || elem(j) < ulen) ? digit(kk[j]) : F;
+        const uint32_t r = atomicAdd(&s_cnt[d], 1u);
+        if (j & 1) rk[j / 2] |= r << 16; else rk[j / 2] = r & 0xffffu;
+      }
+    } else {
+      uint32_t hacc = 0, hbits = 0;
+      const uint32_t lt = lanemask_lt();
+      #pragma unroll
+      for (int j = 0; j < CIT; ++j) {
+        const uint32_t d = (full || elem(j) < ulen) ? digit(kk[j]) : F;
+        const bool ih = d == hot;
+        const uint32_t hm = __ballot_sync(0xffffffffu, ih);
+        const uint32_t r = ih ? hacc + __popc(hm & lt) : atomicAdd(&s_cnt[d], 1u);
+        hacc += __popc(hm);
+        hbits |= (uint32_t)ih << j;
+        if (j & 1) rk[j / 2] |= r << 16; else rk[j / 2] = r & 0xffffu;
+      }
+      if (hacc) {
+        uint32_t base = 0;
+        if (lane == 0) base = atomicAdd(&s_cnt[hot], hacc);
+        base = __shfl_sync(0xffffffffu, base, 0);
+        #pragma unroll
+        for (int j = 0; j < CIT; ++j)
+          if ((hbits >> j) & 1) rk[j / 2] += base << (16 * (j & 1));
+      }
+    }
+    asm volatile("barrier.sync 1, %0;" ::"r"(WS_CT) : "memory");
+
+    // ---- scan + reserve (threads < F) ---------------------------------------------------------
+    unsigned long long* gd = s_gd + (i % 3) * F;
+    // each run's reservation atomic is issued here and its result stored after the shuffle, so
+    // the global atomic's round trip overlaps the shuffle (the writer reads gd after s_ofull)
+    unsigned long long rres = 0;
+    uint32_t rloc = 0;
+    bool rv = false;
+    if (threadIdx.x < nscan) {
+      const uint32_t d = threadIdx.x;
+      const uint32_t c = d < F ? s_cnt[d] : 0u;
+      uint32_t x = c;
+      #pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t y = __shfl_up_sync(0xffffffffu, x, o);
+        if (lane >= o) x += y;
+      }
+      if (lane == 31) s_wt[warp] = x;
+      asm volatile("barrier.sync 2, %0;" ::"r"(nscan) : "memory");
+      uint32_t base = 0;
+      for (int w = 0; w < warp; ++w) base += s_wt[w];
+      const uint32_t loc = base + x - c;
+      if (d < F) {
+        s_loc[d] = loc;
+        s_cnt[d] = 0;
+        if (c) {
+          rres = atomicAdd(D.cur + d, (unsigned long long)c);
+          rloc = loc;
+          rv = true;
+        }
+        if (c > TILE / 4) atomicExch(&s_hot_next, d);  // predicts the next unit's hot digit
+      }
+    }
+    // the output tile is free once the writer finished unit i-1
+    if (i >= 1) mbar_wait(&s_oempty, (i - 1) & 1);
+    asm volatile("barrier.sync 1, %0;" ::"r"(WS_CT) : "memory");
+    if (threadIdx.x == 0) {
+      s_hot = s_hot_next;
+      s_hot_next = 0xffffffffu;
+    }
+    // ---- shuffle the stage into digit order ---------------------------------------------------
+    if (MODE == 1) {
+      #pragma unroll
+      for (int j0 = 0; j0 < CIT; j0 += VEC) {
+        const uint32_t e0 = elem(j0);
+        if (full || e0 < ulen) {
+          const uint4 kv = *reinterpret_cast<const uint4*>(s_k + e0);
+          const uint4 pv = *reinterpret_cast<const uint4*>(s_p + e0);
+          const K* ke = reinterpret_cast<const K*>(&kv);
+          const K* pe = reinterpret_cast<const K*>(&pv);
+          #pragma unroll
+          for (int v = 0; v < VEC; ++v) {
+            const int j = j0 + v;
+            if (full || e0 + v < ulen)
+              s_out[s_loc[digit(ke[v])] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = TT::make(ke[v], pe[v]);
+          }
+        }
+      }
+    } else {
+      #pragma unroll
+      for (int j = 0; j < CIT; ++j) {
+        const uint32_t e = elem(j);
+        if (full || e < ulen) {
+          const T t = s_t[e];
+          s_out[s_loc[digit(TT::key(t))] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = t;
+        }
+      }
+    }
+    if (rv) gd[threadIdx.x] = rres - rloc;
+    __syncwarp();
+    if (lane == 0) {
+      mbar_arrive(&s_empty[stage]);  // the stage may be refilled (unit i+2)
+      mbar_arrive(&s_ofull);         // unit i is in the output tile
+    }
+  }
+}
+
+}  // namespace hj
