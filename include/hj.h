@@ -101,9 +101,11 @@ enum hj_option {
   HJ_OPT_STREAM_CHUNK = 8,  /* hj_join_host: S tuples per streamed chunk (0 = auto = |S|/16, at
                                least 2^22; >= |S| = copy everything, then join)                   */
   HJ_OPT_PASS_WS = 21,      /* partition passes (histogram partitioner, fan-out <= 2^9): 1 (default) =
-                               warp-specialized pipeline (TMA-fed input stages, compute warps that
-                               rank and shuffle, writer warps that stream the previous tile out);
-                               0 = every warp of the block in lock step (round-1 kernel)           */
+                               warp-specialized pipeline (a producer warp feeding three TMA stages,
+                               compute warps that rank and shuffle each stage in place, writer warps
+                               that stream the previous stage out), 20 compute warps; 18/20/22 =
+                               that many compute warps (tuning); 0 = every warp of the block in lock
+                               step (round-1 kernel)                                                */
   HJ_OPT_MAT_CHECKSUM = 20  /* 1 (default) = MATERIALIZE also fills res->checksum (the pairs'
                                signatures are summed by the probe, so every materialized result is
                                self-checking); 0 = checksum left 0 in MATERIALIZE (measurement)   */

@@ -247,12 +247,19 @@ int pass_threads(const Ctx* c, int fanout_bits, int items) {
 // the warp-specialized pass (hj_pass_ws.cuh) for a fan-out of 2^bits: histogram partitioner,
 // fan-out <= WS_MAXF (shared-memory budget); its unit is a 64 KB tile
 bool use_ws(const Ctx* c, int bits) { return c->opt_pass_ws && c->opt_partitioner == 0 && (1 << bits) <= WS_MAXF; }
-// role split: HJ_OPT_PASS_WS = 1 / 2 / 3 -> 16 / 20 / 24 compute warps
-int ws_cw(const Ctx* c) { return c->opt_pass_ws == 3 ? 24 : c->opt_pass_ws == 2 ? 20 : 16; }
+// role split: HJ_OPT_PASS_WS = 1 (default: 20 compute warps; measured on B200, c3 pass 1 / pass 2:
+// 16 warps x 16 tuples 1.01 / 0.97 ms (spills), 18: 0.82 / 0.87, 20: 0.80 / 0.82, 21: 0.81 / 0.83,
+// 22: 0.84 / 0.85, 24 x 8 tuples: 0.93 / 0.93; the lock-step k_pass: 0.94 / 0.85) or an explicit
+// number of compute warps among WS_CWS
+#define WS_CWS(X) X(18) X(20) X(22)
+int ws_cw(const Ctx* c) { return c->opt_pass_ws == 1 ? 20 : (int)c->opt_pass_ws; }
 uint32_t ws_tile(const Ctx* c) {
   const int cw = ws_cw(c);
-  if (c->key_bytes == 4) return cw == 24 ? WsShape<uint32_t, 24>::TILE : cw == 20 ? WsShape<uint32_t, 20>::TILE : WsShape<uint32_t, 16>::TILE;
-  return cw == 24 ? WsShape<uint64_t, 24>::TILE : cw == 20 ? WsShape<uint64_t, 20>::TILE : WsShape<uint64_t, 16>::TILE;
+#define WS_TILE_CASE(N) \
+  if (cw == N) return c->key_bytes == 4 ? WsShape<uint32_t, N>::TILE : WsShape<uint64_t, N>::TILE;
+  WS_CWS(WS_TILE_CASE)
+#undef WS_TILE_CASE
+  return 0;
 }
 
 int choose_bits(unsigned long long nR) {
@@ -351,15 +358,12 @@ void attr_join(F&& attr) {
 
 template <typename K, typename F>
 void for_ws_variants(F&& attr) {
-  attr((const void*)k_pass_ws<K, 1, false, 16>);
-  attr((const void*)k_pass_ws<K, 1, true, 16>);
-  attr((const void*)k_pass_ws<K, 2, false, 16>);
-  attr((const void*)k_pass_ws<K, 1, false, 20>);
-  attr((const void*)k_pass_ws<K, 1, true, 20>);
-  attr((const void*)k_pass_ws<K, 2, false, 20>);
-  attr((const void*)k_pass_ws<K, 1, false, 24>);
-  attr((const void*)k_pass_ws<K, 1, true, 24>);
-  attr((const void*)k_pass_ws<K, 2, false, 24>);
+#define WS_ATTR_CASE(N)                                 \
+  attr((const void*)k_pass_ws<K, 1, false, N>);        \
+  attr((const void*)k_pass_ws<K, 1, true, N>);         \
+  attr((const void*)k_pass_ws<K, 2, false, N>);
+  WS_CWS(WS_ATTR_CASE)
+#undef WS_ATTR_CASE
 }
 
 template <typename K>
@@ -606,11 +610,10 @@ int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
   constexpr int IT = pass_items<K>();
   if (!BC && use_ws(c, fanout_bits) && (MODE == 1 ? hp.tile : hp.C2) == ws_tile(c)) {
     // warp-specialized pipeline: one 1024-thread block per SM
-    switch (ws_cw(c)) {
-      case 24: return launch_pass_ws<K, MODE, GD, 24>(c, hp, P, fanout_bits);
-      case 20: return launch_pass_ws<K, MODE, GD, 20>(c, hp, P, fanout_bits);
-      default: return launch_pass_ws<K, MODE, GD, 16>(c, hp, P, fanout_bits);
-    }
+#define WS_LAUNCH_CASE(N) \
+    if (ws_cw(c) == N) return launch_pass_ws<K, MODE, GD, N>(c, hp, P, fanout_bits);
+    WS_CWS(WS_LAUNCH_CASE)
+#undef WS_LAUNCH_CASE
   }
   const int mask = c->opt_pass_variant > 0 ? (int)c->opt_pass_variant - 1 : (c->key_bytes == 8 ? 1 : 0);
   if (NT == 1024 && ((mask >> (MODE - 1)) & 1) && (1 << fanout_bits) <= 512) {
@@ -1408,7 +1411,8 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
     case HJ_OPT_STREAM_CHUNK: c->opt_stream_chunk = v; break;
     case HJ_OPT_MAT_CHECKSUM: c->opt_mat_chk = v; break;
     case HJ_OPT_PASS_WS:
-      if (v > 3) return fail(c, HJ_ERR_INVALID, "pass_ws must be 0..3");
+      if (v != 0 && v != 1 && v != 18 && v != 20 && v != 22)
+        return fail(c, HJ_ERR_INVALID, "pass_ws must be 0 (off), 1 (auto) or 18/20/22 compute warps");
       c->opt_pass_ws = v;
       break;
     case HJ_OPT_PASS_L2PF: c->opt_pass_l2pf = v; break;

@@ -8,37 +8,40 @@
 // runs rank | write-out of the previous unit | shuffle with every warp of the block in lock step,
 // so each SM's HBM traffic comes in bursts between block barriers (c3 pass 1: 0.95 ms, against
 // 0.68 ms for the same access pattern with no shared-memory work, tools/microbench/mb_scatter.cu).
-// Here one 1024-thread block per SM is three roles joined by mbarriers:
-//   producer (warp 31)   : unit descriptors, and each unit's input copied into one of two
-//                          shared-memory stages by TMA bulk copies (cp.async.bulk, no registers:
-//                          two units of input in flight per SM)
-//   compute  (warps 0-15): rank the stage's keys (shared atomics), scan + reserve (one global
-//                          atomic per digit run), shuffle the stage into the output tile
-//   writer   (warps 16-30): output tile -> HBM, a run per consecutive group of threads
-// so the writer streams unit i-1 while the compute warps rank unit i and TMA fetches unit i+1.
-// Shared memory: 2 input stages + 1 output tile (64 KB each) + run tables: fan-out <= 512.
-// A unit stays in its stage until it is shuffled (only the ranks live in registers). Units whose
-// input is ragged or not 16-byte aligned (the last unit of a relation, a piece whose aligned
-// superset would leave the pass-1 data) are copied into the stage by the compute warps.
+// Here one 1024-thread block per SM is three roles joined by mbarriers, over a ring of three
+// shared-memory stages of one unit (tile) each:
+//   producer (warp 31)    : unit descriptors; each unit's input copied into the next free stage
+//                           by TMA bulk copies (cp.async.bulk: no registers, up to two units of
+//                           input in flight per SM)
+//   compute  (CW warps)   : stage -> registers, rank (shared atomics), scan + reserve (one global
+//                           atomic per digit run), shuffle the registers back into the SAME stage
+//                           in digit order (every read of the stage precedes a compute barrier)
+//   writer   (31-CW warps): stage -> HBM in order, so consecutive threads write consecutive
+//                           addresses of a run; then the stage is free for the producer
+// so while the compute warps rank unit i, the writer streams unit i-1 and TMA fetches unit i+1:
+// no role waits on another's shared-memory buffer except through the three-stage ring.
+// Units whose input is ragged or not 16-byte aligned (the last unit of a relation, a piece whose
+// aligned superset would leave the pass-1 data) are loaded by the compute warps from global.
 #pragma once
 #include "hj_common.cuh"
 #include "hj_plan.cuh"
 
 namespace hj {
 
-constexpr int WS_NT = 1024;       // compute warps + writer warps + producer warp 31
-constexpr int WS_MAXF = 512;      // fan-out bound (shared-memory budget)
+constexpr int WS_NT = 1024;   // compute warps + writer warps + producer warp 31
+constexpr int WS_MAXF = 512;  // fan-out bound (shared-memory budget)
+constexpr int WS_NS = 3;      // stages
 
-// Role split (HJ_OPT_PASS_WS = 1 + variant): CW compute warps, 31 - CW writer warps; each compute
-// thread ranks CIT tuples of a unit, so a unit (tile) has CW * 32 * CIT tuples.
+// Role split (HJ_OPT_PASS_WS): CW compute warps, 31 - CW writer warps; each compute thread ranks
+// CIT tuples of a unit, so a unit (tile) has CW * 32 * CIT tuples (60 KB at CW = 20, the default).
 template <typename K, int CW>
 struct WsShape {
   static constexpr int CT = CW * 32, WT = (31 - CW) * 32;
-  static constexpr int CIT = sizeof(K) == 4 ? (CW == 16 ? 16 : CW == 20 ? 12 : 8) : (CW == 16 ? 8 : CW == 20 ? 6 : 4);
+  static constexpr int CIT = sizeof(K) == 4 ? (CW <= 16 ? 16 : CW <= 23 ? 12 : 8) : (CW <= 16 ? 8 : CW <= 23 ? 6 : 4);
   static constexpr int TILE = CT * CIT;
   static constexpr uint32_t STAGE = (uint32_t)TILE * 2 * sizeof(K) + 16;  // +16: aligned superset of AoS units
-  static constexpr size_t smem(int fanout_bits) {  // 2 stages + output tile + s_gd (3F) + s_cnt + s_loc
-    return 2 * (size_t)STAGE + (size_t)TILE * 2 * sizeof(K) + ((size_t)1 << fanout_bits) * 32 + 16;
+  static constexpr size_t smem(int fanout_bits) {  // stages + s_gd (3F u64) + s_cnt (F + 4) + s_loc (F)
+    return WS_NS * (size_t)STAGE + ((size_t)1 << fanout_bits) * 32 + 16;
   }
 };
 
@@ -62,20 +65,18 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
   using TT = Tup<K>;
   using T = typename TT::T;
   using S = WsShape<K, CW>;
-  constexpr int WS_CT = S::CT, WS_WT = S::WT, CIT = S::CIT, TILE = S::TILE;
-  constexpr uint32_t WS_STAGE = S::STAGE;
+  constexpr int CT = S::CT, WT = S::WT, CIT = S::CIT, TILE = S::TILE;
+  constexpr uint32_t STAGE = S::STAGE;
   constexpr int VEC = 16 / sizeof(K);
   static_assert(CIT % VEC == 0 && CIT % 2 == 0 && TILE < 65536, "tile shape");
   extern __shared__ __align__(128) unsigned char s_raw[];
-  unsigned char* s_in = s_raw;                                    // 2 x WS_STAGE
-  T* s_out = reinterpret_cast<T*>(s_raw + 2 * WS_STAGE);          // TILE tuples
   const uint32_t F = 1u << fanout_bits;
-  unsigned long long* s_gd = reinterpret_cast<unsigned long long*>(s_out + TILE);  // 3 x F: run base - loc
-  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gd + 3 * F);    // F + 1 (spare for ragged lanes)
-  uint32_t* s_loc = s_cnt + F + 4;                                // F
-  __shared__ __align__(8) unsigned long long s_full[2], s_empty[2], s_ofull, s_oempty;
+  unsigned long long* s_gd = reinterpret_cast<unsigned long long*>(s_raw + WS_NS * STAGE);  // 3 x F: run base - loc
+  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gd + 3 * F);  // F + 1 (spare for ragged lanes)
+  uint32_t* s_loc = s_cnt + F + 4;                              // F
+  __shared__ __align__(8) unsigned long long s_full[WS_NS], s_empty[WS_NS], s_done[WS_NS];
   __shared__ WsUnit s_desc[4];
-  __shared__ uint32_t s_wt[WS_CT / 32];
+  __shared__ uint32_t s_wt[CT / 32];
   __shared__ uint32_t s_hot, s_hot_next;
   __shared__ uint32_t s_cst[MODE == 2 ? 2 * 1025 : 1];
 
@@ -106,12 +107,11 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
   if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
   if (threadIdx.x == 0) {
     s_hot = s_hot_next = 0xffffffffu;
-    mbar_init(&s_full[0], 1);
-    mbar_init(&s_full[1], 1);
-    mbar_init(&s_empty[0], WS_CT / 32);
-    mbar_init(&s_empty[1], WS_CT / 32);
-    mbar_init(&s_ofull, WS_CT / 32);
-    mbar_init(&s_oempty, WS_WT / 32);
+    for (int s = 0; s < WS_NS; ++s) {
+      mbar_init(&s_full[s], 1);         // producer (+ TMA bytes)
+      mbar_init(&s_done[s], CT / 32);   // compute warps: the stage holds the shuffled unit
+      mbar_init(&s_empty[s], WT / 32);  // writer warps: the stage is written out
+    }
     fence_mbar_init();
   }
   __syncthreads();
@@ -120,9 +120,11 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
   if (warp == 31) {
     // ---------------------------------------------------------------- producer ----------------
     if (lane != 0) return;
+    const unsigned long long pend[2] = {MODE == 2 ? P.rel[0].pst[P.npieces()] : 0ull,
+                                        MODE == 2 ? P.rel[1].pst[P.npieces()] : 0ull};
     for (uint32_t i = 0;; ++i) {
-      const uint32_t stage = i & 1;
-      if (i >= 2) mbar_wait(&s_empty[stage], ((i >> 1) - 1) & 1);  // compute consumed unit i-2
+      const uint32_t stage = i % WS_NS;
+      if (i >= WS_NS) mbar_wait(&s_empty[stage], ((i / WS_NS) - 1) & 1);  // unit i-3 written out
       const unsigned long long u = blockIdx.x + (unsigned long long)i * G;
       WsUnit D;
       D.valid = u < units;
@@ -159,15 +161,14 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
           // the 16-byte aligned superset must stay inside the relation's pass-1 data
           const uintptr_t a = reinterpret_cast<uintptr_t>(D.src_k), a0 = a & ~(uintptr_t)15;
           const uintptr_t a1 = (a + (uintptr_t)D.len * sizeof(T) + 15) & ~(uintptr_t)15;
-          const uintptr_t end = reinterpret_cast<uintptr_t>((const T*)R.t1 + R.pst[P.npieces()]);
-          D.tma = a1 <= end;
+          D.tma = a1 <= reinterpret_cast<uintptr_t>((const T*)R.t1 + pend[r]);
           D.shift = (uint32_t)((a - a0) / sizeof(T));
         }
       }
       s_desc[i & 3] = D;
-      unsigned char* st = s_in + stage * WS_STAGE;
+      unsigned char* st = s_raw + stage * STAGE;
       if (D.valid && D.tma) {
-        fence_proxy_async();  // the compute warps' reads of this stage (unit i-2) precede the copy
+        fence_proxy_async();  // earlier generic-proxy accesses of this stage precede the copy
         if (MODE == 1) {
           const uint32_t b = TILE * (uint32_t)sizeof(K);
           mbar_arrive_expect_tx(&s_full[stage], 2 * b);
@@ -186,73 +187,87 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
     }
   }
 
-  if (warp >= WS_CT / 32) {
+  if (warp >= CT / 32) {
     // ---------------------------------------------------------------- writer ------------------
-    const uint32_t wt = threadIdx.x - WS_CT;
+    const uint32_t wt = threadIdx.x - CT;
     for (uint32_t i = 0;; ++i) {
-      mbar_wait(&s_ofull, i & 1);  // the compute warps shuffled unit i (or reached the end)
+      const uint32_t stage = i % WS_NS;
+      mbar_wait(&s_done[stage], (i / WS_NS) & 1);  // the compute warps shuffled unit i (or ended)
       const WsUnit& D = s_desc[i & 3];
       if (!D.valid) return;
       T* dst = (T*)D.dst;
       const uint32_t len = D.len;
+      const T* s_t = reinterpret_cast<const T*>(s_raw + stage * STAGE);
       const unsigned long long* gd = s_gd + (i % 3) * F;
       #pragma unroll 4
-      for (uint32_t e = wt; e < len; e += WS_WT) {
-        const T t = s_out[e];
+      for (uint32_t e = wt; e < len; e += WT) {
+        const T t = s_t[e];
         __stcs(dst + (gd[digit(TT::key(t))] + e), t);
       }
       __syncwarp();
-      if (lane == 0) mbar_arrive(&s_oempty);
+      if (lane == 0) mbar_arrive(&s_empty[stage]);
     }
   }
 
   // ------------------------------------------------------------------ compute -----------------
-  // The unit stays in its input stage until the shuffle (keys are read there for the ranks, and
-  // key + payload again for the shuffle): only the ranks live in registers across the barriers.
   const uint32_t nscan = F < 32 ? 32u : F;  // threads in the digit scan (whole warps)
-  // element e of the unit in the stage held by thread (j, v): MODE 1 (j * CT + tid) * VEC + v
-  // (128-bit loads of VEC keys / payloads), MODE 2 j * CT + tid
+  // element e of the unit held by thread (j, v): MODE 1 (j * CT + tid) * VEC + v (128-bit loads of
+  // VEC keys / payloads), MODE 2 j * CT + tid
   auto elem = [&](int j) -> uint32_t {
-    return MODE == 1 ? (uint32_t)((j / VEC) * WS_CT + threadIdx.x) * VEC + (j % VEC) : (uint32_t)(j * WS_CT + threadIdx.x);
+    return MODE == 1 ? (uint32_t)((j / VEC) * CT + threadIdx.x) * VEC + (j % VEC) : (uint32_t)(j * CT + threadIdx.x);
   };
   for (uint32_t i = 0;; ++i) {
-    const uint32_t stage = i & 1;
-    mbar_wait(&s_full[stage], (i >> 1) & 1);
+    const uint32_t stage = i % WS_NS;
+    mbar_wait(&s_full[stage], (i / WS_NS) & 1);
     const WsUnit D = s_desc[i & 3];
     if (!D.valid) {
-      if (i >= 1) mbar_wait(&s_oempty, (i - 1) & 1);  // the writer finished the last unit
       __syncwarp();
-      if (lane == 0) mbar_arrive(&s_ofull);  // end marker for the writer
+      if (lane == 0) mbar_arrive(&s_done[stage]);  // end marker for the writer
       break;
     }
     const uint32_t ulen = D.len;
     const bool full = ulen == TILE;
-    unsigned char* st = s_in + stage * WS_STAGE;
-    const K* s_k = reinterpret_cast<const K*>(st);                   // MODE 1: keys
-    const K* s_p = reinterpret_cast<const K*>(st + TILE * sizeof(K));  //         payloads
-    const T* s_t = reinterpret_cast<const T*>(st) + D.shift;         // MODE 2: tuples
-    if (!D.tma) {  // ragged / unaligned unit: the compute warps copy it into the stage
-      for (uint32_t e = threadIdx.x; e < ulen; e += WS_CT) {
-        if (MODE == 1) {
-          const_cast<K*>(s_k)[e] = ((const K*)D.src_k)[e];
-          const_cast<K*>(s_p)[e] = ((const K*)D.src_p)[e];
-        } else {
-          const_cast<T*>(s_t)[e] = __ldcs((const T*)D.src_k + e);
+    unsigned char* st = s_raw + stage * STAGE;
+    K kk[CIT], pp[CIT];
+    if (D.tma) {
+      if (MODE == 1) {
+        #pragma unroll
+        for (int j = 0; j < CIT / VEC; ++j) {
+          const uint4 kv = reinterpret_cast<const uint4*>(st)[j * CT + threadIdx.x];
+          const uint4 pv = reinterpret_cast<const uint4*>(st + TILE * sizeof(K))[j * CT + threadIdx.x];
+          const K* ke = reinterpret_cast<const K*>(&kv);
+          const K* pe = reinterpret_cast<const K*>(&pv);
+          #pragma unroll
+          for (int v = 0; v < VEC; ++v) {
+            kk[j * VEC + v] = ke[v];
+            pp[j * VEC + v] = pe[v];
+          }
+        }
+      } else {
+        const T* src = reinterpret_cast<const T*>(st) + D.shift;
+        #pragma unroll
+        for (int j = 0; j < CIT; ++j) {
+          if (full || elem(j) < ulen) {
+            const T t = src[elem(j)];
+            kk[j] = TT::key(t);
+            pp[j] = TT::pay(t);
+          }
         }
       }
-      asm volatile("barrier.sync 1, %0;" ::"r"(WS_CT) : "memory");
-    }
-    // this thread's CIT keys (MODE 1: 128-bit loads of VEC consecutive keys, conflict-free)
-    K kk[CIT];
-    #pragma unroll
-    for (int j0 = 0; j0 < CIT; j0 += (MODE == 1 ? VEC : 1)) {
-      if (MODE == 1) {
-        const uint4 kv = *reinterpret_cast<const uint4*>(s_k + elem(j0));
-        const K* ke = reinterpret_cast<const K*>(&kv);
-        #pragma unroll
-        for (int v = 0; v < VEC; ++v) kk[j0 + v] = ke[v];
-      } else {
-        kk[j0] = TT::key(s_t[elem(j0)]);
+    } else {
+      #pragma unroll
+      for (int j = 0; j < CIT; ++j) {
+        const uint32_t e = elem(j);
+        if (e < ulen) {
+          if (MODE == 1) {
+            kk[j] = ((const K*)D.src_k)[e];
+            pp[j] = ((const K*)D.src_p)[e];
+          } else {
+            const T t = __ldcs((const T*)D.src_k + e);
+            kk[j] = TT::key(t);
+            pp[j] = TT::pay(t);
+          }
+        }
       }
     }
 
@@ -288,12 +303,12 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
           if ((hbits >> j) & 1) rk[j / 2] += base << (16 * (j & 1));
       }
     }
-    asm volatile("barrier.sync 1, %0;" ::"r"(WS_CT) : "memory");
+    asm volatile("barrier.sync 1, %0;" ::"r"(CT) : "memory");  // every read of the stage is done
 
     // ---- scan + reserve (threads < F) ---------------------------------------------------------
-    unsigned long long* gd = s_gd + (i % 3) * F;
     // each run's reservation atomic is issued here and its result stored after the shuffle, so
-    // the global atomic's round trip overlaps the shuffle (the writer reads gd after s_ofull)
+    // the global atomic's round trip overlaps the shuffle (the writer reads gd after s_done)
+    unsigned long long* gd = s_gd + (i % 3) * F;
     unsigned long long rres = 0;
     uint32_t rloc = 0;
     bool rv = false;
@@ -322,47 +337,20 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
         if (c > TILE / 4) atomicExch(&s_hot_next, d);  // predicts the next unit's hot digit
       }
     }
-    // the output tile is free once the writer finished unit i-1
-    if (i >= 1) mbar_wait(&s_oempty, (i - 1) & 1);
-    asm volatile("barrier.sync 1, %0;" ::"r"(WS_CT) : "memory");
+    asm volatile("barrier.sync 1, %0;" ::"r"(CT) : "memory");
     if (threadIdx.x == 0) {
       s_hot = s_hot_next;
       s_hot_next = 0xffffffffu;
     }
-    // ---- shuffle the stage into digit order ---------------------------------------------------
-    if (MODE == 1) {
-      #pragma unroll
-      for (int j0 = 0; j0 < CIT; j0 += VEC) {
-        const uint32_t e0 = elem(j0);
-        if (full || e0 < ulen) {
-          const uint4 kv = *reinterpret_cast<const uint4*>(s_k + e0);
-          const uint4 pv = *reinterpret_cast<const uint4*>(s_p + e0);
-          const K* ke = reinterpret_cast<const K*>(&kv);
-          const K* pe = reinterpret_cast<const K*>(&pv);
-          #pragma unroll
-          for (int v = 0; v < VEC; ++v) {
-            const int j = j0 + v;
-            if (full || e0 + v < ulen)
-              s_out[s_loc[digit(ke[v])] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = TT::make(ke[v], pe[v]);
-          }
-        }
-      }
-    } else {
-      #pragma unroll
-      for (int j = 0; j < CIT; ++j) {
-        const uint32_t e = elem(j);
-        if (full || e < ulen) {
-          const T t = s_t[e];
-          s_out[s_loc[digit(TT::key(t))] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = t;
-        }
-      }
-    }
+    // ---- shuffle the registers back into the stage, in digit order ---------------------------
+    T* s_t = reinterpret_cast<T*>(st);
+    #pragma unroll
+    for (int j = 0; j < CIT; ++j)
+      if (full || elem(j) < ulen)
+        s_t[s_loc[digit(kk[j])] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = TT::make(kk[j], pp[j]);
     if (rv) gd[threadIdx.x] = rres - rloc;
     __syncwarp();
-    if (lane == 0) {
-      mbar_arrive(&s_empty[stage]);  // the stage may be refilled (unit i+2)
-      mbar_arrive(&s_ofull);         // unit i is in the output tile
-    }
+    if (lane == 0) mbar_arrive(&s_done[stage]);  // unit i is ready for the writer
   }
 }
 
