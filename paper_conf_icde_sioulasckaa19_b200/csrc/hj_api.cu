@@ -354,6 +354,10 @@ void attr_join(F&& attr) {
   constexpr JoinShape S = JOIN_SHAPES[V];
   attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf>);
   attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf>);
+  if constexpr (sizeof(K) == 4) {
+    attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, true>);
+    attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, true>);
+  }
 }
 
 template <typename K, typename F>
@@ -666,17 +670,24 @@ int launch_pass2(Ctx* c, const HostPlan& hp, const Plan& P) {
   return HJ_OK;
 }
 
-template <typename K, int V>
-int launch_join_v(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
+template <typename K, int V, bool F2>
+int launch_join_f(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   constexpr JoinShape S = JOIN_SHAPES[V];
   cudaStream_t st = c->stream;
-  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf>
-                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf>;
+  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2>
+                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2>;
   int g = grid_for(c, f, S.nt + 32, hp.join_smem, 1ull << 40);
-  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
-  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2><<<g, S.nt + 32, hp.join_smem, st>>>(P);
   CUDA_TRY(c, cudaGetLastError());
   return HJ_OK;
+}
+
+// the two-term slot hash (slot_of2) when it still covers every key bit above the radix field
+template <typename K, int V>
+int launch_join_v(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
+  if (sizeof(K) == 4 && P.H.nfold <= 1) return launch_join_f<K, V, sizeof(K) == 4>(c, hp, P, mat);
+  return launch_join_f<K, V, false>(c, hp, P, mat);
 }
 
 template <typename K>

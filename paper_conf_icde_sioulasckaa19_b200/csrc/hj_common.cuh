@@ -60,6 +60,17 @@ __device__ __forceinline__ uint32_t slot_fold(uint32_t h, const SlotHash& H) {
   return r & ((1u << H.lg) - 1);
 }
 __device__ __forceinline__ uint32_t slot_of(uint32_t key, const SlotHash& H) { return slot_fold(key >> H.B, H); }
+// two-term fold, used when the key bits above B fit in 2 lg bits (H.nfold <= 1, e.g. every 4-byte
+// config of BASELINE.json): 3 instructions instead of 6 per lookup
+__device__ __forceinline__ uint32_t slot_of2(uint32_t key, const SlotHash& H) {
+  const uint32_t h = key >> H.B;
+  return (h ^ (h >> H.lg)) & ((1u << H.lg) - 1);
+}
+template <bool F2, typename K>
+__device__ __forceinline__ uint32_t slot_for(K key, const SlotHash& H) {
+  if constexpr (F2 && sizeof(K) == 4) return slot_of2((uint32_t)key, H);
+  else return slot_of(key, H);
+}
 __device__ __forceinline__ uint32_t slot_of(uint64_t key, const SlotHash& H) {
   const uint64_t h64 = key >> H.B;
   return slot_fold((uint32_t)h64 ^ ((uint32_t)(h64 >> 32) * 0x9E3779B1u), H);

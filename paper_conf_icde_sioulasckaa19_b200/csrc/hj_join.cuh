@@ -147,8 +147,9 @@ __device__ __forceinline__ uint32_t exch16(unsigned short* a, uint32_t v) {
 // compute thread issues a TMA L2 prefetch of rounds 1..SPF, then at round k of rounds k+SPF (one
 // cp.async.bulk.prefetch.L2 of NT*SPT tuples per round), so the bytes in flight per SM no longer
 // depend on the registers of the probing threads.
+// F2: two-term slot hash (slot_of2; the host picks it when the key bits above B fit in 2 lg bits)
 template <typename K, int NT, int SPT, bool MAT, int RBUF, bool H16 = false, bool PF = false, bool L2PF = false,
-          int SPF = 0>
+          int SPF = 0, bool F2 = false>
 __device__ __forceinline__ void join_body(const Plan& P) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -234,8 +235,8 @@ __device__ __forceinline__ void join_body(const Plan& P) {
     // ---- build (a6): wait-free push-front insert (Listing 2) ----------------------
     for (uint32_t i = threadIdx.x; i < job.nr; i += NT) {
       const K k = TT::key(lds_tuple(s_rt_sh + i * (uint32_t)sizeof(T), (T*)nullptr));
-      s_next[i] = H16 ? (uint16_t)exch16(reinterpret_cast<unsigned short*>(&s_head[slot_of(k, H)]), i)
-                      : (uint16_t)atomicExch(reinterpret_cast<uint32_t*>(&s_head[slot_of(k, H)]), i);
+      s_next[i] = H16 ? (uint16_t)exch16(reinterpret_cast<unsigned short*>(&s_head[slot_for<F2>(k, H)]), i)
+                      : (uint16_t)atomicExch(reinterpret_cast<uint32_t*>(&s_head[slot_for<F2>(k, H)]), i);
     }
     bar_compute(NT);
 
@@ -265,13 +266,19 @@ __device__ __forceinline__ void join_body(const Plan& P) {
       }
       uint32_t idx[SPT], m[SPT];
       K rfirst[SPT];
-      // this round's tuples in the item (32-bit: rounds hold NT * SPT tuples)
+      // this round's tuples in the item (32-bit: rounds hold NT * SPT tuples); a full round needs
+      // no per-tuple bounds (block-uniform branch)
       const uint32_t rem = (uint32_t)min(job.se - base, (unsigned long long)NT * SPT);
-      #pragma unroll
-      for (int j = 0; j < SPT; ++j) {
-        idx[j] = ((uint32_t)(j * NT) + threadIdx.x < rem) ? s_head[slot_of(sk[j], H)] : NIL16;
-        m[j] = 0;
+      if (rem == NT * SPT) {
+        #pragma unroll
+        for (int j = 0; j < SPT; ++j) idx[j] = s_head[slot_for<F2>(sk[j], H)];
+      } else {
+        #pragma unroll
+        for (int j = 0; j < SPT; ++j)
+          idx[j] = ((uint32_t)(j * NT) + threadIdx.x < rem) ? s_head[slot_for<F2>(sk[j], H)] : NIL16;
       }
+      #pragma unroll
+      for (int j = 0; j < SPT; ++j) m[j] = 0;
       // first chain step of every tuple without branches (unique build keys: chains of length
       // <= 1, so this is usually the whole probe): the head's tuple is read even for an empty
       // slot (index 0 instead, discarded), the signature is computed for every tuple and added
@@ -288,7 +295,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
         if (MAT) rfirst[j] = TT::pay(r);
         if (!MAT || chk) {
           const uint64_t sg = pair_sig((uint64_t)TT::pay(r), (uint64_t)sp[j]);
-          my_chk += hit ? sg : 0ull;
+          if (hit) my_chk += sg;  // predicated add (no selects)
         }
         m[j] = hit ? 1u : 0u;
         idx[j] = v ? (uint32_t)s_next[i0] : NIL16;
@@ -330,7 +337,12 @@ __device__ __forceinline__ void join_body(const Plan& P) {
           s_base = tot ? atomicAdd(&P.results[RES_CURSOR], (unsigned long long)tot) : 0ull;
         }
         bar_compute(NT);
-        unsigned long long pos0 = s_base + s_wsum[warp];
+        // positions relative to this round's block base: 32-bit (a round emits < 2^32 pairs)
+        const unsigned long long rbase = s_base;
+        K* const o_r = out_r + rbase;
+        K* const o_s = out_s + rbase;
+        const uint32_t room = rbase >= P.out_cap ? 0u : (uint32_t)min(P.out_cap - rbase, 0xffffffffull);
+        uint32_t pos0 = s_wsum[warp];
         #pragma unroll
         for (int j = 0; j < SPT; ++j) {
           // warp-exclusive scan of m[j]; the common case (every m <= 1) is one ballot
@@ -349,20 +361,20 @@ __device__ __forceinline__ void join_body(const Plan& P) {
             excl = x - m[j];
             wtot = __shfl_sync(0xffffffffu, x, 31);
           }
-          unsigned long long pos = pos0 + excl;
+          uint32_t pos = pos0 + excl;
           pos0 += wtot;
           if (m[j] == 1) {
-            if (pos < P.out_cap) {
-              out_r[pos] = rfirst[j];
-              out_s[pos] = sp[j];
+            if (pos < room) {
+              o_r[pos] = rfirst[j];
+              o_s[pos] = sp[j];
             }
           } else if (m[j] > 1) {
-            for (uint32_t i = s_head[slot_of(sk[j], H)]; i != NIL16; i = s_next[i]) {
+            for (uint32_t i = s_head[slot_for<F2>(sk[j], H)]; i != NIL16; i = s_next[i]) {
               const T r = s_rt[i];
               if (TT::key(r) == sk[j]) {
-                if (pos < P.out_cap) {
-                  out_r[pos] = TT::pay(r);
-                  out_s[pos] = sp[j];
+                if (pos < room) {
+                  o_r[pos] = TT::pay(r);
+                  o_s[pos] = sp[j];
                 }
                 ++pos;
               }
@@ -400,9 +412,9 @@ __device__ __forceinline__ void join_body(const Plan& P) {
 }
 
 template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false, bool PF = false,
-          bool L2PF = false, int SPF = 0>
+          bool L2PF = false, int SPF = 0, bool F2 = false>
 __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
-  join_body<K, NT, SPT, MAT, RBUF, H16, PF, L2PF, SPF>(P);
+  join_body<K, NT, SPT, MAT, RBUF, H16, PF, L2PF, SPF, F2>(P);
 }
 
 }  // namespace hj
