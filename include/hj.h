@@ -207,26 +207,33 @@ int hj_partition(hj_ctx* ctx, const void* keys, const void* pays, uint64_t n, in
 /* ---- multi-GPU exchange; the caller runs the collectives in between ------
  * Co-partitions are independent, so G = 2^gpu_bits ranks each own the co-partitions
  * whose radix field is extended by gpu_bits on top: rank j = (key >> local_bits) & (G - 1).
+ * The local field splits into b1 = min(ceil(local_bits / 2), 10 - gpu_bits) pass-1 bits and
+ * local_bits - b1 pass-2 bits (<= 10), the same on sender and receiver.
+ *
+ * Count rows: a sender counts only its pass-1 pieces, (destination rank, d1) = 2^(gpu_bits + b1)
+ * <= 2^10 shared-memory bins, whatever local_bits is; row j (2^b1 uint32, hj_exchange_row_len)
+ * = the tuples of each pass-1 digit d1 sent to rank j. A receiver counts its own 2^local_bits
+ * co-partitions of what it received (after the exchange the keys are dense per bin; c5 at G = 8
+ * would otherwise need 2^19 sender bins in global memory) and checks the rows against it.
  *
  * hj_exchange_pack: rows a1-a3 on this rank's `n` SoA tuples of relation `rel` (0 = R, 1 = S),
  * with the pass-1 digit widened by the rank bits, so the send buffer is grouped by destination
  * rank and, inside each rank's segment, by the local pass-1 digit d1.
  *   *send_out:   device, n AoS tuples (layout as hj_partition), ctx-owned until the next pack of
  *                the same rel; rank j's segment starts at sum_{i<j} dest_counts[i].
- *   *counts_out: device, [G][2^local_bits] uint32 per-co-partition counts (q-order, see the
- *                implementation notes in DESIGN.md §7); row j goes to rank j. ctx-owned.
- *   dest_counts: HOST array of G uint64 (caller-allocated): tuples destined to each rank.
- * The pass-1 digit gets b1 = min(ceil(local_bits / 2), 10 - gpu_bits) local bits (pass 2 the
- * rest, which must stay <= 10), so the fan-out stays <= 2^10 and hj_join_received with
- * nsrc = 2^gpu_bits derives the same split. */
+ *   *counts_out: device, [G][2^b1] uint32 piece counts (row j goes to rank j). ctx-owned.
+ *   dest_counts: HOST array of G uint64 (caller-allocated): tuples destined to each rank. */
 int hj_exchange_pack(hj_ctx* ctx, int rel, const void* keys, const void* pays, uint64_t n, int gpu_bits,
                      int local_bits, const void** send_out, const uint32_t** counts_out, uint64_t* dest_counts);
 
 /* hj_join_received: rows a4-a8 on what this rank received: R_recv / S_recv are device AoS tuples
  * concatenated in source-rank order (each source's segment grouped by d1, as packed), and
- * R_counts / S_counts are device [nsrc][2^local_bits] uint32 count rows (row s = what source s
- * sent, i.e. source s's counts_out row for this rank). Results are this rank's share of the join
- * (sum matches / checksums over ranks mod 2^64; the union of the materialized pairs). */
+ * R_counts / S_counts are device [nsrc][2^b1] uint32 piece-count rows (row s = what source s sent,
+ * i.e. source s's counts_out row for this rank). The rank histograms its own 2^local_bits
+ * co-partitions of the first sum(rows) received tuples; rows that do not match what the buffers
+ * hold (per pass-1 digit), or describe more than nR / nS tuples, fail with HJ_ERR_INVALID and
+ * nothing is written. Results are this rank's share of the join (sum matches / checksums over
+ * ranks mod 2^64; the union of the materialized pairs). */
 int hj_join_received(hj_ctx* ctx, const void* R_recv, uint64_t nR, const uint32_t* R_counts,
                      const void* S_recv, uint64_t nS, const uint32_t* S_counts, int nsrc, int local_bits,
                      int out_mode, hj_result* res);
@@ -251,8 +258,8 @@ int hj_join_received(hj_ctx* ctx, const void* R_recv, uint64_t nR, const uint32_
  *                      rows a4-a8 on what arrived (H = hj_xd_header_bytes(G, local_bits)).
  *
  * Receive window of relation r on rank j (ctx-owned device allocation, exported by IPC):
- *   [0, H)      count rows, [G][2^local_bits] uint32, row s = what source s sent (q-order, as
- *               hj_exchange_pack's counts_out rows)
+ *   [0, H)      piece-count rows, [G][2^b1] uint32, row s = what source s sent per pass-1 digit
+ *               (as hj_exchange_pack's counts_out rows)
  *   [H, ...)    tuples (AoS as hj_partition), source-major: source s's segment starts at
  *               sum_{s' < s} totals[r][s'][j] tuples and is grouped by the local pass-1 digit.
  * Board window (slot 2, HJ_XD_BOARD_BYTES): starts with uint64[HJ_XD_MAX_RANKS] barrier flags,
@@ -275,8 +282,12 @@ int hj_join_received(hj_ctx* ctx, const void* R_recv, uint64_t nR, const uint32_
  *   *grew:       if non-NULL, 1 when the window was (re)allocated (peers must re-open it). */
 int hj_xd_window(hj_ctx* ctx, int slot, uint64_t bytes, void** dptr, void* ipc_handle, int* grew);
 
-/* Bytes of a receive window's count-row header: round_up(G * 2^local_bits * 4, 256). */
+/* Bytes of a receive window's count-row header: round_up(G * hj_exchange_row_len * 4, 256). */
 uint64_t hj_xd_header_bytes(int G, int local_bits);
+
+/* Entries of one exchange count row: 2^b1, b1 = min(ceil(local_bits / 2), 10 - log2 G). 0 for
+ * invalid arguments. */
+uint32_t hj_exchange_row_len(int G, int local_bits);
 
 /* hj_ipc_open: map a peer's window (64-byte handle from its hj_xd_window) into this process on
  * ctx's device (cudaIpcMemLazyEnablePeerAccess); hj_ipc_close unmaps it. A handle exported by

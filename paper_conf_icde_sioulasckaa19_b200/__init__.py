@@ -53,7 +53,8 @@ _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4:
 
 # every symbol include/hj.h declares (checked by tests/test_abi.py)
 EXPORTS = ("hj_create", "hj_destroy", "hj_last_error", "hj_set_stream", "hj_set_option", "hj_join",
-           "hj_workspace_bytes", "hj_set_workspace", "hj_join_host", "hj_partition", "hj_exchange_pack", "hj_join_received", "hj_xd_window",
+           "hj_workspace_bytes", "hj_set_workspace", "hj_join_host", "hj_partition", "hj_exchange_pack",
+           "hj_exchange_row_len", "hj_join_received", "hj_xd_window",
            "hj_xd_header_bytes", "hj_ipc_open", "hj_ipc_close", "hj_xd_count", "hj_xd_store", "hj_xd_barrier",
            "hj_xd_join", "hj_xd_reserve", "hj_version")
 XD_MAX_RANKS = 64
@@ -109,6 +110,8 @@ def _load_lib():
     lib.hj_xd_window.restype = i32
     lib.hj_xd_header_bytes.argtypes = [i32, i32]
     lib.hj_xd_header_bytes.restype = u64
+    lib.hj_exchange_row_len.argtypes = [i32, i32]
+    lib.hj_exchange_row_len.restype = ctypes.c_uint32
     lib.hj_ipc_open.argtypes = [vp, vp, ctypes.POINTER(vp)]
     lib.hj_ipc_open.restype = i32
     lib.hj_ipc_close.argtypes = [vp, vp]
@@ -304,9 +307,10 @@ class Context:
     def exchange_pack(self, rel: int, keys, pays, gpu_bits: int, local_bits: int):
         """Rows a1-a3 with the pass-1 digit widened by `gpu_bits` rank bits (hj_exchange_pack).
         Returns (send, counts, dest): send = int64 tensor view of the AoS send buffer (one word per
-        4/4 tuple, two per 8/8 tuple), counts = int32 tensor [G, 2^local_bits] (row j goes to rank
-        j), dest = numpy uint64 [G] tuples per destination. Views are ctx-owned (valid until the
-        next pack of the same relation)."""
+        4/4 tuple, two per 8/8 tuple), counts = int32 tensor [G, row_len] of piece counts (row j
+        goes to rank j: its tuples per pass-1 digit d1, row_len = exchange_row_len(G, local_bits)),
+        dest = numpy uint64 [G] tuples per destination. Views are ctx-owned (valid until the next
+        pack of the same relation)."""
         import torch
 
         k = _as_device_col(keys, self.key_bytes)
@@ -320,7 +324,8 @@ class Context:
         words = k.numel() * (self.key_bytes + self.pay_bytes) // 8
         send_t = (_wrap_device(send.value, words, 8, k.device) if words
                   else torch.zeros(0, dtype=torch.int64, device=k.device))
-        cnt_t = _wrap_device(cnt.value, G << local_bits, 4, k.device).view(G, 1 << local_bits)
+        rl = exchange_row_len(G, local_bits)
+        cnt_t = _wrap_device(cnt.value, G * rl, 4, k.device).view(G, rl)
         return send_t, cnt_t, np.frombuffer(dest, dtype=np.uint64).copy()
 
     def join_received(self, R_recv, nR: int, R_counts, S_recv, nS: int, S_counts, nsrc: int, local_bits: int,
@@ -385,11 +390,12 @@ class Context:
         return xd_header_bytes(G, local_bits)
 
     def xd_views(self, dptr: int, G: int, local_bits: int, n: int, device):
-        """Torch views of a receive window: (tuples as int64 words, count rows int32 [G, 2^local_bits])."""
+        """Torch views of a receive window: (tuples as int64 words, piece-count rows int32 [G, row_len])."""
         H = xd_header_bytes(G, local_bits)
         words = n * (self.key_bytes + self.pay_bytes) // 8
         recv = _wrap_device(dptr + H, max(words, 1), 8, device)[:words]
-        cnt = _wrap_device(dptr, G << local_bits, 4, device).view(G, 1 << local_bits)
+        rl = exchange_row_len(G, local_bits)
+        cnt = _wrap_device(dptr, G * rl, 4, device).view(G, rl)
         return recv, cnt
 
     def xd_barrier(self, rank: int, flags, timeout_ms: int = 10000):
@@ -444,6 +450,11 @@ class Context:
 
 def xd_header_bytes(G: int, local_bits: int) -> int:
     return int(_lib.hj_xd_header_bytes(G, local_bits))
+
+
+def exchange_row_len(G: int, local_bits: int) -> int:
+    """Entries per count row of the exchange: 2^b1, the pass-1 digits of one destination."""
+    return int(_lib.hj_exchange_row_len(G, local_bits))
 
 
 def _result(res: _Result) -> JoinResult:

@@ -166,7 +166,10 @@ int ensure(Ctx* c, DevBuf& b, size_t bytes) {
     return HJ_OK;
   }
   if (b.bytes >= bytes && b.p && !b.ws) return HJ_OK;
-  if (b.p && !b.ws) cudaFree(b.p);
+  if (b.p && !b.ws) {  // earlier work of this ctx may still read it (e.g. an asynchronous pass 1)
+    cudaStreamSynchronize(c->stream);
+    cudaFree(b.p);
+  }
   b.p = nullptr;
   b.bytes = 0;
   b.ws = false;
@@ -203,7 +206,7 @@ int ilog2_ceil(unsigned long long x) {
 
 // Host-side plan of one call: radix bits, capacities, launch shapes, metadata layout.
 struct HostPlan {
-  int B = 0, b1 = 0, b2 = 0;
+  int B = 0, b1 = 0, b2 = 0, gsh = 0;
   int g = 0, nsrc = 1, mode = PLAN_FULL;
   uint32_t CR = 0, CS = 0, C2 = 0;
   int lg_nb = 6;
@@ -269,21 +272,33 @@ int choose_bits(unsigned long long nR) {
   return std::min(B, 20);
 }
 
+// pass-1 bits of the exchange: pass 1's fan-out (rank bits + b1) and the
+// receiver's pieces (sources x 2^b1) stay <= 2^10, so b1 = min(ceil(B/2), 10 - log2 G); sender
+// and receiver derive the same b1 (c5 at G = 8: B = 16 -> 7 + 9)
+int xchg_b1(int G, int B) {
+  const int gl = ilog2_ceil((unsigned long long)std::max(G, 1));
+  int b1 = (B + 1) / 2;
+  if (gl > 0 && b1 > 10 - gl) b1 = std::max(0, 10 - gl);
+  return b1;
+}
+
 // mode PLAN_FULL: one GPU; PLAN_SEND: exchange sender (g rank bits); PLAN_RECV: exchange
-// receiver (nsrc count rows). nR / nS are the tuples this GPU partitions / joins.
+// receiver (nsrc sources). nR / nS are the tuples this GPU partitions / joins.
 int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS, int radix_bits, bool mat, int g = 0,
               int nsrc = 1, int mode = PLAN_FULL) {
   const size_t tb = (size_t)c->key_bytes + c->pay_bytes;  // AoS tuple bytes
   hp.B = radix_bits < 0 ? choose_bits(nR) : radix_bits;
   if (hp.B > 20) return fail(c, HJ_ERR_UNSUPPORTED, "radix_bits %d > 20", hp.B);
-  hp.b1 = (hp.B + 1) / 2;  // reading S6; HJ_OPT_PASS1_BITS overrides (results never change)
-  if (c->opt_pass1_bits > 0 && hp.B >= 2) hp.b1 = (int)std::min<int64_t>(c->opt_pass1_bits, hp.B - 1);
-  // multi-GPU: pass 1's fan-out (rank bits + b1) and the receiver's pass-2 pieces
-  // (sources x 2^b1) stay <= 2^10, so b1 = min(ceil(B/2), 10 - log2 G); sender (g rank bits)
-  // and receiver (nsrc = G sources) derive the same b1 (c5 at G = 8: B = 16 -> 7 + 9)
-  const int gl = std::max(g, ilog2_ceil((unsigned long long)std::max(nsrc, 1)));
-  if (gl > 0 && hp.b1 > 10 - gl) hp.b1 = std::max(0, 10 - gl);
+  hp.b1 = (hp.B + 1) / 2;  // reading S6; HJ_OPT_PASS1_BITS overrides on one GPU (results never change)
+  const bool xchg = mode != PLAN_FULL || g > 0 || nsrc > 1;
+  if (xchg) hp.b1 = xchg_b1(std::max(1 << g, nsrc), hp.B);
+  else if (c->opt_pass1_bits > 0 && hp.B >= 2) hp.b1 = (int)std::min<int64_t>(c->opt_pass1_bits, hp.B - 1);
   hp.b2 = hp.B - hp.b1;
+  hp.gsh = hp.B;
+  if (mode == PLAN_SEND) {  // the sender counts and lays out only its (rank, d1) pieces
+    hp.B = hp.b1;
+    hp.b2 = 0;
+  }
   hp.g = g;
   hp.nsrc = nsrc;
   hp.mode = mode;
@@ -334,7 +349,7 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   // zeroed region first
   hp.o_counters = take(64);
   hp.o_results = take(64);
-  for (int r = 0; r < 2; ++r) hp.o_cnt[r] = take(mode == PLAN_RECV ? 0 : nq * 4);
+  for (int r = 0; r < 2; ++r) hp.o_cnt[r] = take(nq * 4);  // (the receiver's own histogram too)
   hp.zero_bytes = o;
   for (int r = 0; r < 2; ++r) {
     hp.o_off[r] = take((nq + 1) * 8);
@@ -403,6 +418,9 @@ int set_kernel_attrs(Ctx* c) {
   attr((const void*)k_hist<K, true, true, true>);
   attr((const void*)k_hist<K, true, false, false>);
   attr((const void*)k_hist<K, true, true, false>);
+  load((const void*)k_hist_recv<K, false, false>);
+  attr((const void*)k_hist_recv<K, true, true>);
+  attr((const void*)k_hist_recv<K, true, false>);
   for_ws_variants<K>(attr);
   attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), false>);
   attr((const void*)k_pass<K, 1, 1024, pass_items<K>(), true>);
@@ -480,6 +498,7 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   P.b1 = hp.b1;
   P.b2 = hp.b2;
   P.g = hp.g;
+  P.gsh = hp.gsh;
   P.nsrc = hp.nsrc;
   P.mode = hp.mode;
   P.C2 = hp.C2;
@@ -530,6 +549,26 @@ int launch_plan(Ctx* c, const HostPlan& hp, const Plan& P) {
   return HJ_OK;
 }
 
+// a1 on the exchange receiver: its own histogram of what it received (k_hist_recv)
+template <typename K>
+int launch_hist_recv(Ctx* c, const HostPlan& hp, const Plan& P) {
+  cudaStream_t st = c->stream;
+  const bool smem = hp.B <= 16, c32 = hp.B <= 15;
+  const size_t sm = smem ? (c32 ? ((size_t)4 << hp.B) : ((size_t)2 << hp.B)) : 0;
+  const unsigned long long nR = P.rel[0].n, nS = P.rel[1].n;
+  const void* f = !smem ? (const void*)k_hist_recv<K, false, false>
+                        : c32 ? (const void*)k_hist_recv<K, true, true> : (const void*)k_hist_recv<K, true, false>;
+  const int g = std::max(2, grid_for(c, f, HIST_NT, sm, (nR + nS + 4095) / 4096 + 2));
+  uint32_t gr = (uint32_t)((double)g * (double)nR / (double)std::max<unsigned long long>(nR + nS, 1) + 0.5);
+  gr = std::min<uint32_t>(std::max<uint32_t>(gr, 1), (uint32_t)g - 1);
+  if (!smem) k_hist_recv<K, false, false><<<g, HIST_NT, 0, st>>>(P, gr);
+  else if (c32) k_hist_recv<K, true, true><<<g, HIST_NT, sm, st>>>(P, gr);
+  else k_hist_recv<K, true, false><<<g, HIST_NT, sm, st>>>(P, gr);
+  CUDA_TRY(c, cudaGetLastError());
+  c->launches += 1;
+  return HJ_OK;
+}
+
 // stage: 0 = all of a1-a3; 1 = a1-a2 only (hj_xd_count); 2 = a3 only (hj_xd_store, after stage 1
 // with the same plan)
 template <typename K>
@@ -572,6 +611,8 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false, 
     else k_hist<K, false, false><<<g, HIST_NT, 0, st>>>(P, gr);
     CUDA_TRY(c, cudaGetLastError());
     c->launches += 1;
+  } else if (int rc = launch_hist_recv<K>(c, hp, P)) {  // exchange receiver: its own histogram
+    return rc;
   }
   mark(c, 1);
   if (int rc = launch_plan(c, hp, P)) return rc;
@@ -1652,8 +1693,8 @@ int hj_join_received(hj_ctx* h, const void* R_recv, uint64_t nR, const uint32_t*
     Plan P = device_plan(c, hp, nullptr, nullptr, nR, nullptr, nullptr, nS);
     P.rel[0].t1 = const_cast<void*>(R_recv);
     P.rel[1].t1 = const_cast<void*>(S_recv);
-    P.rel[0].cnt = const_cast<uint32_t*>(R_counts);
-    P.rel[1].cnt = const_cast<uint32_t*>(S_counts);
+    P.prow[0] = R_counts;
+    P.prow[1] = S_counts;
     c->launches = 0;
     rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P) : launch_front<uint64_t>(c, hp, P);
     if (rc == HJ_OK) rc = c->key_bytes == 4 ? launch_pass2<uint32_t>(c, hp, P) : launch_pass2<uint64_t>(c, hp, P);
@@ -1715,7 +1756,12 @@ int hj_xd_window(hj_ctx* h, int slot, uint64_t bytes, void** dptr, void* ipc_han
 
 uint64_t hj_xd_header_bytes(int G, int local_bits) {
   if (G < 1 || local_bits < 0 || local_bits > 20) return 0;
-  return align_up((size_t)G * ((size_t)4 << local_bits), 256);
+  return align_up((size_t)G * ((size_t)4 << xchg_b1(G, local_bits)), 256);
+}
+
+uint32_t hj_exchange_row_len(int G, int local_bits) {
+  if (G < 1 || local_bits < 0 || local_bits > 20) return 0;
+  return 1u << xchg_b1(G, local_bits);
 }
 
 int hj_ipc_open(hj_ctx* h, const void* ipc_handle, void** dptr) {
@@ -1766,6 +1812,9 @@ int hj_xd_count(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const vo
   }
   HostPlan& hp = *c->xd_hp;
   int rc = prepare(c, hp, nR, nS, local_bits, false, gpu_bits, 1, PLAN_SEND);
+  // the send plan lives in its own buffer: hj_xd_store's pass 1 still reads it (asynchronously)
+  // when this rank's hj_join_received prepares its receive plan in c->meta
+  if (rc == HJ_OK) rc = ensure(c, c->xd_meta, hp.meta_bytes);
   if (rc == HJ_OK && !c->h_xd_cur) {
     if (cudaMallocHost(&c->h_xd_cur, (size_t)XD_MAX * 2 * XD_MAX * 8) != cudaSuccess ||
         cudaHostAlloc(&c->h_xd_err, 64, cudaHostAllocMapped) != cudaSuccess ||
@@ -1776,7 +1825,7 @@ int hj_xd_count(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const vo
   }
   if (rc == HJ_OK) {
     Plan& P = *c->xd_P;
-    P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
+    P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS, c->xd_meta.p);
     c->launches = 0;
     rc = c->key_bytes == 4 ? launch_front<uint32_t>(c, hp, P, false, 1) : launch_front<uint64_t>(c, hp, P, false, 1);
     const uint32_t F1 = 1u << hp.pb();
@@ -1816,7 +1865,7 @@ int hj_xd_store(hj_ctx* h, int rank, const uint64_t* totals, void* const* win_R,
     for (int j = 0; j < G; ++j)
       if (!win[r][j]) return fail(c, HJ_ERR_INVALID, "null window pointer (relation %d, rank %d)", r, j);
   const long long tb = c->key_bytes + c->pay_bytes;
-  const size_t H = hj_xd_header_bytes(G, hp.B);
+  const size_t H = hj_xd_header_bytes(G, hp.gsh);  // (the send plan's B is its b1; gsh = local bits)
   const uint32_t F1 = 1u << hp.pb();
   // cursor of pass-1 digit D = (j, d1): element offset, from this rank's own window tuples, of
   // where this rank's d1 run for rank j starts in rank j's window (source-major layout, then d1)
@@ -1962,7 +2011,7 @@ int hj_xd_join(hj_ctx* h, int rank, int gpu_bits, const void* Rk, const void* Rp
     char* own = (char*)win[r][rank];
     Ps.rel[r].t1 = own + H;
     Pr.rel[r].t1 = own + H;
-    Pr.rel[r].cnt = (uint32_t*)own;
+    Pr.prow[r] = (const uint32_t*)own;  // the senders' piece rows; rel[r].cnt: this rank's own histogram
     a.pst[r] = Ps.rel[r].pst;
     a.cur1[r] = Ps.rel[r].cur1;
     a.rows0[r] = (uint32_t*)own;
@@ -1978,7 +2027,7 @@ int hj_xd_join(hj_ctx* h, int rank, int gpu_bits, const void* Rk, const void* Rp
   a.err = c->d_xd_err;
   a.epoch = ++c->xd_epoch;
   a.timeout_ns = (unsigned long long)timeout_ms * 1000000ull;
-  a.rows_words = (uint32_t)G << local_bits;
+  a.rows_words = (uint32_t)G << xchg_b1(G, local_bits);
   a.G = G;
   a.rank = rank;
   a.b1 = hs.b1;
@@ -2050,6 +2099,7 @@ int hj_xd_join(hj_ctx* h, int rank, int gpu_bits, const void* Rk, const void* Rp
     CUDA_TRY(c, cudaGetLastError());
     c->launches += 1;
     mark(c, 3);
+    if (int e1 = k4 ? launch_hist_recv<uint32_t>(c, hr, Pr) : launch_hist_recv<uint64_t>(c, hr, Pr)) return e1;
     if (int e1 = launch_plan(c, hr, Pr)) return e1;
     e = k4 ? launch_pass2<uint32_t>(c, hr, Pr) : launch_pass2<uint64_t>(c, hr, Pr);
     if (e) return e;

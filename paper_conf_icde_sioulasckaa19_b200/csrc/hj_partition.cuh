@@ -131,6 +131,65 @@ __global__ void __launch_bounds__(1024) k_hist(Plan P, uint32_t blocks_r) {
 }
 
 // ------------------------------------------------------------------------------------------
+// a1 on the exchange receiver: this rank's own histogram of the 2^B co-partitions of the AoS
+// tuples it received (rel.t1, the first sum(prow) of them), in shared memory as k_hist (u32 bins
+// up to 2^15, packed 16-bit bins at 2^16). After the exchange every key in the buffer belongs to
+// this rank's 2^B co-partitions, so the counts are dense per bin; the senders then only count
+// their (rank, d1) pieces (<= 2^10 bins) instead of 2^(g+B) bins in global memory.
+// grid: blocks [0, blocks_r) count R, the rest S.
+// ------------------------------------------------------------------------------------------
+template <typename K, bool SMEM, bool C32>
+__global__ void __launch_bounds__(1024) k_hist_recv(Plan P, uint32_t blocks_r) {
+  using TT = Tup<K>;
+  using T = typename TT::T;
+  extern __shared__ uint32_t s_hist[];
+  __shared__ unsigned long long s_tot;
+  const uint32_t np = 1u << P.B;
+  const uint32_t nwords = !SMEM ? 0u : C32 ? np : np / 2;
+  const int rel = blockIdx.x < blocks_r ? 0 : 1;
+  for (uint32_t i = threadIdx.x; i < nwords; i += blockDim.x) s_hist[i] = 0;
+  if (threadIdx.x == 0) s_tot = 0;
+  __syncthreads();
+  {  // tuples received = sum of the piece rows (<= 1024 words)
+    unsigned long long t = 0;
+    for (uint32_t i = threadIdx.x; i < P.npieces(); i += blockDim.x) t += P.prow[rel][i];
+    #pragma unroll
+    for (int o = 16; o; o >>= 1) t += __shfl_xor_sync(0xffffffffu, t, o);
+    if ((threadIdx.x & 31) == 0 && t) atomicAdd(&s_tot, t);
+  }
+  __syncthreads();
+  const unsigned long long n = min(s_tot, P.rel[rel].n);
+  const uint32_t nblk = rel ? gridDim.x - blocks_r : blocks_r;
+  const uint32_t bid = rel ? blockIdx.x - blocks_r : blockIdx.x;
+  const unsigned long long per = (n + nblk - 1) / nblk;
+  const unsigned long long lo = min((unsigned long long)bid * per, n), hi = min(lo + per, n);
+  const T* t1 = (const T*)P.rel[rel].t1;
+  uint32_t* gcnt = P.rel[rel].cnt;
+  auto add = [&](K key) {
+    const uint32_t b = qbin<false>(key, P);
+    if (!SMEM) atomicAdd(&gcnt[b], 1u);  // more than 2^16 bins: global atomics (correct, slower)
+    else if (C32) atomicAdd(&s_hist[b], 1u);
+    else hist_add<false>(s_hist, b, gcnt);
+  };
+  constexpr int U = 4;  // tuples per thread per batch (loaded before any atomic)
+  unsigned long long i = lo + threadIdx.x;
+  for (; i + (U - 1) * blockDim.x < hi; i += U * (unsigned long long)blockDim.x) {
+    K k[U];
+    #pragma unroll
+    for (int u = 0; u < U; ++u) k[u] = TT::key(__ldcs(t1 + i + u * blockDim.x));
+    #pragma unroll
+    for (int u = 0; u < U; ++u) add(k[u]);
+  }
+  for (; i < hi; i += blockDim.x) add(TT::key(__ldcs(t1 + i)));
+  if (!SMEM) return;
+  __syncthreads();
+  for (uint32_t q = threadIdx.x; q < np; q += blockDim.x) {
+    const uint32_t c = C32 ? s_hist[q] : ((s_hist[q >> 1] >> ((q & 1) << 4)) & 0xffffu);
+    if (c) atomicAdd(&gcnt[q], c);
+  }
+}
+
+// ------------------------------------------------------------------------------------------
 // a2 + a5: the planner. grid = ceil(2^qbits / 1024) blocks of 1024 threads.
 //   off[q]  = exclusive scan over q of sum_s cnt[s][q]             (co-partition starts in T2)
 //   cur2[q] = off[q]                                               (pass-2 reservation cursors)
@@ -152,12 +211,7 @@ __device__ __forceinline__ unsigned long long plan_items(const Plan& P, unsigned
   return ((cr + P.CR - 1) / P.CR) * ((cs + P.CS - 1) / P.CS);
 }
 
-__device__ __forceinline__ unsigned long long plan_count(const RelDev& R, int nsrc, uint32_t np, uint32_t q) {
-  if (nsrc == 1) return R.cnt[q];
-  unsigned long long c = 0;
-  for (int s = 0; s < nsrc; ++s) c += R.cnt[(size_t)s * np + q];
-  return c;
-}
+__device__ __forceinline__ unsigned long long plan_count(const RelDev& R, int, uint32_t, uint32_t q) { return R.cnt[q]; }
 
 // MS: several sources (exchange receiver); IT: join items (not on the exchange sender). Specialised so each launch runs (and fetches) only its own code.
 template <bool MS, bool IT>
@@ -226,24 +280,6 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
     }
     if (items) P.ist[np] = bad ? 0u : (uint32_t)(bI + tI);
   }
-  // ---- several sources: piece sizes, a warp per piece (stored in pst[i + 1]) --------------
-  const uint32_t npieces = P.npieces();
-  const int pb = P.pb(), b2 = P.b2;
-  if (MS && nsrc > 1) {
-    const uint32_t lane = threadIdx.x & 31, gw = b * (NT / 32) + (threadIdx.x >> 5), nw = gridDim.x * (NT / 32);
-    for (int rel = 0; rel < 2; ++rel) {
-      const RelDev& R = P.rel[rel];
-      for (uint32_t i = gw; i < npieces; i += nw) {
-        const uint32_t src = i >> pb, D = i & ((1u << pb) - 1);
-        const uint32_t* row = R.cnt + (size_t)src * np + ((size_t)D << b2);
-        unsigned long long c = 0;
-        for (uint32_t t = lane; t < (1u << b2); t += 32) c += row[t];
-        #pragma unroll
-        for (int o = 16; o; o >>= 1) c += __shfl_xor_sync(0xffffffffu, c, o);
-        if (lane == 0) R.pst[i + 1] = c;
-      }
-    }
-  }
   // ---- last block: piece starts, pass-1 cursors, pass-2 chunk lists (npieces <= 1024) ------
   __threadfence();
   __syncthreads();
@@ -251,6 +287,8 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   __syncthreads();
   if (!s_last) return;
   __threadfence();
+  const uint32_t npieces = P.npieces();
+  const int b2 = P.b2;
   const uint32_t i = threadIdx.x;
   unsigned long long pv[4], ptt[4];  // (piece size, its pass-2 chunks) of R, then of S
   #pragma unroll
@@ -261,10 +299,26 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
       if (nsrc == 1)
         sz = __ldcg(&R.off[(unsigned long long)(i + 1) << b2]) - __ldcg(&R.off[(unsigned long long)i << b2]);
       else
-        sz = __ldcg(&R.pst[i + 1]);
+        sz = P.prow[rel][i];  // exchange receiver: piece i = (source i >> pb, digit) as sent
     }
     pv[2 * rel] = sz;
     pv[2 * rel + 1] = (sz + P.C2 - 1) / P.C2;
+  }
+  if (P.mode == PLAN_RECV) {
+    // the pieces of pass-1 digit D (one per source) must hold exactly what this rank's own
+    // histogram counted in D's co-partitions; else the rows describe other tuples than the
+    // buffers hold (pass 2 and the join then do nothing, hj_join_received fails)
+    const uint32_t F1 = 1u << P.pb();
+    for (int rel = 0; rel < 2 && i < F1; ++rel) {
+      unsigned long long sent = 0;
+      for (int sr = 0; sr < nsrc; ++sr) sent += P.prow[rel][(size_t)sr * F1 + i];
+      const RelDev& R = P.rel[rel];
+      const unsigned long long got = __ldcg(&R.off[(unsigned long long)(i + 1) << b2]) - __ldcg(&R.off[(unsigned long long)i << b2]);
+      if (sent != got) {
+        P.counters[CNT_BAD_COUNTS] = 1u;
+        if (rel == 0) P.ist[1u << P.B] = 0u;
+      }
+    }
   }
   block_exclusive_scan64xM<NT, 4>(pv, s_tmp6, ptt);
   #pragma unroll
@@ -520,7 +574,7 @@ __device__ __forceinline__ void pass_body(const Plan& P, int fanout_bits) {
   // shifts and masks live in registers (not re-read from the parameter struct per tuple)
   const uint32_t dsh = MODE == 1 ? 0u : (uint32_t)P.b1;
   const uint32_t dmask = MODE == 1 ? ((1u << P.b1) - 1) : ((1u << P.b2) - 1);
-  const uint32_t gsh = (uint32_t)P.B, gmask = (1u << P.g) - 1, gup = (uint32_t)P.b1;
+  const uint32_t gsh = (uint32_t)P.gsh, gmask = (1u << P.g) - 1, gup = (uint32_t)P.b1;
   auto digit = [=](K key) -> uint32_t {
     uint32_t d = (uint32_t)(key >> dsh) & dmask;
     if (MODE == 1 && GD) d |= ((uint32_t)(key >> gsh) & gmask) << gup;

@@ -84,7 +84,7 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
   if (MODE == 2 && P.mode == PLAN_RECV && *(volatile const uint32_t*)&P.counters[CNT_BAD_COUNTS]) return;
   const uint32_t dsh = MODE == 1 ? 0u : (uint32_t)P.b1;
   const uint32_t dmask = MODE == 1 ? ((1u << P.b1) - 1) : ((1u << P.b2) - 1);
-  const uint32_t gsh = (uint32_t)P.B, gmask = (1u << P.g) - 1, gup = (uint32_t)P.b1;
+  const uint32_t gsh = (uint32_t)P.gsh, gmask = (1u << P.g) - 1, gup = (uint32_t)P.b1;
   auto digit = [=](K key) -> uint32_t {
     uint32_t d = (uint32_t)(key >> dsh) & dmask;
     if (MODE == 1 && GD) d |= ((uint32_t)(key >> gsh) & gmask) << gup;

@@ -7,12 +7,14 @@
 namespace hj {
 
 // Radix field and co-partition order. The local radix field p = key & (2^B - 1) splits into
-// d1 = p & (2^b1 - 1) (pass 1) and d2 = p >> b1 (pass 2). On the multi-GPU exchange sender the
-// pass-1 digit is widened by g rank bits taken from just above the local field:
-//   D = ((key >> B) & (2^g - 1)) << b1 | d1        (pb = g + b1 bits)
-// Counts, offsets and cursors use q-order q = D << b2 | d2 over a q-space of qbits = pb + b2
-// bits, so pass-1 partition D is the contiguous q range [D << b2, (D + 1) << b2) and, on the
-// sender, rank j's co-partitions are the contiguous range [j << B, (j + 1) << B).
+// d1 = p & (2^b1 - 1) (pass 1) and d2 = p >> b1 (pass 2). Counts, offsets and cursors use q-order
+// q = d1 << b2 | d2, so pass-1 partition d1 is the contiguous q range [d1 << b2, (d1 + 1) << b2).
+// Multi-GPU exchange: the sender only needs its pass-1 layout, so its plan has
+// B = b1, b2 = 0 and the pass-1 digit widened by g rank bits taken from just above the LOCAL field:
+//   D = ((key >> gsh) & (2^g - 1)) << b1 | d1        (pb = g + b1 <= 10 bits, gsh = local bits)
+// -- a histogram of <= 2^10 bins whatever the local field (c5 at G = 8: 3 + 7 bits, not 3 + 16).
+// The receiver counts the 2^B co-partitions of what it received itself (k_hist_recv: keys are
+// dense per bin only after the exchange) and takes the pieces' sizes from the senders' rows.
 // Pass 2 reads "pieces": piece i = (source s, D) = (i >> pb, i & (2^pb - 1)); on one GPU the
 // pieces are the pass-1 partitions, on the exchange receiver the d1-segments sent by each rank.
 enum { PLAN_FULL = 0, PLAN_SEND = 1, PLAN_RECV = 2 };
@@ -66,8 +68,12 @@ struct Plan {
   RelDev rel[2];  // 0 = R (build), 1 = S (probe)
   int bc;         // 1: bucket-chain partitioner (NEXT-1), rel[r].t2 = bc[r].pool2
   BcRel bc_rel[2];
-  int B, b1, b2;  // local radix field
+  int B, b1, b2;  // radix field of this plan's histogram / passes (the exchange sender: B = b1, b2 = 0)
   int g;          // rank bits in the pass-1 digit (PLAN_SEND), else 0
+  int gsh;        // PLAN_SEND: the rank digit is (key >> gsh) & (2^g - 1), gsh = the local radix bits
+  const uint32_t* prow[2];  // PLAN_RECV: received piece counts [nsrc][2^b1] per relation (row s = what
+                            // source s sent, by pass-1 digit); rel[r].cnt is then this rank's own
+                            // histogram of what it received
   int nsrc;       // count rows / piece sources (PLAN_RECV: ranks), else 1
   int mode;       // PLAN_FULL, PLAN_SEND, PLAN_RECV
   int skip_r;     // streaming S chunks: R is already partitioned (its pass-2 units are skipped)
@@ -94,7 +100,7 @@ struct Plan {
 template <bool GD, typename K>
 __device__ __forceinline__ uint32_t dig1(K key, const Plan& P) {
   uint32_t d = (uint32_t)key & ((1u << P.b1) - 1);
-  if (GD) d |= ((uint32_t)(key >> P.B) & ((1u << P.g) - 1)) << P.b1;
+  if (GD) d |= ((uint32_t)(key >> P.gsh) & ((1u << P.g) - 1)) << P.b1;
   return d;
 }
 template <typename K>

@@ -29,41 +29,41 @@ class NumpyExchangeCtx:
         self.sent_rows = {}
 
     @staticmethod
-    def _split(lb):
-        return (lb + 1) // 2, lb // 2
+    def _b1(G, lb):  # hj_exchange_row_len's rule: b1 = min(ceil(lb / 2), 10 - log2 G)
+        g = G.bit_length() - 1
+        b1 = (lb + 1) // 2
+        return max(0, 10 - g) if g > 0 and b1 > 10 - g else b1
 
     def exchange_pack(self, rel, keys, pays, gpu_bits, local_bits):
         k = keys.numpy().view(np.uint32).astype(np.uint64)
         p = pays.numpy().view(np.uint32).astype(np.uint64)
         G = 1 << gpu_bits
-        b1, b2 = self._split(local_bits)
+        b1 = self._b1(G, local_bits)
         j = (k >> np.uint64(local_bits)) & np.uint64(G - 1)
         d1 = k & np.uint64((1 << b1) - 1)
-        d2 = (k >> np.uint64(b1)) & np.uint64((1 << b2) - 1)
         order = np.lexsort((d1, j))  # grouped by destination, then by d1
         words = (k | (p << np.uint64(32)))[order].view(np.int64)
-        q = (d1 << np.uint64(b2)) | d2
-        cnt = np.zeros((G, 1 << local_bits), dtype=np.int64)
-        np.add.at(cnt, (j.astype(np.int64), q.astype(np.int64)), 1)
+        cnt = np.zeros((G, 1 << b1), dtype=np.int64)  # piece counts: tuples per (destination, d1)
+        np.add.at(cnt, (j.astype(np.int64), d1.astype(np.int64)), 1)
         dest = np.bincount(j.astype(np.int64), minlength=G).astype(np.uint64)
         return torch.from_numpy(words.copy()), torch.from_numpy(cnt.astype(np.int32)), dest
 
     def join_received(self, R_recv, nR, R_counts, S_recv, nS, S_counts, nsrc, local_bits, out_mode=0):
-        b1, b2 = self._split(local_bits)
+        b1 = self._b1(nsrc, local_bits)
         cols = []
         for buf, n, cnt in ((R_recv, nR, R_counts), (S_recv, nS, S_counts)):
             w = buf.numpy().view(np.uint64)
             assert len(w) == n
             k = (w & np.uint64(0xFFFFFFFF)).astype(np.uint32)
             p = (w >> np.uint64(32)).astype(np.uint32)
-            # the received count rows describe the received segments exactly
+            # the received piece rows describe the received segments exactly (source-major, d1-grouped)
             c = cnt.numpy().astype(np.int64)
             pos = 0
             for s in range(nsrc):
-                seg = k[pos:pos + c[s].sum()].astype(np.uint64)
-                q = ((seg & np.uint64((1 << b1) - 1)) << np.uint64(b2)) | ((seg >> np.uint64(b1)) & np.uint64((1 << b2) - 1))
-                assert np.array_equal(np.bincount(q.astype(np.int64), minlength=1 << local_bits), c[s])
-                pos += c[s].sum()
+                for d in range(1 << b1):
+                    seg = k[pos:pos + c[s, d]].astype(np.uint64)
+                    assert np.all((seg & np.uint64((1 << b1) - 1)) == np.uint64(d))
+                    pos += c[s, d]
             assert pos == n
             cols += [k, p]
         m, chk = oracle.hash_join(*cols)
@@ -147,7 +147,7 @@ class NumpyDirectCtx(NumpyExchangeCtx):
         return np.ndarray((self.seg[base].size,), dtype=np.uint8, buffer=self.seg[base].buf), addr - base
 
     def xd_header_bytes(self, G, lb):
-        return -(-G * (4 << lb) // 256) * 256
+        return -(-G * (4 << self._b1(G, lb)) // 256) * 256
 
     def xd_window(self, slot, nbytes, want_handle=True):
         from multiprocessing import shared_memory
@@ -207,7 +207,8 @@ class NumpyDirectCtx(NumpyExchangeCtx):
         for r, win in ((0, win_R), (1, win_S)):
             n = int(totals[r, :, rank].sum())
             buf, o = self._buf(int(win[rank]))
-            cnt = buf[o:o + G * (4 << lb)].view(np.int32).reshape(G, 1 << lb).copy()
+            rl = 1 << self._b1(G, lb)
+            cnt = buf[o:o + G * 4 * rl].view(np.int32).reshape(G, rl).copy()
             recv = buf[o + H:o + H + 8 * n].view(np.int64).copy()
             ins += [torch.from_numpy(recv), n, torch.from_numpy(cnt)]
         res = self.join_received(*ins, G, lb, out_mode)
@@ -455,7 +456,8 @@ def _direct_virtual(hj, w, G, lb, out_mode, width=4):
         for r in (0, 1):
             words = nin[r] * tb // 8
             recv = hj._wrap_device(win[r][v] + H, max(words, 1), 8, torch.device("cuda", 0))[:words]
-            cnt = hj._wrap_device(win[r][v], G << lb, 4, torch.device("cuda", 0)).view(G, 1 << lb)
+            rl = hj.exchange_row_len(G, lb)
+            cnt = hj._wrap_device(win[r][v], G * rl, 4, torch.device("cuda", 0)).view(G, rl)
             ins += [recv, nin[r], cnt]
         with torch.cuda.stream(streams[v]):
             res = ctxs[v].join_received(*ins, G, lb, out_mode)

@@ -526,7 +526,11 @@ def test_compute_sanitizer_clean(hj, tool):
     import sys
 
     root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
-    out = subprocess.run(["compute-sanitizer", "--tool", tool, sys.executable,
+    # racecheck does not model mbarrier hand-offs between warps: it reports hazards on a correct
+    # two-warp ping-pong (tools/microbench/mb_mbar_race.cu, profiles/r02_sanitizers.md), so the
+    # warp-specialized pass (stages handed over by mbarriers) is excluded from racecheck only
+    extra = ["--kernel-name-exclude", "kns=k_pass_ws"] if tool == "racecheck" else []
+    out = subprocess.run(["compute-sanitizer", "--tool", tool, *extra, sys.executable,
                           os.path.join(root, "tools", "sanitize_cases.py"), "core"],
                          capture_output=True, text=True, timeout=1800)
     txt = out.stdout + out.stderr

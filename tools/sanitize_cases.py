@@ -37,6 +37,9 @@ for w in cases:
     for bits in (-1, 0, 5, 11):
         check(ctx4, w, bits)
 check(ctx8, W.Workload("d", 9000, 12000, "1to1", keys="k8", seed=403).with_(nS=9000))
+cw = hj.Context(0, 4, 4)
+cw.set_option(hj.OPT_PASS_WS, 0)  # the lock-step partition passes (racecheck covers them; see test)
+check(cw, W.Workload("h", 20000, 30011, "zipf", z=1.2, keys="sparse", seed=407))
 if which == "all":
     w = W.Workload("e", 30000, 40000, "fk", keys="sparse", seed=404)
     Rk, Rp, Sk, Sp = W.np_generate(w)
