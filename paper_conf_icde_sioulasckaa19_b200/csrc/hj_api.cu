@@ -36,16 +36,19 @@ struct JoinShape {
   bool pf;                        // next probe round's S loads issued before the current walk
   bool l2pf;                      // claimed item's R chunk + first S round prefetched into L2
   int spf = 0;                    // S stream prefetched into L2 this many probe rounds ahead (0 = off)
+  bool bf = true;                 // branch-free first chain step for every tuple of a round
 };
 // 0-2 are the defaults (join_variant below); 3-5 are kept as measured alternatives (round 1 swept
 // 46 shapes; the slower ones were removed)
 constexpr JoinShape JOIN_SHAPES[] = {
     {256, 6, 3, 1, 1, false, true, true},      // 0: 4 B count
     {256, 8, 3, 1, 1, false, false, true, 2},  // 1: 4 B materialize
-    {512, 1, 2, 1, 1, false, true, true},      // 2: 8 B (both modes)
+    {512, 1, 2, 1, 1, false, true, true, 0, false},  // 2: 8 B (both modes), round-1 shape
     {256, 8, 3, 1, 1},                         // 3: no prefetching
     {256, 8, 2, 2, 1},                         // 4: double-buffered R tile
     {224, 8, 4, 1, 1, true},                   // 5: 16-bit heads, 4 blocks / SM
+    {512, 2, 2, 1, 1, false, true, true, 0, false},  // 6: 8 B, two tuples per thread (c5_gpu join 2.71 vs 2.45 ms)
+    {512, 2, 2, 1, 1, false, true, true},             // 7: 8 B, branch-free first step (2.60 ms; 256 x 4: 3.23)
 };
 constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
@@ -367,11 +370,11 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
 template <typename K, int V, typename F>
 void attr_join(F&& attr) {
   constexpr JoinShape S = JOIN_SHAPES[V];
-  attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf>);
-  attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf>);
+  attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, true, S.bf>);
+  attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, true, S.bf>);
   if constexpr (sizeof(K) == 4) {
-    attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, true>);
-    attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, true>);
+    attr((const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, false, S.bf>);
+    attr((const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, false, S.bf>);
   }
 }
 
@@ -443,6 +446,8 @@ int set_kernel_attrs(Ctx* c) {
   attr_join<K, 3>(attr);
   attr_join<K, 4>(attr);
   attr_join<K, 5>(attr);
+  attr_join<K, 6>(attr);
+  attr_join<K, 7>(attr);
   return rc;
 }
 
@@ -715,20 +720,23 @@ template <typename K, int V, bool F2>
 int launch_join_f(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
   constexpr JoinShape S = JOIN_SHAPES[V];
   cudaStream_t st = c->stream;
-  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2>
-                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2>;
+  const void* f = mat ? (const void*)k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2, S.bf>
+                      : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2, S.bf>;
   int g = grid_for(c, f, S.nt + 32, hp.join_smem, 1ull << 40);
-  if (mat) k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2><<<g, S.nt + 32, hp.join_smem, st>>>(P);
-  else k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  if (mat)
+    k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2, S.bf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+  else
+    k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2, S.bf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
   CUDA_TRY(c, cudaGetLastError());
   return HJ_OK;
 }
 
-// the two-term slot hash (slot_of2) when it still covers every key bit above the radix field
+// the cheaper slot hash (slot_of2): 8-byte keys always, 4-byte keys when the two-term fold still
+// covers every key bit above the radix field
 template <typename K, int V>
 int launch_join_v(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
-  if (sizeof(K) == 4 && P.H.nfold <= 1) return launch_join_f<K, V, sizeof(K) == 4>(c, hp, P, mat);
-  return launch_join_f<K, V, false>(c, hp, P, mat);
+  if (sizeof(K) == 8 || P.H.nfold <= 1) return launch_join_f<K, V, true>(c, hp, P, mat);
+  return launch_join_f<K, V, sizeof(K) == 8>(c, hp, P, mat);
 }
 
 template <typename K>
@@ -751,6 +759,9 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
     case 3: rc = launch_join_v<K, 3>(c, hp, P, mat); break;
     case 4: rc = launch_join_v<K, 4>(c, hp, P, mat); break;
     case 5: rc = launch_join_v<K, 5>(c, hp, P, mat); break;
+    case 6: rc = launch_join_v<K, 6>(c, hp, P, mat); break;
+    case 7: rc = launch_join_v<K, 7>(c, hp, P, mat); break;
+
     default: rc = launch_join_v<K, 0>(c, hp, P, mat); break;
   }
   if (rc) return rc;

@@ -66,9 +66,16 @@ __device__ __forceinline__ uint32_t slot_of2(uint32_t key, const SlotHash& H) {
   const uint32_t h = key >> H.B;
   return (h ^ (h >> H.lg)) & ((1u << H.lg) - 1);
 }
+// 64-bit keys: the bits above B folded to 32 by a multiply-xor, then one xor-shift (6 instructions
+// instead of 10; any hash gives the same join, chains always compare full keys)
+__device__ __forceinline__ uint32_t slot_of2(uint64_t key, const SlotHash& H) {
+  const uint64_t h64 = key >> H.B;
+  const uint32_t h = (uint32_t)h64 ^ ((uint32_t)(h64 >> 32) * 0x9E3779B1u);
+  return (h ^ (h >> H.lg)) & ((1u << H.lg) - 1);
+}
 template <bool F2, typename K>
 __device__ __forceinline__ uint32_t slot_for(K key, const SlotHash& H) {
-  if constexpr (F2 && sizeof(K) == 4) return slot_of2((uint32_t)key, H);
+  if constexpr (F2) return slot_of2(key, H);
   else return slot_of(key, H);
 }
 __device__ __forceinline__ uint32_t slot_of(uint64_t key, const SlotHash& H) {

@@ -147,9 +147,10 @@ __device__ __forceinline__ uint32_t exch16(unsigned short* a, uint32_t v) {
 // compute thread issues a TMA L2 prefetch of rounds 1..SPF, then at round k of rounds k+SPF (one
 // cp.async.bulk.prefetch.L2 of NT*SPT tuples per round), so the bytes in flight per SM no longer
 // depend on the registers of the probing threads.
-// F2: two-term slot hash (slot_of2; the host picks it when the key bits above B fit in 2 lg bits)
+// F2: the cheaper slot hash (slot_of2; the host picks it for 8-byte keys and for 4-byte keys whose
+// bits above B fit in 2 lg bits). BF: branch-free first chain step for all SPT tuples of a round.
 template <typename K, int NT, int SPT, bool MAT, int RBUF, bool H16 = false, bool PF = false, bool L2PF = false,
-          int SPF = 0, bool F2 = false>
+          int SPF = 0, bool F2 = false, bool BF = true>
 __device__ __forceinline__ void join_body(const Plan& P) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -205,28 +206,30 @@ __device__ __forceinline__ void join_body(const Plan& P) {
     }
 
     // ---- first probe round's S loads (in flight during the build) --------------------------
+    // S offsets are 32-bit, relative to the item's first S tuple (an item has <= C_S < 2^31)
+    constexpr uint32_t RND = (uint32_t)NT * SPT;
+    const T* const sitem = ssrc + job.sb + threadIdx.x;
+    const uint32_t slen = (uint32_t)(job.se - job.sb);
     K sk[SPT], sp[SPT];
-    auto load_s = [&](unsigned long long base) {
-      const uint32_t rem = (uint32_t)min(job.se - base, (unsigned long long)NT * SPT);
-      const T* src = ssrc + base + threadIdx.x;
+    auto load_s = [&](uint32_t off) {
+      const uint32_t rem = min(slen - off, RND);
       #pragma unroll
       for (int j = 0; j < SPT; ++j) {
         if ((uint32_t)(j * NT) + threadIdx.x < rem) {
-          const T t = __ldcs(src + j * NT);
+          const T t = __ldcs(sitem + off + j * NT);
           sk[j] = TT::key(t);
           sp[j] = TT::pay(t);
         }
       }
     };
     T nx[PF ? SPT : 1];  // PF: the next round's tuples
-    auto load_next = [&](unsigned long long base) {
-      const uint32_t rem = (uint32_t)min(job.se - base, (unsigned long long)NT * SPT);
-      const T* src = ssrc + base + threadIdx.x;
+    auto load_next = [&](uint32_t off) {
+      const uint32_t rem = min(slen - off, RND);
       #pragma unroll
       for (int j = 0; j < SPT; ++j)
-        if ((uint32_t)(j * NT) + threadIdx.x < rem) nx[j] = __ldcs(src + j * NT);
+        if ((uint32_t)(j * NT) + threadIdx.x < rem) nx[j] = __ldcs(sitem + off + j * NT);
     };
-    load_s(job.sb);
+    load_s(0);
     for (uint32_t i = threadIdx.x; i < nb; i += NT) s_head[i] = NIL16;
     const T* s_rt = s_rtb + (RBUF == 2 ? (it & 1) * cap : 0) + job.shift;
     const uint32_t s_rt_sh = (uint32_t)__cvta_generic_to_shared(s_rt);
@@ -241,35 +244,34 @@ __device__ __forceinline__ void join_body(const Plan& P) {
     bar_compute(NT);
 
     // ---- probe (a7) + output (a8), SPT tuples per thread per round --------------------------
-    for (unsigned long long base = job.sb; base < job.se; base += (unsigned long long)NT * SPT) {
+    for (uint32_t off = 0; off < slen; off += RND) {
       if (SPF > 0 && threadIdx.x == 0) {
-        constexpr unsigned long long RND = (unsigned long long)NT * SPT;
-        const unsigned long long lo = base == job.sb ? base + RND : base + SPF * RND;
-        const unsigned long long hi = min(base + (SPF + 1) * RND, job.se);
+        const uint32_t lo = off == 0 ? RND : off + SPF * RND;
+        const uint32_t hi = min(off + (SPF + 1) * RND, slen);
         if (lo < hi) {
-          const uintptr_t a = reinterpret_cast<uintptr_t>(ssrc + lo), a0 = a & ~(uintptr_t)15;
-          const uintptr_t a1 = (reinterpret_cast<uintptr_t>(ssrc + hi) + 15) & ~(uintptr_t)15;
+          const T* sbase = ssrc + job.sb;
+          const uintptr_t a = reinterpret_cast<uintptr_t>(sbase + lo), a0 = a & ~(uintptr_t)15;
+          const uintptr_t a1 = (reinterpret_cast<uintptr_t>(sbase + hi) + 15) & ~(uintptr_t)15;
           bulk_prefetch_l2(reinterpret_cast<const void*>(a0), (uint32_t)(a1 - a0));
         }
       }
       if (PF) {
-        if (base != job.sb) {
+        if (off != 0) {
           #pragma unroll
           for (int j = 0; j < SPT; ++j) {
             sk[j] = TT::key(nx[j]);
             sp[j] = TT::pay(nx[j]);
           }
         }
-        if (base + (unsigned long long)NT * SPT < job.se) load_next(base + (unsigned long long)NT * SPT);
-      } else if (base != job.sb) {
-        load_s(base);
+        if (off + RND < slen) load_next(off + RND);
+      } else if (off != 0) {
+        load_s(off);
       }
       uint32_t idx[SPT], m[SPT];
       K rfirst[SPT];
-      // this round's tuples in the item (32-bit: rounds hold NT * SPT tuples); a full round needs
-      // no per-tuple bounds (block-uniform branch)
-      const uint32_t rem = (uint32_t)min(job.se - base, (unsigned long long)NT * SPT);
-      if (rem == NT * SPT) {
+      // this round's tuples; a full round needs no per-tuple bounds (block-uniform branch)
+      const uint32_t rem = min(slen - off, RND);
+      if (rem == RND) {
         #pragma unroll
         for (int j = 0; j < SPT; ++j) idx[j] = s_head[slot_for<F2>(sk[j], H)];
       } else {
@@ -282,12 +284,11 @@ __device__ __forceinline__ void join_body(const Plan& P) {
       // first chain step of every tuple without branches (unique build keys: chains of length
       // <= 1, so this is usually the whole probe): the head's tuple is read even for an empty
       // slot (index 0 instead, discarded), the signature is computed for every tuple and added
-      // only on a hit; the general walk below runs only while some lane still has a chain
-      // (4-byte tuples; for 8-byte tuples the branchy walk below measured faster: c5_gpu join
-      // 2.69 vs 2.84-2.90 ms)
-      bool live = sizeof(K) != 4;
+      // only on a hit; the general walk below runs only while some lane still has a chain.
+      // BF = false (the round-1 8-byte shape, one tuple per thread): every step branchy.
+      bool live = !BF;
       #pragma unroll
-      for (int j = 0; j < SPT && sizeof(K) == 4; ++j) {
+      for (int j = 0; j < SPT && BF; ++j) {
         const bool v = idx[j] != NIL16;
         const uint32_t i0 = v ? idx[j] : 0u;
         const T r = lds_tuple(s_rt_sh + i0 * (uint32_t)sizeof(T), (T*)nullptr);
@@ -302,7 +303,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
         live |= idx[j] != NIL16;
       }
       // chains of all SPT tuples advance together (independent shared-memory loads in flight)
-      while (sizeof(K) == 4 ? __any_sync(0xffffffffu, live) : live) {
+      while (BF ? __any_sync(0xffffffffu, live) : live) {
         live = false;
         #pragma unroll
         for (int j = 0; j < SPT; ++j) {
@@ -412,9 +413,9 @@ __device__ __forceinline__ void join_body(const Plan& P) {
 }
 
 template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false, bool PF = false,
-          bool L2PF = false, int SPF = 0, bool F2 = false>
+          bool L2PF = false, int SPF = 0, bool F2 = false, bool BF = true>
 __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
-  join_body<K, NT, SPT, MAT, RBUF, H16, PF, L2PF, SPF, F2>(P);
+  join_body<K, NT, SPT, MAT, RBUF, H16, PF, L2PF, SPF, F2, BF>(P);
 }
 
 }  // namespace hj
