@@ -10,7 +10,8 @@ WANT = ["gpu__time_duration.sum", "dram__bytes_read.sum", "dram__bytes_write.sum
         "l1tex__data_bank_conflicts_pipe_lsu_mem_shared_op_ld.sum",
         "l1tex__data_bank_conflicts_pipe_lsu_mem_shared_op_st.sum",
         "l1tex__data_bank_conflicts_pipe_lsu_mem_shared_op_atom.sum",
-        "lts__t_sectors_op_write.sum", "lts__t_sectors_op_read.sum"]
+        "lts__t_sectors_op_write.sum", "lts__t_requests_op_write.sum", "lts__t_sectors_op_read.sum",
+        "smsp__sass_inst_executed_op_shared_atom.sum", "l1tex__data_pipe_lsu_wavefronts_mem_shared.sum"]
 
 
 def main(path, as_json=False):
@@ -38,6 +39,9 @@ def main(path, as_json=False):
         t = val("gpu__time_duration.sum", 1e-9)
         if rd is not None and wr is not None and t:
             d["achieved_dram_GBps"] = f"{(rd + wr) / t / 1e9:.0f} GB/s (read + write / duration; cold-cache replay)"
+        ws, wq = val("lts__t_sectors_op_write.sum", 1), val("lts__t_requests_op_write.sum", 1)
+        if ws and wq:
+            d["l2_write_sectors_per_request"] = f"{ws / wq:.2f} (4 = full 128-byte lines per request)"
         st = sorted(((float(r[i] or 0), hdr[i].replace("smsp__average_warps_issue_stalled_", "")
                       .replace("_per_issue_active.ratio", "")) for i in stall), reverse=True)[:6]
         d["top_stalls"] = ", ".join(f"{n}={v:.2f}" for v, n in st)
