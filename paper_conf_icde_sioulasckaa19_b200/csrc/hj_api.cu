@@ -329,7 +329,7 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
   const size_t head_bytes = JS.h16 ? 2 : 4;
   int lg_nb = std::max(6, ilog2_ceil(CR) - nbsh);
   auto join_smem = [&](uint32_t cr, int lg) {  // R tile buffer(s) (TMA) + heads + next
-    return (size_t)rbuf * ((cr + 3) & ~1u) * tb + (head_bytes << lg) + (size_t)cr * 2;
+    return (size_t)rbuf * ((cr + 3) & ~1u) * tb + (head_bytes << lg) + (size_t)(cr + 1) * 2;
   };
   const size_t join_cap = cap_max_smem - 8 * 1024;
   while (join_smem(CR, lg_nb) > join_cap && CR > 256) {

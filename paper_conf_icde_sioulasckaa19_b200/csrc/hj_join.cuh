@@ -20,7 +20,6 @@
 
 namespace hj {
 
-constexpr uint32_t NIL16 = 0xffffu;
 
 struct JoinJob {
   uint32_t item, nr, shift;  // shift: tuples between the 16-byte aligned copy start and rb
@@ -161,7 +160,13 @@ __device__ __forceinline__ void join_body(const Plan& P) {
   T* s_rtb = reinterpret_cast<T*>(s_raw);                             // RBUF x cap tuples
   using HT = typename std::conditional<H16, unsigned short, uint32_t>::type;
   HT* s_head = reinterpret_cast<HT*>(s_rtb + RBUF * cap);             // nb
-  uint16_t* s_next = reinterpret_cast<uint16_t*>(s_head + nb);       // CR
+  uint16_t* s_next = reinterpret_cast<uint16_t*>(s_head + nb);       // CR + 1
+  // chain end. SENT (count mode with the branch-free first step): the sentinel index CR, so an
+  // empty slot's "tuple" s_rt[CR] is the tile's spare slot (read and discarded) and s_next[CR] = CR:
+  // the probe step needs no selects (c2 join 0.628 -> 0.589 ms). Materialize mode keeps 0xffff and
+  // the selects (the sentinel cost it a spill at 72 registers: c3 0.690 -> 0.707)
+  constexpr bool SENT = BF && !MAT;
+  const uint32_t NIL = SENT ? P.CR : 0xffffu;
   __shared__ JoinJob s_jobs[2];
   __shared__ __align__(8) unsigned long long s_bar[2];
   __shared__ unsigned long long s_base;
@@ -230,7 +235,8 @@ __device__ __forceinline__ void join_body(const Plan& P) {
         if ((uint32_t)(j * NT) + threadIdx.x < rem) nx[j] = __ldcs(sitem + off + j * NT);
     };
     load_s(0);
-    for (uint32_t i = threadIdx.x; i < nb; i += NT) s_head[i] = NIL16;
+    for (uint32_t i = threadIdx.x; i < nb; i += NT) s_head[i] = (HT)NIL;
+    if (SENT && threadIdx.x == 0) s_next[NIL] = (uint16_t)NIL;
     const T* s_rt = s_rtb + (RBUF == 2 ? (it & 1) * cap : 0) + job.shift;
     const uint32_t s_rt_sh = (uint32_t)__cvta_generic_to_shared(s_rt);
     mbar_wait(&s_bar[it & 1], (it >> 1) & 1);  // R chunk landed (TMA)
@@ -277,7 +283,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
       } else {
         #pragma unroll
         for (int j = 0; j < SPT; ++j)
-          idx[j] = ((uint32_t)(j * NT) + threadIdx.x < rem) ? s_head[slot_for<F2>(sk[j], H)] : NIL16;
+          idx[j] = ((uint32_t)(j * NT) + threadIdx.x < rem) ? (uint32_t)s_head[slot_for<F2>(sk[j], H)] : NIL;
       }
       #pragma unroll
       for (int j = 0; j < SPT; ++j) m[j] = 0;
@@ -289,8 +295,8 @@ __device__ __forceinline__ void join_body(const Plan& P) {
       bool live = !BF;
       #pragma unroll
       for (int j = 0; j < SPT && BF; ++j) {
-        const bool v = idx[j] != NIL16;
-        const uint32_t i0 = v ? idx[j] : 0u;
+        const bool v = idx[j] != NIL;
+        const uint32_t i0 = SENT ? idx[j] : (v ? idx[j] : 0u);  // SENT: NIL reads the spare slot (discarded)
         const T r = lds_tuple(s_rt_sh + i0 * (uint32_t)sizeof(T), (T*)nullptr);
         const bool hit = v && TT::key(r) == sk[j];
         if (MAT) rfirst[j] = TT::pay(r);
@@ -299,15 +305,15 @@ __device__ __forceinline__ void join_body(const Plan& P) {
           if (hit) my_chk += sg;  // predicated add (no selects)
         }
         m[j] = hit ? 1u : 0u;
-        idx[j] = v ? (uint32_t)s_next[i0] : NIL16;
-        live |= idx[j] != NIL16;
+        idx[j] = SENT ? (uint32_t)s_next[i0] : (v ? (uint32_t)s_next[i0] : NIL);  // SENT: s_next[NIL] = NIL
+        live |= idx[j] != NIL;
       }
       // chains of all SPT tuples advance together (independent shared-memory loads in flight)
       while (BF ? __any_sync(0xffffffffu, live) : live) {
         live = false;
         #pragma unroll
         for (int j = 0; j < SPT; ++j) {
-          if (idx[j] != NIL16) {
+          if (idx[j] != NIL) {
             const T r = lds_tuple(s_rt_sh + idx[j] * (uint32_t)sizeof(T), (T*)nullptr);
             if (TT::key(r) == sk[j]) {
               if (MAT && m[j] == 0) rfirst[j] = TT::pay(r);
@@ -315,7 +321,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
               ++m[j];
             }
             idx[j] = s_next[idx[j]];
-            live |= idx[j] != NIL16;
+            live |= idx[j] != NIL;
           }
         }
       }
@@ -370,7 +376,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
               o_s[pos] = sp[j];
             }
           } else if (m[j] > 1) {
-            for (uint32_t i = s_head[slot_for<F2>(sk[j], H)]; i != NIL16; i = s_next[i]) {
+            for (uint32_t i = s_head[slot_for<F2>(sk[j], H)]; i != NIL; i = s_next[i]) {
               const T r = s_rt[i];
               if (TT::key(r) == sk[j]) {
                 if (pos < room) {
