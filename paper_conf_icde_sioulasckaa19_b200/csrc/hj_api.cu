@@ -522,6 +522,7 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   P.out_cap = std::min(c->out_r.bytes, c->out_s.bytes) / c->pay_bytes;
   P.H.B = hp.B;
   P.H.lg = hp.lg_nb;
+  P.one = 1;
   {
     const int rem = 8 * c->key_bytes - hp.B;  // key bits above the radix field (64-bit keys fold to 32 first)
     const int bits = std::min(rem, 32);

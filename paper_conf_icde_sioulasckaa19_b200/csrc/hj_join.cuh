@@ -107,6 +107,17 @@ __device__ __forceinline__ ulonglong2 lds_tuple(uint32_t a, ulonglong2*) {
   return v;
 }
 
+__device__ __forceinline__ uint32_t lds_u32(uint32_t a) {
+  uint32_t v;
+  asm volatile("ld.shared.u32 %0, [%1];" : "=r"(v) : "r"(a));
+  return v;
+}
+__device__ __forceinline__ uint32_t lds_u16(uint32_t a) {
+  unsigned short v;
+  asm volatile("ld.shared.u16 %0, [%1];" : "=h"(v) : "r"(a));
+  return v;
+}
+
 __device__ __forceinline__ void bar_compute(int nthreads) {  // named barrier 1: compute warps only
   asm volatile("barrier.sync 1, %0;" ::"r"(nthreads) : "memory");
 }
@@ -167,6 +178,11 @@ __device__ __forceinline__ void join_body(const Plan& P) {
   // the selects (the sentinel cost it a spill at 72 registers: c3 0.690 -> 0.707)
   constexpr bool SENT = BF && !MAT;
   const uint32_t NIL = SENT ? P.CR : 0xffffu;
+  // SENT: shared addresses as base + index * size with the sizes runtime values (P.one == 1), so
+  // they are IMADs on the FMA pipe rather than LEAs on the ALU pipe (the count probe is ALU-bound)
+  const uint32_t tmul = (uint32_t)sizeof(T) * P.one, hmul = (uint32_t)sizeof(HT) * P.one, nmul = 2u * P.one;
+  const uint32_t s_head_sh = (uint32_t)__cvta_generic_to_shared(s_head);
+  const uint32_t s_next_sh = (uint32_t)__cvta_generic_to_shared(s_next);
   __shared__ JoinJob s_jobs[2];
   __shared__ __align__(8) unsigned long long s_bar[2];
   __shared__ unsigned long long s_base;
@@ -279,7 +295,9 @@ __device__ __forceinline__ void join_body(const Plan& P) {
       const uint32_t rem = min(slen - off, RND);
       if (rem == RND) {
         #pragma unroll
-        for (int j = 0; j < SPT; ++j) idx[j] = s_head[slot_for<F2>(sk[j], H)];
+        for (int j = 0; j < SPT; ++j)
+          idx[j] = SENT ? (H16 ? lds_u16(s_head_sh + slot_for<F2>(sk[j], H) * hmul) : lds_u32(s_head_sh + slot_for<F2>(sk[j], H) * hmul))
+                        : (uint32_t)s_head[slot_for<F2>(sk[j], H)];
       } else {
         #pragma unroll
         for (int j = 0; j < SPT; ++j)
@@ -297,7 +315,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
       for (int j = 0; j < SPT && BF; ++j) {
         const bool v = idx[j] != NIL;
         const uint32_t i0 = SENT ? idx[j] : (v ? idx[j] : 0u);  // SENT: NIL reads the spare slot (discarded)
-        const T r = lds_tuple(s_rt_sh + i0 * (uint32_t)sizeof(T), (T*)nullptr);
+        const T r = lds_tuple(s_rt_sh + i0 * (SENT ? tmul : (uint32_t)sizeof(T)), (T*)nullptr);
         const bool hit = v && TT::key(r) == sk[j];
         if (MAT) rfirst[j] = TT::pay(r);
         if (!MAT || chk) {
@@ -305,7 +323,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
           if (hit) my_chk += sg;  // predicated add (no selects)
         }
         m[j] = hit ? 1u : 0u;
-        idx[j] = SENT ? (uint32_t)s_next[i0] : (v ? (uint32_t)s_next[i0] : NIL);  // SENT: s_next[NIL] = NIL
+        idx[j] = SENT ? lds_u16(s_next_sh + i0 * nmul) : (v ? (uint32_t)s_next[i0] : NIL);  // SENT: s_next[NIL] = NIL
         live |= idx[j] != NIL;
       }
       // chains of all SPT tuples advance together (independent shared-memory loads in flight)

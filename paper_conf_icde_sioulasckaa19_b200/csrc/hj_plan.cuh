@@ -90,6 +90,7 @@ struct Plan {
   unsigned long long out_cap;
   unsigned long long tiles1[2];  // pass-1 tiles per relation (host-known)
   SlotHash H;            // in-partition slot hash (lg = log2 of hash-table slots per join item)
+  uint32_t one;          // 1 (a runtime multiplier: keeps index * size an IMAD, see k_join)
   int mat_chk;           // MATERIALIZE also accumulates the checksum (HJ_OPT_MAT_CHECKSUM, default 1)
   __host__ __device__ int pb() const { return g + b1; }
   __host__ __device__ int qbits() const { return g + B; }
