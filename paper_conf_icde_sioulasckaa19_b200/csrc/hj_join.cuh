@@ -196,6 +196,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
   K* out_s = (K*)P.out_s;
   const T* ssrc = (const T*)P.rel[1].t2;
   unsigned long long my_cnt = 0, my_chk = 0;
+  uint32_t my_cnt32 = 0;  // count mode: this thread's matches in the current round
   // checksum in MATERIALIZE mode too (block-uniform; the pairs' signatures are summed in the first
   // chain walk, so re-walks of multi-match tuples only write)
   const bool chk = !MAT || P.mat_chk != 0;
@@ -322,7 +323,8 @@ __device__ __forceinline__ void join_body(const Plan& P) {
           const uint64_t sg = pair_sig((uint64_t)TT::pay(r), (uint64_t)sp[j]);
           if (hit) my_chk += sg;  // predicated add (no selects)
         }
-        m[j] = hit ? 1u : 0u;
+        if (MAT) m[j] = hit ? 1u : 0u;
+        else if (hit) ++my_cnt32;  // count mode: one predicated add, no per-tuple match counts
         idx[j] = SENT ? lds_u16(s_next_sh + i0 * nmul) : (v ? (uint32_t)s_next[i0] : NIL);  // SENT: s_next[NIL] = NIL
         live |= idx[j] != NIL;
       }
@@ -336,18 +338,23 @@ __device__ __forceinline__ void join_body(const Plan& P) {
             if (TT::key(r) == sk[j]) {
               if (MAT && m[j] == 0) rfirst[j] = TT::pay(r);
               if (!MAT || chk) my_chk += pair_sig((uint64_t)TT::pay(r), (uint64_t)sp[j]);
-              ++m[j];
+              if (MAT) ++m[j];
+              else ++my_cnt32;
             }
             idx[j] = s_next[idx[j]];
             live |= idx[j] != NIL;
           }
         }
       }
-      uint32_t mt = 0;
-      #pragma unroll
-      for (int j = 0; j < SPT; ++j) mt += m[j];
-      my_cnt += mt;
+      if (!MAT) {  // a round adds < SPT * C_R <= 2^20 matches per thread
+        my_cnt += my_cnt32;
+        my_cnt32 = 0;
+      }
       if (MAT) {
+        uint32_t mt = 0;
+        #pragma unroll
+        for (int j = 0; j < SPT; ++j) mt += m[j];
+        my_cnt += mt;
         const uint32_t wsum = __reduce_add_sync(0xffffffffu, mt);
         if (lane == 0) s_wsum[warp] = wsum;
         bar_compute(NT);
