@@ -26,8 +26,11 @@ def main():
     ap.add_argument("--opt", default="join_variant")
     ap.add_argument("--values", type=int, nargs="+", default=[0])
     ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--bits", type=int, default=None, help="radix bits instead of the config's")
     a = ap.parse_args()
     w = W.CONFIGS[a.config]
+    if a.bits is not None:
+        w = w.with_(radix_bits=a.bits)
     cols = W.torch_generate(w, device="cuda")
     ref = None
     for v in a.values:  # join_variant: 0 = auto, k = shape k-1
