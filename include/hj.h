@@ -68,7 +68,7 @@ enum hj_option {
   HJ_OPT_TIMING = 4,       /* 1 = record per-phase CUDA events into hj_result (default 1)     */
   HJ_OPT_BLOCKS_PER_SM = 5, /* persistent-grid residency override for the passes (0 = auto)   */
   HJ_OPT_JOIN_VARIANT = 6,  /* join kernel shape (tuning; 0 = auto, k = shape k-1 of hj_api.cu's
-                               JOIN_SHAPES, 1..8)                                                */
+                               JOIN_SHAPES, 1..9)                                                */
   HJ_OPT_PASS_THREADS = 7,  /* partition-pass block size 512 / 1024 (0 = auto)                   */
   HJ_OPT_JOIN_ALGO = 9,     /* 0 = radix-partitioned + smem hash table (default); 1 = radix-
                                partitioned + ballot nested loops (Listing 1); 2 = non-

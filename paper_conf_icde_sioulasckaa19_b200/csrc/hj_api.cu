@@ -49,6 +49,7 @@ constexpr JoinShape JOIN_SHAPES[] = {
     {224, 8, 4, 1, 1, true},                   // 5: 16-bit heads, 4 blocks / SM
     {512, 2, 2, 1, 1, false, true, true, 0, false},  // 6: 8 B, two tuples per thread (c5_gpu join 2.71 vs 2.45 ms)
     {512, 2, 2, 1, 1, false, true, true},             // 7: 8 B, branch-free first step (2.60 ms; 256 x 4: 3.23)
+    {512, 1, 2, 1, 0, false, true, true, 0, false},  // 8: 8 B default: shape 2 with twice the hash slots
 };
 constexpr int JOIN_NVARIANTS = sizeof(JOIN_SHAPES) / sizeof(JOIN_SHAPES[0]);
 constexpr int HIST_NT = 1024;
@@ -235,13 +236,16 @@ constexpr int pass_items() {
 //                      probe, 0.646 after)
 //   4 B count       -> shape 0 (256 x 6, next round's S in registers + L2 prefetch of the next
 //                      item: c2 0.873 -> 0.814 ms; streaming S through L2 was slower here)
-//   8 B             -> shape 2 (512 x 1, two blocks per SM: the 16-byte R tile limits blocks to
+//   8 B             -> shape 8 (512 x 1, two blocks per SM: the 16-byte R tile limits blocks to
 //                      two per SM, so more threads per block -- not more tuples per thread --
-//                      hide the chain-walk latency: c5_gpu join 3.54 -> 2.69 ms; 512 x 2: 2.90,
-//                      640 x 1: 2.85, 768 x 1: 3.34)
+//                      hide the chain-walk latency: c5_gpu join 3.54 -> 2.69 ms in round 1; 512 x 2:
+//                      2.90, 640 x 1: 2.85, 768 x 1: 3.34) with twice the hash slots: fmix64 keys hash
+//                      to random slots, so chains at load factor 1 average 1.5 entries per hit (2.45
+//                      -> 2.16 ms; 16-bit heads with 2x / 4x slots 2.56 / 2.82, branch-free first
+//                      step 2.30-2.40; 4-byte dense keys hash without collisions: c2 2x slots 0.58 -> 0.63)
 int join_variant(const Ctx* c, bool mat) {
   if (c->opt_join_variant >= 0) return (int)c->opt_join_variant;
-  if (c->key_bytes == 8) return 2;
+  if (c->key_bytes == 8) return 8;
   return mat ? 1 : 0;
 }
 
@@ -448,6 +452,7 @@ int set_kernel_attrs(Ctx* c) {
   attr_join<K, 5>(attr);
   attr_join<K, 6>(attr);
   attr_join<K, 7>(attr);
+  attr_join<K, 8>(attr);
   return rc;
 }
 
@@ -762,6 +767,8 @@ int launch_join(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
     case 5: rc = launch_join_v<K, 5>(c, hp, P, mat); break;
     case 6: rc = launch_join_v<K, 6>(c, hp, P, mat); break;
     case 7: rc = launch_join_v<K, 7>(c, hp, P, mat); break;
+    case 8: rc = launch_join_v<K, 8>(c, hp, P, mat); break;
+
 
     default: rc = launch_join_v<K, 0>(c, hp, P, mat); break;
   }

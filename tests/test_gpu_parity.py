@@ -123,7 +123,7 @@ def test_knob_invariance_block_nested_loops(hj, cap_r, chunk_s):
     ctx.close()
 
 
-JOIN_SHAPES = 8  # number of k_join shapes in hj_api.cu (HJ_OPT_JOIN_VARIANT 1..8)
+JOIN_SHAPES = 9  # number of k_join shapes in hj_api.cu (HJ_OPT_JOIN_VARIANT 1..9)
 
 
 @pytest.mark.parametrize("variant", range(1, JOIN_SHAPES + 1))
