@@ -39,5 +39,6 @@ for graph in (0, 1):
                          ctypes.byref(res))
     raw = (time.perf_counter() - t1) / N * 1e3
     print(f"{w.name} graph={graph}: device events {e0.elapsed_time(e1) / N:.3f} ms/call, in-call ms_total "
-          f"{dev / N:.3f}, wall {wall:.3f} ms/call, raw C-ABI call {raw:.3f} ms/call", flush=True)
+          f"{dev / N:.3f}, wall {wall:.3f} ms/call, raw C-ABI call {raw:.3f} ms/call, "
+          f"kernels {[round(x, 3) for x in r.ms_kernel]}", flush=True)
     ctx.close()
