@@ -254,9 +254,12 @@ int pass_threads(const Ctx* c, int fanout_bits, int items) {
   return (512 * items) >> fanout_bits >= 32 ? 512 : 1024;
 }
 
-// the warp-specialized pass (hj_pass_ws.cuh) for a fan-out of 2^bits: histogram partitioner,
-// fan-out <= WS_MAXF (shared-memory budget); its unit is a 64 KB tile
-bool use_ws(const Ctx* c, int bits) { return c->opt_pass_ws && c->opt_partitioner == 0 && (1 << bits) <= WS_MAXF; }
+// the warp-specialized pass (hj_pass_ws.cuh) for a fan-out of 2^bits: fan-out <= WS_MAXF
+// (shared-memory budget); its unit is a 60 KB tile. The bucket-chain partitioner has it for the
+// default role split only.
+bool use_ws(const Ctx* c, int bits) {
+  return c->opt_pass_ws && (1 << bits) <= WS_MAXF && (c->opt_partitioner == 0 || c->opt_pass_ws == 1);
+}
 // role split: HJ_OPT_PASS_WS = 1 (default: 20 compute warps; measured on B200, c3 pass 1 / pass 2:
 // 16 warps x 16 tuples 1.01 / 0.97 ms (spills), 18: 0.82 / 0.87, 20: 0.80 / 0.82, 21: 0.81 / 0.83,
 // 22: 0.84 / 0.85, 24 x 8 tuples: 0.93 / 0.93; the lock-step k_pass: 0.94 / 0.85) or an explicit
@@ -390,6 +393,8 @@ void for_ws_variants(F&& attr) {
   attr((const void*)k_pass_ws<K, 2, false, N>);
   WS_CWS(WS_ATTR_CASE)
 #undef WS_ATTR_CASE
+  attr((const void*)k_pass_ws<K, 1, false, 20, true>);
+  attr((const void*)k_pass_ws<K, 2, false, 20, true>);
 }
 
 template <typename K>
@@ -640,22 +645,23 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false, 
 }
 
 // a3 / a4: one partition pass (launch shape per pass and width).
-template <typename K, int MODE, bool GD, int CW>
+template <typename K, int MODE, bool GD, int CW, bool BC = false>
 int launch_pass_ws(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
   using S = WsShape<K, CW>;
-  const void* f = (const void*)k_pass_ws<K, MODE, GD, CW>;
+  const void* f = (const void*)k_pass_ws<K, MODE, GD, CW, BC>;
   const size_t sm = S::smem(fanout_bits);
   const unsigned long long tile = S::TILE;
   Plan Q = P;
   Q.C2 = (uint32_t)tile;
-  const unsigned long long units = MODE == 1 ? (P.rel[0].n + tile - 1) / tile + (P.rel[1].n + tile - 1) / tile
-                                             : (P.rel[0].n + P.rel[1].n) / tile + 2ull * hp.npieces() + 2;
+  unsigned long long units = MODE == 1 ? (P.rel[0].n + tile - 1) / tile + (P.rel[1].n + tile - 1) / tile
+                                       : (P.rel[0].n + P.rel[1].n) / tile + 2ull * hp.npieces() + 2;
+  if (BC && MODE == 2) units = (P.rel[0].n + P.rel[1].n) / tile + P.bc_rel[0].nbmax1 + P.bc_rel[1].nbmax1 + 2;
   if (MODE == 1) {
     Q.tiles1[0] = (P.rel[0].n + tile - 1) / tile;
     Q.tiles1[1] = (P.rel[1].n + tile - 1) / tile;
   }
   const int g = grid_for(c, f, WS_NT, sm, units);
-  k_pass_ws<K, MODE, GD, CW><<<g, WS_NT, sm, c->stream>>>(Q, fanout_bits);
+  k_pass_ws<K, MODE, GD, CW, BC><<<g, WS_NT, sm, c->stream>>>(Q, fanout_bits);
   CUDA_TRY(c, cudaGetLastError());
   c->launches += 1;
   return HJ_OK;
@@ -664,6 +670,11 @@ int launch_pass_ws(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
 template <typename K, int MODE, int NT, bool GD, bool BC>
 int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
   constexpr int IT = pass_items<K>();
+  if constexpr (BC && !GD) {
+    // pass 2 keeps the pass-1 bucket list in static shared memory (32 KB): fan-out <= 2^8
+    if (use_ws(c, fanout_bits) && (MODE == 1 ? hp.tile : hp.C2) == ws_tile(c) && (MODE == 1 || fanout_bits <= 8))
+      return launch_pass_ws<K, MODE, GD, 20, true>(c, hp, P, fanout_bits);
+  }
   if (!BC && use_ws(c, fanout_bits) && (MODE == 1 ? hp.tile : hp.C2) == ws_tile(c)) {
     // warp-specialized pipeline: one 1024-thread block per SM
 #define WS_LAUNCH_CASE(N) \

@@ -22,8 +22,12 @@
 // no role waits on another's shared-memory buffer except through the three-stage ring.
 // Units whose input is ragged or not 16-byte aligned (the last unit of a relation, a piece whose
 // aligned superset would leave the pass-1 data) are loaded by the compute warps from global.
+// BC = true: the paper's bucket-chain partitioner (hj_bucket.cuh, NEXT-1): runs are reserved in
+// the partitions' buckets (bc_reserve) instead of at histogram offsets, and pass 2's units are
+// the pass-1 buckets cut into tiles (bucket at a time); the roles are unchanged.
 #pragma once
 #include "hj_common.cuh"
+#include "hj_partition.cuh"
 #include "hj_plan.cuh"
 
 namespace hj {
@@ -58,9 +62,11 @@ struct WsUnit {
   uint32_t valid;
   uint32_t tma;    // input is in the stage (else: load from global)
   uint32_t shift;  // MODE 2: tuples between the stage start and the unit's first tuple
+  uint32_t rel;    // bucket chains: relation, and the partition index of the unit's digit 0
+  uint32_t pbase;
 };
 
-template <typename K, int MODE, bool GD, int CW>
+template <typename K, int MODE, bool GD, int CW, bool BC = false>
 __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -78,7 +84,10 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
   __shared__ WsUnit s_desc[4];
   __shared__ uint32_t s_wt[CT / 32];
   __shared__ uint32_t s_hot, s_hot_next;
-  __shared__ uint32_t s_cst[MODE == 2 ? 2 * 1025 : 1];
+  __shared__ uint32_t s_cst[MODE == 2 ? (BC ? 2 * BC_MAX_NB1 : 2 * 1025) : 1];
+  __shared__ uint32_t s_bfill[MODE == 2 && BC ? 2 * BC_MAX_NB1 : 1];  // bucket chains: pass-1 bucket fills
+  __shared__ uint16_t s_bd[MODE == 2 && BC ? 2 * BC_MAX_NB1 : 1];     // and their partitions D
+  __shared__ BcRel s_bc[BC ? 2 : 1];
 
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   if (MODE == 2 && P.mode == PLAN_RECV && *(volatile const uint32_t*)&P.counters[CNT_BAD_COUNTS]) return;
@@ -92,9 +101,21 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
   };
 
   unsigned long long units0, units;
+  if (BC) {
+    if (threadIdx.x == 0) {
+      s_bc[0] = P.bc_rel[0];
+      s_bc[1] = P.bc_rel[1];
+    }
+    __syncthreads();
+  }
   if (MODE == 1) {
     units0 = P.tiles1[0];
     units = units0 + P.tiles1[1];
+  } else if (BC) {  // pass-1 buckets -> shared unit prefix (all threads)
+    bc_pass2_units<WS_NT, TILE>(s_bc, P.counters, 1u << P.b1, s_cst, s_bfill, s_bd);
+    __syncthreads();
+    units0 = s_cst[2 * BC_MAX_NB1 - 3];
+    units = s_cst[2 * BC_MAX_NB1 - 4];
   } else {
     const uint32_t npc = P.npieces();  // <= 1024
     for (uint32_t i = threadIdx.x; i <= npc; i += WS_NT) {
@@ -130,15 +151,36 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
       D.valid = u < units;
       D.tma = 0;
       D.shift = 0;
+      D.pbase = 0;
       if (D.valid) {
         const int r = u < units0 ? 0 : 1;
         const RelDev& R = P.rel[r];
         const unsigned long long ul = r ? u - units0 : u;
-        if (MODE == 1) {
+        D.rel = r;
+        if (BC && MODE == 2) {  // unit -> (pass-1 bucket, tile) by binary search over the unit prefix
+          const BcRel& Bc = s_bc[r];
+          const uint32_t* cst = s_cst + r * BC_MAX_NB1;
+          const uint32_t uc = (uint32_t)ul;
+          uint32_t lo = 0, hi = s_cst[2 * BC_MAX_NB1 - 1 - r];  // buckets of r; largest with cst[b] <= uc
+          while (hi - lo > 1) {
+            const uint32_t mid = (lo + hi) >> 1;
+            if (cst[mid] <= uc) lo = mid; else hi = mid;
+          }
+          const uint32_t k = uc - cst[lo];
+          D.src_k = (const T*)Bc.pool1 + (unsigned long long)lo * Bc.bsz1 + (unsigned long long)k * TILE;
+          D.src_p = nullptr;
+          D.dst = Bc.pool2;
+          D.pbase = (uint32_t)s_bd[r * BC_MAX_NB1 + lo] << P.b2;
+          D.cur = nullptr;
+          D.len = min((uint32_t)TILE, s_bfill[r * BC_MAX_NB1 + lo] - k * TILE);
+          // bucket strides are tile multiples (16-byte aligned); the rounded-up copy stays inside
+          // the bucket's stride (fill < cap + tile = bsz1)
+          D.tma = 1;
+        } else if (MODE == 1) {
           const unsigned long long s0 = ul * TILE;
           D.src_k = (const K*)R.keys + s0;
           D.src_p = (const K*)R.pays + s0;
-          D.dst = R.t1;
+          D.dst = BC ? P.bc_rel[r].pool1 : R.t1;
           D.cur = R.cur1;
           D.len = (uint32_t)min((unsigned long long)TILE, R.n - s0);
           D.tma = D.len == TILE && ((reinterpret_cast<uintptr_t>(D.src_k) | reinterpret_cast<uintptr_t>(D.src_p)) & 15) == 0;
@@ -314,7 +356,7 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
     // the global atomic's round trip overlaps the shuffle (the writer reads gd after s_done)
     unsigned long long* gd = s_gd + (i % 3) * F;
     unsigned long long rres = 0;
-    uint32_t rloc = 0;
+    uint32_t rloc = 0, rcnt = 0;
     bool rv = false;
     if (threadIdx.x < nscan) {
       const uint32_t d = threadIdx.x;
@@ -334,8 +376,12 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
         s_loc[d] = loc;
         s_cnt[d] = 0;
         if (c) {
-          rres = atomicAdd(D.cur + d, (unsigned long long)c);
+          if (BC)  // the state's old value: finished (fast path or close / wait) after the shuffle
+            rres = bc_reserve_issue<MODE>(&s_bc[D.rel], D.pbase + d, c);
+          else
+            rres = atomicAdd(D.cur + d, (unsigned long long)c);
           rloc = loc;
+          rcnt = c;
           rv = true;
         }
         if (c > TILE / 4) atomicExch(&s_hot_next, d);  // predicts the next unit's hot digit
@@ -356,6 +402,9 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
 #else
         s_t[s_loc[digit(kk[j])] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = TT::make(kk[j], pp[j]);
 #endif
+    if (BC && rv)
+      rres = bc_reserve_finish<MODE>(&s_bc[D.rel], &P.counters[(MODE == 1 ? CNT_BC_NB1 : CNT_BC_NB2) + D.rel],
+                                     &P.results[RES_BC_OVERFLOW], D.pbase + threadIdx.x, rcnt, rres);
     if (rv) gd[threadIdx.x] = rres - rloc;
     __syncwarp();
     if (lane == 0) mbar_arrive(&s_done[stage]);  // unit i is ready for the writer
