@@ -46,6 +46,8 @@ def parse():
     ap.add_argument("--e2e-steps", type=int, default=3)
     ap.add_argument("--clock-period", type=float, default=0.01,
                     help="NVML clock / throttle sampling period (s) during the timed region; 0 = off (testing only)")
+    ap.add_argument("--sync-calls", action="store_true",
+                    help="one synchronous hj_join per timed step instead of K queued hj_join_async calls")
     ap.add_argument("--dist", action="store_true", help="use the multi-GPU exchange path even at N=1")
     ap.add_argument("--debug-one-device", action="store_true",
                     help="testing only: every rank on cuda:0 with a gloo process group (validates the multi-rank "
@@ -341,15 +343,23 @@ def main():
         e1 = torch.cuda.Event(enable_timing=True)
         e0.record(stream)
         results = []
-        for _ in range(args.steps):
-            res = step()
+        if not use_dist and not args.sync_calls:
+            # hj_join_async: the K joins are queued back to back on the stream (each call's host
+            # preparation overlaps the previous call's kernels); hj_sync returns every step's result
+            for _ in range(args.steps):
+                ctx.join_async(Rk, Rp, Sk, Sp, radix_bits=w.radix_bits, out_mode=w.out_mode)
+            e1.record(stream)
+            outs = ctx.sync()
+        else:
+            outs = [step() for _ in range(args.steps)]
+            e1.record(stream)
+        for res in outs:
             results.append((res.matches, res.checksum))
             loc = res if not use_dist else res.local
             per_k += np.array(loc.ms_kernel)
             # + the sender side: direct = hist, plan, count rows, pass 1, barrier; nccl = (hist, plan, pass 1) x 2
             launches += loc.kernels if not use_dist else loc.kernels + (5 if args.exchange == "direct" else 6)
             sent += 0 if not use_dist else res.sent_bytes
-        e1.record(stream)
         barrier()
     bad = [k for k, r in enumerate(results) if r != expect]
     assert not bad, f"timed steps {bad[:5]} differ from the closed form {expect}"
@@ -392,6 +402,9 @@ def main():
            "config": {"workload": workload_desc(w), "radix_bits": loc.radix_bits, "passes": loc.passes,
                       "join_items": loc.n_items,
                       "l2": "inputs larger than L2 (2 GiB in + 4 GiB partition buffers vs 126 MB L2); no flush",
+                      "calls": ("hj_join_async x K queued on the stream, one hj_sync; every step's result "
+                                "returned and validated" if not use_dist and not args.sync_calls else
+                                "one synchronous call per step"),
                       "parallelism": "1 GPU" if not use_dist else
                       f"{ws} rank(s): rows sharded, radix exchange "
                       + ("fused into pass 1 (direct peer stores, hj_xd_*)" if args.exchange == "direct"

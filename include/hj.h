@@ -165,6 +165,28 @@ int hj_join(hj_ctx* ctx,
             const void* S_keys, const void* S_pay, uint64_t nS,
             int radix_bits, int out_mode, hj_result* res);
 
+/* Asynchronous hj_join: the same work, enqueued on ctx's stream; returns once it is enqueued
+ * (host preparation of the next call overlaps this one's kernels: queued back to back, the
+ * kernels of consecutive joins leave no host round trip between them). *res is caller-owned and
+ * is filled by hj_sync (or by any later call on ctx that completes it); the column pointers must
+ * stay valid until then. At most HJ_MAX_PENDING calls are pending per ctx: one more first
+ * completes the oldest. Every other call on ctx that touches its buffers (hj_join, hj_join_host,
+ * hj_partition, the exchange calls, hj_set_workspace, hj_set_stream to another stream, hj_destroy)
+ * first completes all pending calls and fails with the first of their errors, if any.
+ * MATERIALIZE: pending calls share the ctx's output buffer, so once hj_sync returns it holds the
+ * pairs of the LAST call; a call whose pairs outgrew HJ_OPT_OUT_CAPACITY is not re-run -- its
+ * completion fails with HJ_ERR_WORKSPACE and res->matches = the exact count. Graph mode
+ * (HJ_OPT_GRAPH) and HJ_OPT_JOIN_ALGO = 2 run synchronously (res filled on return). */
+#define HJ_MAX_PENDING 8
+int hj_join_async(hj_ctx* ctx,
+                  const void* R_keys, const void* R_pay, uint64_t nR,
+                  const void* S_keys, const void* S_pay, uint64_t nS,
+                  int radix_bits, int out_mode, hj_result* res);
+
+/* Complete every pending hj_join_async call of ctx, in issue order (each one's *res filled).
+ * Returns HJ_OK or the first failure among them (hj_last_error: its message). */
+int hj_sync(hj_ctx* ctx);
+
 /* Caller-provided device workspace (device buffers reserved up front).
  * hj_workspace_bytes: the device bytes hj_join(ctx, nR, nS, radix_bits, out_mode) needs with the
  *   ctx's current options (partitioner, join algorithm, HJ_OPT_OUT_CAPACITY); 0 if nR or nS is 0

@@ -53,11 +53,13 @@ _ERRORS = {-1: "HJ_ERR_INVALID", -2: "HJ_ERR_UNSUPPORTED", -3: "HJ_ERR_OOM", -4:
 
 # every symbol include/hj.h declares (checked by tests/test_abi.py)
 EXPORTS = ("hj_create", "hj_destroy", "hj_last_error", "hj_set_stream", "hj_set_option", "hj_join",
+           "hj_join_async", "hj_sync",
            "hj_workspace_bytes", "hj_set_workspace", "hj_join_host", "hj_partition", "hj_exchange_pack",
            "hj_exchange_row_len", "hj_join_received", "hj_xd_window",
            "hj_xd_header_bytes", "hj_ipc_open", "hj_ipc_close", "hj_xd_count", "hj_xd_store", "hj_xd_barrier",
            "hj_xd_join", "hj_xd_reserve", "hj_version")
 XD_MAX_RANKS = 64
+MAX_PENDING = 8         # HJ_MAX_PENDING
 XD_BOARD_BYTES = 69632  # HJ_XD_BOARD_BYTES
 XD_REGROW = 1           # HJ_XD_REGROW
 
@@ -92,9 +94,11 @@ def _load_lib():
     lib.hj_set_stream.restype = i32
     lib.hj_set_option.argtypes = [vp, i32, i64]
     lib.hj_set_option.restype = i32
-    for f in (lib.hj_join, lib.hj_join_host):
+    for f in (lib.hj_join, lib.hj_join_host, lib.hj_join_async):
         f.argtypes = [vp, vp, vp, u64, vp, vp, u64, i32, i32, ctypes.POINTER(_Result)]
         f.restype = i32
+    lib.hj_sync.argtypes = [vp]
+    lib.hj_sync.restype = i32
     lib.hj_workspace_bytes.argtypes = [vp, u64, u64, i32, i32]
     lib.hj_workspace_bytes.restype = u64
     lib.hj_set_workspace.argtypes = [vp, vp, u64]
@@ -179,12 +183,14 @@ class Context:
         self.pay_bytes = pay_bytes
         self.use_workspace = workspace
         self._ws = None  # torch uint8 tensor backing hj_join's buffers
+        self._pending = []  # join_async calls not yet returned by sync(): (result struct, columns, mode, device)
 
     def close(self):
         self._view_key = self._view_val = None  # views of memory hj_destroy frees
         if getattr(self, "_h", None):
-            _lib.hj_destroy(self._h)
+            _lib.hj_destroy(self._h)  # completes pending join_async calls first
             self._h = None
+        self._pending = []
         self._ws = None  # after hj_destroy: the ctx no longer touches it
 
     def __del__(self):
@@ -242,6 +248,37 @@ class Context:
         out = _result(res)
         if out_mode == OUT_MATERIALIZE and res.matches:
             out.r_pay, out.s_pay = self._views(res, dev_)
+        return out
+
+    def join_async(self, Rk, Rp, Sk, Sp, radix_bits: int = -1, out_mode: int = OUT_COUNT_CHECKSUM) -> int:
+        """hj_join_async: enqueue the join on torch's current stream and return at once; sync()
+        returns the results of every pending call in issue order. The columns are kept alive
+        until then. Returns the call's index in the next sync() list."""
+        import torch
+
+        cols = [_as_device_col(t, self.key_bytes if i % 2 == 0 else self.pay_bytes) for i, t in enumerate((Rk, Rp, Sk, Sp))]
+        if cols[0].numel() != cols[1].numel() or cols[2].numel() != cols[3].numel():
+            raise ValueError("key and payload columns differ in length")
+        dev_ = cols[0].device
+        self.set_stream(torch.cuda.current_stream(dev_).cuda_stream)
+        nR, nS = cols[0].numel(), cols[2].numel()
+        if self.use_workspace and nR and nS:
+            self._ensure_workspace(self.workspace_bytes(nR, nS, radix_bits, out_mode), dev_)
+        res = _Result()
+        self._check(_lib.hj_join_async(self._h, _ptr(cols[0]), _ptr(cols[1]), nR, _ptr(cols[2]), _ptr(cols[3]), nS,
+                                       radix_bits, out_mode, ctypes.byref(res)))
+        self._pending.append((res, cols, out_mode, dev_))
+        return len(self._pending) - 1
+
+    def sync(self) -> list:
+        """hj_sync: wait for every pending join_async call; their JoinResults in issue order.
+        MATERIALIZE: the pending calls share the output buffer, so only the last result carries
+        the pair views (the last call's pairs)."""
+        pend, self._pending = self._pending, []
+        self._check(_lib.hj_sync(self._h))
+        out = [_result(r) for r, _, _, _ in pend]
+        if pend and pend[-1][2] == OUT_MATERIALIZE and pend[-1][0].matches:
+            out[-1].r_pay, out[-1].s_pay = self._views(pend[-1][0], pend[-1][3])
         return out
 
     def _views(self, res, device):

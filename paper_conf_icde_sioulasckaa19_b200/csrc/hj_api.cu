@@ -62,6 +62,21 @@ struct DevBuf {
 
 struct HostPlan;
 
+// hj_join_async: a call whose result readback is enqueued but not yet waited for. Each slot owns
+// its events and pinned result words, so calls can be queued back to back on the stream.
+constexpr int MAX_PENDING = HJ_MAX_PENDING;
+struct Pending {
+  hj_result* res = nullptr;
+  cudaEvent_t ev[7] = {};
+  unsigned long long* h = nullptr;  // pinned: results readback of this call
+  int B = 0;
+  bool mat = false, bc = false, recv = false, timing = false;
+  unsigned long long out_cap = 0;
+  const void* out_r = nullptr;
+  const void* out_s = nullptr;
+  uint32_t launches = 0;
+};
+
 struct Ctx {
   int device = 0;
   int key_bytes = 4, pay_bytes = 4;
@@ -113,6 +128,12 @@ struct Ctx {
   unsigned long long graph_key[16] = {};
   bool capturing = false;  // a graph capture is in progress on c->stream
   uint32_t graph_launches = 0;
+  // hj_join_async: ring of pending calls (issue order from pend_head); `async` = the slot the
+  // call being enqueued fills (finish_join then enqueues its readback and returns)
+  Pending pend[MAX_PENDING];
+  int pend_head = 0, pend_n = 0;
+  Pending* async = nullptr;
+  cudaEvent_t ev_own[7] = {};  // the ctx's own timing events (c->ev[0..6] outside async calls)
 };
 
 int fail(Ctx* c, int code, const char* fmt, ...) {
@@ -816,7 +837,7 @@ int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res, c
   const bool timing = c->opt_timing != 0;
   int rc = c->key_bytes == 4 ? launch_join<uint32_t>(c, hp, P, mat) : launch_join<uint64_t>(c, hp, P, mat);
   if (rc) return rc;
-  unsigned long long* h = (unsigned long long*)c->h_res;
+  unsigned long long* h = c->async ? c->async->h : (unsigned long long*)c->h_res;
   if (xd) {  // hj_xd_join: phase C (results of every rank summed on the device) before the readback
     k_xd_results<<<1, XD_MAX, 0, st>>>(*xd);
     CUDA_TRY(c, cudaGetLastError());
@@ -828,6 +849,20 @@ int finish_join(Ctx* c, const HostPlan& hp, Plan& P, bool mat, hj_result* res, c
   h[5] = 0;
   if (P.mode == PLAN_RECV)
     CUDA_TRY(c, cudaMemcpyAsync(h + 5, P.counters + CNT_BAD_COUNTS, sizeof(uint32_t), cudaMemcpyDeviceToHost, st));
+  if (c->async) {  // hj_join_async: the readback is enqueued; complete_pending() finishes the call
+    Pending& q = *c->async;
+    CUDA_TRY(c, cudaEventRecord(c->ev[6], st));
+    q.B = hp.B;
+    q.mat = mat;
+    q.bc = P.bc != 0;
+    q.recv = P.mode == PLAN_RECV;
+    q.timing = timing;
+    q.out_cap = P.out_cap;
+    q.out_r = c->out_r.p;
+    q.out_s = c->out_s.p;
+    q.launches = c->launches;
+    return HJ_OK;
+  }
   if (timing) CUDA_TRY(c, cudaEventRecord(c->ev[6], st));
   CUDA_TRY(c, cudaStreamSynchronize(st));
   if (P.bc && h[RES_BC_OVERFLOW]) return fail(c, HJ_ERR_CUDA, "bucket pool overflow (pool bound violated)");
@@ -949,6 +984,58 @@ int run_join_np(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, c
     return HJ_OK;
   }
   return HJ_OK;
+}
+
+// Wait for the oldest pending hj_join_async call and fill its result (as finish_join's tail).
+// Post-hoc failures (bucket pool, received rows, output capacity) are reported here.
+int complete_pending(Ctx* c) {
+  Pending& q = c->pend[c->pend_head];
+  c->pend_head = (c->pend_head + 1) % MAX_PENDING;
+  c->pend_n--;
+  hj_result* res = q.res;
+  const unsigned long long* h = q.h;
+  CUDA_TRY(c, cudaEventSynchronize(q.ev[6]));
+  memset(res, 0, sizeof *res);
+  if (q.bc && h[RES_BC_OVERFLOW]) return fail(c, HJ_ERR_CUDA, "bucket pool overflow (pool bound violated)");
+  if (q.recv && (uint32_t)h[5])
+    return fail(c, HJ_ERR_INVALID, "received count rows describe more tuples than the received buffers hold");
+  res->matches = h[RES_MATCHES];
+  if (q.mat && res->matches > q.out_cap)  // no re-run: later calls have reused the buffers
+    return fail(c, HJ_ERR_WORKSPACE, "materialized output needs %llu pairs (capacity %llu): set "
+                "HJ_OPT_OUT_CAPACITY >= matches and call again", res->matches, q.out_cap);
+  res->checksum = h[RES_CHECKSUM];
+  res->n_items = (uint32_t)h[4];
+  res->radix_bits = q.B;
+  res->passes = q.B >= 2 ? 2 : (q.B == 1 ? 1 : 0);
+  if (q.mat) {
+    res->r_pay_out = q.out_r;
+    res->s_pay_out = q.out_s;
+  }
+  res->kernels = q.launches;
+  if (q.timing) {
+    cudaEventElapsedTime(&res->ms_total, q.ev[0], q.ev[6]);
+    cudaEventElapsedTime(&res->ms_partition, q.ev[0], q.ev[4]);
+    cudaEventElapsedTime(&res->ms_join, q.ev[4], q.ev[6]);
+    for (int k = 0; k < 5; ++k) cudaEventElapsedTime(&res->ms_kernel[k], q.ev[k], q.ev[k + 1]);
+    cudaGetLastError();
+  }
+  return HJ_OK;
+}
+
+// Complete every pending call in issue order; the first failure's code (its message stays in
+// c->err unless a later one overwrites it -- the first is kept).
+int drain_pending(Ctx* c) {
+  int first = HJ_OK;
+  std::string msg;
+  while (c->pend_n > 0) {
+    const int rc = complete_pending(c);
+    if (rc && first == HJ_OK) {
+      first = rc;
+      msg = c->err;
+    }
+  }
+  if (first) c->err = msg;
+  return first;
 }
 
 // One-shot graph path (HJ_OPT_GRAPH): kernels + result readback captured from the ctx stream;
@@ -1422,6 +1509,7 @@ int hj_create(hj_ctx** out, int device, int key_bytes, int pay_bytes, void* cuda
   }
   c->stream = cuda_stream ? (cudaStream_t)cuda_stream : c->own_stream;
   for (auto& ev : c->ev) cudaEventCreate(&ev);
+  for (int k = 0; k < 7; ++k) c->ev_own[k] = c->ev[k];
   for (auto& ev : c->sev) cudaEventCreate(&ev);
   cudaStreamCreateWithFlags(&c->h2d_stream, cudaStreamNonBlocking);
   cudaStreamCreateWithFlags(&c->d2h_stream, cudaStreamNonBlocking);
@@ -1437,6 +1525,7 @@ void hj_destroy(hj_ctx* h) {
   int prev = 0;
   cudaGetDevice(&prev);
   cudaSetDevice(c->device);
+  drain_pending(c);  // fills the results of pending hj_join_async calls
   // drain every stream this ctx issued work on before its memory is freed
   for (cudaStream_t s : {c->stream, c->own_stream, c->h2d_stream, c->d2h_stream})
     if (s) cudaStreamSynchronize(s);
@@ -1458,6 +1547,11 @@ void hj_destroy(hj_ctx* h) {
   if (c->h_out) cudaFreeHost(c->h_out);
   for (auto& ev : c->ev)
     if (ev) cudaEventDestroy(ev);
+  for (Pending& q : c->pend) {
+    for (auto& ev : q.ev)
+      if (ev) cudaEventDestroy(ev);
+    if (q.h) cudaFreeHost(q.h);
+  }
   for (auto& ev : c->sev)
     if (ev) cudaEventDestroy(ev);
   if (c->h_cur) cudaFreeHost(c->h_cur);
@@ -1475,7 +1569,12 @@ int hj_set_stream(hj_ctx* h, void* s) {
   // NULL is the caller's "stream 0", the legacy default stream (torch's default stream handle is
   // 0): work is then ordered after every kernel the caller issued there (mapping NULL
   // to the ctx's non-blocking stream let the join read columns still being written)
-  h->c.stream = s ? (cudaStream_t)s : cudaStreamLegacy;
+  const cudaStream_t ns = s ? (cudaStream_t)s : cudaStreamLegacy;
+  // pending hj_join_async calls use the ctx's buffers on the old stream: finish them before work
+  // on another stream could overlap them
+  if (ns != h->c.stream)
+    if (const int rc_ = drain_pending(&h->c)) return rc_;
+  h->c.stream = ns;
   return HJ_OK;
 }
 
@@ -1539,6 +1638,7 @@ int hj_join(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const void* 
   int rc = check_args(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode);
   if (rc) return rc;
   memset(res, 0, sizeof *res);
+  if ((rc = drain_pending(c))) return rc;
   if (nR == 0 || nS == 0) return HJ_OK;
   int prev = 0;
   cudaGetDevice(&prev);
@@ -1549,6 +1649,62 @@ int hj_join(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const void* 
   }
   rc = run_join(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
   c->use_ws = false;
+  cudaSetDevice(prev);
+  return rc;
+}
+
+int hj_join_async(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const void* Sk, const void* Sp,
+                  uint64_t nS, int radix_bits, int out_mode, hj_result* res) {
+  if (!h || !res) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  c->err.clear();
+  int rc = check_args(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode);
+  if (rc) return rc;
+  memset(res, 0, sizeof *res);
+  if (nR == 0 || nS == 0) return HJ_OK;
+  // graph replays and the non-partitioned join wait inside the call: run them synchronously
+  if (c->opt_graph || c->opt_join_algo == 2) {
+    if ((rc = drain_pending(c))) return rc;
+    return hj_join(h, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
+  }
+  if (c->pend_n == MAX_PENDING && (rc = complete_pending(c))) return rc;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  Pending& q = c->pend[(c->pend_head + c->pend_n) % MAX_PENDING];
+  if (!q.h) {
+    for (auto& ev : q.ev)
+      if (cudaEventCreate(&ev) != cudaSuccess) ev = nullptr;
+    if (cudaMallocHost(&q.h, 16 * sizeof(unsigned long long)) != cudaSuccess) q.h = nullptr;
+    if (!q.h || !q.ev[6]) {
+      cudaSetDevice(prev);
+      return fail(c, HJ_ERR_OOM, "async slot: event / pinned allocation failed");
+    }
+  }
+  q.res = res;
+  q.h[5] = 0;
+  for (int k = 0; k < 7; ++k) c->ev[k] = q.ev[k];
+  c->async = &q;
+  if (c->ws) {
+    ws_begin(c);
+    c->use_ws = true;
+  }
+  rc = run_join(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode, res);
+  c->use_ws = false;
+  c->async = nullptr;
+  for (int k = 0; k < 7; ++k) c->ev[k] = c->ev_own[k];
+  if (!rc) c->pend_n++;
+  cudaSetDevice(prev);
+  return rc;
+}
+
+int hj_sync(hj_ctx* h) {
+  if (!h) return HJ_ERR_INVALID;
+  Ctx* c = &h->c;
+  int prev = 0;
+  cudaGetDevice(&prev);
+  cudaSetDevice(c->device);
+  const int rc = drain_pending(c);
   cudaSetDevice(prev);
   return rc;
 }
@@ -1571,6 +1727,7 @@ int hj_set_workspace(hj_ctx* h, void* dptr, uint64_t bytes) {
   if (!h) return HJ_ERR_INVALID;
   Ctx* c = &h->c;
   c->err.clear();
+  if (const int rc_ = drain_pending(c)) return rc_;  // pending hj_join_async calls first
   if (dptr && ((uintptr_t)dptr & 255)) return fail(c, HJ_ERR_INVALID, "workspace must be 256-byte aligned");
   int prev = 0;
   cudaGetDevice(&prev);
@@ -1601,6 +1758,7 @@ int hj_join_host(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const v
   if (!h || !res) return HJ_ERR_INVALID;
   Ctx* c = &h->c;
   c->err.clear();
+  if (const int rc_ = drain_pending(c)) return rc_;  // pending hj_join_async calls first
   int rc = check_args(c, Rk, Rp, nR, Sk, Sp, nS, radix_bits, out_mode);
   if (rc) return rc;
   memset(res, 0, sizeof *res);
@@ -1623,6 +1781,7 @@ int hj_partition(hj_ctx* h, const void* keys, const void* pays, uint64_t n, int 
   if (!h || !tuples_out || !part_start || !part_count) return HJ_ERR_INVALID;
   Ctx* c = &h->c;
   c->err.clear();
+  if (const int rc_ = drain_pending(c)) return rc_;  // pending hj_join_async calls first
   if (radix_bits < 0 || radix_bits > 20) return fail(c, HJ_ERR_INVALID, "radix_bits must be 0..20");
   if (n && (!keys || !pays)) return fail(c, HJ_ERR_INVALID, "null column with n > 0");
   int prev = 0;
@@ -1662,6 +1821,7 @@ int hj_exchange_pack(hj_ctx* h, int rel, const void* keys, const void* pays, uin
   if (!h || !send_out || !counts_out || !dest_counts) return HJ_ERR_INVALID;
   Ctx* c = &h->c;
   c->err.clear();
+  if (const int rc_ = drain_pending(c)) return rc_;  // pending hj_join_async calls first
   if (rel != 0 && rel != 1) return fail(c, HJ_ERR_INVALID, "rel must be 0 (R) or 1 (S)");
   if (gpu_bits < 0 || gpu_bits > 10 || local_bits < 0 || local_bits > 20)
     return fail(c, HJ_ERR_INVALID, "gpu_bits 0..10, local_bits 0..20");
@@ -1706,6 +1866,7 @@ int hj_join_received(hj_ctx* h, const void* R_recv, uint64_t nR, const uint32_t*
   if (!h || !res) return HJ_ERR_INVALID;
   Ctx* c = &h->c;
   c->err.clear();
+  if (const int rc_ = drain_pending(c)) return rc_;  // pending hj_join_async calls first
   if (out_mode != HJ_OUT_COUNT_CHECKSUM && out_mode != HJ_OUT_MATERIALIZE)
     return fail(c, HJ_ERR_INVALID, "bad out_mode %d", out_mode);
   if (nsrc < 1 || nsrc > 1024 || local_bits < 0 || local_bits > 20)
@@ -1830,6 +1991,7 @@ int hj_xd_count(hj_ctx* h, const void* Rk, const void* Rp, uint64_t nR, const vo
   if (!h || !dest_counts) return HJ_ERR_INVALID;
   Ctx* c = &h->c;
   c->err.clear();
+  if (const int rc_ = drain_pending(c)) return rc_;  // pending hj_join_async calls first
   if (gpu_bits < 0 || (1 << gpu_bits) > XD_MAX || local_bits < 0 || local_bits > 20)
     return fail(c, HJ_ERR_INVALID, "gpu_bits 0..6, local_bits 0..20");
   if ((nR && (!Rk || !Rp)) || (nS && (!Sk || !Sp))) return fail(c, HJ_ERR_INVALID, "null column with n > 0");
@@ -1885,6 +2047,7 @@ int hj_xd_store(hj_ctx* h, int rank, const uint64_t* totals, void* const* win_R,
   if (!h || !totals || !win_R || !win_S) return HJ_ERR_INVALID;
   Ctx* c = &h->c;
   c->err.clear();
+  if (const int rc_ = drain_pending(c)) return rc_;  // pending hj_join_async calls first
   if (!c->xd_hp || c->xd_pst[0].empty()) return fail(c, HJ_ERR_INVALID, "hj_xd_store without hj_xd_count");
   HostPlan& hp = *c->xd_hp;
   Plan P = *c->xd_P;
@@ -1999,6 +2162,7 @@ int hj_xd_join(hj_ctx* h, int rank, int gpu_bits, const void* Rk, const void* Rp
   if (!h || !win_R || !win_S || !board || !win_bytes || !res || !totals || !all) return HJ_ERR_INVALID;
   Ctx* c = &h->c;
   c->err.clear();
+  if (const int rc_ = drain_pending(c)) return rc_;  // pending hj_join_async calls first
   if (out_mode != HJ_OUT_COUNT_CHECKSUM && out_mode != HJ_OUT_MATERIALIZE)
     return fail(c, HJ_ERR_INVALID, "bad out_mode %d", out_mode);
   if (gpu_bits < 0 || (1 << gpu_bits) > XD_MAX || local_bits < 0 || local_bits > 20)

@@ -692,3 +692,55 @@ def test_workspace_api(hj):
                                bits=3, mat=True, ctx=ctx)
     assert res.matches == 50 * 40 * 30
     ctx.close()
+
+
+def test_join_async_queue_vs_oracle(hj):
+    """hj_join_async / hj_sync: more queued calls than HJ_MAX_PENDING (the ring completes the
+    oldest), different inputs, sizes, modes and both partitioners on one ctx; every result
+    equals the oracle's, in issue order, and the last MATERIALIZE call's pairs are returned."""
+    specs = [W.Workload("a%d" % i, n, n if d == "1to1" else 3 * n + i, d, keys=k, z=1.0, seed=140 + i)
+             for i, (n, d, k) in enumerate([(1 << 15, "fk", "dense"), (40000, "zipf", "sparse"),
+                                            (1 << 16, "1to1", "sparse"), (777, "fk", "sparse")])]
+    data = [W.np_generate(w) for w in specs]
+    refs = [oracle.hash_join(*a, materialize=True) for a in data]
+    cols = [[dev(x) for x in a] for a in data]
+    for part, kb in ((0, 4), (1, 4)):
+        ctx = hj.Context(0, kb, kb)
+        ctx.set_option(hj.OPT_PARTITIONER, part)
+        order = [(i % 4, i % 3 == 2) for i in range(2 * hj.MAX_PENDING + 2)] + [(2, True)]
+        for i, mat in order:
+            ctx.join_async(*cols[i], out_mode=hj.OUT_MATERIALIZE if mat else hj.OUT_COUNT_CHECKSUM)
+        out = ctx.sync()
+        assert len(out) == len(order)
+        for (i, mat), r in zip(order, out):
+            assert (r.matches, r.checksum) == refs[i][:2], (part, i, mat)
+            assert r.kernels > 0 and r.ms_kernel[4] > 0
+        i, mat = order[-1]
+        assert mat and np.array_equal(oracle.pairs_sorted(to_np(out[-1].r_pay, 4), to_np(out[-1].s_pay, 4)),
+                                      oracle.pairs_sorted(refs[i][2], refs[i][3]))
+        # a synchronous call completes pending async calls first (their structs are filled)
+        ctx.join_async(*cols[0])
+        r = ctx.join(*cols[1])
+        assert (r.matches, r.checksum) == refs[1][:2]
+        assert [(x.matches, x.checksum) for x in ctx.sync()] == [refs[0][:2]]
+        assert ctx.sync() == []
+        ctx.close()
+
+
+def test_join_async_output_overflow_reported_at_sync(hj):
+    """A queued MATERIALIZE call whose pairs outgrow the capacity is not re-run (later calls
+    reuse the buffers): its completion fails with HJ_ERR_WORKSPACE and the exact count."""
+    lib = hj.lib()
+    ctx = hj.Context(0, 4, 4, workspace=False)
+    ctx.set_option(hj.OPT_OUT_CAPACITY, 1000)
+    Rk = np.repeat(np.arange(50, dtype=np.uint32), 40)
+    Sk = np.repeat(np.arange(60, dtype=np.uint32), 30)
+    cols = [dev(a) for a in (Rk, np.arange(len(Rk), dtype=np.uint32), Sk, np.arange(len(Sk), dtype=np.uint32))]
+    res = hj._Result()
+    ptrs = [ctypes.c_void_p(c.data_ptr()) for c in cols]
+    assert lib.hj_join_async(ctx._h, ptrs[0], ptrs[1], len(Rk), ptrs[2], ptrs[3], len(Sk), 3, 1, ctypes.byref(res)) == 0
+    assert lib.hj_sync(ctx._h) == hj.ERR_WORKSPACE
+    assert res.matches == 50 * 40 * 30
+    assert b"HJ_OPT_OUT_CAPACITY" in lib.hj_last_error(ctx._h)
+    assert lib.hj_sync(ctx._h) == 0  # nothing pending any more
+    ctx.close()
