@@ -206,6 +206,7 @@ __global__ void __launch_bounds__(1024) k_hist_recv(Plan P, uint32_t blocks_r) {
 // ------------------------------------------------------------------------------------------
 __device__ __forceinline__ unsigned long long plan_items(const Plan& P, unsigned long long cr, unsigned long long cs) {
   if (!cr || !cs) return 0ull;
+  if (cr <= P.CR && cs <= P.CS) return 1ull;  // the common case: no division (~20 instructions each)
   if (((cr | cs) >> 31) == 0)  // 32-bit division (a 64-bit one is ~10x the instructions)
     return (unsigned long long)(((uint32_t)cr + P.CR - 1) / P.CR) * (((uint32_t)cs + P.CS - 1) / P.CS);
   return ((cr + P.CR - 1) / P.CR) * ((cs + P.CS - 1) / P.CS);
@@ -225,18 +226,18 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   constexpr bool items = IT;
   // ---- prefix of everything below this block's range -------------------------------------
   unsigned long long sR = 0, sS = 0, sI = 0;
-  // batches of 8 earlier blocks: all 16 count loads are issued before any is used (the loop is
+  // batches of 16 earlier blocks: all 32 count loads are issued before any is used (the loop is
   // latency-bound: one L2 round trip per batch instead of per block)
-  for (uint32_t k0 = 0; k0 < b; k0 += 8) {
-    unsigned long long cr[8], cs[8];
+  for (uint32_t k0 = 0; k0 < b; k0 += 16) {
+    uint32_t cr[16], cs[16];
     #pragma unroll
-    for (int u = 0; u < 8; ++u) {
+    for (int u = 0; u < 16; ++u) {
       const bool ok = k0 + u < b;
-      cr[u] = ok ? plan_count(P.rel[0], nsrc, np, (k0 + u) * NT + threadIdx.x) : 0ull;
-      cs[u] = ok ? plan_count(P.rel[1], nsrc, np, (k0 + u) * NT + threadIdx.x) : 0ull;
+      cr[u] = ok ? (uint32_t)plan_count(P.rel[0], nsrc, np, (k0 + u) * NT + threadIdx.x) : 0u;
+      cs[u] = ok ? (uint32_t)plan_count(P.rel[1], nsrc, np, (k0 + u) * NT + threadIdx.x) : 0u;
     }
     #pragma unroll
-    for (int u = 0; u < 8; ++u) {
+    for (int u = 0; u < 16; ++u) {
       sR += cr[u];
       sS += cs[u];
       if (items) sI += plan_items(P, cr[u], cs[u]);
