@@ -46,6 +46,9 @@ def parse():
     ap.add_argument("--e2e-steps", type=int, default=3)
     ap.add_argument("--clock-period", type=float, default=0.01,
                     help="NVML clock / throttle sampling period (s) during the timed region; 0 = off (testing only)")
+    ap.add_argument("--partitioner", default="histogram", choices=["histogram", "bucket-chains"],
+                    help="HJ_OPT_PARTITIONER: histogram + exact placement (default) or the paper's bucket chains "
+                         "(NEXT-1; more device memory)")
     ap.add_argument("--sync-calls", action="store_true",
                     help="one synchronous hj_join per timed step instead of K queued hj_join_async calls")
     ap.add_argument("--dist", action="store_true", help="use the multi-GPU exchange path even at N=1")
@@ -290,6 +293,8 @@ def main():
     import paper_conf_icde_sioulasckaa19_b200 as hj
 
     ctx = hj.Context(local, w.key_bytes, w.key_bytes)
+    if args.partitioner == "bucket-chains":
+        ctx.set_option(hj.OPT_PARTITIONER, 1)
     Rk, Rp, Sk, Sp = W.torch_generate(w, device=dev)
     if ws > 1:
         # strong scaling: the same workload, rows sharded across ranks (inputs start row-sharded)
@@ -402,6 +407,7 @@ def main():
            "config": {"workload": workload_desc(w), "radix_bits": loc.radix_bits, "passes": loc.passes,
                       "join_items": loc.n_items,
                       "l2": "inputs larger than L2 (2 GiB in + 4 GiB partition buffers vs 126 MB L2); no flush",
+                      "partitioner": args.partitioner,
                       "calls": ("hj_join_async x K queued on the stream, one hj_sync; every step's result "
                                 "returned and validated" if not use_dist and not args.sync_calls else
                                 "one synchronous call per step"),
