@@ -45,6 +45,7 @@ OPT_PASS1_BITS = 18
 OPT_PASS_VARIANT = 19
 OPT_MAT_CHECKSUM = 20  # 1 (default): MATERIALIZE also returns the checksum
 OPT_PASS_WS = 21  # 1 (default): warp-specialized partition passes
+OPT_PASS_RANK = 22  # 0 (default): lane-private ranking at fan-outs <= 2^8; 1: one counter per digit
 ALGO_HASH, ALGO_NLJ, ALGO_NONPARTITIONED = 0, 1, 2
 
 ERR_WORKSPACE = -6
