@@ -106,10 +106,6 @@ enum hj_option {
                                that stream the previous stage out), 20 compute warps; 18/20/22 =
                                that many compute warps (tuning); 0 = every warp of the block in lock
                                step (round-1 kernel)                                                */
-  HJ_OPT_PASS_RANK = 22,    /* warp-specialized passes: 0 (default) = lane-private ranking where the
-                               fan-out is <= 2^8 (every lane counts into its own shared-memory word
-                               column: conflict-free rank atomics and base lookups); 1 = one shared
-                               counter per digit (round-1 ranking)                                 */
   HJ_OPT_MAT_CHECKSUM = 20  /* 1 (default) = MATERIALIZE also fills res->checksum (the pairs'
                                signatures are summed by the probe, so every materialized result is
                                self-checking); 0 = checksum left 0 in MATERIALIZE (measurement)   */

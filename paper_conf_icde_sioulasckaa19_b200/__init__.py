@@ -24,7 +24,7 @@ import threading
 import numpy as np
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libhj.so")
+LIB_PATH = os.environ.get("HJ_LIB") or os.path.join(_HERE, "libhj.so")  # HJ_LIB: an experimental build
 
 OUT_COUNT_CHECKSUM = 0
 OUT_MATERIALIZE = 1
@@ -45,7 +45,6 @@ OPT_PASS1_BITS = 18
 OPT_PASS_VARIANT = 19
 OPT_MAT_CHECKSUM = 20  # 1 (default): MATERIALIZE also returns the checksum
 OPT_PASS_WS = 21  # 1 (default): warp-specialized partition passes
-OPT_PASS_RANK = 22  # 0 (default): lane-private ranking at fan-outs <= 2^8; 1: one counter per digit
 ALGO_HASH, ALGO_NLJ, ALGO_NONPARTITIONED = 0, 1, 2
 
 ERR_WORKSPACE = -6

@@ -92,7 +92,7 @@ struct Ctx {
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
           opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_graph = 0, opt_pass_l2pf = 2, opt_pass1_bits = 0,
-          opt_partitioner = 0, opt_pass_variant = 0, opt_mat_chk = 1, opt_pass_ws = 1, opt_pass_rank = 0;
+          opt_partitioner = 0, opt_pass_variant = 0, opt_mat_chk = 1, opt_pass_ws = 1;
   DevBuf bc_pool1[2], bc_pool2[2], bc_meta;  // HJ_OPT_PARTITIONER = 1 (NEXT-1 bucket chains)
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2], np_heads, np_next;
@@ -411,16 +411,11 @@ void for_ws_variants(F&& attr) {
 #define WS_ATTR_CASE(N)                                 \
   attr((const void*)k_pass_ws<K, 1, false, N>);        \
   attr((const void*)k_pass_ws<K, 1, true, N>);         \
-  attr((const void*)k_pass_ws<K, 2, false, N>);        \
-  attr((const void*)k_pass_ws<K, 1, false, N, false, true>); \
-  attr((const void*)k_pass_ws<K, 1, true, N, false, true>);  \
-  attr((const void*)k_pass_ws<K, 2, false, N, false, true>);
+  attr((const void*)k_pass_ws<K, 2, false, N>);
   WS_CWS(WS_ATTR_CASE)
 #undef WS_ATTR_CASE
   attr((const void*)k_pass_ws<K, 1, false, 20, true>);
   attr((const void*)k_pass_ws<K, 2, false, 20, true>);
-  attr((const void*)k_pass_ws<K, 1, false, 20, true, true>);
-  attr((const void*)k_pass_ws<K, 2, false, 20, true, true>);
 }
 
 template <typename K>
@@ -671,11 +666,11 @@ int launch_front(Ctx* c, const HostPlan& hp, const Plan& P, bool chunk = false, 
 }
 
 // a3 / a4: one partition pass (launch shape per pass and width).
-template <typename K, int MODE, bool GD, int CW, bool BC, bool LP>
+template <typename K, int MODE, bool GD, int CW, bool BC = false>
 int launch_pass_ws(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
   using S = WsShape<K, CW>;
-  const void* f = (const void*)k_pass_ws<K, MODE, GD, CW, BC, LP>;
-  const size_t sm = S::smem(fanout_bits, LP);
+  const void* f = (const void*)k_pass_ws<K, MODE, GD, CW, BC>;
+  const size_t sm = S::smem(fanout_bits);
   const unsigned long long tile = S::TILE;
   Plan Q = P;
   Q.C2 = (uint32_t)tile;
@@ -687,28 +682,11 @@ int launch_pass_ws(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
     Q.tiles1[1] = (P.rel[1].n + tile - 1) / tile;
   }
   const int g = grid_for(c, f, WS_NT, sm, units);
-  k_pass_ws<K, MODE, GD, CW, BC, LP><<<g, WS_NT, sm, c->stream>>>(Q, fanout_bits);
+  k_pass_ws<K, MODE, GD, CW, BC><<<g, WS_NT, sm, c->stream>>>(Q, fanout_bits);
   CUDA_TRY(c, cudaGetLastError());
   c->launches += 1;
   return HJ_OK;
 }
-
-// LP (lane-private ranking) for fan-outs <= 2^WS_LP_MAXB when its counters fit next to the
-// kernel's static shared memory (HJ_OPT_PASS_RANK)
-template <typename K, int MODE, bool GD, int CW, bool BC>
-bool ws_lp(Ctx* c, int fanout_bits) {
-  if (c->opt_pass_rank == 1 || fanout_bits > WS_LP_MAXB) return false;
-  cudaFuncAttributes fa;
-  if (cudaFuncGetAttributes(&fa, (const void*)k_pass_ws<K, MODE, GD, CW, BC, true>) != cudaSuccess) return false;
-  return WsShape<K, CW>::smem(fanout_bits, true) + fa.sharedSizeBytes <= c->smem_optin;
-}
-
-template <typename K, int MODE, bool GD, int CW, bool BC = false>
-int launch_pass_ws(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
-  if (ws_lp<K, MODE, GD, CW, BC>(c, fanout_bits)) return launch_pass_ws<K, MODE, GD, CW, BC, true>(c, hp, P, fanout_bits);
-  return launch_pass_ws<K, MODE, GD, CW, BC, false>(c, hp, P, fanout_bits);
-}
-
 
 template <typename K, int MODE, int NT, bool GD, bool BC>
 int launch_pass(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
@@ -1617,10 +1595,6 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
       if (v != 0 && v != 1 && v != 18 && v != 20 && v != 22)
         return fail(c, HJ_ERR_INVALID, "pass_ws must be 0 (off), 1 (auto) or 18/20/22 compute warps");
       c->opt_pass_ws = v;
-      break;
-    case HJ_OPT_PASS_RANK:
-      if (v > 1) return fail(c, HJ_ERR_INVALID, "pass rank must be 0 (auto) or 1 (digit counters)");
-      c->opt_pass_rank = v;
       break;
     case HJ_OPT_PASS_L2PF: c->opt_pass_l2pf = v; break;
     case HJ_OPT_PASS1_BITS: c->opt_pass1_bits = v; break;

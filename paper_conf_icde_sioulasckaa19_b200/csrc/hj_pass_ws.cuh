@@ -35,7 +35,6 @@ namespace hj {
 constexpr int WS_NT = 1024;   // compute warps + writer warps + producer warp 31
 constexpr int WS_MAXF = 512;  // fan-out bound (shared-memory budget)
 constexpr int WS_NS = 3;      // stages
-constexpr int WS_LP_MAXB = 8; // lane-private ranking (LP): fan-out <= 2^8 (two 16 KB counter arrays)
 
 // Role split (HJ_OPT_PASS_WS): CW compute warps, 31 - CW writer warps; each compute thread ranks
 // CIT tuples of a unit, so a unit (tile) has CW * 32 * CIT tuples (60 KB at CW = 20, the default).
@@ -45,13 +44,9 @@ struct WsShape {
   static constexpr int CIT = sizeof(K) == 4 ? (CW <= 16 ? 16 : CW <= 23 ? 12 : 8) : (CW <= 16 ? 8 : CW <= 23 ? 6 : 4);
   static constexpr int TILE = CT * CIT;
   static constexpr uint32_t STAGE = (uint32_t)TILE * 2 * sizeof(K) + 16;  // +16: aligned superset of AoS units
-  static constexpr size_t smem(int fanout_bits, bool lp = false) {
-    // stages + s_gd (3F u64) + either s_cnt (F + 4) + s_loc (F) or, LP, two lane-counter arrays
-    // of F/2 rows x 32 words
-    return WS_NS * (size_t)STAGE + ((size_t)1 << fanout_bits) * (lp ? 24 + 128 : 32) + 16;
+  static constexpr size_t smem(int fanout_bits) {  // stages + s_gd (3F u64) + s_cnt (F + 4) + s_loc (F)
+    return WS_NS * (size_t)STAGE + ((size_t)1 << fanout_bits) * 32 + 16;
   }
-  // LP: rows of lane counters per compute warp at the largest fan-out (2^WS_LP_MAXB)
-  static constexpr int LP_RMAX = ((1 << 7) + CW - 1) / CW;
 };
 
 __device__ __forceinline__ void mbar_arrive(unsigned long long* bar) {
@@ -71,7 +66,7 @@ struct WsUnit {
   uint32_t pbase;
 };
 
-template <typename K, int MODE, bool GD, int CW, bool BC = false, bool LP = false>
+template <typename K, int MODE, bool GD, int CW, bool BC = false>
 __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -85,9 +80,6 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
   unsigned long long* s_gd = reinterpret_cast<unsigned long long*>(s_raw + WS_NS * STAGE);  // 3 x F: run base - loc
   uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_gd + 3 * F);  // F + 1 (spare for ragged lanes)
   uint32_t* s_loc = s_cnt + F + 4;                              // F
-  // LP: two arrays [F/2][32] of packed 16-bit counters, word (d >> 1) * 32 + lane holds the count
-  // of digit d among the tuples ranked by lane `lane` of any compute warp (half d & 1)
-  uint32_t* s_lc = reinterpret_cast<uint32_t*>(s_gd + 3 * F);
   __shared__ __align__(8) unsigned long long s_full[WS_NS], s_empty[WS_NS], s_done[WS_NS];
   __shared__ WsUnit s_desc[4];
   __shared__ uint32_t s_wt[CT / 32];
@@ -133,11 +125,7 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
     units0 = P.skip_r ? 0ull : P.rel[0].cst[npc];
     units = units0 + P.rel[1].cst[npc];
   }
-  if (LP) {
-    for (uint32_t i = threadIdx.x; i < 32 * F; i += WS_NT) s_lc[i] = 0;
-  } else if (threadIdx.x < F) {
-    s_cnt[threadIdx.x] = 0;
-  }
+  if (threadIdx.x < F) s_cnt[threadIdx.x] = 0;
   if (threadIdx.x == 0) {
     s_hot = s_hot_next = 0xffffffffu;
     for (int s = 0; s < WS_NS; ++s) {
