@@ -238,7 +238,7 @@ struct HostPlan {
   size_t join_smem = 0;
   int tile = 0;
   // metadata offsets (bytes) inside ctx->meta
-  size_t o_cnt[2], o_off[2], o_cur1[2], o_cur2[2], o_pst[2], o_cst[2], o_ist, o_counters, o_results;
+  size_t o_cnt[2], o_off[2], o_cur1[2], o_cur2[2], o_pst[2], o_cst[2], o_hot[2], o_ist, o_counters, o_results;
   size_t zero_bytes = 0;  // [0, zero_bytes) is memset to 0 per call
   size_t meta_bytes = 0;
   int pb() const { return g + b1; }
@@ -388,6 +388,7 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
     hp.o_cur2[r] = take(nq * 8);
     hp.o_pst[r] = take((npc + 1) * 8);
     hp.o_cst[r] = take((npc + 1) * 4);
+    hp.o_hot[r] = take((F1 + 1) * 4);
   }
   hp.o_ist = take((((size_t)1 << hp.B) + 1) * 4);
   hp.meta_bytes = o;
@@ -528,6 +529,7 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
     d.cur2 = (unsigned long long*)(m + hp.o_cur2[r]);
     d.pst = (unsigned long long*)(m + hp.o_pst[r]);
     d.cst = (uint32_t*)(m + hp.o_cst[r]);
+    d.hot = (uint32_t*)(m + hp.o_hot[r]);
     P.tiles1[r] = (ns[r] + hp.tile - 1) / hp.tile;
   }
   P.B = hp.B;

@@ -271,6 +271,40 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
     P.rel[1].cur2[q] = oS;
     if (items) P.ist[q] = (uint32_t)oI;
   }
+  // ---- pass-2 skew hints: the d2 digit holding > 1/4 of its pass-1 partition ----------------
+  // (a partition's 2^b2 bins lie in one block: b2 <= 10). k_pass_ws ranks that digit's tuples by
+  // ballot instead of on one shared counter (c4: the Zipf keys' partitions).
+  if (P.b2 > 0) {
+    __shared__ unsigned long long s_psz[2][NT];  // sizes of this block's partitions (local index)
+    __shared__ uint32_t s_hot2[2][NT];
+    const uint32_t lp = threadIdx.x >> P.b2, d2 = threadIdx.x & ((1u << P.b2) - 1);
+    s_psz[0][threadIdx.x] = s_psz[1][threadIdx.x] = 0ull;
+    s_hot2[0][threadIdx.x] = s_hot2[1][threadIdx.x] = HOT_NONE;
+    __syncthreads();
+    if (P.b2 >= 5) {  // a warp's 32 bins lie in one partition: one shared atomic per warp
+      unsigned long long wr = cr, ws = cs;
+      #pragma unroll
+      for (int o = 16; o; o >>= 1) {
+        wr += __shfl_xor_sync(0xffffffffu, wr, o);
+        ws += __shfl_xor_sync(0xffffffffu, ws, o);
+      }
+      if ((threadIdx.x & 31) == 0) {
+        if (wr) atomicAdd(&s_psz[0][lp], wr);
+        if (ws) atomicAdd(&s_psz[1][lp], ws);
+      }
+    } else {
+      if (cr) atomicAdd(&s_psz[0][lp], cr);
+      if (cs) atomicAdd(&s_psz[1][lp], cs);
+    }
+    __syncthreads();
+    if (cr && 4 * cr > s_psz[0][lp]) s_hot2[0][lp] = d2;  // at most three digits qualify; any one wins
+    if (cs && 4 * cs > s_psz[1][lp]) s_hot2[1][lp] = d2;
+    __syncthreads();
+    if (q < np && d2 == 0) {
+      P.rel[0].hot[1 + (q >> P.b2)] = s_hot2[0][lp];
+      P.rel[1].hot[1 + (q >> P.b2)] = s_hot2[1][lp];
+    }
+  }
   if (b == gridDim.x - 1 && threadIdx.x == 0) {
     P.rel[0].off[np] = bR + tR;
     P.rel[1].off[np] = bS + tS;
@@ -321,10 +355,18 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
       }
     }
   }
-  block_exclusive_scan64xM<NT, 4>(pv, s_tmp6, ptt);
+  // pass-1 skew hints: the pass-1 digit holding > 1/4 of the relation (one source only: the
+  // receiver runs no pass 1); the defaults are written before the scan, whose barriers order them
+  // before the hints written after it
+  bool hot1[2];
+  #pragma unroll
+  for (int rel = 0; rel < 2; ++rel) hot1[rel] = nsrc == 1 && i < npieces && pv[2 * rel] && 4 * pv[2 * rel] > P.rel[rel].n;
+  if (i == 0) P.rel[0].hot[0] = P.rel[1].hot[0] = HOT_NONE;
+  block_exclusive_scan64xM<NT, 4>(pv, s_tmp6, ptt);  // pv becomes the exclusive prefix
   #pragma unroll
   for (int rel = 0; rel < 2; ++rel) {
     const RelDev& R = P.rel[rel];
+    if (hot1[rel]) R.hot[0] = i;
     if (i < npieces) {
       R.pst[i] = pv[2 * rel];
       R.cst[i] = (uint32_t)pv[2 * rel + 1];

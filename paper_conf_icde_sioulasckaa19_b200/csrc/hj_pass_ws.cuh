@@ -64,6 +64,7 @@ struct WsUnit {
   uint32_t shift;  // MODE 2: tuples between the stage start and the unit's first tuple
   uint32_t rel;    // bucket chains: relation, and the partition index of the unit's digit 0
   uint32_t pbase;
+  uint32_t hot;    // the planner's skew hint for this unit's digits (RelDev::hot), HOT_NONE if none
 };
 
 template <typename K, int MODE, bool GD, int CW, bool BC = false>
@@ -85,6 +86,7 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
   __shared__ uint32_t s_wt[CT / 32];
   __shared__ uint32_t s_hot, s_hot_next;
   __shared__ uint32_t s_cst[MODE == 2 ? (BC ? 2 * BC_MAX_NB1 : 2 * 1025) : 1];
+  __shared__ uint32_t s_hint2[MODE == 2 && !BC ? 2 * 1024 : 1];  // pass-2 skew hints per piece digit
   __shared__ uint32_t s_bfill[MODE == 2 && BC ? 2 * BC_MAX_NB1 : 1];  // bucket chains: pass-1 bucket fills
   __shared__ uint16_t s_bd[MODE == 2 && BC ? 2 * BC_MAX_NB1 : 1];     // and their partitions D
   __shared__ BcRel s_bc[BC ? 2 : 1];
@@ -122,6 +124,10 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
       s_cst[i] = P.rel[0].cst[i];
       s_cst[1025 + i] = P.rel[1].cst[i];
     }
+    for (uint32_t i = threadIdx.x; i < (1u << P.pb()); i += WS_NT) {
+      s_hint2[i] = P.rel[0].hot[1 + i];
+      s_hint2[1024 + i] = P.rel[1].hot[1 + i];
+    }
     units0 = P.skip_r ? 0ull : P.rel[0].cst[npc];
     units = units0 + P.rel[1].cst[npc];
   }
@@ -143,6 +149,8 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
     if (lane != 0) return;
     const unsigned long long pend[2] = {MODE == 2 ? P.rel[0].pst[P.npieces()] : 0ull,
                                         MODE == 2 ? P.rel[1].pst[P.npieces()] : 0ull};
+    const uint32_t hint1r = MODE == 1 && !BC ? P.rel[0].hot[0] : HOT_NONE;  // pass-1 skew hints
+    const uint32_t hint1s = MODE == 1 && !BC ? P.rel[1].hot[0] : HOT_NONE;
     for (uint32_t i = 0;; ++i) {
       const uint32_t stage = i % WS_NS;
       if (i >= WS_NS) mbar_wait(&s_empty[stage], ((i / WS_NS) - 1) & 1);  // unit i-3 written out
@@ -152,6 +160,7 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
       D.tma = 0;
       D.shift = 0;
       D.pbase = 0;
+      D.hot = HOT_NONE;
       if (D.valid) {
         const int r = u < units0 ? 0 : 1;
         const RelDev& R = P.rel[r];
@@ -184,6 +193,7 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
           D.cur = R.cur1;
           D.len = (uint32_t)min((unsigned long long)TILE, R.n - s0);
           D.tma = D.len == TILE && ((reinterpret_cast<uintptr_t>(D.src_k) | reinterpret_cast<uintptr_t>(D.src_p)) & 15) == 0;
+          D.hot = r ? hint1s : hint1r;
         } else {
           const uint32_t* cst = s_cst + r * 1025;
           const uint32_t uc = (uint32_t)ul;
@@ -199,6 +209,7 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
           D.src_p = nullptr;
           D.dst = R.t2;
           D.cur = R.cur2 + ((unsigned long long)Dg << P.b2);
+          D.hot = s_hint2[r * 1024 + Dg];
           D.len = (uint32_t)min((unsigned long long)TILE, pb - s0);
           // the 16-byte aligned superset must stay inside the relation's pass-1 data
           const uintptr_t a = reinterpret_cast<uintptr_t>(D.src_k), a0 = a & ~(uintptr_t)15;
@@ -319,7 +330,10 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
 
     // ---- rank (as k_pass: lanes on the predicted hot digit are ranked by ballot) -------------
     uint32_t rk[CIT / 2];
-    const uint32_t hot = s_hot;
+    // the hot digit: the planner's hint from the histogram (exact; pass 2 takes only the hint, as
+    // its units change partition from one to the next), else in pass 1 the previous unit's
+    // (bucket chains: no histogram)
+    const uint32_t hot = D.hot != HOT_NONE ? D.hot : (MODE == 1 || BC ? s_hot : HOT_NONE);
     if (hot > F) {
       #pragma unroll
       for (int j = 0; j < CIT; ++j) {

@@ -31,7 +31,11 @@ struct RelDev {
   unsigned long long* cur2;   // [2^qbits] pass-2 reservation cursors
   unsigned long long* pst;    // [npieces + 1] pass-2 input piece starts in t1
   uint32_t* cst;              // [npieces + 1] pass-2 chunk prefix (chunks of C2 tuples per piece)
+  uint32_t* hot;              // [1 + 2^pb] skew hints from the histogram (k_plan; HOT_NONE = none):
+                              // [0] the pass-1 digit holding > 1/4 of the relation, [1 + D] the
+                              // d2 digit holding > 1/4 of pass-1 partition D (pass 2)
 };
+constexpr uint32_t HOT_NONE = 0xffffffffu;
 
 // NEXT-1: the paper's histogram-free partitioner (§III-A). Each pass writes,
 // per output partition, a chain of fixed-capacity buckets taken from a pool with atomics; no

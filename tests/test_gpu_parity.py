@@ -308,6 +308,39 @@ def test_partition_vs_oracle(hj, bits, width):
     assert int(start.max() + count[np.argmax(start)]) <= n
 
 
+@pytest.mark.parametrize("bits", [8, 11, 15])
+@pytest.mark.parametrize("width", [4, 8])
+def test_partition_skewed_vs_oracle(hj, bits, width):
+    """Steps a1-a4 on skewed keys: the planner's hot-digit hints (one pass-1 digit with > 1/4 of
+    a relation, one d2 digit with > 1/4 of a pass-1 partition) switch the passes to ballot ranking
+    for those digits; the partitions must still equal the oracle's multisets."""
+    rng = np.random.default_rng(300 + bits + width)
+    dt = np.uint32 if width == 4 else np.uint64
+    n = 400_003
+    keys = rng.integers(0, 1 << (8 * width - 1), n, dtype=np.uint64).astype(dt)
+    u = rng.random(n)
+    keys[u < 0.40] = dt(0x5A5A5A5A)          # > 1/4 of the relation: a pass-1 hint
+    keys[(u >= 0.40) & (u < 0.55)] = dt(77)  # 15 %: its pass-1 partition is mostly one d2 digit
+    pays = np.arange(n, dtype=dt)
+    ok, op, offs = oracle.radix_partition(keys, pays, 0, bits)
+    ctx = hj.context(0, width, width)
+    t, start, count = ctx.partition(dev(keys), dev(pays), bits)
+    torch.cuda.synchronize()
+    assert np.array_equal(count, np.diff(offs.astype(np.int64)).astype(np.uint64))
+    tt = t.cpu().numpy()
+    if width == 4:
+        gk = (tt.view(np.uint64) & np.uint64(0xFFFFFFFF)).astype(np.uint32)
+        gp = (tt.view(np.uint64) >> np.uint64(32)).astype(np.uint32)
+    else:
+        gk = tt[:, 0].view(np.uint64)
+        gp = tt[:, 1].view(np.uint64)
+    for p in range(1 << bits):
+        a, c = int(start[p]), int(count[p])
+        o0 = int(offs[p])
+        assert np.array_equal(np.sort(gp[a:a + c]), np.sort(op[o0:o0 + c])), f"partition {p}"
+    assert np.array_equal(gk, keys[gp.astype(np.int64)])
+
+
 def test_join_host_matches_device(hj):
     w = W.Workload("t", 1 << 15, 1 << 16, "fk", seed=121)
     Rk, Rp, Sk, Sp = W.np_generate(w)
