@@ -106,6 +106,10 @@ enum hj_option {
                                that stream the previous stage out), 20 compute warps; 18/20/22 =
                                that many compute warps (tuning); 0 = every warp of the block in lock
                                step (round-1 kernel)                                                */
+  HJ_OPT_PDL = 22,          /* 1 = the planner, the passes and the join are launched with programmatic
+                               dependent launch (each starts while its predecessor's last blocks
+                               run and waits in-kernel for its results); 0 (default) = plain
+                               stream order                                                         */
   HJ_OPT_MAT_CHECKSUM = 20  /* 1 (default) = MATERIALIZE also fills res->checksum (the pairs'
                                signatures are summed by the probe, so every materialized result is
                                self-checking); 0 = checksum left 0 in MATERIALIZE (measurement)   */

@@ -45,6 +45,7 @@ OPT_PASS1_BITS = 18
 OPT_PASS_VARIANT = 19
 OPT_MAT_CHECKSUM = 20  # 1 (default): MATERIALIZE also returns the checksum
 OPT_PASS_WS = 21  # 1 (default): warp-specialized partition passes
+OPT_PDL = 22  # 1: programmatic dependent launch between the kernels of a call
 ALGO_HASH, ALGO_NLJ, ALGO_NONPARTITIONED = 0, 1, 2
 
 ERR_WORKSPACE = -6

@@ -92,7 +92,7 @@ struct Ctx {
   // options
   int64_t opt_cap_r = 0, opt_chunk_s = 0, opt_out_cap = 0, opt_timing = 1, opt_bps = 0, opt_join_variant = -1,
           opt_pass_nt = 0, opt_stream_chunk = 0, opt_join_algo = 0, opt_graph = 0, opt_pass_l2pf = 2, opt_pass1_bits = 0,
-          opt_partitioner = 0, opt_pass_variant = 0, opt_mat_chk = 1, opt_pass_ws = 1;
+          opt_partitioner = 0, opt_pass_variant = 0, opt_mat_chk = 1, opt_pass_ws = 1, opt_pdl = 0;
   DevBuf bc_pool1[2], bc_pool2[2], bc_meta;  // HJ_OPT_PARTITIONER = 1 (NEXT-1 bucket chains)
   // workspace
   DevBuf t1[2], t2[2], meta, out_r, out_s, in[4], xsend[2], xcnt[2], np_heads, np_next;
@@ -564,6 +564,23 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   return P;
 }
 
+// launch on the ctx stream; HJ_OPT_PDL = 1: with programmatic stream serialization, so the
+// kernel (which starts with pdl_wait) is scheduled while its predecessor's last blocks run
+template <typename... KArgs, typename... Args>
+cudaError_t launch_k(Ctx* c, void (*f)(KArgs...), dim3 grid, dim3 block, size_t smem, Args... args) {
+  cudaLaunchConfig_t cfg = {};
+  cfg.gridDim = grid;
+  cfg.blockDim = block;
+  cfg.dynamicSmemBytes = smem;
+  cfg.stream = c->stream;
+  cudaLaunchAttribute at[1];
+  at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+  at[0].val.programmaticStreamSerializationAllowed = 1;
+  cfg.attrs = at;
+  cfg.numAttrs = c->opt_pdl ? 1 : 0;
+  return cudaLaunchKernelEx(&cfg, f, args...);
+}
+
 void mark(Ctx* c, int i) {
   // inside a graph capture the record must be an external event-record node to be timed
   if (c->opt_timing)
@@ -580,9 +597,9 @@ int launch_plan(Ctx* c, const HostPlan& hp, const Plan& P) {
   const unsigned g = (unsigned)((((size_t)1 << hp.qbits()) + 1023) / 1024);
   const bool ms = P.nsrc > 1, it = P.mode != PLAN_SEND;
   cudaStream_t st = c->stream;
-  if (ms) k_plan<true, true><<<g, 1024, 0, st>>>(P);
-  else if (it) k_plan<false, true><<<g, 1024, 0, st>>>(P);
-  else k_plan<false, false><<<g, 1024, 0, st>>>(P);
+  if (ms) CUDA_TRY(c, launch_k(c, k_plan<true, true>, g, 1024, 0, P));
+  else if (it) CUDA_TRY(c, launch_k(c, k_plan<false, true>, g, 1024, 0, P));
+  else CUDA_TRY(c, launch_k(c, k_plan<false, false>, g, 1024, 0, P));
   CUDA_TRY(c, cudaGetLastError());
   c->launches += 1;
   return HJ_OK;
@@ -684,7 +701,7 @@ int launch_pass_ws(Ctx* c, const HostPlan& hp, const Plan& P, int fanout_bits) {
     Q.tiles1[1] = (P.rel[1].n + tile - 1) / tile;
   }
   const int g = grid_for(c, f, WS_NT, sm, units);
-  k_pass_ws<K, MODE, GD, CW, BC><<<g, WS_NT, sm, c->stream>>>(Q, fanout_bits);
+  CUDA_TRY(c, launch_k(c, k_pass_ws<K, MODE, GD, CW, BC>, g, WS_NT, sm, Q, fanout_bits));
   CUDA_TRY(c, cudaGetLastError());
   c->launches += 1;
   return HJ_OK;
@@ -764,9 +781,11 @@ int launch_join_f(Ctx* c, const HostPlan& hp, const Plan& P, bool mat) {
                       : (const void*)k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2, S.bf>;
   int g = grid_for(c, f, S.nt + 32, hp.join_smem, 1ull << 40);
   if (mat)
-    k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2, S.bf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+    CUDA_TRY(c, launch_k(c, k_join<K, S.nt, S.spt, true, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2, S.bf>, g,
+                         S.nt + 32, hp.join_smem, P));
   else
-    k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2, S.bf><<<g, S.nt + 32, hp.join_smem, st>>>(P);
+    CUDA_TRY(c, launch_k(c, k_join<K, S.nt, S.spt, false, S.minb, S.rbuf, S.h16, S.pf, S.l2pf, S.spf, F2, S.bf>, g,
+                         S.nt + 32, hp.join_smem, P));
   CUDA_TRY(c, cudaGetLastError());
   return HJ_OK;
 }
@@ -1598,6 +1617,7 @@ int hj_set_option(hj_ctx* h, int opt, int64_t v) {
         return fail(c, HJ_ERR_INVALID, "pass_ws must be 0 (off), 1 (auto) or 18/20/22 compute warps");
       c->opt_pass_ws = v;
       break;
+    case HJ_OPT_PDL: c->opt_pdl = v ? 1 : 0; break;
     case HJ_OPT_PASS_L2PF: c->opt_pass_l2pf = v; break;
     case HJ_OPT_PASS1_BITS: c->opt_pass1_bits = v; break;
     case HJ_OPT_PARTITIONER:

@@ -234,4 +234,9 @@ __device__ __forceinline__ void block_exclusive_scan64xM(unsigned long long (&v)
   __syncthreads();
 }
 
+// Programmatic dependent launch (HJ_OPT_PDL): a kernel launched with programmatic stream
+// serialization may start while its predecessor's last blocks still run; it waits here, before
+// its first read of anything the predecessor wrote. A no-op for a normal launch.
+__device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+
 }  // namespace hj

@@ -464,6 +464,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
 template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = false, bool PF = false,
           bool L2PF = false, int SPF = 0, bool F2 = false, bool BF = true>
 __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
+  pdl_wait();
   join_body<K, NT, SPT, MAT, RBUF, H16, PF, L2PF, SPF, F2, BF>(P);
 }
 

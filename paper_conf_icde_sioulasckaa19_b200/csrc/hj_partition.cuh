@@ -217,6 +217,7 @@ __device__ __forceinline__ unsigned long long plan_count(const RelDev& R, int, u
 // MS: several sources (exchange receiver); IT: join items (not on the exchange sender). Specialised so each launch runs (and fetches) only its own code.
 template <bool MS, bool IT>
 __global__ void __launch_bounds__(1024) k_plan(Plan P) {
+  pdl_wait();
   constexpr int NT = 1024;
   __shared__ unsigned long long s_tmp6[6 * (NT / 32 + 1)];
   __shared__ bool s_last;

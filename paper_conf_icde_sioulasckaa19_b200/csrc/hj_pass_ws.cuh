@@ -91,6 +91,7 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
   __shared__ uint16_t s_bd[MODE == 2 && BC ? 2 * BC_MAX_NB1 : 1];     // and their partitions D
   __shared__ BcRel s_bc[BC ? 2 : 1];
 
+  pdl_wait();
   const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
   if (MODE == 2 && P.mode == PLAN_RECV && *(volatile const uint32_t*)&P.counters[CNT_BAD_COUNTS]) return;
   const uint32_t dsh = MODE == 1 ? 0u : (uint32_t)P.b1;

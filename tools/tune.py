@@ -18,7 +18,7 @@ OPTS = {"join_variant": hj.OPT_JOIN_VARIANT, "cap_r": hj.OPT_CAP_R, "chunk_s": h
         "stream_chunk": hj.OPT_STREAM_CHUNK, "partitioner": hj.OPT_PARTITIONER,
         "pass_l2pf": hj.OPT_PASS_L2PF, "pass1_bits": hj.OPT_PASS1_BITS,
         "pass_variant": hj.OPT_PASS_VARIANT, "mat_checksum": hj.OPT_MAT_CHECKSUM, "pass_ws": hj.OPT_PASS_WS,
-        "pass_rank": hj.OPT_PASS_RANK}
+        "pdl": hj.OPT_PDL, "timing": hj.OPT_TIMING}
 
 
 def main():
