@@ -573,6 +573,30 @@ def test_compute_sanitizer_clean(hj, tool):
     assert ("ERROR SUMMARY: 0 errors" in txt) or ("RACECHECK SUMMARY: 0 hazards" in txt), txt[-2000:]
 
 
+@pytest.mark.parametrize("timing", [1, 0])
+def test_pdl_launch_matches_oracle(hj, timing):
+    """HJ_OPT_PDL: the planner, passes and join launched with programmatic dependent launch
+    (each waits in-kernel for its predecessor) give the oracle's results, synchronous and queued,
+    with and without the per-kernel timing events between the launches."""
+    ctx = hj.Context(0, 4, 4)
+    ctx.set_option(hj.OPT_PDL, 1)
+    ctx.set_option(hj.OPT_TIMING, timing)
+    w = W.Workload("pdl", 1 << 16, 1 << 18, "zipf", keys="sparse", z=1.0, seed=197)
+    Rk, Rp, Sk, Sp = W.np_generate(w)
+    m, c, r, s = oracle.hash_join(Rk, Rp, Sk, Sp, materialize=True)
+    cols = [dev(a) for a in (Rk, Rp, Sk, Sp)]
+    for _ in range(3):
+        res = ctx.join(*cols)
+        assert (res.matches, res.checksum) == (m, c)
+    for _ in range(4):
+        ctx.join_async(*cols, out_mode=hj.OUT_MATERIALIZE)
+    for res in ctx.sync():
+        assert (res.matches, res.checksum) == (m, c)
+    res = ctx.join(*cols, out_mode=hj.OUT_MATERIALIZE)
+    assert np.array_equal(oracle.pairs_sorted(to_np(res.r_pay, 4), to_np(res.s_pay, 4)), oracle.pairs_sorted(r, s))
+    ctx.close()
+
+
 def test_graph_replay_matches_oracle(hj):
     """HJ_OPT_GRAPH: the captured launch sequence replays with identical results; a new call
     signature recaptures; materialize overflow falls back to the normal path."""

@@ -1,8 +1,8 @@
 """Turn the round's ncu captures into the committed evidence under profiles/.
 
     python tools/profile_summary.py ROUND LAUNCHES.csv FULL.ncu-rep CONFIG
-writes profiles/<ROUND>_launches.csv (our kernels only: name, grid, block, ms, DRAM bytes),
-profiles/<ROUND>_ncu_summary.md and profiles/traffic_<CONFIG>.json (DRAM bytes per launch of
+writes profiles/<ROUND>_launches_<CONFIG>.csv (our kernels only: name, grid, block, ms, DRAM bytes),
+profiles/<ROUND>_ncu_<CONFIG>.md and profiles/traffic_<CONFIG>.json (DRAM bytes per launch of
 each kernel of the last complete step, read by bench.py as roofline.traffic).
 """
 import csv
@@ -26,7 +26,7 @@ def short(name):
     return None
 
 
-def main(rnd, launches, rep, cfg):
+def main(rnd, launches, rep, cfg, outdir="profiles"):
     rows = list(csv.reader(open(launches)))
     rows = [r for r in rows if len(r) > 14 and r[0].isdigit()]
     hdr = ["ID", "Process ID", "Process Name", "Host Name", "Kernel Name", "Context", "Stream", "Block Size",
@@ -45,7 +45,7 @@ def main(rnd, launches, rep, cfg):
         else:
             scale = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9}.get(unit, 1)
             e[d["Metric Name"]] = v * scale
-    out = os.path.join("profiles", f"{rnd}_launches.csv")
+    out = os.path.join(outdir, f"{rnd}_launches_{cfg}.csv")
     with open(out, "w") as f:
         w = csv.writer(f)
         w.writerow(["launch_id", "kernel", "grid", "block", "ms", "dram_read_bytes", "dram_write_bytes", "name"])
@@ -57,7 +57,7 @@ def main(rnd, launches, rep, cfg):
     last = {}
     for k in sorted(per, key=int):
         last[per[k]["kernel"]] = per[k].get("dram__bytes_read.sum", 0) + per[k].get("dram__bytes_write.sum", 0)
-    json.dump({k: int(v) for k, v in last.items()}, open(os.path.join("profiles", f"traffic_{cfg}.json"), "w"),
+    json.dump({k: int(v) for k, v in last.items()}, open(os.path.join(outdir, f"traffic_{cfg}.json"), "w"),
               indent=1)
     # full-set summary
     import io
@@ -66,7 +66,7 @@ def main(rnd, launches, rep, cfg):
     buf = io.StringIO()
     with redirect_stdout(buf):
         ncu_main(rep)
-    with open(os.path.join("profiles", f"{rnd}_ncu_summary.md"), "w") as f:
+    with open(os.path.join(outdir, f"{rnd}_ncu_{cfg}.md"), "w") as f:
         f.write(f"# ncu --set full summary, {rnd}, config {cfg} (one step, cold-cache serialized replays)\n\n")
         f.write("```\n" + buf.getvalue() + "```\n")
     print(open(out).read())
@@ -74,4 +74,10 @@ def main(rnd, launches, rep, cfg):
 
 
 if __name__ == "__main__":
-    main(*sys.argv[1:5])
+    a = sys.argv[1:]
+    od = "profiles"
+    if "--outdir" in a:
+        i = a.index("--outdir")
+        od = a[i + 1]
+        del a[i:i + 2]
+    main(*a[:4], outdir=od)
