@@ -279,8 +279,10 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
     __shared__ unsigned long long s_psz[2][NT];  // sizes of this block's partitions (local index)
     __shared__ uint32_t s_hot2[2][NT];
     const uint32_t lp = threadIdx.x >> P.b2, d2 = threadIdx.x & ((1u << P.b2) - 1);
-    s_psz[0][threadIdx.x] = s_psz[1][threadIdx.x] = 0ull;
-    s_hot2[0][threadIdx.x] = s_hot2[1][threadIdx.x] = HOT_NONE;
+    if (threadIdx.x < (NT >> P.b2)) {  // this block's partitions
+      s_psz[0][threadIdx.x] = s_psz[1][threadIdx.x] = 0ull;
+      s_hot2[0][threadIdx.x] = s_hot2[1][threadIdx.x] = HOT_NONE;
+    }
     __syncthreads();
     if (P.b2 >= 5) {  // a warp's 32 bins lie in one partition: one shared atomic per warp
       unsigned long long wr = cr, ws = cs;
