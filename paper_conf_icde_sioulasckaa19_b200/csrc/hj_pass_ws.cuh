@@ -154,7 +154,9 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
     const uint32_t hint1s = MODE == 1 && !BC ? P.rel[1].hot[0] : HOT_NONE;
     for (uint32_t i = 0;; ++i) {
       const uint32_t stage = i % WS_NS;
-      if (i >= WS_NS) mbar_wait(&s_empty[stage], ((i / WS_NS) - 1) & 1);  // unit i-3 written out
+      // the descriptor is built before the wait for a free stage (its loads -- the unit search,
+      // the piece bounds -- overlap the wait instead of delaying the copy); it is published
+      // after the wait: slot i & 3 may still be read by the writer for unit i - 4 until then
       const unsigned long long u = blockIdx.x + (unsigned long long)i * G;
       WsUnit D;
       D.valid = u < units;
@@ -219,6 +221,7 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
           D.shift = (uint32_t)((a - a0) / sizeof(T));
         }
       }
+      if (i >= WS_NS) mbar_wait(&s_empty[stage], ((i / WS_NS) - 1) & 1);  // unit i-3 written out
       s_desc[i & 3] = D;
       unsigned char* st = s_raw + stage * STAGE;
       if (D.valid && D.tma) {
