@@ -103,7 +103,8 @@ enum hj_option {
   HJ_OPT_PASS_WS = 21,      /* partition passes (histogram partitioner, fan-out <= 2^9): 1 (default) =
                                warp-specialized pipeline (a producer warp feeding three TMA stages,
                                compute warps that rank and shuffle each stage in place, writer warps
-                               that stream the previous stage out), 20 compute warps; 18/20/22 =
+                               that stream the previous stage out), 20 compute warps (18 for 8-byte
+                               tuples on the histogram partitioner); 18/20/22 =
                                that many compute warps (tuning); 0 = every warp of the block in lock
                                step (round-1 kernel)                                                */
   HJ_OPT_PDL = 22,          /* 1 = the planner, the passes and the join are launched with programmatic
