@@ -259,11 +259,7 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
       #pragma unroll 4
       for (uint32_t e = wt; e < len; e += WT) {
         const T t = s_t[e];
-#if defined(HJ_WS_DIAG) && (HJ_WS_DIAG & 4)  // timing experiment only: no run bases, sequential stores
-        __stcs(dst + e, t);  // (every tile to the same place: the writes stay in L2)
-#else
         __stcs(dst + (gd[digit(TT::key(t))] + e), t);
-#endif
       }
       __syncwarp();
       if (lane == 0) mbar_arrive(&s_empty[stage]);
@@ -415,11 +411,7 @@ __global__ void __launch_bounds__(WS_NT, 1) k_pass_ws(Plan P, int fanout_bits) {
     #pragma unroll
     for (int j = 0; j < CIT; ++j)
       if (full || elem(j) < ulen)
-#if defined(HJ_WS_DIAG) && (HJ_WS_DIAG & 2)  // timing experiment only: conflict-free shuffle
-        s_t[elem(j)] = TT::make(kk[j], pp[j] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu) + s_loc[digit(kk[j]) & 7]);
-#else
         s_t[s_loc[digit(kk[j])] + ((rk[j / 2] >> (16 * (j & 1))) & 0xffffu)] = TT::make(kk[j], pp[j]);
-#endif
     if (BC && rv)
       rres = bc_reserve_finish<MODE>(&s_bc[D.rel], &P.counters[(MODE == 1 ? CNT_BC_NB1 : CNT_BC_NB2) + D.rel],
                                      &P.results[RES_BC_OVERFLOW], D.pbase + threadIdx.x, rcnt, rres);
