@@ -238,7 +238,7 @@ struct HostPlan {
   size_t join_smem = 0;
   int tile = 0;
   // metadata offsets (bytes) inside ctx->meta
-  size_t o_cnt[2], o_off[2], o_cur1[2], o_cur2[2], o_pst[2], o_cst[2], o_hot[2], o_ist, o_counters, o_results;
+  size_t o_cnt[2], o_off[2], o_cur1[2], o_cur2[2], o_pst[2], o_cst[2], o_hot[2], o_ist, o_ist2, o_counters, o_results;
   size_t zero_bytes = 0;  // [0, zero_bytes) is memset to 0 per call
   size_t meta_bytes = 0;
   int pb() const { return g + b1; }
@@ -399,6 +399,7 @@ int make_plan(Ctx* c, HostPlan& hp, unsigned long long nR, unsigned long long nS
     hp.o_hot[r] = take((F1 + 1) * 4);
   }
   hp.o_ist = take((((size_t)1 << hp.B) + 1) * 4);
+  hp.o_ist2 = take((((size_t)1 << hp.B) + 1) * 4);
   hp.meta_bytes = o;
   (void)nS;
   return HJ_OK;
@@ -555,6 +556,7 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   P.CR = hp.CR;
   P.CS = hp.CS;
   P.ist = (uint32_t*)(m + hp.o_ist);
+  P.ist2 = (uint32_t*)(m + hp.o_ist2);
   P.counters = (uint32_t*)(m + hp.o_counters);
   P.results = (unsigned long long*)(m + hp.o_results);
   P.mat_chk = c->opt_mat_chk ? 1 : 0;
@@ -1169,6 +1171,7 @@ int run_join_bc(Ctx* c, const void* Rk, const void* Rp, unsigned long long nR, c
   }
   Plan P = device_plan(c, hp, Rk, Rp, nR, Sk, Sp, nS);
   P.bc = 1;
+  P.ist2 = nullptr;  // the bucket-chain planner makes no swapped items
   const size_t tb = sizeof(typename Tup<K>::T);
   const unsigned long long ns[2] = {nR, nS}, F1 = 1ull << hp.b1, np = 1ull << hp.B;
   const uint32_t tile1 = (uint32_t)hp.tile, C2 = hp.C2;

@@ -29,21 +29,24 @@ struct JoinJob {
 
 // Claim the next work item and decode it (item -> co-partition q by binary search over the
 // planner's item prefix; then the R chunk and S chunk of q it covers). One lane.
-template <typename T>
+// SWAP: an item of a swapped co-partition (P.ist2): the build chunk is its S side (one chunk), the
+// probe chunk one C_S-sized chunk of its R side.
+template <typename T, bool SWAP = false>
 __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items) {
   JoinJob j;
-  j.item = atomicAdd(&P.counters[CNT_NEXT_ITEM], 1u);
+  j.item = atomicAdd(&P.counters[SWAP ? CNT_NEXT_ITEM2 : CNT_NEXT_ITEM], 1u);
   j.nr = j.shift = 0;
   j.rb = j.sb = j.se = 0;
   if (j.item < total_items) {
     const uint32_t np = 1u << P.B;
+    const uint32_t* ist = SWAP ? P.ist2 : P.ist;
     uint32_t lo = 0, hi = np;  // largest q with ist[q] <= item
     while (hi - lo > 1) {
       const uint32_t mid = (lo + hi) >> 1;
-      if (P.ist[mid] <= j.item) lo = mid; else hi = mid;
+      if (ist[mid] <= j.item) lo = mid; else hi = mid;
     }
     const uint32_t q = lo;
-    if (P.bc) {  // bucket chains (NEXT-1): item = (R slice, S slice) of q, slices from k_bc_slices
+    if (!SWAP && P.bc) {  // bucket chains (NEXT-1): item = (R slice, S slice) of q, slices from k_bc_slices
       const uint32_t loc = j.item - P.ist[q], nsch = P.bc_rel[1].sst[q + 1] - P.bc_rel[1].sst[q];
       const uint4 rs = P.bc_rel[0].sl[P.bc_rel[0].sst[q] + loc / nsch];
       const uint4 ss = P.bc_rel[1].sl[P.bc_rel[1].sst[q] + loc % nsch];
@@ -55,25 +58,26 @@ __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items
       j.shift = (uint32_t)((a & 15) / sizeof(T));
       return j;
     }
-    const unsigned long long r0 = P.rel[0].off[q], rn = P.rel[0].off[q + 1] - r0;
-    const unsigned long long s0 = P.rel[1].off[q], sn = P.rel[1].off[q + 1] - s0;
+    // build side (rel SWAP) and probe side (rel !SWAP)
+    const unsigned long long r0 = P.rel[SWAP ? 1 : 0].off[q], rn = P.rel[SWAP ? 1 : 0].off[q + 1] - r0;
+    const unsigned long long s0 = P.rel[SWAP ? 0 : 1].off[q], sn = P.rel[SWAP ? 0 : 1].off[q + 1] - s0;
     const unsigned long long nsch = (sn + P.CS - 1) / P.CS;
-    const unsigned long long loc = j.item - P.ist[q];
+    const unsigned long long loc = j.item - ist[q];
     const unsigned long long rc = loc / nsch, sc = loc % nsch;
     j.rb = r0 + rc * P.CR;
     j.nr = (uint32_t)min((unsigned long long)P.CR, rn - rc * P.CR);
     j.sb = s0 + sc * P.CS;
     j.se = j.sb + min((unsigned long long)P.CS, sn - sc * P.CS);
-    const uintptr_t a = reinterpret_cast<uintptr_t>((const T*)P.rel[0].t2 + j.rb);
+    const uintptr_t a = reinterpret_cast<uintptr_t>((const T*)P.rel[SWAP ? 1 : 0].t2 + j.rb);
     j.shift = (uint32_t)((a & 15) / sizeof(T));  // tuples between the 16 B aligned copy start and rb
   }
   return j;
 }
 
 // TMA bulk copy of a job's R chunk (the 16-byte aligned superset) into an smem tile buffer.
-template <typename T>
+template <typename T, bool SWAP = false>
 __device__ __forceinline__ void issue_r_copy(const Plan& P, const JoinJob& j, T* buf, unsigned long long* bar) {
-  const uintptr_t a = reinterpret_cast<uintptr_t>((const T*)P.rel[0].t2 + j.rb);
+  const uintptr_t a = reinterpret_cast<uintptr_t>((const T*)P.rel[SWAP ? 1 : 0].t2 + j.rb);
   const uintptr_t a0 = a & ~(uintptr_t)15;
   const uint32_t bytes = (uint32_t)(((a + (uintptr_t)j.nr * sizeof(T) - a0) + 15) & ~(uintptr_t)15);
   fence_proxy_async();  // prior generic-proxy reads of buf (the item before last) are ordered before
@@ -83,15 +87,15 @@ __device__ __forceinline__ void issue_r_copy(const Plan& P, const JoinJob& j, T*
 
 // L2 prefetch of a claimed item's R chunk and first probe round (TMA prefetch, no smem): the
 // R copy issued after the end-of-item barrier and the first S loads then hit L2.
-template <typename T>
+template <typename T, bool SWAP = false>
 __device__ __forceinline__ void prefetch_item_l2(const Plan& P, const JoinJob& j, uint32_t s_round) {
   auto pf = [](const T* b, unsigned long long n) {
     const uintptr_t a = reinterpret_cast<uintptr_t>(b), a0 = a & ~(uintptr_t)15;
     const uintptr_t a1 = (a + n * sizeof(T) + 15) & ~(uintptr_t)15;
     if (a1 > a0) bulk_prefetch_l2(reinterpret_cast<const void*>(a0), (uint32_t)(a1 - a0));
   };
-  pf((const T*)P.rel[0].t2 + j.rb, j.nr);
-  pf((const T*)P.rel[1].t2 + j.sb, min((unsigned long long)s_round, j.se - j.sb));
+  pf((const T*)P.rel[SWAP ? 1 : 0].t2 + j.rb, j.nr);
+  pf((const T*)P.rel[SWAP ? 0 : 1].t2 + j.sb, min((unsigned long long)s_round, j.se - j.sb));
 }
 
 // a tuple of the R tile from its 32-bit shared-window address (keeps the tile base in a register:
@@ -160,8 +164,15 @@ __device__ __forceinline__ uint32_t exch16(unsigned short* a, uint32_t v) {
 // depend on the registers of the probing threads.
 // F2: the cheaper slot hash (slot_of2; the host picks it for 8-byte keys and for 4-byte keys whose
 // bits above B fit in 2 lg bits). BF: branch-free first chain step for all SPT tuples of a round.
+// the pair signature of (build tuple, probe tuple) payloads: sig(r_pay, s_pay) (SWAP: the build
+// side is S)
+template <bool SWAP>
+__device__ __forceinline__ uint64_t sig_bp(uint64_t build_pay, uint64_t probe_pay) {
+  return SWAP ? pair_sig(probe_pay, build_pay) : pair_sig(build_pay, probe_pay);
+}
+
 template <typename K, int NT, int SPT, bool MAT, int RBUF, bool H16 = false, bool PF = false, bool L2PF = false,
-          int SPF = 0, bool F2 = false, bool BF = true>
+          int SPF = 0, bool F2 = false, bool BF = true, bool SWAP = false>
 __device__ __forceinline__ void join_body(const Plan& P) {
   using TT = Tup<K>;
   using T = typename TT::T;
@@ -188,12 +199,12 @@ __device__ __forceinline__ void join_body(const Plan& P) {
   __shared__ __align__(8) unsigned long long s_bar[2];
   __shared__ unsigned long long s_red[2][NT / 32 + 1];
 
-  const uint32_t total_items = P.ist[1u << P.B];
+  const uint32_t total_items = (SWAP ? P.ist2 : P.ist)[1u << P.B];
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   const bool sched = threadIdx.x >= NT;
   K* out_r = (K*)P.out_r;
   K* out_s = (K*)P.out_s;
-  const T* ssrc = (const T*)P.rel[1].t2;
+  const T* ssrc = (const T*)P.rel[SWAP ? 0 : 1].t2;  // the probe side
   unsigned long long my_cnt = 0, my_chk = 0;
   uint32_t my_cnt32 = 0;  // count mode: this thread's matches in the current round
   // checksum in MATERIALIZE mode too (block-uniform; the pairs' signatures are summed in the first
@@ -204,8 +215,8 @@ __device__ __forceinline__ void join_body(const Plan& P) {
     mbar_init(&s_bar[0], 1);
     mbar_init(&s_bar[1], 1);
     fence_mbar_init();
-    JoinJob j = claim_job<T>(P, total_items);
-    if (j.item < total_items) issue_r_copy<T>(P, j, s_rtb, &s_bar[0]);
+    JoinJob j = claim_job<T, SWAP>(P, total_items);
+    if (j.item < total_items) issue_r_copy<T, SWAP>(P, j, s_rtb, &s_bar[0]);
     s_jobs[0] = j;
   }
   __syncthreads();
@@ -216,13 +227,14 @@ __device__ __forceinline__ void join_body(const Plan& P) {
     if (sched) {
       JoinJob j;
       if (lane == 0) {
-        j = claim_job<T>(P, total_items);
-        if (L2PF && RBUF == 1 && j.item < total_items) prefetch_item_l2<T>(P, j, NT * SPT);
-        if (RBUF == 2 && j.item < total_items) issue_r_copy<T>(P, j, s_rtb + ((it + 1) & 1) * cap, &s_bar[(it + 1) & 1]);
+        j = claim_job<T, SWAP>(P, total_items);
+        if (L2PF && RBUF == 1 && j.item < total_items) prefetch_item_l2<T, SWAP>(P, j, NT * SPT);
+        if (RBUF == 2 && j.item < total_items)
+          issue_r_copy<T, SWAP>(P, j, s_rtb + ((it + 1) & 1) * cap, &s_bar[(it + 1) & 1]);
         s_jobs[(it + 1) & 1] = j;
       }
       bar_item(NT + 32);  // end-of-item barrier (matches the compute warps' one below)
-      if (RBUF == 1 && lane == 0 && j.item < total_items) issue_r_copy<T>(P, j, s_rtb, &s_bar[(it + 1) & 1]);
+      if (RBUF == 1 && lane == 0 && j.item < total_items) issue_r_copy<T, SWAP>(P, j, s_rtb, &s_bar[(it + 1) & 1]);
       continue;
     }
 
@@ -319,7 +331,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
         const bool hit = v && TT::key(r) == sk[j];
         if (MAT) rfirst[j] = TT::pay(r);
         if (!MAT || chk) {
-          const uint64_t sg = pair_sig((uint64_t)TT::pay(r), (uint64_t)sp[j]);
+          const uint64_t sg = sig_bp<SWAP>((uint64_t)TT::pay(r), (uint64_t)sp[j]);
           if (hit) my_chk += sg;  // predicated add (no selects)
         }
         if (MAT) m[j] = hit ? 1u : 0u;
@@ -337,7 +349,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
               const T r = lds_tuple(s_rt_sh + idx[j] * (uint32_t)sizeof(T), (T*)nullptr);
               if (TT::key(r) == sk[j]) {
                 if (MAT && m[j] == 0) rfirst[j] = TT::pay(r);
-                if (!MAT || chk) my_chk += pair_sig((uint64_t)TT::pay(r), (uint64_t)sp[j]);
+                if (!MAT || chk) my_chk += sig_bp<SWAP>((uint64_t)TT::pay(r), (uint64_t)sp[j]);
                 if (MAT) ++m[j];
                 else ++my_cnt32;
               }
@@ -359,7 +371,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
               const T r = lds_tuple(s_rt_sh + idx[j] * (uint32_t)sizeof(T), (T*)nullptr);
               if (TT::key(r) == sk[j]) {
                 if (m[j] == 0) rfirst[j] = TT::pay(r);
-                else if (!MAT || chk) my_chk += pair_sig((uint64_t)TT::pay(r), (uint64_t)sp[j]);
+                else if (!MAT || chk) my_chk += sig_bp<SWAP>((uint64_t)TT::pay(r), (uint64_t)sp[j]);
                 ++m[j];
               }
               idx[j] = s_next[idx[j]];
@@ -370,7 +382,7 @@ __device__ __forceinline__ void join_body(const Plan& P) {
         #pragma unroll
         for (int j = 0; j < SPT; ++j) {
           if (!MAT || chk) {
-            const uint64_t sg = pair_sig((uint64_t)rfirst[j], (uint64_t)sp[j]);
+            const uint64_t sg = sig_bp<SWAP>((uint64_t)rfirst[j], (uint64_t)sp[j]);
             if (m[j]) my_chk += sg;
           }
           if (!MAT) my_cnt32 += m[j];
@@ -416,16 +428,16 @@ __device__ __forceinline__ void join_body(const Plan& P) {
           pos0 += wtot;
           if (m[j] == 1) {
             if (pos < room) {
-              o_r[pos] = rfirst[j];
-              o_s[pos] = sp[j];
+              o_r[pos] = SWAP ? sp[j] : rfirst[j];
+              o_s[pos] = SWAP ? rfirst[j] : sp[j];
             }
           } else if (m[j] > 1) {
             for (uint32_t i = s_head[slot_for<F2>(sk[j], H)]; i != NIL; i = s_next[i]) {
               const T r = s_rt[i];
               if (TT::key(r) == sk[j]) {
                 if (pos < room) {
-                  o_r[pos] = TT::pay(r);
-                  o_s[pos] = sp[j];
+                  o_r[pos] = SWAP ? sp[j] : TT::pay(r);
+                  o_s[pos] = SWAP ? TT::pay(r) : sp[j];
                 }
                 ++pos;
               }
@@ -466,6 +478,10 @@ template <typename K, int NT, int SPT, bool MAT, int MINB, int RBUF, bool H16 = 
 __global__ void __launch_bounds__(NT + 32, MINB) k_join(Plan P) {
   pdl_wait();
   join_body<K, NT, SPT, MAT, RBUF, H16, PF, L2PF, SPF, F2, BF>(P);
+  if (P.ist2 != nullptr && !P.bc) {  // then the swapped items (usually none: one load, then exit)
+    __syncthreads();
+    join_body<K, NT, SPT, MAT, RBUF, H16, PF, L2PF, SPF, F2, BF, true>(P);
+  }
 }
 
 }  // namespace hj

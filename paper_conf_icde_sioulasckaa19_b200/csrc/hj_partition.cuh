@@ -214,6 +214,17 @@ __device__ __forceinline__ unsigned long long plan_items(const Plan& P, unsigned
 
 __device__ __forceinline__ unsigned long long plan_count(const RelDev& R, int, uint32_t, uint32_t q) { return R.cnt[q]; }
 
+// a co-partition is swapped when its R side needs several C_R chunks while its S side fits one:
+// its items build on S and probe with C_S-sized R chunks (a duplicate-heavy build side would
+// otherwise walk chains of identical keys in single lanes)
+__device__ __forceinline__ bool plan_swapped(const Plan& P, unsigned long long cr, unsigned long long cs) {
+  return P.ist2 != nullptr && cr > P.CR && cs && cs <= P.CR;
+}
+__device__ __forceinline__ unsigned long long plan_items_swapped(const Plan& P, unsigned long long cr) {
+  if ((cr >> 31) == 0) return ((uint32_t)cr + P.CS - 1) / P.CS;  // 32-bit division (the common case)
+  return (cr + P.CS - 1) / P.CS;
+}
+
 // MS: several sources (exchange receiver); IT: join items (not on the exchange sender). Specialised so each launch runs (and fetches) only its own code.
 template <bool MS, bool IT>
 __global__ void __launch_bounds__(1024) k_plan(Plan P) {
@@ -226,7 +237,7 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   const int nsrc = MS ? P.nsrc : 1;
   constexpr bool items = IT;
   // ---- prefix of everything below this block's range -------------------------------------
-  unsigned long long sR = 0, sS = 0, sI = 0;
+  unsigned long long sR = 0, sS = 0, sI = 0, sI2 = 0;
   // batches of 16 earlier blocks: all 32 count loads are issued before any is used (the loop is
   // latency-bound: one L2 round trip per batch instead of per block)
   for (uint32_t k0 = 0; k0 < b; k0 += 16) {
@@ -241,7 +252,10 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
     for (int u = 0; u < 16; ++u) {
       sR += cr[u];
       sS += cs[u];
-      if (items) sI += plan_items(P, cr[u], cs[u]);
+      if (items) {
+        if (plan_swapped(P, cr[u], cs[u])) sI2 += plan_items_swapped(P, cr[u]);
+        else sI += plan_items(P, cr[u], cs[u]);
+      }
     }
   }
   // T2's 64-byte tails (the join's 16-byte aligned R copies may read into them; streaming S
@@ -260,17 +274,24 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
   }
   // the block totals of the prefix (reductions: exclusive scans whose totals are used) and this
   // range's three scans, all in ONE multi-value scan (one pair of barriers)
-  unsigned long long v[6] = {sR, sS, sI, cr, cs, items ? plan_items(P, cr, cs) : 0ull}, tt[6];
+  // the normal and the swapped item counts share one scan value (low / high 32 bits: the item
+  // totals are < 2^32, the join's item indices are u32)
+  const bool swp = items && plan_swapped(P, cr, cs);
+  const unsigned long long it2 = (items && !swp ? plan_items(P, cr, cs) : 0ull) |
+                                 (swp ? plan_items_swapped(P, cr) : 0ull) << 32;
+  unsigned long long v[6] = {sR, sS, sI | sI2 << 32, cr, cs, it2}, tt[6];
   block_exclusive_scan64xM<NT, 6>(v, s_tmp6, tt);
-  const unsigned long long bR = tt[0], bS = tt[1], bI = tt[2];
-  const unsigned long long tR = tt[3], tS = tt[4], tI = tt[5];
-  const unsigned long long oR = bR + v[3], oS = bS + v[4], oI = bI + v[5];
+  const unsigned long long bR = tt[0], bS = tt[1], bI = tt[2] & 0xffffffffull, bI2 = tt[2] >> 32;
+  const unsigned long long tR = tt[3], tS = tt[4], tI = tt[5] & 0xffffffffull, tI2 = tt[5] >> 32;
+  const unsigned long long oR = bR + v[3], oS = bS + v[4];
+  const unsigned long long oI = bI + (v[5] & 0xffffffffull), oI2 = bI2 + (v[5] >> 32);
   if (q < np) {
     P.rel[0].off[q] = oR;
     P.rel[0].cur2[q] = oR;
     P.rel[1].off[q] = oS;
     P.rel[1].cur2[q] = oS;
     if (items) P.ist[q] = (uint32_t)oI;
+    if (items && P.ist2) P.ist2[q] = (uint32_t)oI2;
   }
   // ---- pass-2 skew hints: the d2 digit holding > 1/4 of its pass-1 partition ----------------
   // (a partition's 2^b2 bins lie in one block: b2 <= 10). k_pass_ws ranks that digit's tuples by
@@ -317,6 +338,7 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
       if (bad) P.counters[CNT_BAD_COUNTS] = 1u;  // pass 2 and the join then do nothing
     }
     if (items) P.ist[np] = bad ? 0u : (uint32_t)(bI + tI);
+    if (items && P.ist2) P.ist2[np] = bad ? 0u : (uint32_t)(bI2 + tI2);
   }
   // ---- last block: piece starts, pass-1 cursors, pass-2 chunk lists (npieces <= 1024) ------
   __threadfence();
@@ -354,7 +376,10 @@ __global__ void __launch_bounds__(1024) k_plan(Plan P) {
       const unsigned long long got = __ldcg(&R.off[(unsigned long long)(i + 1) << b2]) - __ldcg(&R.off[(unsigned long long)i << b2]);
       if (sent != got) {
         P.counters[CNT_BAD_COUNTS] = 1u;
-        if (rel == 0) P.ist[1u << P.B] = 0u;
+        if (rel == 0) {
+          P.ist[1u << P.B] = 0u;
+          if (P.ist2) P.ist2[1u << P.B] = 0u;
+        }
       }
     }
   }

@@ -86,6 +86,9 @@ struct Plan {
   uint32_t C2;           // pass-2 chunk (tile) size in tuples
   uint32_t CR, CS;       // join item capacities: R tuples (smem build) and S tuples per item
   uint32_t* ist;         // [2^B + 1] join item prefix (q-order)
+  uint32_t* ist2;        // [2^B + 1] prefix of the SWAPPED items (null: none): co-partitions whose R
+                         // side needs more than one C_R chunk while S fits one (duplicate-heavy
+                         // build side) are joined building on S and probing with R chunks
   uint32_t* counters;    // [8]: 0 next join item, 1 planner blocks done, 2..5 bucket-chain counters,
                          //      6 bad received counts
   unsigned long long* results;  // [4]: 0 matches, 1 checksum, 2 output cursor, 3 bucket pool overflow
@@ -119,7 +122,7 @@ __device__ __forceinline__ uint32_t qbin(K key, const Plan& P) {
 
 // counters[CNT_BAD_COUNTS]: the exchange receiver's planner found count rows that do not sum
 // to the tuples received (pass 2 and the join then do nothing; hj_join_received fails)
-enum { CNT_NEXT_ITEM = 0, CNT_PLAN_DONE = 1, CNT_BAD_COUNTS = 6 };
+enum { CNT_NEXT_ITEM = 0, CNT_PLAN_DONE = 1, CNT_BAD_COUNTS = 6, CNT_NEXT_ITEM2 = 7 };
 enum { RES_MATCHES = 0, RES_CHECKSUM = 1, RES_CURSOR = 2 };
 
 }  // namespace hj
