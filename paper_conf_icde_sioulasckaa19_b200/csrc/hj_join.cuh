@@ -61,13 +61,16 @@ __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items
     // build side (rel SWAP) and probe side (rel !SWAP)
     const unsigned long long r0 = P.rel[SWAP ? 1 : 0].off[q], rn = P.rel[SWAP ? 1 : 0].off[q + 1] - r0;
     const unsigned long long s0 = P.rel[SWAP ? 0 : 1].off[q], sn = P.rel[SWAP ? 0 : 1].off[q + 1] - s0;
-    const unsigned long long nsch = (sn + P.CS - 1) / P.CS;
+    // probe chunks: C_S tuples; swapped items probe C_R-sized R chunks (more items: a duplicate-
+    // heavy probe side keeps many blocks busy)
+    const unsigned long long CSx = SWAP ? P.CR : P.CS;
+    const unsigned long long nsch = (sn + CSx - 1) / CSx;
     const unsigned long long loc = j.item - ist[q];
     const unsigned long long rc = loc / nsch, sc = loc % nsch;
     j.rb = r0 + rc * P.CR;
     j.nr = (uint32_t)min((unsigned long long)P.CR, rn - rc * P.CR);
-    j.sb = s0 + sc * P.CS;
-    j.se = j.sb + min((unsigned long long)P.CS, sn - sc * P.CS);
+    j.sb = s0 + sc * CSx;
+    j.se = j.sb + min(CSx, sn - sc * CSx);
     const uintptr_t a = reinterpret_cast<uintptr_t>((const T*)P.rel[SWAP ? 1 : 0].t2 + j.rb);
     j.shift = (uint32_t)((a & 15) / sizeof(T));  // tuples between the 16 B aligned copy start and rb
   }
