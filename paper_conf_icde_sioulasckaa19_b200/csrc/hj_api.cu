@@ -554,6 +554,8 @@ Plan device_plan(Ctx* c, const HostPlan& hp, const void* Rk, const void* Rp, uns
   // slower (c3 0.939 -> 0.983), pass 2 unchanged -> auto (2) = on for 8-byte keys only
   P.pass_l2pf = c->opt_pass_l2pf == 2 ? (c->key_bytes == 8) : (c->opt_pass_l2pf ? 1 : 0);
   P.CR = hp.CR;
+  P.lgCRp = 0;
+  while ((2u << P.lgCRp) <= hp.CR) ++P.lgCRp;
   P.CS = hp.CS;
   P.ist = (uint32_t*)(m + hp.o_ist);
   P.ist2 = (uint32_t*)(m + hp.o_ist2);

@@ -61,9 +61,9 @@ __device__ __forceinline__ JoinJob claim_job(const Plan& P, uint32_t total_items
     // build side (rel SWAP) and probe side (rel !SWAP)
     const unsigned long long r0 = P.rel[SWAP ? 1 : 0].off[q], rn = P.rel[SWAP ? 1 : 0].off[q + 1] - r0;
     const unsigned long long s0 = P.rel[SWAP ? 0 : 1].off[q], sn = P.rel[SWAP ? 0 : 1].off[q + 1] - s0;
-    // probe chunks: C_S tuples; swapped items probe C_R-sized R chunks (more items: a duplicate-
-    // heavy probe side keeps many blocks busy)
-    const unsigned long long CSx = SWAP ? P.CR : P.CS;
+    // probe chunks: C_S tuples; swapped items probe R chunks of 2^lgCRp <= C_R tuples (more items:
+    // a duplicate-heavy probe side keeps many blocks busy)
+    const unsigned long long CSx = SWAP ? 1ull << P.lgCRp : (unsigned long long)P.CS;
     const unsigned long long nsch = (sn + CSx - 1) / CSx;
     const unsigned long long loc = j.item - ist[q];
     const unsigned long long rc = loc / nsch, sc = loc % nsch;

@@ -215,15 +215,14 @@ __device__ __forceinline__ unsigned long long plan_items(const Plan& P, unsigned
 __device__ __forceinline__ unsigned long long plan_count(const RelDev& R, int, uint32_t, uint32_t q) { return R.cnt[q]; }
 
 // a co-partition is swapped when its R side needs several C_R chunks while its S side fits one:
-// its items build on S and probe with C_R-sized R chunks (a duplicate-heavy build side would
+// its items build on S and probe with R chunks of 2^lgCRp <= C_R tuples (a duplicate-heavy build side would
 // otherwise walk chains of identical keys in single lanes)
 __device__ __forceinline__ bool plan_swapped(const Plan& P, unsigned long long cr, unsigned long long cs) {
   return P.ist2 != nullptr && cr > P.CR && cs && cs <= P.CR;
 }
 __device__ __forceinline__ unsigned long long plan_items_swapped(const Plan& P, unsigned long long cr) {
-  // probe chunks of C_R R tuples (k_join's claim_job<SWAP>)
-  if ((cr >> 31) == 0) return ((uint32_t)cr + P.CR - 1) / P.CR;  // 32-bit division (the common case)
-  return (cr + P.CR - 1) / P.CR;
+  // probe chunks of 2^lgCRp <= C_R R tuples (k_join's claim_job<SWAP>)
+  return (cr + (1ull << P.lgCRp) - 1) >> P.lgCRp;
 }
 
 // MS: several sources (exchange receiver); IT: join items (not on the exchange sender). Specialised so each launch runs (and fetches) only its own code.

@@ -85,6 +85,8 @@ struct Plan {
   int tuple_bytes;  // AoS tuple size (8 or 16): the planner zeroes each T2's 64-byte tail
   uint32_t C2;           // pass-2 chunk (tile) size in tuples
   uint32_t CR, CS;       // join item capacities: R tuples (smem build) and S tuples per item
+  uint32_t lgCRp;        // log2 of the largest power of two <= CR: swapped items probe R chunks of
+                         // 2^lgCRp tuples (a shift, not a division, in the planner's prefix loop)
   uint32_t* ist;         // [2^B + 1] join item prefix (q-order)
   uint32_t* ist2;        // [2^B + 1] prefix of the SWAPPED items (null: none): co-partitions whose R
                          // side needs more than one C_R chunk while S fits one (duplicate-heavy
